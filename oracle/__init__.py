@@ -1,0 +1,119 @@
+"""CPU oracle for the hybrid radix sort (arXiv 1611.01137) -- TEST INFRASTRUCTURE.
+
+Only tests/, __graft_entry__.smoke() and bench.py's cpu_baseline / --impl reference
+legs may import this package.  The product library (paper_1611_01137_b200) never
+imports it, and the two share no code: the only common module is gen/ (seeded
+input generators, none of the method's arithmetic).
+
+Contents
+  oracle.c (built to liboracle.so, loaded with ctypes):
+      histogram       -- digit histogram, P:293-296 / P:503-505
+      partition_pass  -- one stable counting-sort pass, P:293-301 / P:503-509
+      sort            -- LSD radix sort, 8-bit digits, P:304-311 (the definition of
+                         the unique stable sort by bits [begin, end))
+  plan.py (pure Python):
+      classify_bucket -- rules R1-R3 and tiny-bucket merging, P:552-561, P:805-811
+      simulate_msd    -- the MSD hybrid recursion step by step (Fig 1),
+                         giving the pass / bucket / local-sort structure
+
+Pinning (none of these re-run the oracle's own formula): tests/test_oracle.py
+checks the paper's worked example (Table 2, tests/golden/table2.txt),
+brute force against insertion sort on every short sequence over a 4-letter
+alphabet, numpy's stable argsort (a library routine), and the invariants
+non-decreasing / multiset equality / stability.
+"""
+from __future__ import annotations
+
+import ctypes
+import os
+import subprocess
+
+import numpy as np
+
+_HERE = os.path.dirname(os.path.abspath(__file__))
+_SRC = os.path.join(_HERE, "oracle.c")
+_LIB = os.path.join(_HERE, "liboracle.so")
+_lib = None
+
+
+def build(force: bool = False) -> str:
+    """Compile oracle.c with gcc (plain C, -O2, single thread)."""
+    if force or not os.path.exists(_LIB) or os.path.getmtime(_LIB) < os.path.getmtime(_SRC):
+        subprocess.check_call(["gcc", "-O2", "-std=c99", "-shared", "-fPIC", "-o", _LIB, _SRC])
+    return _LIB
+
+
+def _load():
+    global _lib
+    if _lib is None:
+        build()
+        lib = ctypes.CDLL(_LIB)
+        P = ctypes.c_void_p
+        U = ctypes.c_uint64
+        I = ctypes.c_int
+        lib.oracle_digit_histogram.argtypes = [P, U, I, I, P]
+        lib.oracle_partition_pass.argtypes = [P, P, U, I, I, P, P, P]
+        lib.oracle_lsd_sort.argtypes = [P, P, U, I, I, P, P]
+        for f in (lib.oracle_digit_histogram, lib.oracle_partition_pass, lib.oracle_lsd_sort):
+            f.restype = I
+        _lib = lib
+    return _lib
+
+
+def _u64(a) -> np.ndarray:
+    """Widen any unsigned integer array (numpy or torch CPU tensor) to contiguous uint64."""
+    if hasattr(a, "numpy"):  # torch tensor
+        a = a.cpu()
+        if str(a.dtype) == "torch.uint32":
+            a = a.view(dtype=__import__("torch").int32).numpy().view(np.uint32)
+        elif str(a.dtype) == "torch.uint64":
+            a = a.view(dtype=__import__("torch").int64).numpy().view(np.uint64)
+        else:
+            a = a.numpy()
+    a = np.asarray(a)
+    if a.dtype.kind not in "ui":
+        raise TypeError(a.dtype)
+    return np.ascontiguousarray(a.astype(np.uint64, copy=False))
+
+
+def _ptr(a: np.ndarray):
+    return a.ctypes.data_as(ctypes.c_void_p) if a is not None else None
+
+
+def histogram(keys, lo: int, hi: int) -> np.ndarray:
+    k = _u64(keys)
+    h = np.zeros(1 << (hi - lo), dtype=np.uint64)
+    rc = _load().oracle_digit_histogram(_ptr(k), k.size, lo, hi, _ptr(h))
+    if rc:
+        raise ValueError(f"oracle_digit_histogram rc={rc}")
+    return h
+
+
+def partition_pass(keys, vals, lo: int, hi: int):
+    """One stable counting pass on digit bits [lo, hi): (keys_out, vals_out, offsets[r+1])."""
+    k = _u64(keys)
+    v = _u64(vals) if vals is not None else None
+    ko = np.empty_like(k)
+    vo = np.empty_like(v) if v is not None else None
+    offs = np.zeros((1 << (hi - lo)) + 1, dtype=np.uint64)
+    rc = _load().oracle_partition_pass(_ptr(k), _ptr(v), k.size, lo, hi, _ptr(ko), _ptr(vo), _ptr(offs))
+    if rc:
+        raise ValueError(f"oracle_partition_pass rc={rc}")
+    return ko, vo, offs
+
+
+def sort(keys, vals=None, begin_bit: int = 0, end_bit: int | None = None, key_bits: int | None = None):
+    """The stable sort by bits [begin_bit, end_bit) -> (keys_out, vals_out) as uint64 arrays."""
+    k = _u64(keys)
+    if end_bit is None:
+        end_bit = key_bits if key_bits is not None else 64
+    v = _u64(vals) if vals is not None else None
+    ko = np.empty_like(k)
+    vo = np.empty_like(v) if v is not None else None
+    rc = _load().oracle_lsd_sort(_ptr(k), _ptr(v), k.size, begin_bit, end_bit, _ptr(ko), _ptr(vo))
+    if rc:
+        raise ValueError(f"oracle_lsd_sort rc={rc}")
+    return ko, vo
+
+
+from .plan import classify_bucket, simulate_msd, size_class  # noqa: E402,F401
