@@ -1,0 +1,356 @@
+#!/usr/bin/env python
+"""Benchmark of the stable hybrid MSD radix sort on B200 (one JSON line on rank 0).
+
+    python bench.py [--gpus N] [--steps K] [--warmup W] [--config c2] [--dist uniform]
+    python bench.py --impl reference ...      # the CPU oracle on a bounded sample
+
+Metric (BASELINE.json): sorted records/s and the fraction of the HBM roofline.  A
+"step" is one full sort (every counting pass, the classification and every local
+sort) of the configured synthetic workload, inputs resident in HBM.  Default config
+c2 = 2^28 uint32 keys + uint32 values, uniform (BASELINE.json configs[1]); the
+inputs (2 GiB + outputs + aux) are far larger than the 126 MB L2, so no flush is
+needed between steps.
+
+Multi-GPU (torchrun, N > 1): every rank sorts its own 2^28-record shard of a global
+N * 2^28 input through the distributed driver (first-digit histogram all-gather,
+bucket assignment, stable partition, NCCL all-to-all, local sort); value = N * 2^28
+records / max-over-ranks step time ("weak" scaling).
+"""
+from __future__ import annotations
+
+import argparse
+import json
+import os
+import statistics
+import subprocess
+import sys
+import threading
+import time
+
+ROOT = os.path.dirname(os.path.abspath(__file__))
+sys.path.insert(0, ROOT)
+
+CONFIGS = {
+    # name: (log2 n, key bits, value bits, description)
+    "c1": (20, 32, 0, "2^20 uniform uint32 keys, keys-only"),
+    "c2": (28, 32, 32, "2^28 uint32 key + uint32 value pairs"),
+    "c3": (28, 32, 32, "2^28 uint32 key + uint32 value pairs, AND-skewed"),
+    "c4": (28, 64, 64, "2^28 uint64 key + uint64 value pairs"),
+}
+METRIC = "sorted records/sec and % of B200 HBM roofline (1/2/4/8 GPU)"
+
+
+def _peaks():
+    try:
+        with open(os.path.join(ROOT, "MEASURED_PEAKS.json")) as f:
+            p = json.load(f)
+        return float(p["hbm_gbs"]), "measured"
+    except Exception:
+        return 6650.0, "fallback"
+
+
+class ClockSampler:
+    """nvidia-smi clocks and throttle reasons sampled during the timed region."""
+
+    FIELDS = ("clocks.sm,clocks.max.sm,clocks_event_reasons.hw_slowdown,"
+              "clocks_event_reasons.hw_thermal_slowdown,clocks_event_reasons.sw_thermal_slowdown,"
+              "clocks_event_reasons.sw_power_cap")
+
+    def __init__(self, index: int):
+        self.index = index
+        self.samples = []
+        self.proc = None
+        self.thread = None
+
+    def start(self):
+        try:
+            self.proc = subprocess.Popen(
+                ["nvidia-smi", "-i", str(self.index), f"--query-gpu={self.FIELDS}", "--format=csv,noheader,nounits",
+                 "-lms", "100"], stdout=subprocess.PIPE, stderr=subprocess.DEVNULL, text=True)
+        except Exception:
+            self.proc = None
+            return
+        self.thread = threading.Thread(target=self._read, daemon=True)
+        self.thread.start()
+
+    def _read(self):
+        for line in self.proc.stdout:
+            parts = [x.strip() for x in line.split(",")]
+            if len(parts) == 6:
+                self.samples.append(parts)
+
+    def stop(self) -> dict:
+        if self.proc is None:
+            return {"sm_mhz": None, "sm_max_mhz": None, "reasons": ["nvidia-smi unavailable"]}
+        time.sleep(0.25)
+        self.proc.terminate()
+        try:
+            self.proc.wait(timeout=2)
+        except Exception:
+            self.proc.kill()
+        sm = [float(s[0]) for s in self.samples if s[0].replace(".", "").isdigit()]
+        mx = [float(s[1]) for s in self.samples if s[1].replace(".", "").isdigit()]
+        names = ["hw_slowdown", "hw_thermal_slowdown", "sw_thermal_slowdown", "sw_power_cap"]
+        reasons = sorted({names[i] for s in self.samples for i in range(4) if s[2 + i].lower() == "active"})
+        return {"sm_mhz": statistics.median(sm) if sm else None, "sm_max_mhz": max(mx) if mx else None,
+                "reasons": reasons, "samples": len(self.samples)}
+
+
+def _env_rank():
+    return int(os.environ.get("RANK", "0")), int(os.environ.get("WORLD_SIZE", "1")), \
+        int(os.environ.get("LOCAL_RANK", "0"))
+
+
+# ---------------------------------------------------------------------------- reference arm
+
+def run_reference(args):
+    """The CPU oracle (oracle/oracle.c, single-threaded LSD) as it stands, one bounded
+    sample of the configured workload per step."""
+    rank, world, _ = _env_rank()
+    if rank != 0:
+        return 0
+    import numpy as np
+    import gen
+    import oracle
+    logn, kbits, vbits, desc = CONFIGS[args.config]
+    n = min(1 << logn, 1 << args.ref_log2)
+    k = oracle._u64(gen.keys(n, kbits, args.dist))
+    v = np.arange(n, dtype=np.uint64) if vbits else None
+    for _ in range(args.warmup):
+        oracle.sort(k, v, 0, kbits)
+    times = []
+    for _ in range(args.steps):
+        t0 = time.perf_counter()
+        oracle.sort(k, v, 0, kbits)
+        times.append(time.perf_counter() - t0)
+    t = sum(times) / len(times)
+    value = n / t
+    unit = "records/s"
+    sample = f"{n} records ({args.dist}) of the {desc} workload per step, single-threaded LSD oracle"
+    line = {
+        "impl": "reference", "metric": METRIC, "value": value, "unit": unit, "n_gpus": world,
+        "steps": args.steps, "warmup": args.warmup, "ms_per_step": t * 1e3, "higher_is_better": True,
+        "scaling": "weak", "vs_baseline": None, "dtype": "u32" if kbits == 32 else "u64", "data": "synthetic",
+        "config": {"workload": f"{args.config}:{desc}, {args.dist}", "n": n, "key_bits": kbits,
+                   "value_bits": vbits, "parallelism": f"cpu1"},
+        "cpu_baseline": {"value": value, "unit": unit, "cores": 1, "kind": "oracle", "sample": sample},
+        "e2e": {"value": value, "unit": unit, "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0},
+    }
+    print(json.dumps(line), flush=True)
+    return 0
+
+
+# ---------------------------------------------------------------------------- product arm
+
+def _events(torch, k):
+    return [torch.cuda.Event(enable_timing=True) for _ in range(k)]
+
+
+def run_hrs(args):
+    import torch
+
+    import gen
+    import paper_1611_01137_b200 as hrs
+
+    rank, world, local_rank = _env_rank()
+    torch.cuda.set_device(local_rank)
+    dev = torch.device("cuda", local_rank)
+    logn, kbits, vbits, desc = CONFIGS[args.config]
+    dist_name = args.dist
+    if args.config == "c3" and dist_name == "uniform":
+        dist_name = "and3"
+    n = 1 << logn
+    kb, vb = kbits // 8, vbits // 8
+    pg = None
+    if world > 1:
+        import torch.distributed as dist
+        dist.init_process_group("nccl", device_id=dev)
+        pg = dist.group.WORLD
+
+    seed = gen.SEEDS[0]
+    keys = gen.keys(n, kbits, dist_name, seed=seed, start=rank * n, device=dev)
+    vals = gen.values(n, vbits, "index", start=rank * n, device=dev) if vbits else None
+    stream = torch.cuda.current_stream()
+
+    if world > 1:
+        from paper_1611_01137_b200 import dist as hdist
+        sorter = hdist.DistributedSorter(keys, vals, group=pg)
+        step = sorter.step
+    else:
+        keys_out = torch.empty_like(keys)
+        vals_out = torch.empty_like(vals) if vals is not None else None
+        temp = torch.empty(hrs.temp_bytes(n, kb, vb), dtype=torch.uint8, device=dev)
+
+        def step():
+            hrs.sort(keys, vals, keys_out=keys_out, values_out=vals_out, temp=temp)
+
+    for _ in range(args.warmup):
+        step()
+    torch.cuda.synchronize()
+
+    # ---------------- timed region: K steps, barrier + synchronize on both sides
+    sampler = ClockSampler(local_rank)
+    sampler.start()
+    time.sleep(0.3)
+    if pg is not None:
+        torch.distributed.barrier()
+    torch.cuda.synchronize()
+    l0 = hrs.launch_count()
+    ev = _events(torch, args.steps + 1)
+    ev[0].record(stream)
+    for i in range(args.steps):
+        step()
+        ev[i + 1].record(stream)
+    torch.cuda.synchronize()
+    launches = hrs.launch_count() - l0
+    if pg is not None:
+        torch.distributed.barrier()
+    clocks = sampler.stop()
+    step_ms = [ev[i].elapsed_time(ev[i + 1]) for i in range(args.steps)]
+    t_ms = sum(step_ms) / len(step_ms)
+    if pg is not None:
+        tt = torch.tensor([t_ms], dtype=torch.float64, device=dev)
+        torch.distributed.all_reduce(tt, op=torch.distributed.ReduceOp.MAX)
+        t_ms = float(tt.item())
+    total = n * world
+    value = total / (t_ms * 1e-3)
+
+    peak, peak_kind = _peaks()
+    out = {"metric": METRIC, "value": value, "unit": "records/s", "n_gpus": world, "steps": args.steps,
+           "warmup": args.warmup, "ms_per_step": t_ms, "higher_is_better": True, "scaling": "weak",
+           "vs_baseline": None, "dtype": "u32" if kbits == 32 else "u64", "data": "synthetic",
+           "config": {"workload": f"{args.config}:{desc}, {dist_name}", "n_per_gpu": n, "key_bits": kbits,
+                      "value_bits": vbits, "bits": [0, kbits], "values": "input index",
+                      "parallelism": f"dp{world}" if world > 1 else "single",
+                      "l2": "inputs (>= 2 GiB) larger than the 126 MB L2; no flush"},
+           "gpu_launches": launches, "clocks": clocks,
+           "step_ms": {"median": statistics.median(step_ms), "min": min(step_ms), "max": max(step_ms)}}
+
+    if world == 1:
+        st = hrs.get_stats(temp)
+        bmin = st["bytes_min"]
+        out["sort_roofline"] = {
+            "bytes_min": bmin, "bytes_per_record": bmin / n, "peak_gbs": peak, "peak": peak_kind,
+            "achieved_gbs": bmin / (t_ms * 1e-3) / 1e9, "frac": bmin / (t_ms * 1e-3) / (peak * 1e9),
+            "frac_of_8tbs": bmin / (t_ms * 1e-3) / 8.0e12, "sort_rate_GBps": n * (kb + vb) / (t_ms * 1e-3) / 1e9,
+            "counting_passes": st["counting_passes"], "recs_in_pass": st["recs_in_pass"],
+            "local_recs": st["local_recs"], "local_buckets": st["local_buckets"],
+            "merged_groups": st["merged_groups"]}
+        # ---------------- per-kernel breakdown: the same K steps again, each launch bracketed by events
+        hrs.profile_enable(True)
+        for _ in range(args.steps):
+            step()
+        recs = hrs.profile_collect()
+        hrs.profile_enable(False)
+        per = {}
+        for kind, p, ms in recs:
+            key = f"{kind}{p}" if kind in ("hist", "scatter", "local") else kind
+            per.setdefault(key, []).append(ms)
+        kern = {k2: sum(v2) / args.steps for k2, v2 in per.items()}
+        out["kernels_ms_per_step"] = {k2: round(v2, 4) for k2, v2 in sorted(kern.items())}
+        # dominant kernel: the scatter (2(K+V) bytes per record of every counting pass)
+        sc_bytes = sum(r * 2 * (kb + vb) for r in st["recs_in_pass"])
+        sc_ms = sum(v2 for k2, v2 in kern.items() if k2.startswith("scatter"))
+        traffic = None
+        tpath = os.path.join(ROOT, "profiles", "traffic.json")
+        if os.path.exists(tpath):
+            try:
+                tj = json.load(open(tpath))
+                traffic = tj.get(f"{args.config}:{dist_name}", {}).get("scatter_dram_bytes_per_step")
+            except Exception:
+                traffic = None
+        if sc_ms > 0:
+            ach = sc_bytes / (sc_ms * 1e-3) / 1e9
+            out["roofline"] = {"bound": "hbm", "kernel": "k_scatter (all counting passes)", "achieved": ach,
+                               "peak": peak, "unit": "GB/s", "frac": ach / peak, "traffic": traffic,
+                               "algorithmic_bytes": sc_bytes, "share_of_step": sc_ms / sum(kern.values()),
+                               "peak_source": peak_kind}
+        # ---------------- end to end through the public API with host buffers
+        if not args.no_e2e:
+            out["e2e"] = run_e2e(torch, hrs, keys, vals, temp, args, n, kb, vb)
+        # ---------------- CPU baseline: the oracle as it stands on a bounded sample
+        if not args.no_cpu:
+            out["cpu_baseline"] = cpu_baseline(args, kbits, vbits, dist_name)
+    if rank == 0:
+        print(json.dumps(out), flush=True)
+    if pg is not None:
+        torch.distributed.destroy_process_group()
+    return 0
+
+
+def run_e2e(torch, hrs, keys, vals, temp, args, n, kb, vb):
+    hk = torch.empty(keys.shape, dtype=keys.dtype, pin_memory=True)
+    hk.copy_(keys)
+    hv = None
+    if vals is not None:
+        hv = torch.empty(vals.shape, dtype=vals.dtype, pin_memory=True)
+        hv.copy_(vals)
+    hko = torch.empty_like(hk, pin_memory=True)
+    hvo = torch.empty_like(hv, pin_memory=True) if hv is not None else None
+    dk, dko = torch.empty_like(keys), torch.empty_like(keys)
+    dv = torch.empty_like(vals) if vals is not None else None
+    dvo = torch.empty_like(vals) if vals is not None else None
+    stream = torch.cuda.current_stream()
+
+    def step():
+        dk.copy_(hk, non_blocking=True)
+        if hv is not None:
+            dv.copy_(hv, non_blocking=True)
+        hrs.sort(dk, dv, keys_out=dko, values_out=dvo, temp=temp)
+        hko.copy_(dko, non_blocking=True)
+        if hvo is not None:
+            hvo.copy_(dvo, non_blocking=True)
+
+    for _ in range(2):
+        step()
+    torch.cuda.synchronize()
+    k = max(2, min(args.steps, 5))
+    ev = _events(torch, 2)
+    ev[0].record(stream)
+    for _ in range(k):
+        step()
+    ev[1].record(stream)
+    torch.cuda.synchronize()
+    t = ev[0].elapsed_time(ev[1]) / k
+    nb = n * (kb + vb)
+    return {"value": n / (t * 1e-3), "unit": "records/s", "ms_per_step": t, "h2d_bytes_per_step": nb,
+            "d2h_bytes_per_step": nb, "steps": k, "path": "pinned host -> H2D -> hrs.sort (C ABI) -> D2H"}
+
+
+def cpu_baseline(args, kbits, vbits, dist_name):
+    import numpy as np
+    import gen
+    import oracle
+    n = 1 << args.cpu_log2
+    k = oracle._u64(gen.keys(n, kbits, dist_name))
+    v = np.arange(n, dtype=np.uint64) if vbits else None
+    t0 = time.perf_counter()
+    oracle.sort(k, v, 0, kbits)
+    t = time.perf_counter() - t0
+    return {"value": n / t, "unit": "records/s", "cores": 1, "kind": "oracle",
+            "sample": f"{n} records of the same workload ({dist_name}), single-threaded LSD oracle "
+                      f"(oracle/oracle.c), {t:.2f} s"}
+
+
+def main(argv=None):
+    ap = argparse.ArgumentParser()
+    ap.add_argument("--gpus", type=int, default=1)
+    ap.add_argument("--steps", type=int, default=10)
+    ap.add_argument("--warmup", type=int, default=3)
+    ap.add_argument("--impl", default="hrs", choices=["hrs", "reference"])
+    ap.add_argument("--config", default="c2", choices=sorted(CONFIGS))
+    ap.add_argument("--dist", default="uniform", choices=["uniform", "and2", "and3", "and4", "const"])
+    ap.add_argument("--no-e2e", action="store_true")
+    ap.add_argument("--no-cpu", action="store_true")
+    ap.add_argument("--cpu-log2", type=int, default=26)
+    ap.add_argument("--ref-log2", type=int, default=24)
+    args = ap.parse_args(argv)
+    if args.warmup < 3:
+        args.warmup = 3
+    if args.impl == "reference":
+        return run_reference(args)
+    return run_hrs(args)
+
+
+if __name__ == "__main__":
+    sys.exit(main())

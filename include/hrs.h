@@ -1,0 +1,183 @@
+/*
+ * hrs.h -- C ABI of the B200-native (sm_100a) hybrid radix sort.
+ *
+ * Method: Stehle & Jacobsen, "A Memory Bandwidth-Efficient Hybrid Radix Sort on
+ * GPUs", SIGMOD'17 (arXiv 1611.01137).  PAPER.md line citations are P:<line>.
+ *   - MSD radix sort with 8-bit digits (d = 8): every bucket larger than
+ *     the local-sort threshold ∂ˆ is partitioned by a counting sort -- histogram,
+ *     exclusive prefix sum into sub-bucket offsets, scatter -- and
+ *     every bucket of at most ∂ˆ records is finished by an on-chip local sort
+ *     (R1/R2 P:805-808).  Tiny neighbouring sub-buckets are merged while
+ *     their total is below ∂ (R3 P:809-811).
+ *   - Departure from the paper: every pass is STABLE, so
+ *     the output is the unique stable sort and is bit-identical run to run.
+ *
+ * Semantics of every hrs_sort_* call:
+ *   With W = end_bit - begin_bit and sk(x) = (x >> begin_bit) mod 2^W, the output
+ *   is keys_in[pi(i)] (and vals_in[pi(i)]) for the unique permutation pi such that
+ *   (sk(keys_in[pi(i)]), pi(i)) is strictly increasing: ties keep input order.
+ *   Key bits outside [begin_bit, end_bit) are carried unchanged.  n == 0 is a no-op;
+ *   begin_bit == end_bit is a stable copy.
+ *
+ * Conventions
+ *   Memory:    every data pointer (keys, values, temp, d_hist, d_offsets) is a CUDA
+ *              device pointer owned by the caller, naturally aligned for its type
+ *              (temp: 256 bytes).  The library never allocates, frees or retains
+ *              device memory.  Inputs are const; keys_in/keys_out/vals_in/vals_out/
+ *              temp must not overlap (HRS_ERROR_ALIASING).
+ *   Temp:      two-phase protocol: with d_temp == NULL the call stores the required
+ *              size in *temp_bytes, enqueues nothing and returns HRS_SUCCESS.
+ *              Otherwise *temp_bytes is the size of d_temp.
+ *   Streams:   work is enqueued on `stream` (NULL = legacy default stream) and the
+ *              call returns without synchronising (no device->host reads inside the
+ *              sort, so calls can be captured in CUDA graphs).  hrs_get_stats is the
+ *              only entry point that synchronises its stream.
+ *   Errors:    argument errors are returned synchronously; a CUDA launch error maps
+ *              to HRS_ERROR_CUDA with the cudaError_t in hrs_last_cuda_error()
+ *              (thread-local).  Device faults surface at the caller's next sync.
+ *              No C++ exception crosses this ABI.
+ *   Devices:   the library contains sm_100a code only; on any other device the
+ *              calls fail with HRS_ERROR_NO_DEVICE.  There is no CPU fallback.
+ *   Threads:   stateless apart from the thread-local last error and per-device
+ *              launch-configuration caches; concurrent calls on different streams
+ *              with different temp buffers are safe.
+ *   Limits:    n <= HRS_MAX_ITEMS.
+ */
+#ifndef HRS_H_
+#define HRS_H_
+
+#include <stddef.h>
+#include <stdint.h>
+
+#ifdef __cplusplus
+extern "C" {
+#endif
+#if defined(__GNUC__)
+#pragma GCC visibility push(default) /* the library is built with -fvisibility=hidden */
+#endif
+
+#define HRS_MAX_ITEMS 0xFFFFFFFFull /* counts are 32-bit inside the kernels ("easily adjusted") */
+
+typedef struct CUstream_st *hrs_stream_t; /* identical to cudaStream_t */
+
+typedef enum {
+    HRS_SUCCESS = 0,
+    HRS_ERROR_INVALID_VALUE = 1,  /* NULL pointer with n > 0, NULL temp_bytes, misaligned pointer, bad tuning */
+    HRS_ERROR_INVALID_BITS = 2,   /* not 0 <= begin_bit <= end_bit <= key bits (digit range for building blocks) */
+    HRS_ERROR_ALIASING = 3,       /* any overlap among the data buffers and temp */
+    HRS_ERROR_TEMP_TOO_SMALL = 4, /* *temp_bytes smaller than required */
+    HRS_ERROR_TOO_LARGE = 5,      /* n > HRS_MAX_ITEMS */
+    HRS_ERROR_NO_DEVICE = 6,      /* current device is not an sm_100 GPU */
+    HRS_ERROR_CUDA = 7            /* a CUDA call failed; see hrs_last_cuda_error() */
+} hrs_status;
+
+/* Tuning override (tests and ablations).  0 in a field = the default for the
+ * key/value types.  Thresholds change performance, never results.
+ *   local_threshold  ∂ˆ  buckets with <= ∂ˆ records are local-sorted (1 .. hrs_max_local_threshold)
+ *   merge_threshold  ∂   neighbouring sub-buckets merge while their total < ∂ (1 .. ∂ˆ; 1 = no merging)
+ *   keys_per_tile    KPB records per tile ("key block") (1 .. hrs_max_keys_per_tile)
+ *   local_classes    0 = size classes [1,128], (128,256], ...; 1 = a single
+ *                    local-sort configuration for every bucket (the ablation of Figs 11-14) */
+typedef struct {
+    uint32_t local_threshold;
+    uint32_t merge_threshold;
+    uint32_t keys_per_tile;
+    uint32_t local_classes;
+} hrs_tuning;
+
+#define HRS_MAX_PASSES 8
+#define HRS_NUM_CLASSES 8
+
+/* Observability block kept inside temp and filled on the device during a sort. */
+typedef struct {
+    uint64_t n;
+    uint32_t key_bytes, value_bytes;
+    uint32_t counting_passes;                  /* counting-sort passes executed */
+    uint32_t overflow;                         /* non-zero: an internal table bound was exceeded (bug) */
+    uint64_t recs_in_pass[HRS_MAX_PASSES];     /* records in buckets partitioned by pass p+1 */
+    uint64_t tiles_in_pass[HRS_MAX_PASSES];    /* tiles (key blocks) of pass p+1 */
+    uint64_t buckets_in_pass[HRS_MAX_PASSES];  /* buckets partitioned by pass p+1 */
+    uint64_t local_buckets;                    /* local-sort entries (after merging) */
+    uint64_t local_recs;                       /* records finished by a local sort */
+    uint64_t merged_groups;                    /* local entries made of >= 2 merged sub-buckets */
+    uint64_t local_in_class[HRS_NUM_CLASSES];  /* local entries per size class */
+    uint64_t bytes_min;                        /* sum_p R_p (K + 2(K+V)) + R_L 2(K+V) */
+} hrs_stats;
+
+/* ---- full sorts; arguments: temp, size, keys in/out, [values in/out], n, bit range, stream ---- */
+hrs_status hrs_sort_keys_u32(void *d_temp, size_t *temp_bytes, const uint32_t *keys_in, uint32_t *keys_out,
+                             uint64_t n, int begin_bit, int end_bit, hrs_stream_t stream);
+hrs_status hrs_sort_keys_u64(void *d_temp, size_t *temp_bytes, const uint64_t *keys_in, uint64_t *keys_out,
+                             uint64_t n, int begin_bit, int end_bit, hrs_stream_t stream);
+hrs_status hrs_sort_pairs_u32_u32(void *d_temp, size_t *temp_bytes, const uint32_t *keys_in, uint32_t *keys_out,
+                                  const uint32_t *vals_in, uint32_t *vals_out, uint64_t n, int begin_bit,
+                                  int end_bit, hrs_stream_t stream);
+hrs_status hrs_sort_pairs_u32_u64(void *d_temp, size_t *temp_bytes, const uint32_t *keys_in, uint32_t *keys_out,
+                                  const uint64_t *vals_in, uint64_t *vals_out, uint64_t n, int begin_bit,
+                                  int end_bit, hrs_stream_t stream);
+hrs_status hrs_sort_pairs_u64_u32(void *d_temp, size_t *temp_bytes, const uint64_t *keys_in, uint64_t *keys_out,
+                                  const uint32_t *vals_in, uint32_t *vals_out, uint64_t n, int begin_bit,
+                                  int end_bit, hrs_stream_t stream);
+hrs_status hrs_sort_pairs_u64_u64(void *d_temp, size_t *temp_bytes, const uint64_t *keys_in, uint64_t *keys_out,
+                                  const uint64_t *vals_in, uint64_t *vals_out, uint64_t n, int begin_bit,
+                                  int end_bit, hrs_stream_t stream);
+
+/* Generic form behind the typed entry points.  key_bytes in {4, 8}; value_bytes in
+ * {0, 4, 8} (0: vals_in/vals_out ignored, may be NULL); tuning may be NULL. */
+hrs_status hrs_sort_ex(void *d_temp, size_t *temp_bytes, const void *keys_in, void *keys_out,
+                       const void *vals_in, void *vals_out, uint64_t n, int key_bytes, int value_bytes,
+                       int begin_bit, int end_bit, const hrs_tuning *tuning, hrs_stream_t stream);
+
+/* Copies the stats block of the last sort that used d_temp to *out.  Synchronises
+ * `stream`; call it outside any timed region. */
+hrs_status hrs_get_stats(const void *d_temp, hrs_stats *out, hrs_stream_t stream);
+
+/* Largest accepted local_threshold / keys_per_tile for the key/value widths. */
+uint32_t hrs_max_local_threshold(int key_bytes, int value_bytes);
+uint32_t hrs_max_keys_per_tile(int key_bytes, int value_bytes);
+/* Default tuning for the key/value widths (written to *out). */
+hrs_status hrs_default_tuning(int key_bytes, int value_bytes, hrs_tuning *out);
+
+/* ---- building blocks (kernel-level tests, the distributed driver) ---- */
+
+/* Histogram of digit bits [lo_bit, hi_bit) (1 <= hi_bit - lo_bit <= 8) over all n keys:
+ * step (1) of a counting sort.  d_hist receives 2^(hi-lo) uint64 counts. */
+hrs_status hrs_digit_histogram(void *d_temp, size_t *temp_bytes, const void *keys, uint64_t n, int key_bytes,
+                               int lo_bit, int hi_bit, uint64_t *d_hist, hrs_stream_t stream);
+
+/* One STABLE counting-sort pass of the whole input on digit bits [lo_bit, hi_bit):
+ * histogram, exclusive prefix sum, scatter.  d_offsets receives the
+ * 2^(hi-lo) + 1 uint64 bucket starts (the last entry is n).  d_offsets may be NULL. */
+hrs_status hrs_partition_pass(void *d_temp, size_t *temp_bytes, const void *keys_in, void *keys_out,
+                              const void *vals_in, void *vals_out, uint64_t n, int key_bytes, int value_bytes,
+                              int lo_bit, int hi_bit, uint64_t *d_offsets, hrs_stream_t stream);
+
+/* ---- observability ---- */
+
+/* Per-launch device timing for benchmarks (thread-local, off by default).  While
+ * enabled, every kernel this thread enqueues is bracketed by CUDA events recorded
+ * on the launch stream.  hrs_profile_collect synchronises on those events, writes
+ * up to `max` records in launch order, returns how many it wrote, and clears the
+ * list.  kind: 0 init, 1 histogram/look-back/classify (k_hist), 2 scatter
+ * (k_scatter), 3 local sort (pass = size class), 4 copy/fill. */
+typedef struct {
+    int kind;
+    int pass;
+    float ms;
+} hrs_profile_record;
+void hrs_profile_enable(int on);
+int hrs_profile_collect(hrs_profile_record *out, int max);
+/* Number of kernel launches this thread has enqueued through the library. */
+uint64_t hrs_launch_count(void);
+
+const char *hrs_status_string(hrs_status status);
+int hrs_last_cuda_error(void);
+int hrs_version(void);
+
+#if defined(__GNUC__)
+#pragma GCC visibility pop
+#endif
+#ifdef __cplusplus
+}
+#endif
+#endif /* HRS_H_ */

@@ -1,0 +1,195 @@
+"""B200-native (sm_100a) stable hybrid MSD radix sort -- Python binding.
+
+Implements the hot path of Stehle & Jacobsen, "A Memory Bandwidth-Efficient Hybrid
+Radix Sort on GPUs" (arXiv 1611.01137): MSD counting-sort passes on 8-bit digits
+(histogram -> exclusive prefix sum -> shared-memory staged scatter), recursion on
+buckets above the local-sort threshold, tiny-bucket merging and an on-chip local
+sort.  Every step runs in the CUDA kernels of libhrs.so (include/hrs.h); this
+module only allocates with torch and marshals arguments through ctypes.
+"""
+from __future__ import annotations
+
+import ctypes
+
+import torch
+
+from ._lib import HRS_MAX_ITEMS, HrsError, Stats, Tuning, check, lib  # noqa: F401
+
+__all__ = ["sort", "temp_bytes", "get_stats", "digit_histogram", "partition_pass", "HrsError", "Tuning",
+           "default_tuning", "max_local_threshold", "max_keys_per_tile", "lib"]
+
+_KEY_DTYPES = {torch.uint32: 4, torch.uint64: 8}
+
+
+def _nbytes(t: torch.Tensor | None, what: str) -> int:
+    if t is None:
+        return 0
+    if t.dtype not in _KEY_DTYPES:
+        raise TypeError(f"{what} must be torch.uint32 or torch.uint64, got {t.dtype}")
+    return _KEY_DTYPES[t.dtype]
+
+
+def _check_tensor(t: torch.Tensor, what: str) -> None:
+    if not t.is_cuda:
+        raise ValueError(f"{what} must be a CUDA tensor (there is no CPU path)")
+    if not t.is_contiguous():
+        raise ValueError(f"{what} must be contiguous")
+    if t.dim() != 1:
+        raise ValueError(f"{what} must be 1-D")
+
+
+def _ptr(t: torch.Tensor | None):
+    return ctypes.c_void_p(t.data_ptr()) if t is not None and t.numel() > 0 else ctypes.c_void_p(0)
+
+
+def _stream(stream) -> ctypes.c_void_p:
+    if stream is None:
+        stream = torch.cuda.current_stream()
+    return ctypes.c_void_p(stream.cuda_stream if hasattr(stream, "cuda_stream") else int(stream))
+
+
+def _tuning(tuning) -> ctypes.POINTER(Tuning) | None:
+    if tuning is None:
+        return None
+    if isinstance(tuning, dict):
+        tuning = Tuning(**tuning)
+    return ctypes.pointer(tuning)
+
+
+def temp_bytes(n: int, key_bytes: int, value_bytes: int = 0, begin_bit: int = 0, end_bit: int | None = None,
+               tuning=None) -> int:
+    """Required temp size for a sort (the library's two-phase temp protocol)."""
+    if end_bit is None:
+        end_bit = 8 * key_bytes
+    sz = ctypes.c_size_t(0)
+    check(lib.hrs_sort_ex(None, ctypes.byref(sz), None, None, None, None, n, key_bytes, value_bytes, begin_bit,
+                          end_bit, _tuning(tuning), None), "hrs_sort_ex(size query)")
+    return sz.value
+
+
+def alloc_temp(nbytes: int, device) -> torch.Tensor:
+    return torch.empty(max(nbytes, 256), dtype=torch.uint8, device=device)
+
+
+def sort(keys: torch.Tensor, values: torch.Tensor | None = None, begin_bit: int = 0, end_bit: int | None = None,
+         *, tuning=None, keys_out: torch.Tensor | None = None, values_out: torch.Tensor | None = None,
+         temp: torch.Tensor | None = None, stream=None):
+    """Stable sort of `keys` (and `values`) by key bits [begin_bit, end_bit).
+
+    Returns (keys_out, values_out); values_out is None for keys-only sorts.
+    Enqueued on `stream` (default: torch's current stream); nothing synchronises.
+    """
+    _check_tensor(keys, "keys")
+    kb = _nbytes(keys, "keys")
+    vb = 0
+    if values is not None:
+        _check_tensor(values, "values")
+        vb = _nbytes(values, "values")
+        if values.numel() != keys.numel():
+            raise ValueError("keys and values differ in length")
+        if values.device != keys.device:
+            raise ValueError("keys and values are on different devices")
+    n = keys.numel()
+    if end_bit is None:
+        end_bit = 8 * kb
+    if keys_out is None:
+        keys_out = torch.empty_like(keys)
+    if values is not None and values_out is None:
+        values_out = torch.empty_like(values)
+    tb = temp_bytes(n, kb, vb, begin_bit, end_bit, tuning)
+    if temp is None or temp.numel() < tb:
+        temp = alloc_temp(tb, keys.device)
+    sz = ctypes.c_size_t(temp.numel())
+    with torch.cuda.device(keys.device):
+        check(lib.hrs_sort_ex(_ptr(temp), ctypes.byref(sz), _ptr(keys), _ptr(keys_out), _ptr(values),
+                              _ptr(values_out), n, kb, vb, begin_bit, end_bit, _tuning(tuning), _stream(stream)),
+              "hrs_sort_ex")
+    return keys_out, (values_out if values is not None else None)
+
+
+def get_stats(temp: torch.Tensor, stream=None) -> dict:
+    """Statistics of the last sort that used `temp` (synchronises the stream)."""
+    st = Stats()
+    with torch.cuda.device(temp.device):
+        check(lib.hrs_get_stats(_ptr(temp), ctypes.byref(st), _stream(stream)), "hrs_get_stats")
+    return st.to_dict()
+
+
+def digit_histogram(keys: torch.Tensor, lo_bit: int, hi_bit: int, *, temp: torch.Tensor | None = None,
+                    stream=None) -> torch.Tensor:
+    """2^(hi-lo) uint64 counts of digit bits [lo_bit, hi_bit) (device tensor)."""
+    _check_tensor(keys, "keys")
+    kb = _nbytes(keys, "keys")
+    n = keys.numel()
+    sz = ctypes.c_size_t(0)
+    check(lib.hrs_digit_histogram(None, ctypes.byref(sz), None, n, kb, lo_bit, hi_bit, None, None),
+          "hrs_digit_histogram(size query)")
+    if temp is None or temp.numel() < sz.value:
+        temp = alloc_temp(sz.value, keys.device)
+    hist = torch.empty(1 << (hi_bit - lo_bit), dtype=torch.uint64, device=keys.device)
+    sz = ctypes.c_size_t(temp.numel())
+    with torch.cuda.device(keys.device):
+        check(lib.hrs_digit_histogram(_ptr(temp), ctypes.byref(sz), _ptr(keys), n, kb, lo_bit, hi_bit, _ptr(hist),
+                                      _stream(stream)), "hrs_digit_histogram")
+    return hist
+
+
+def partition_pass(keys: torch.Tensor, values: torch.Tensor | None, lo_bit: int, hi_bit: int, *,
+                   keys_out: torch.Tensor | None = None, values_out: torch.Tensor | None = None,
+                   temp: torch.Tensor | None = None, stream=None):
+    """One stable counting pass on digit bits [lo_bit, hi_bit): (keys_out, values_out, offsets[r+1])."""
+    _check_tensor(keys, "keys")
+    kb = _nbytes(keys, "keys")
+    vb = 0
+    if values is not None:
+        _check_tensor(values, "values")
+        vb = _nbytes(values, "values")
+    n = keys.numel()
+    sz = ctypes.c_size_t(0)
+    check(lib.hrs_partition_pass(None, ctypes.byref(sz), None, None, None, None, n, kb, vb, lo_bit, hi_bit, None,
+                                 None), "hrs_partition_pass(size query)")
+    if temp is None or temp.numel() < sz.value:
+        temp = alloc_temp(sz.value, keys.device)
+    if keys_out is None:
+        keys_out = torch.empty_like(keys)
+    if values is not None and values_out is None:
+        values_out = torch.empty_like(values)
+    offs = torch.empty((1 << (hi_bit - lo_bit)) + 1, dtype=torch.uint64, device=keys.device)
+    sz = ctypes.c_size_t(temp.numel())
+    with torch.cuda.device(keys.device):
+        check(lib.hrs_partition_pass(_ptr(temp), ctypes.byref(sz), _ptr(keys), _ptr(keys_out), _ptr(values),
+                                     _ptr(values_out), n, kb, vb, lo_bit, hi_bit, _ptr(offs), _stream(stream)),
+              "hrs_partition_pass")
+    return keys_out, (values_out if values is not None else None), offs
+
+
+def default_tuning(key_bytes: int, value_bytes: int) -> dict:
+    t = Tuning()
+    check(lib.hrs_default_tuning(key_bytes, value_bytes, ctypes.byref(t)), "hrs_default_tuning")
+    return {f: getattr(t, f) for f, _ in Tuning._fields_}
+
+
+def max_local_threshold(key_bytes: int, value_bytes: int) -> int:
+    return lib.hrs_max_local_threshold(key_bytes, value_bytes)
+
+
+def max_keys_per_tile(key_bytes: int, value_bytes: int) -> int:
+    return lib.hrs_max_keys_per_tile(key_bytes, value_bytes)
+
+
+def profile_enable(on: bool = True) -> None:
+    """Per-launch CUDA-event timing of this thread's library launches (see hrs.h)."""
+    lib.hrs_profile_enable(1 if on else 0)
+
+
+def profile_collect(max_records: int = 1 << 16) -> list:
+    """[(kind, pass, ms)] of the launches since profile_enable; clears the list."""
+    from ._lib import PROFILE_KINDS, ProfileRecord
+    buf = (ProfileRecord * max_records)()
+    k = lib.hrs_profile_collect(buf, max_records)
+    return [(PROFILE_KINDS.get(r.kind, str(r.kind)), r.pass_, r.ms) for r in buf[:k]]
+
+
+def launch_count() -> int:
+    """Kernel launches this thread has enqueued through the library."""
+    return lib.hrs_launch_count()

@@ -1,0 +1,771 @@
+// hrs.cu -- host planner, launch dispatch and C ABI of the hybrid radix sort.
+//
+// See include/hrs.h for the contract and hrs_device.cuh for the kernels.  The
+// host side only validates arguments, computes the digit plan and the temp
+// layout from the analytical bounds of P:815-874 (I1-I4, M1-M5), and enqueues a
+// constant number of launches per pass.  It never reads device memory
+// during a sort.
+#include <cuda_runtime.h>
+
+#include <algorithm>
+#include <cstdint>
+#include <cstring>
+#include <mutex>
+#include <type_traits>
+#include <unordered_map>
+#include <vector>
+
+#include "hrs_device.cuh"
+
+using namespace hrs;
+
+namespace {
+
+thread_local int g_last_cuda = 0;
+thread_local uint64_t g_launches = 0;
+
+// ------------------------------------------------------------------ per-launch profiling (opt-in)
+struct ProfRec {
+    cudaEvent_t a, b;
+    int kind, pass;
+};
+thread_local bool g_prof = false;
+thread_local std::vector<ProfRec> g_prof_recs;
+thread_local std::vector<cudaEvent_t> g_prof_pool;
+
+cudaEvent_t prof_event() {
+    if (!g_prof_pool.empty()) {
+        cudaEvent_t e = g_prof_pool.back();
+        g_prof_pool.pop_back();
+        return e;
+    }
+    cudaEvent_t e = nullptr;
+    cudaEventCreate(&e);
+    return e;
+}
+
+// RAII bracket around one launch: counts it and, when profiling, records events
+struct LaunchScope {
+    cudaStream_t st;
+    ProfRec rec;
+    LaunchScope(cudaStream_t s, int kind, int pass) : st(s) {
+        ++g_launches;
+        if (g_prof) {
+            rec.kind = kind;
+            rec.pass = pass;
+            rec.a = prof_event();
+            rec.b = prof_event();
+            cudaEventRecord(rec.a, st);
+        }
+    }
+    ~LaunchScope() {
+        if (g_prof) {
+            cudaEventRecord(rec.b, st);
+            g_prof_recs.push_back(rec);
+        }
+    }
+};
+
+constexpr uint32_t DEFAULT_MT_DIV = 4;
+
+// ------------------------------------------------------------------ compile-time configurations
+
+// scatter: THREADS x KPT records per tile; MINB resident CTAs per SM requested
+template <int KB, int VB>
+struct ScatterCfg {
+    static constexpr int THREADS = (KB == 4 && VB <= 4) ? 256 : 512;
+    static constexpr int KPT = (KB == 4 && VB <= 4) ? 16 : 8;
+    static constexpr int MINB = (KB == 4 && VB <= 4) ? 3 : 2;
+};
+constexpr int HIST_THREADS = 512;
+
+template <int C>
+struct LocalCfg;
+template <> struct LocalCfg<0> { static constexpr int THREADS = 32, KPT = 4; };
+template <> struct LocalCfg<1> { static constexpr int THREADS = 64, KPT = 4; };
+template <> struct LocalCfg<2> { static constexpr int THREADS = 64, KPT = 8; };
+template <> struct LocalCfg<3> { static constexpr int THREADS = 128, KPT = 8; };
+template <> struct LocalCfg<4> { static constexpr int THREADS = 128, KPT = 16; };
+template <> struct LocalCfg<5> { static constexpr int THREADS = 256, KPT = 16; };
+template <> struct LocalCfg<6> { static constexpr int THREADS = 512, KPT = 16; };
+template <> struct LocalCfg<7> { static constexpr int THREADS = 1024, KPT = 16; };
+
+int max_class(int kb, int vb) { return (kb == 4 && vb <= 4) ? 7 : 6; }
+
+uint32_t max_kpb(int kb, int vb) {
+    if (kb == 4 && vb <= 4) return ScatterCfg<4, 4>::THREADS * ScatterCfg<4, 4>::KPT;
+    return ScatterCfg<8, 8>::THREADS * ScatterCfg<8, 8>::KPT;
+}
+uint32_t max_lt(int kb, int vb) { return 128u << max_class(kb, vb); }
+
+// ------------------------------------------------------------------ launch helpers
+
+struct KernelInfo {
+    int grid = 0;
+};
+std::mutex g_mu;
+std::unordered_map<uint64_t, KernelInfo> g_kinfo;  // key: (device << 48) ^ fn pointer
+std::unordered_map<int, int> g_dev_ok;             // device -> 1 ok / 0 not sm_100
+std::unordered_map<int, int> g_dev_sms;
+
+hrs_status cuda_fail(cudaError_t e) {
+    g_last_cuda = static_cast<int>(e);
+    return HRS_ERROR_CUDA;
+}
+
+hrs_status check_device(int *dev_out, int *sms_out) {
+    int dev = 0;
+    cudaError_t e = cudaGetDevice(&dev);
+    if (e != cudaSuccess) return cuda_fail(e);
+    std::lock_guard<std::mutex> lk(g_mu);
+    auto it = g_dev_ok.find(dev);
+    if (it == g_dev_ok.end()) {
+        cudaDeviceProp prop;
+        e = cudaGetDeviceProperties(&prop, dev);
+        if (e != cudaSuccess) return cuda_fail(e);
+        g_dev_ok[dev] = (prop.major == 10 && prop.minor == 0) ? 1 : 0;
+        g_dev_sms[dev] = prop.multiProcessorCount;
+        it = g_dev_ok.find(dev);
+    }
+    if (!it->second) return HRS_ERROR_NO_DEVICE;
+    *dev_out = dev;
+    *sms_out = g_dev_sms[dev];
+    return HRS_SUCCESS;
+}
+
+// persistent grid = SMs x resident CTAs per SM (occupancy API), cached per kernel
+template <typename F>
+hrs_status grid_for(F *fn, int threads, size_t smem, int dev, int sms, int *grid) {
+    const uint64_t key = (static_cast<uint64_t>(dev) << 56) ^ reinterpret_cast<uint64_t>(fn);
+    {
+        std::lock_guard<std::mutex> lk(g_mu);
+        auto it = g_kinfo.find(key);
+        if (it != g_kinfo.end()) {
+            *grid = it->second.grid;
+            return HRS_SUCCESS;
+        }
+    }
+    cudaError_t e = cudaSuccess;
+    if (smem > 48 * 1024) {
+        e = cudaFuncSetAttribute(reinterpret_cast<const void *>(fn), cudaFuncAttributeMaxDynamicSharedMemorySize,
+                                 static_cast<int>(smem));
+        if (e != cudaSuccess) return cuda_fail(e);
+    }
+    int per_sm = 0;
+    e = cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, reinterpret_cast<const void *>(fn), threads, smem);
+    if (e != cudaSuccess) return cuda_fail(e);
+    if (per_sm < 1) return cuda_fail(cudaErrorInvalidConfiguration);
+    KernelInfo ki;
+    ki.grid = per_sm * sms;
+    {
+        std::lock_guard<std::mutex> lk(g_mu);
+        g_kinfo[key] = ki;
+    }
+    *grid = ki.grid;
+    return HRS_SUCCESS;
+}
+
+hrs_status last_launch() {
+    cudaError_t e = cudaGetLastError();
+    if (e != cudaSuccess) return cuda_fail(e);
+    return HRS_SUCCESS;
+}
+
+// ------------------------------------------------------------------ plan + temp layout
+
+enum Mode { MODE_SORT = 0, MODE_HIST = 1, MODE_PARTITION = 2 };
+
+struct Plan {
+    uint64_t n = 0;
+    int kb = 4, vb = 0;
+    int begin = 0, end = 0;
+    int D = 0;
+    int lo[HRS_MAX_PASSES] = {0}, hi[HRS_MAX_PASSES] = {0};
+    uint32_t lt = 0, mt = 0, kpb = 0;
+    int single_class = -1;
+    bool counting = false;
+    bool wide = false;  // 64-bit look-back status words
+    uint32_t tile_cap = 0, bucket_cap = 0;
+    uint32_t local_cap[HRS_NUM_CLASSES] = {0};
+    size_t off_auxk = 0, off_auxv = 0, off_tiles[2] = {0, 0}, off_buckets[2] = {0, 0}, off_subrel = 0,
+           off_status[2] = {0, 0}, off_local[HRS_NUM_CLASSES] = {0}, total = 0;
+};
+
+size_t align_up(size_t x, size_t a) { return (x + a - 1) / a * a; }
+
+hrs_status make_plan(Plan &pl, uint64_t n, int kb, int vb, int begin, int end, const hrs_tuning *tu, Mode mode) {
+    pl.n = n;
+    pl.kb = kb;
+    pl.vb = vb;
+    pl.begin = begin;
+    pl.end = end;
+    hrs_tuning t;
+    t.local_threshold = 8192;
+    t.merge_threshold = 8192 / DEFAULT_MT_DIV;
+    t.keys_per_tile = max_kpb(kb, vb);
+    t.local_classes = 0;
+    if (tu) {
+        if (tu->local_threshold) t.local_threshold = tu->local_threshold;
+        if (tu->merge_threshold) t.merge_threshold = tu->merge_threshold;
+        else if (tu->local_threshold) t.merge_threshold = std::max<uint32_t>(1, t.local_threshold / DEFAULT_MT_DIV);
+        if (tu->keys_per_tile) t.keys_per_tile = tu->keys_per_tile;
+        t.local_classes = tu->local_classes;
+    }
+    if (t.local_threshold < 1 || t.local_threshold > max_lt(kb, vb)) return HRS_ERROR_INVALID_VALUE;
+    if (t.merge_threshold < 1 || t.merge_threshold > t.local_threshold) return HRS_ERROR_INVALID_VALUE;
+    if (t.keys_per_tile < 1 || t.keys_per_tile > max_kpb(kb, vb)) return HRS_ERROR_INVALID_VALUE;
+    if (t.local_classes > 1) return HRS_ERROR_INVALID_VALUE;
+    pl.lt = t.local_threshold;
+    pl.mt = t.merge_threshold;
+    pl.kpb = t.keys_per_tile;
+    pl.single_class = t.local_classes ? size_class_of(pl.lt) : -1;
+    pl.wide = n >= (1ull << 30);
+
+    // digit plan: 8-bit digits aligned to end_bit, most-significant first (reading #3)
+    pl.D = 0;
+    for (int h = end; h > begin; h -= 8) {
+        pl.hi[pl.D] = h;
+        pl.lo[pl.D] = std::max(begin, h - 8);
+        ++pl.D;
+    }
+    if (mode != MODE_SORT) pl.D = 1;
+    pl.counting = (mode != MODE_SORT) ? (n > 0) : (n > pl.lt && begin < end);
+
+    // analytical bounds: I1 buckets <= n/∂ˆ, I4 tiles <= n/KPB + n/∂ˆ
+    const uint64_t lt = pl.lt, kpb = pl.kpb;
+    uint64_t tiles = n / kpb + n / lt + 2;
+    uint64_t buckets = n / lt + 2;
+    if (mode != MODE_SORT) {
+        tiles = n / kpb + 2;
+        buckets = 2;
+    }
+    pl.tile_cap = static_cast<uint32_t>(std::min<uint64_t>(tiles, 0xFFFFFFFFull));
+    pl.bucket_cap = static_cast<uint32_t>(std::min<uint64_t>(buckets, 0xFFFFFFFFull));
+    // local lists: class c >= 1 entries hold > 64 * 2^c records; class 0 bounded by the
+    // merge rule (I3: any two neighbouring groups hold >= ∂ records)
+    for (int c = 0; c < HRS_NUM_CLASSES; ++c) {
+        uint64_t cap = 0;
+        if (mode == MODE_SORT) {
+            if (pl.single_class >= 0) {
+                cap = c == pl.single_class ? std::min<uint64_t>(n, 2 * n / pl.mt + 2 * pl.D * (n / lt + 1)) + 2 : 0;
+            } else if (c == 0) {
+                cap = std::min<uint64_t>(n, 2 * n / pl.mt + 2 * pl.D * (n / lt + 1)) + 2;
+            } else if ((64u << c) < pl.lt) {
+                cap = n / (64ull << c) + 2;  // entries of class c hold > 64 * 2^c records
+            }
+            if (!pl.counting) cap = (c == (pl.single_class >= 0 ? pl.single_class : size_class_of((uint32_t)std::max<uint64_t>(n, 1)))) ? 1 : 0;
+        }
+        pl.local_cap[c] = static_cast<uint32_t>(std::min<uint64_t>(cap, 0xFFFFFFFFull));
+    }
+
+    // temp layout
+    size_t off = align_up(sizeof(Ctl), 256);
+    const bool need_aux = (mode == MODE_SORT) && pl.counting && pl.D >= 2;
+    pl.off_auxk = off;
+    if (need_aux) off = align_up(off + n * kb, 256);
+    pl.off_auxv = off;
+    if (need_aux && vb) off = align_up(off + n * vb, 256);
+    const size_t sbytes = pl.wide ? 8 : 4;
+    for (int i = 0; i < 2; ++i) {
+        pl.off_tiles[i] = off;
+        off = align_up(off + sizeof(Tile) * static_cast<size_t>(pl.tile_cap), 256);
+        pl.off_buckets[i] = off;
+        off = align_up(off + sizeof(Bucket) * static_cast<size_t>(pl.bucket_cap), 256);
+        pl.off_status[i] = off;
+        off = align_up(off + sbytes * RADIX * static_cast<size_t>(pl.tile_cap), 256);
+    }
+    pl.off_subrel = off;
+    off = align_up(off + sizeof(uint32_t) * RADIX * static_cast<size_t>(pl.bucket_cap), 256);
+    for (int c = 0; c < HRS_NUM_CLASSES; ++c) {
+        pl.off_local[c] = off;
+        off = align_up(off + sizeof(LocalEntry) * static_cast<size_t>(pl.local_cap[c]), 256);
+    }
+    pl.total = off;
+    return HRS_SUCCESS;
+}
+
+bool overlap(const void *a, size_t na, const void *b, size_t nb) {
+    if (!a || !b || !na || !nb) return false;
+    const uintptr_t x = reinterpret_cast<uintptr_t>(a), y = reinterpret_cast<uintptr_t>(b);
+    return x < y + nb && y < x + na;
+}
+
+template <typename P>
+P *at(void *base, size_t off) {
+    return reinterpret_cast<P *>(static_cast<unsigned char *>(base) + off);
+}
+
+// ------------------------------------------------------------------ typed launch sequences
+
+template <typename K, typename V, typename S>
+struct Runner {
+    static constexpr int KB = sizeof(K);
+    static constexpr int VB = HasVal<V>::value ? sizeof(V) : 0;
+    using SC = ScatterCfg<KB, (VB == 0 ? 4 : VB)>;
+
+    static hrs_status init(const Plan &pl, void *temp, cudaStream_t st, int dev, int sms, int root_class,
+                           int counting) {
+        InitParams ip;
+        ip.ctl = at<Ctl>(temp, 0);
+        ip.tiles = at<Tile>(temp, pl.off_tiles[1]);
+        ip.buckets = at<Bucket>(temp, pl.off_buckets[1]);
+        ip.status = at<void>(temp, pl.off_status[1]);
+        ip.status_bytes = sizeof(S);
+        ip.root_local = root_class >= 0 ? at<LocalEntry>(temp, pl.off_local[root_class]) : nullptr;
+        ip.root_class = root_class;
+        ip.n = pl.n;
+        ip.kpb = pl.kpb;
+        ip.counting = counting;
+        ip.end_bit = pl.end;
+        ip.key_bytes = pl.kb;
+        ip.value_bytes = pl.vb;
+        const uint64_t T1 = counting ? (pl.n + pl.kpb - 1) / pl.kpb : 0;
+        const uint64_t work = std::max<uint64_t>(T1 * RADIX * sizeof(S) / 16, 1);
+        const int grid = static_cast<int>(std::min<uint64_t>((work + 255) / 256, static_cast<uint64_t>(sms) * 8));
+        LaunchScope ls(st, 0, 0);
+        k_init<<<std::max(grid, 1), 256, 0, st>>>(ip);
+        return last_launch();
+    }
+
+    static hrs_status hist(const Plan &pl, void *temp, cudaStream_t st, int dev, int sms, int p, const void *xin,
+                           uint16_t src_code, uint64_t *out_hist, uint64_t *out_offsets, bool last) {
+        HistParams hp;
+        std::memset(&hp, 0, sizeof(hp));
+        hp.keys = xin;
+        hp.p = p;
+        hp.last = last ? 1 : 0;
+        hp.lo = pl.lo[p - 1];
+        hp.width = pl.hi[p - 1] - pl.lo[p - 1];
+        hp.mask = (1u << hp.width) - 1u;
+        hp.tiles = at<Tile>(temp, pl.off_tiles[p & 1]);
+        hp.buckets = at<Bucket>(temp, pl.off_buckets[p & 1]);
+        hp.next_tiles = at<Tile>(temp, pl.off_tiles[(p + 1) & 1]);
+        hp.next_buckets = at<Bucket>(temp, pl.off_buckets[(p + 1) & 1]);
+        hp.status = at<void>(temp, pl.off_status[p & 1]);
+        hp.sub_rel = at<uint32_t>(temp, pl.off_subrel);
+        hp.ctl = at<Ctl>(temp, 0);
+        for (int c = 0; c < HRS_NUM_CLASSES; ++c) {
+            hp.local[c] = at<LocalEntry>(temp, pl.off_local[c]);
+            hp.local_cap[c] = pl.local_cap[c];
+        }
+        hp.tile_cap = pl.tile_cap;
+        hp.bucket_cap = pl.bucket_cap;
+        hp.lt = pl.lt;
+        hp.mt = pl.mt;
+        hp.kpb = pl.kpb;
+        hp.single_class = pl.single_class;
+        hp.src_code = src_code;
+        hp.out_hist = out_hist;
+        hp.out_offsets = out_offsets;
+        auto fn = k_hist<K, S, HIST_THREADS>;
+        int grid = 0;
+        hrs_status s = grid_for(fn, HIST_THREADS, 0, dev, sms, &grid);
+        if (s) return s;
+        LaunchScope ls(st, 1, p);
+        fn<<<grid, HIST_THREADS, 0, st>>>(hp);
+        return last_launch();
+    }
+
+    static hrs_status scatter(const Plan &pl, void *temp, cudaStream_t st, int dev, int sms, int p, const void *kin,
+                              void *kout, const void *vin, void *vout) {
+        ScatterParams sp;
+        sp.keys_in = kin;
+        sp.keys_out = kout;
+        sp.vals_in = vin;
+        sp.vals_out = vout;
+        sp.p = p;
+        sp.lo = pl.lo[p - 1];
+        sp.mask = (1u << (pl.hi[p - 1] - pl.lo[p - 1])) - 1u;
+        sp.tiles = at<Tile>(temp, pl.off_tiles[p & 1]);
+        sp.buckets = at<Bucket>(temp, pl.off_buckets[p & 1]);
+        sp.status = at<void>(temp, pl.off_status[p & 1]);
+        sp.sub_rel = at<uint32_t>(temp, pl.off_subrel);
+        sp.status_next = p < pl.D ? at<void>(temp, pl.off_status[(p + 1) & 1]) : nullptr;
+        sp.status_bytes = sizeof(S);
+        sp.ctl = at<Ctl>(temp, 0);
+        auto fn = k_scatter<K, V, S, SC::THREADS, SC::KPT, SC::MINB>;
+        const size_t smem = ScatterSmem<K, V, SC::THREADS, SC::KPT>::bytes;
+        int grid = 0;
+        hrs_status s = grid_for(fn, SC::THREADS, smem, dev, sms, &grid);
+        if (s) return s;
+        LaunchScope ls(st, 2, p);
+        fn<<<grid, SC::THREADS, smem, st>>>(sp);
+        return last_launch();
+    }
+
+    template <int C>
+    static hrs_status local_one(const Plan &pl, void *temp, cudaStream_t st, int dev, int sms, const void *kin,
+                                void *kout, const void *vin, void *vout) {
+        if constexpr (C > 7) {
+            return HRS_ERROR_INVALID_VALUE;
+        } else {
+            using LC = LocalCfg<C>;
+            using LS = LocalSmem<K, V, LC::THREADS, LC::KPT>;
+            if constexpr (LS::bytes > 220 * 1024) {
+                return HRS_ERROR_INVALID_VALUE;
+            } else {
+                LocalParams lp;
+                lp.src_keys[SRC_IN] = kin;
+                lp.src_keys[SRC_AUX] = at<void>(temp, pl.off_auxk);
+                lp.src_keys[SRC_OUT] = kout;
+                lp.src_vals[SRC_IN] = vin;
+                lp.src_vals[SRC_AUX] = VB ? at<void>(temp, pl.off_auxv) : nullptr;
+                lp.src_vals[SRC_OUT] = vout;
+                lp.keys_out = kout;
+                lp.vals_out = vout;
+                lp.list = at<LocalEntry>(temp, pl.off_local[C]);
+                lp.count = &at<Ctl>(temp, 0)->nlocal[C];
+                lp.begin_bit = pl.begin;
+                auto fn = k_local<K, V, LC::THREADS, LC::KPT, 1>;
+                int grid = 0;
+                hrs_status s = grid_for(fn, LC::THREADS, LS::bytes, dev, sms, &grid);
+                if (s) return s;
+                grid = static_cast<int>(std::min<uint64_t>(grid, std::max<uint32_t>(pl.local_cap[C], 1)));
+                LaunchScope ls(st, 3, C);
+                fn<<<grid, LC::THREADS, LS::bytes, st>>>(lp);
+                return last_launch();
+            }
+        }
+    }
+
+    static hrs_status local(const Plan &pl, void *temp, cudaStream_t st, int dev, int sms, int c, const void *kin,
+                            void *kout, const void *vin, void *vout) {
+        switch (c) {
+            case 0: return local_one<0>(pl, temp, st, dev, sms, kin, kout, vin, vout);
+            case 1: return local_one<1>(pl, temp, st, dev, sms, kin, kout, vin, vout);
+            case 2: return local_one<2>(pl, temp, st, dev, sms, kin, kout, vin, vout);
+            case 3: return local_one<3>(pl, temp, st, dev, sms, kin, kout, vin, vout);
+            case 4: return local_one<4>(pl, temp, st, dev, sms, kin, kout, vin, vout);
+            case 5: return local_one<5>(pl, temp, st, dev, sms, kin, kout, vin, vout);
+            case 6: return local_one<6>(pl, temp, st, dev, sms, kin, kout, vin, vout);
+            case 7: return local_one<7>(pl, temp, st, dev, sms, kin, kout, vin, vout);
+        }
+        return HRS_ERROR_INVALID_VALUE;
+    }
+
+    static hrs_status sort(const Plan &pl, void *temp, const void *kin, void *kout, const void *vin, void *vout,
+                           cudaStream_t st, int dev, int sms) {
+        hrs_status s;
+        const int root_class = pl.counting ? -1 : (pl.single_class >= 0 ? pl.single_class
+                                                                        : size_class_of((uint32_t)std::max<uint64_t>(pl.n, 1)));
+        if ((s = init(pl, temp, st, dev, sms, pl.n > 0 && pl.begin < pl.end ? root_class : -1, pl.counting ? 1 : 0)))
+            return s;
+        if (pl.n == 0) return HRS_SUCCESS;
+        if (pl.begin == pl.end) {
+            const int grid = static_cast<int>(std::min<uint64_t>((pl.n + 255) / 256, static_cast<uint64_t>(sms) * 8));
+            {
+                LaunchScope ls(st, 4, 0);
+                k_copy<K><<<grid, 256, 0, st>>>(static_cast<const K *>(kin), static_cast<K *>(kout), pl.n);
+            }
+            if ((s = last_launch())) return s;
+            if (VB) {
+                LaunchScope ls(st, 4, 0);
+                k_copy<typename std::conditional<VB == 8, uint64_t, uint32_t>::type><<<grid, 256, 0, st>>>(
+                    static_cast<const typename std::conditional<VB == 8, uint64_t, uint32_t>::type *>(vin),
+                    static_cast<typename std::conditional<VB == 8, uint64_t, uint32_t>::type *>(vout), pl.n);
+                if ((s = last_launch())) return s;
+            }
+            return HRS_SUCCESS;
+        }
+        void *auxk = at<void>(temp, pl.off_auxk);
+        void *auxv = VB ? at<void>(temp, pl.off_auxv) : nullptr;
+        if (pl.counting) {
+            const void *xk = kin, *xv = vin;
+            for (int p = 1; p <= pl.D; ++p) {
+                const bool to_out = ((pl.D - p) % 2) == 0;
+                void *yk = to_out ? kout : auxk;
+                void *yv = to_out ? vout : auxv;
+                if ((s = hist(pl, temp, st, dev, sms, p, xk, to_out ? SRC_OUT : SRC_AUX, nullptr, nullptr,
+                              p == pl.D)))
+                    return s;
+                if ((s = scatter(pl, temp, st, dev, sms, p, xk, yk, xv, yv))) return s;
+                xk = yk;
+                xv = yv;
+            }
+            const int cmax = pl.single_class >= 0 ? pl.single_class : size_class_of(pl.lt);
+            for (int c = (pl.single_class >= 0 ? pl.single_class : 0); c <= cmax; ++c)
+                if ((s = local(pl, temp, st, dev, sms, c, kin, kout, vin, vout))) return s;
+        } else {
+            if ((s = local(pl, temp, st, dev, sms, root_class, kin, kout, vin, vout))) return s;
+        }
+        return HRS_SUCCESS;
+    }
+
+    static hrs_status building_block(const Plan &pl, void *temp, const void *kin, void *kout, const void *vin,
+                                     void *vout, uint64_t *out_hist, uint64_t *out_offsets, bool do_scatter,
+                                     cudaStream_t st, int dev, int sms) {
+        hrs_status s;
+        if ((s = init(pl, temp, st, dev, sms, -1, pl.n > 0 ? 1 : 0))) return s;
+        const int r = 1 << (pl.hi[0] - pl.lo[0]);
+        if (pl.n == 0) {
+            uint64_t *p = out_hist ? out_hist : out_offsets;
+            if (p) {
+                LaunchScope ls(st, 4, 0);
+                k_fill_u64<<<1, 256, 0, st>>>(p, static_cast<uint64_t>(r) + (out_hist ? 0 : 1), 0);
+                return last_launch();
+            }
+            return HRS_SUCCESS;
+        }
+        if ((s = hist(pl, temp, st, dev, sms, 1, kin, SRC_OUT, out_hist, out_offsets, true))) return s;
+        if (do_scatter && (s = scatter(pl, temp, st, dev, sms, 1, kin, kout, vin, vout))) return s;
+        return HRS_SUCCESS;
+    }
+};
+
+template <typename K, typename V>
+hrs_status run_sort(const Plan &pl, void *temp, const void *kin, void *kout, const void *vin, void *vout,
+                    cudaStream_t st, int dev, int sms) {
+    if (pl.wide) return Runner<K, V, unsigned long long>::sort(pl, temp, kin, kout, vin, vout, st, dev, sms);
+    return Runner<K, V, uint32_t>::sort(pl, temp, kin, kout, vin, vout, st, dev, sms);
+}
+
+template <typename K, typename V>
+hrs_status run_block(const Plan &pl, void *temp, const void *kin, void *kout, const void *vin, void *vout,
+                     uint64_t *h, uint64_t *o, bool sc, cudaStream_t st, int dev, int sms) {
+    if (pl.wide)
+        return Runner<K, V, unsigned long long>::building_block(pl, temp, kin, kout, vin, vout, h, o, sc, st, dev, sms);
+    return Runner<K, V, uint32_t>::building_block(pl, temp, kin, kout, vin, vout, h, o, sc, st, dev, sms);
+}
+
+hrs_status sort_dispatch(int kb, int vb, const Plan &pl, void *temp, const void *kin, void *kout, const void *vin,
+                         void *vout, cudaStream_t st, int dev, int sms) {
+    if (kb == 4) {
+        if (vb == 0) return run_sort<uint32_t, NoVal>(pl, temp, kin, kout, vin, vout, st, dev, sms);
+        if (vb == 4) return run_sort<uint32_t, uint32_t>(pl, temp, kin, kout, vin, vout, st, dev, sms);
+        return run_sort<uint32_t, unsigned long long>(pl, temp, kin, kout, vin, vout, st, dev, sms);
+    }
+    if (vb == 0) return run_sort<unsigned long long, NoVal>(pl, temp, kin, kout, vin, vout, st, dev, sms);
+    if (vb == 4) return run_sort<unsigned long long, uint32_t>(pl, temp, kin, kout, vin, vout, st, dev, sms);
+    return run_sort<unsigned long long, unsigned long long>(pl, temp, kin, kout, vin, vout, st, dev, sms);
+}
+
+hrs_status block_dispatch(int kb, int vb, const Plan &pl, void *temp, const void *kin, void *kout, const void *vin,
+                          void *vout, uint64_t *h, uint64_t *o, bool sc, cudaStream_t st, int dev, int sms) {
+    if (kb == 4) {
+        if (vb == 0) return run_block<uint32_t, NoVal>(pl, temp, kin, kout, vin, vout, h, o, sc, st, dev, sms);
+        if (vb == 4) return run_block<uint32_t, uint32_t>(pl, temp, kin, kout, vin, vout, h, o, sc, st, dev, sms);
+        return run_block<uint32_t, unsigned long long>(pl, temp, kin, kout, vin, vout, h, o, sc, st, dev, sms);
+    }
+    if (vb == 0) return run_block<unsigned long long, NoVal>(pl, temp, kin, kout, vin, vout, h, o, sc, st, dev, sms);
+    if (vb == 4) return run_block<unsigned long long, uint32_t>(pl, temp, kin, kout, vin, vout, h, o, sc, st, dev, sms);
+    return run_block<unsigned long long, unsigned long long>(pl, temp, kin, kout, vin, vout, h, o, sc, st, dev, sms);
+}
+
+bool aligned(const void *p, size_t a) { return (reinterpret_cast<uintptr_t>(p) % a) == 0; }
+
+}  // namespace
+
+// ====================================================================== C ABI
+
+extern "C" {
+
+hrs_status hrs_sort_ex(void *d_temp, size_t *temp_bytes, const void *keys_in, void *keys_out, const void *vals_in,
+                       void *vals_out, uint64_t n, int key_bytes, int value_bytes, int begin_bit, int end_bit,
+                       const hrs_tuning *tuning, hrs_stream_t stream) {
+    if (!temp_bytes) return HRS_ERROR_INVALID_VALUE;
+    if (key_bytes != 4 && key_bytes != 8) return HRS_ERROR_INVALID_VALUE;
+    if (value_bytes != 0 && value_bytes != 4 && value_bytes != 8) return HRS_ERROR_INVALID_VALUE;
+    if (begin_bit < 0 || end_bit > 8 * key_bytes || begin_bit > end_bit) return HRS_ERROR_INVALID_BITS;
+    if (n > HRS_MAX_ITEMS) return HRS_ERROR_TOO_LARGE;
+    Plan pl;
+    hrs_status s = make_plan(pl, n, key_bytes, value_bytes, begin_bit, end_bit, tuning, MODE_SORT);
+    if (s) return s;
+    if (!d_temp) {
+        *temp_bytes = pl.total;
+        return HRS_SUCCESS;
+    }
+    if (*temp_bytes < pl.total) return HRS_ERROR_TEMP_TOO_SMALL;
+    if (!aligned(d_temp, 256)) return HRS_ERROR_INVALID_VALUE;
+    if (n > 0) {
+        if (!keys_in || !keys_out) return HRS_ERROR_INVALID_VALUE;
+        if (value_bytes && (!vals_in || !vals_out)) return HRS_ERROR_INVALID_VALUE;
+        if (!aligned(keys_in, key_bytes) || !aligned(keys_out, key_bytes)) return HRS_ERROR_INVALID_VALUE;
+        if (value_bytes && (!aligned(vals_in, value_bytes) || !aligned(vals_out, value_bytes)))
+            return HRS_ERROR_INVALID_VALUE;
+        const size_t nk = n * key_bytes, nv = n * value_bytes;
+        const void *bufs[5] = {keys_in, keys_out, value_bytes ? vals_in : nullptr, value_bytes ? vals_out : nullptr,
+                               d_temp};
+        const size_t lens[5] = {nk, nk, nv, nv, pl.total};
+        for (int i = 0; i < 5; ++i)
+            for (int j = i + 1; j < 5; ++j)
+                if (overlap(bufs[i], lens[i], bufs[j], lens[j])) return HRS_ERROR_ALIASING;
+    }
+    int dev = 0, sms = 0;
+    if ((s = check_device(&dev, &sms))) return s;
+    return sort_dispatch(key_bytes, value_bytes, pl, d_temp, keys_in, keys_out, vals_in, vals_out,
+                         reinterpret_cast<cudaStream_t>(stream), dev, sms);
+}
+
+hrs_status hrs_sort_keys_u32(void *t, size_t *tb, const uint32_t *ki, uint32_t *ko, uint64_t n, int b, int e,
+                             hrs_stream_t s) {
+    return hrs_sort_ex(t, tb, ki, ko, nullptr, nullptr, n, 4, 0, b, e, nullptr, s);
+}
+hrs_status hrs_sort_keys_u64(void *t, size_t *tb, const uint64_t *ki, uint64_t *ko, uint64_t n, int b, int e,
+                             hrs_stream_t s) {
+    return hrs_sort_ex(t, tb, ki, ko, nullptr, nullptr, n, 8, 0, b, e, nullptr, s);
+}
+hrs_status hrs_sort_pairs_u32_u32(void *t, size_t *tb, const uint32_t *ki, uint32_t *ko, const uint32_t *vi,
+                                  uint32_t *vo, uint64_t n, int b, int e, hrs_stream_t s) {
+    return hrs_sort_ex(t, tb, ki, ko, vi, vo, n, 4, 4, b, e, nullptr, s);
+}
+hrs_status hrs_sort_pairs_u32_u64(void *t, size_t *tb, const uint32_t *ki, uint32_t *ko, const uint64_t *vi,
+                                  uint64_t *vo, uint64_t n, int b, int e, hrs_stream_t s) {
+    return hrs_sort_ex(t, tb, ki, ko, vi, vo, n, 4, 8, b, e, nullptr, s);
+}
+hrs_status hrs_sort_pairs_u64_u32(void *t, size_t *tb, const uint64_t *ki, uint64_t *ko, const uint32_t *vi,
+                                  uint32_t *vo, uint64_t n, int b, int e, hrs_stream_t s) {
+    return hrs_sort_ex(t, tb, ki, ko, vi, vo, n, 8, 4, b, e, nullptr, s);
+}
+hrs_status hrs_sort_pairs_u64_u64(void *t, size_t *tb, const uint64_t *ki, uint64_t *ko, const uint64_t *vi,
+                                  uint64_t *vo, uint64_t n, int b, int e, hrs_stream_t s) {
+    return hrs_sort_ex(t, tb, ki, ko, vi, vo, n, 8, 8, b, e, nullptr, s);
+}
+
+hrs_status hrs_get_stats(const void *d_temp, hrs_stats *out, hrs_stream_t stream) {
+    if (!d_temp || !out) return HRS_ERROR_INVALID_VALUE;
+    Ctl c;
+    cudaStream_t st = reinterpret_cast<cudaStream_t>(stream);
+    cudaError_t e = cudaMemcpyAsync(&c, d_temp, sizeof(Ctl), cudaMemcpyDeviceToHost, st);
+    if (e != cudaSuccess) return cuda_fail(e);
+    e = cudaStreamSynchronize(st);
+    if (e != cudaSuccess) return cuda_fail(e);
+    if (c.magic != CTL_MAGIC) return HRS_ERROR_INVALID_VALUE;
+    std::memset(out, 0, sizeof(*out));
+    out->n = c.n;
+    out->key_bytes = c.key_bytes;
+    out->value_bytes = c.value_bytes;
+    out->overflow = c.overflow;
+    const uint64_t K = c.key_bytes, R = c.key_bytes + c.value_bytes;
+    uint64_t bytes = 0;
+    for (int p = 1; p <= HRS_MAX_PASSES; ++p) {
+        if (c.ntiles[p] == 0) continue;
+        out->counting_passes = p;
+        out->recs_in_pass[p - 1] = c.recs_in_pass[p];
+        out->tiles_in_pass[p - 1] = c.ntiles[p];
+        out->buckets_in_pass[p - 1] = c.nbuckets[p];
+        bytes += c.recs_in_pass[p] * (K + 2 * R);
+    }
+    for (int k = 0; k < HRS_NUM_CLASSES; ++k) {
+        out->local_in_class[k] = c.nlocal[k];
+        out->local_buckets += c.nlocal[k];
+    }
+    out->local_recs = c.local_recs;
+    out->merged_groups = c.merged_groups;
+    out->bytes_min = bytes + c.local_recs * 2 * R;
+    return HRS_SUCCESS;
+}
+
+uint32_t hrs_max_local_threshold(int key_bytes, int value_bytes) { return max_lt(key_bytes, value_bytes); }
+uint32_t hrs_max_keys_per_tile(int key_bytes, int value_bytes) { return max_kpb(key_bytes, value_bytes); }
+
+hrs_status hrs_default_tuning(int key_bytes, int value_bytes, hrs_tuning *out) {
+    if (!out || (key_bytes != 4 && key_bytes != 8) || (value_bytes != 0 && value_bytes != 4 && value_bytes != 8))
+        return HRS_ERROR_INVALID_VALUE;
+    Plan pl;
+    hrs_status s = make_plan(pl, 0, key_bytes, value_bytes, 0, 8 * key_bytes, nullptr, MODE_SORT);
+    if (s) return s;
+    out->local_threshold = pl.lt;
+    out->merge_threshold = pl.mt;
+    out->keys_per_tile = pl.kpb;
+    out->local_classes = 0;
+    return HRS_SUCCESS;
+}
+
+static hrs_status block_common(void *d_temp, size_t *temp_bytes, const void *keys_in, void *keys_out,
+                               const void *vals_in, void *vals_out, uint64_t n, int kb, int vb, int lo, int hi,
+                               uint64_t *h, uint64_t *o, bool scatter, hrs_stream_t stream) {
+    if (!temp_bytes) return HRS_ERROR_INVALID_VALUE;
+    if (kb != 4 && kb != 8) return HRS_ERROR_INVALID_VALUE;
+    if (vb != 0 && vb != 4 && vb != 8) return HRS_ERROR_INVALID_VALUE;
+    if (lo < 0 || hi > 8 * kb || hi - lo < 1 || hi - lo > 8) return HRS_ERROR_INVALID_BITS;
+    if (n > HRS_MAX_ITEMS) return HRS_ERROR_TOO_LARGE;
+    Plan pl;
+    hrs_status s = make_plan(pl, n, kb, vb, lo, hi, nullptr, scatter ? MODE_PARTITION : MODE_HIST);
+    if (s) return s;
+    pl.lo[0] = lo;
+    pl.hi[0] = hi;
+    if (!d_temp) {
+        *temp_bytes = pl.total;
+        return HRS_SUCCESS;
+    }
+    if (*temp_bytes < pl.total) return HRS_ERROR_TEMP_TOO_SMALL;
+    if (!aligned(d_temp, 256)) return HRS_ERROR_INVALID_VALUE;
+    if (!scatter && !h) return HRS_ERROR_INVALID_VALUE;
+    if (n > 0) {
+        if (!keys_in || (scatter && !keys_out)) return HRS_ERROR_INVALID_VALUE;
+        if (scatter && vb && (!vals_in || !vals_out)) return HRS_ERROR_INVALID_VALUE;
+        if (!aligned(keys_in, kb) || (scatter && !aligned(keys_out, kb))) return HRS_ERROR_INVALID_VALUE;
+        const size_t nk = n * kb, nv = n * vb;
+        const void *bufs[5] = {keys_in, scatter ? keys_out : nullptr, vb ? vals_in : nullptr,
+                               vb ? vals_out : nullptr, d_temp};
+        const size_t lens[5] = {nk, nk, nv, nv, pl.total};
+        for (int i = 0; i < 5; ++i)
+            for (int j = i + 1; j < 5; ++j)
+                if (overlap(bufs[i], lens[i], bufs[j], lens[j])) return HRS_ERROR_ALIASING;
+    }
+    int dev = 0, sms = 0;
+    if ((s = check_device(&dev, &sms))) return s;
+    return block_dispatch(kb, vb, pl, d_temp, keys_in, keys_out, vals_in, vals_out, h, o, scatter,
+                          reinterpret_cast<cudaStream_t>(stream), dev, sms);
+}
+
+hrs_status hrs_digit_histogram(void *d_temp, size_t *temp_bytes, const void *keys, uint64_t n, int key_bytes,
+                               int lo_bit, int hi_bit, uint64_t *d_hist, hrs_stream_t stream) {
+    return block_common(d_temp, temp_bytes, keys, nullptr, nullptr, nullptr, n, key_bytes, 0, lo_bit, hi_bit,
+                        d_hist, nullptr, false, stream);
+}
+
+hrs_status hrs_partition_pass(void *d_temp, size_t *temp_bytes, const void *keys_in, void *keys_out,
+                              const void *vals_in, void *vals_out, uint64_t n, int key_bytes, int value_bytes,
+                              int lo_bit, int hi_bit, uint64_t *d_offsets, hrs_stream_t stream) {
+    return block_common(d_temp, temp_bytes, keys_in, keys_out, vals_in, vals_out, n, key_bytes, value_bytes, lo_bit,
+                        hi_bit, nullptr, d_offsets, true, stream);
+}
+
+const char *hrs_status_string(hrs_status s) {
+    switch (s) {
+        case HRS_SUCCESS: return "success";
+        case HRS_ERROR_INVALID_VALUE: return "invalid value";
+        case HRS_ERROR_INVALID_BITS: return "invalid bit range";
+        case HRS_ERROR_ALIASING: return "buffers overlap";
+        case HRS_ERROR_TEMP_TOO_SMALL: return "temp storage too small";
+        case HRS_ERROR_TOO_LARGE: return "n exceeds HRS_MAX_ITEMS";
+        case HRS_ERROR_NO_DEVICE: return "current device is not an sm_100 GPU";
+        case HRS_ERROR_CUDA: return "CUDA error";
+    }
+    return "unknown status";
+}
+
+int hrs_last_cuda_error(void) { return g_last_cuda; }
+uint64_t hrs_launch_count(void) { return g_launches; }
+
+void hrs_profile_enable(int on) {
+    for (auto &r : g_prof_recs) {
+        g_prof_pool.push_back(r.a);
+        g_prof_pool.push_back(r.b);
+    }
+    g_prof_recs.clear();
+    g_prof = on != 0;
+}
+
+int hrs_profile_collect(hrs_profile_record *out, int max) {
+    int k = 0;
+    for (auto &r : g_prof_recs) {
+        if (out && k < max) {
+            float ms = 0.f;
+            cudaEventSynchronize(r.b);
+            cudaEventElapsedTime(&ms, r.a, r.b);
+            out[k].kind = r.kind;
+            out[k].pass = r.pass;
+            out[k].ms = ms;
+            ++k;
+        }
+        g_prof_pool.push_back(r.a);
+        g_prof_pool.push_back(r.b);
+    }
+    g_prof_recs.clear();
+    return k;
+}
+int hrs_version(void) { return 1; }
+
+}  // extern "C"

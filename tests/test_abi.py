@@ -1,0 +1,103 @@
+"""C-ABI checks that need no GPU: the library loads, exports every symbol the header
+declares with the binding's arity, and rejects bad arguments before touching a device."""
+import ctypes
+import os
+import re
+
+import pytest
+
+ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+HEADER = os.path.join(ROOT, "include", "hrs.h")
+
+
+def _header_functions():
+    src = open(HEADER, encoding="utf-8").read()
+    src = re.sub(r"/\*.*?\*/", "", src, flags=re.S)
+    src = re.sub(r"#[^\n]*", "", src)
+    funcs = {}
+    for m in re.finditer(r"\b(hrs_\w+)\s*\(([^;{]*?)\)\s*;", src):
+        name, args = m.group(1), m.group(2).strip()
+        n = 0 if args in ("void", "") else args.count(",") + 1
+        funcs[name] = n
+    return funcs
+
+
+def test_header_parses():
+    f = _header_functions()
+    for name in ("hrs_sort_keys_u32", "hrs_sort_keys_u64", "hrs_sort_pairs_u32_u32", "hrs_sort_pairs_u32_u64",
+                 "hrs_sort_pairs_u64_u32", "hrs_sort_pairs_u64_u64", "hrs_get_stats", "hrs_digit_histogram",
+                 "hrs_partition_pass", "hrs_sort_ex"):
+        assert name in f
+
+
+def test_library_exports_every_declared_symbol():
+    import paper_1611_01137_b200 as hrs
+    from paper_1611_01137_b200 import _lib
+    decl = _header_functions()
+    raw = ctypes.CDLL(_lib.LIB_PATH)
+    for name, nargs in decl.items():
+        assert hasattr(raw, name), f"{name} declared in hrs.h but not exported"
+        assert name in _lib.SIGNATURES, f"{name} missing from the Python binding"
+        assert len(_lib.SIGNATURES[name][1]) == nargs, name
+    assert set(_lib.SIGNATURES) == set(decl)
+    assert hrs.lib.hrs_version() >= 1
+
+
+def test_library_is_sm100a_only():
+    from paper_1611_01137_b200 import _lib
+    import subprocess
+    out = subprocess.run(["/usr/local/cuda/bin/cuobjdump", "--list-elf", _lib.LIB_PATH], capture_output=True,
+                         text=True).stdout
+    assert "sm_100a" in out
+    for other in ("sm_80", "sm_90", "sm_103"):
+        assert other + "." not in out and other + "a." not in out
+
+
+def _sz(fn, *args):
+    sz = ctypes.c_size_t(0)
+    return fn(None, ctypes.byref(sz), *args), sz.value
+
+
+def test_size_query_and_validation_without_gpu():
+    from paper_1611_01137_b200 import _lib
+    lib = _lib.lib
+    st, size = _sz(lib.hrs_sort_ex, None, None, None, None, 1 << 20, 4, 4, 0, 32, None, None)
+    assert st == 0 and size > (1 << 20) * 8  # aux buffers for the double buffering (M1)
+    # M2..M5 (metadata) stay a small fraction of M1 = input + aux (the paper's 5 %
+    # is for its 16-byte tables, ours keep two look-back status arrays): < 10 % of M1
+    assert size - (1 << 20) * 8 < 0.10 * 2 * (1 << 20) * 8
+    assert _sz(lib.hrs_sort_ex, None, None, None, None, 10, 4, 0, 0, 33, None, None)[0] == 2   # bits
+    assert _sz(lib.hrs_sort_ex, None, None, None, None, 10, 4, 0, 5, 4, None, None)[0] == 2
+    assert _sz(lib.hrs_sort_ex, None, None, None, None, 10, 3, 0, 0, 24, None, None)[0] == 1   # key bytes
+    assert _sz(lib.hrs_sort_ex, None, None, None, None, 10, 4, 2, 0, 32, None, None)[0] == 1   # value bytes
+    assert _sz(lib.hrs_sort_ex, None, None, None, None, 1 << 33, 8, 8, 0, 64, None, None)[0] == 5
+    assert lib.hrs_sort_ex(None, None, None, None, None, None, 1, 4, 0, 0, 32, None, None) == 1
+    bad = _lib.Tuning(local_threshold=10, merge_threshold=11)   # ∂ > ∂ˆ
+    assert _sz(lib.hrs_sort_ex, None, None, None, None, 10, 4, 0, 0, 32, ctypes.byref(bad), None)[0] == 1
+    too_big = _lib.Tuning(local_threshold=1 << 20)
+    assert _sz(lib.hrs_sort_ex, None, None, None, None, 10, 4, 0, 0, 32, ctypes.byref(too_big), None)[0] == 1
+    # temp too small is detected before any device work
+    small = ctypes.c_size_t(16)
+    buf = ctypes.create_string_buffer(512)
+    p = ctypes.cast(ctypes.addressof(buf) + (-ctypes.addressof(buf)) % 256, ctypes.c_void_p)
+    assert lib.hrs_sort_ex(p, ctypes.byref(small), p, p, None, None, 100, 4, 0, 0, 32, None, None) == 4
+    # building blocks: digit width 1..8
+    assert _sz(lib.hrs_digit_histogram, None, 10, 4, 0, 9, None, None)[0] == 2
+    assert _sz(lib.hrs_digit_histogram, None, 10, 4, 28, 36, None, None)[0] == 2
+    assert _sz(lib.hrs_partition_pass, None, None, None, None, 10, 8, 8, 56, 64, None, None)[0] == 0
+    assert lib.hrs_status_string(3) == b"buffers overlap"
+
+
+def test_default_tuning_within_limits():
+    import paper_1611_01137_b200 as hrs
+    for kb, vb in ((4, 0), (4, 4), (4, 8), (8, 0), (8, 4), (8, 8)):
+        t = hrs.default_tuning(kb, vb)
+        assert 1 <= t["merge_threshold"] <= t["local_threshold"] <= hrs.max_local_threshold(kb, vb)
+        assert 1 <= t["keys_per_tile"] <= hrs.max_keys_per_tile(kb, vb)
+
+
+def test_python_wrapper_rejects_cpu_tensors():
+    import torch
+    import paper_1611_01137_b200 as hrs
+    with pytest.raises(ValueError, match="CUDA"):
+        hrs.sort(torch.zeros(4, dtype=torch.uint32))

@@ -1,0 +1,233 @@
+"""GPU parity: the CUDA path through the C ABI against the CPU oracle, element by element.
+
+All integer work, so the bar is bit-exact keys and values (BJ north_star).  Inputs are
+seeded synthetic workloads from gen/ (uniform and AND-m skew)."""
+import numpy as np
+import pytest
+import torch
+
+import gen
+import oracle
+from oracle import plan
+
+pytestmark = pytest.mark.gpu
+
+DEV = "cuda:0"
+TYPES = [(32, 0), (32, 32), (32, 64), (64, 0), (64, 32), (64, 64)]
+
+
+def _np(t: torch.Tensor) -> np.ndarray:
+    return oracle._u64(t.cpu())
+
+
+def _inputs(n, kbits, vbits, dist, seed, vkind="random"):
+    k = gen.keys(n, kbits, dist, seed=seed)
+    v = gen.values(n, vbits, vkind, seed=seed) if vbits else None
+    return k, v
+
+
+def _run_and_check(k, v, b, e, tuning=None, stats_expect=None):
+    import paper_1611_01137_b200 as hrs
+    kd = k.to(DEV)
+    vd = v.to(DEV) if v is not None else None
+    ko, vo = hrs.sort(kd, vd, b, e, tuning=tuning)
+    torch.cuda.synchronize()
+    ek, ev = oracle.sort(k, v, b, e)
+    got_k = _np(ko)
+    assert np.array_equal(got_k, ek), f"keys differ (n={k.numel()}, bits=[{b},{e}))"
+    if v is not None:
+        assert np.array_equal(_np(vo), ev), f"values differ (n={k.numel()}, bits=[{b},{e}))"
+    return ko, vo
+
+
+@pytest.mark.parametrize("kbits,vbits", TYPES)
+@pytest.mark.parametrize("n", [0, 1, 2, 31, 32, 33, 1000, 4095, 4096, 4097, 8192, 8193, 12289, 100003])
+def test_sizes_uniform(kbits, vbits, n):
+    k, v = _inputs(n, kbits, vbits, "uniform", seed=n + 1)
+    _run_and_check(k, v, 0, kbits)
+
+
+@pytest.mark.parametrize("kbits,vbits", TYPES)
+@pytest.mark.parametrize("dist", ["and2", "and3", "and4", "const"])
+def test_skewed(kbits, vbits, dist):
+    k, v = _inputs(300001, kbits, vbits, dist, seed=7)
+    _run_and_check(k, v, 0, kbits)
+
+
+@pytest.mark.parametrize("kbits,vbits", [(32, 32), (64, 64), (64, 0)])
+def test_one_million_and_odd_values(kbits, vbits):
+    for dist in ("uniform", "and3"):
+        k, v = _inputs((1 << 20) + 17, kbits, vbits, dist, seed=3)
+        _run_and_check(k, v, 0, kbits)
+
+
+@pytest.mark.parametrize("kbits,vbits", [(32, 32), (64, 32)])
+def test_bit_ranges(kbits, vbits):
+    k, v = _inputs(50000, kbits, vbits, "and2", seed=4)
+    ranges = [(0, 1), (7, 9), (3, 29), (8, 16), (kbits - 1, kbits), (5, 5), (0, 8), (1, kbits), (0, kbits - 3)]
+    if kbits == 64:
+        ranges += [(0, 33), (17, 61), (32, 64), (56, 64)]
+    for b, e in ranges:
+        _run_and_check(k, v, b, e)
+
+
+def test_tie_heavy_stability():
+    """Constant and two-valued keys: only stability decides the value order."""
+    n = 200000
+    for keys in (torch.zeros(n, dtype=torch.int32).view(torch.uint32),
+                 (torch.arange(n, dtype=torch.int32) % 2).view(torch.uint32),
+                 torch.full((n,), -1, dtype=torch.int32).view(torch.uint32),
+                 torch.full((n,), 0x5A5A5A5A, dtype=torch.int32).view(torch.uint32)):
+        v = gen.values(n, 32, "index")
+        _run_and_check(keys, v, 0, 32)
+
+
+def test_sorted_and_reverse_inputs():
+    n = 123457
+    k = gen.keys(n, 32, "uniform", seed=2)
+    ks, _ = oracle.sort(k, None, 0, 32)
+    ks_t = torch.from_numpy(ks.astype(np.uint32).view(np.int32)).view(torch.uint32)
+    _run_and_check(ks_t, gen.values(n, 32, "index"), 0, 32)
+    _run_and_check(ks_t.flip(0).contiguous(), gen.values(n, 32, "index"), 0, 32)
+
+
+# ------------------------------------------------------------- deep recursion via tuning overrides
+
+TUNINGS = [
+    dict(local_threshold=64, merge_threshold=40, keys_per_tile=32),
+    dict(local_threshold=300, merge_threshold=100, keys_per_tile=128),
+    dict(local_threshold=3, merge_threshold=2, keys_per_tile=4),
+    dict(local_threshold=200, merge_threshold=1, keys_per_tile=1),
+    dict(local_threshold=4096, merge_threshold=4096, keys_per_tile=4096),
+]
+
+
+@pytest.mark.parametrize("tuning", TUNINGS)
+@pytest.mark.parametrize("dist", ["uniform", "and2", "and4", "const"])
+@pytest.mark.parametrize("kbits,vbits", [(32, 32), (64, 64)])
+def test_threshold_overrides_and_structure(tuning, dist, kbits, vbits):
+    """Forcing tiny thresholds exercises deep recursion, merging, every size class and
+    last-digit exhaustion; the pass/bucket/local structure must equal the paper-order
+    MSD simulation (oracle/plan.py) exactly."""
+    import paper_1611_01137_b200 as hrs
+    n = 5000
+    k, v = _inputs(n, kbits, vbits, dist, seed=11)
+    kd, vd = k.to(DEV), v.to(DEV)
+    tb = hrs.temp_bytes(n, kbits // 8, vbits // 8, 0, kbits, tuning)
+    temp = torch.empty(tb, dtype=torch.uint8, device=DEV)
+    ko, vo = hrs.sort(kd, vd, 0, kbits, tuning=tuning, temp=temp)
+    st = hrs.get_stats(temp)
+    ek, ev = oracle.sort(k, v, 0, kbits)
+    assert np.array_equal(_np(ko), ek) and np.array_equal(_np(vo), ev)
+    sim = plan.simulate_msd(oracle._u64(k), None, 0, kbits, tuning["local_threshold"],
+                            tuning["merge_threshold"], tuning["keys_per_tile"])
+    assert st["overflow"] == 0
+    assert st["counting_passes"] == sim.counting_passes
+    assert st["recs_in_pass"] == sim.recs_in_pass
+    assert st["tiles_in_pass"] == sim.tiles_in_pass
+    assert st["buckets_in_pass"] == sim.buckets_in_pass
+    assert st["local_buckets"] == sim.local_buckets
+    assert st["local_recs"] == sim.local_recs
+    assert st["merged_groups"] == sim.merged_groups
+    per_class = [0] * 8
+    for e in sim.local_entries:
+        per_class[e[3]] += 1
+    assert st["local_in_class"] == per_class
+    assert st["bytes_min"] == plan.bytes_min(sim, kbits // 8, vbits // 8)
+
+
+def test_single_local_config_ablation():
+    n = 40000
+    k, v = _inputs(n, 32, 32, "and2", seed=12)
+    _run_and_check(k, v, 0, 32, tuning=dict(local_threshold=2048, merge_threshold=1, keys_per_tile=512,
+                                            local_classes=1))
+
+
+def test_table2_worked_example_on_gpu():
+    """Table 2 with keys (a << 8) | b, ∂ˆ = 3, no merging, KPB = 4."""
+    import paper_1611_01137_b200 as hrs
+    toks = "31 12 01 23 12 22 12 00 11 10 10 31 03 13 12 03".split()
+    final = "00 01 03 03 10 10 11 12 12 12 12 13 22 23 31 31".split()
+    enc = [(int(t[0]) << 8) | int(t[1]) for t in toks]
+    k = torch.tensor(enc, dtype=torch.int32).view(torch.uint32).to(DEV)
+    v = torch.arange(16, dtype=torch.int32).view(torch.uint32).to(DEV)
+    tun = dict(local_threshold=3, merge_threshold=1, keys_per_tile=4)
+    temp = torch.empty(hrs.temp_bytes(16, 4, 4, 0, 16, tun), dtype=torch.uint8, device=DEV)
+    ko, vo = hrs.sort(k, v, 0, 16, tuning=tun, temp=temp)
+    assert ko.view(torch.int32).cpu().tolist() == [(int(t[0]) << 8) | int(t[1]) for t in final]
+    assert vo.view(torch.int32).cpu().tolist() == [7, 2, 12, 15, 9, 10, 8, 1, 4, 6, 14, 13, 5, 3, 0, 11]
+    st = hrs.get_stats(temp)
+    assert st["counting_passes"] == 2 and st["recs_in_pass"] == [16, 12] and st["local_buckets"] == 2
+    # pass 1 alone: the partition building block reproduces Table 2 row 5 and the offsets
+    k1, v1, offs = hrs.partition_pass(k, v, 8, 16)
+    assert v1.view(torch.int32).cpu().tolist() == [2, 7, 12, 15, 1, 4, 6, 8, 9, 10, 13, 14, 3, 5, 0, 11]
+    assert offs.view(torch.int64).cpu().tolist()[:5] == [0, 4, 12, 14, 16]
+    h = hrs.digit_histogram(k, 8, 16)
+    assert h.view(torch.int64).cpu().tolist()[:4] == [4, 8, 2, 2]
+
+
+# ------------------------------------------------------------- building blocks
+
+@pytest.mark.parametrize("kbits", [32, 64])
+@pytest.mark.parametrize("n", [0, 1, 4097, 1000003])
+def test_digit_histogram(kbits, n):
+    import paper_1611_01137_b200 as hrs
+    k = gen.keys(n, kbits, "and2", seed=5)
+    kd = k.to(DEV)
+    for lo, hi in ((kbits - 8, kbits), (0, 8), (3, 7), (kbits - 1, kbits)):
+        h = hrs.digit_histogram(kd, lo, hi)
+        exp = oracle.histogram(k, lo, hi)
+        assert np.array_equal(_np(h), exp), (lo, hi)
+
+
+@pytest.mark.parametrize("kbits,vbits", TYPES)
+def test_partition_pass(kbits, vbits):
+    import paper_1611_01137_b200 as hrs
+    for n in (1, 4097, 654321):
+        k, v = _inputs(n, kbits, vbits, "and3", seed=n)
+        kd = k.to(DEV)
+        vd = v.to(DEV) if v is not None else None
+        for lo, hi in ((kbits - 8, kbits), (5, 11)):
+            ko, vo, offs = hrs.partition_pass(kd, vd, lo, hi)
+            ek, ev, eo = oracle.partition_pass(k, v, lo, hi)
+            assert np.array_equal(_np(ko), ek)
+            if v is not None:
+                assert np.array_equal(_np(vo), ev)
+            assert np.array_equal(_np(offs), eo)
+
+
+# ------------------------------------------------------------- properties
+
+def test_deterministic_repeats():
+    import paper_1611_01137_b200 as hrs
+    n = 1 << 21
+    k = gen.keys(n, 32, "and3", seed=9, device=DEV)
+    v = gen.values(n, 32, "index", device=DEV)
+    ref = None
+    for _ in range(5):
+        ko, vo = hrs.sort(k, v)
+        cur = (ko.clone(), vo.clone())
+        if ref is None:
+            ref = cur
+        else:
+            assert torch.equal(cur[0].view(torch.int32), ref[0].view(torch.int32))
+            assert torch.equal(cur[1].view(torch.int32), ref[1].view(torch.int32))
+
+
+def test_errors_on_gpu():
+    import paper_1611_01137_b200 as hrs
+    k = torch.zeros(100, dtype=torch.uint32, device=DEV)
+    with pytest.raises(hrs.HrsError):
+        hrs.sort(k, None, 0, 33)
+    # aliasing: output overlapping input
+    with pytest.raises(hrs.HrsError, match="ALIASING"):
+        hrs.sort(k, None, keys_out=k)
+    # misaligned u32 pointer (view starting one byte in)
+    raw = torch.zeros(404, dtype=torch.uint8, device=DEV)
+    with pytest.raises(hrs.HrsError):
+        import ctypes
+        sz = ctypes.c_size_t(1 << 20)
+        t = torch.empty(1 << 20, dtype=torch.uint8, device=DEV)
+        hrs.check(hrs.lib.hrs_sort_ex(ctypes.c_void_p(t.data_ptr()), ctypes.byref(sz),
+                                      ctypes.c_void_p(raw.data_ptr() + 1), ctypes.c_void_p(raw.data_ptr() + 404),
+                                      None, None, 10, 4, 0, 0, 32, None, None), "misaligned")
