@@ -88,7 +88,7 @@ def test_sorted_and_reverse_inputs():
     ks, _ = oracle.sort(k, None, 0, 32)
     ks_t = torch.from_numpy(ks.astype(np.uint32).view(np.int32)).view(torch.uint32)
     _run_and_check(ks_t, gen.values(n, 32, "index"), 0, 32)
-    _run_and_check(ks_t.flip(0).contiguous(), gen.values(n, 32, "index"), 0, 32)
+    _run_and_check(ks_t.view(torch.int32).flip(0).contiguous().view(torch.uint32), gen.values(n, 32, "index"), 0, 32)
 
 
 # ------------------------------------------------------------- deep recursion via tuning overrides
