@@ -244,7 +244,7 @@ def run_hrs(args):
         hrs.profile_enable(False)
         per = {}
         for kind, p, ms in recs:
-            key = f"{kind}{p}" if kind in ("hist", "scatter", "local") else kind
+            key = f"{kind}{p}" if kind in ("hist", "scatter", "local", "classify") else kind
             per.setdefault(key, []).append(ms)
         kern = {k2: sum(v2) / args.steps for k2, v2 in per.items()}
         out["kernels_ms_per_step"] = {k2: round(v2, 4) for k2, v2 in sorted(kern.items())}

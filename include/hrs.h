@@ -158,8 +158,9 @@ hrs_status hrs_partition_pass(void *d_temp, size_t *temp_bytes, const void *keys
  * enabled, every kernel this thread enqueues is bracketed by CUDA events recorded
  * on the launch stream.  hrs_profile_collect synchronises on those events, writes
  * up to `max` records in launch order, returns how many it wrote, and clears the
- * list.  kind: 0 init, 1 histogram/look-back/classify (k_hist), 2 scatter
- * (k_scatter), 3 local sort (pass = size class), 4 copy/fill. */
+ * list.  kind: 0 init, 1 digit histogram (k_hist), 2 rank + look-back + scatter
+ * (k_scatter), 3 local sort (pass = size class), 4 copy/fill, 5 bucket
+ * classification (k_classify). */
 typedef struct {
     int kind;
     int pass;

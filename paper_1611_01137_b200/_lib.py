@@ -83,7 +83,7 @@ class ProfileRecord(ctypes.Structure):
     _fields_ = [("kind", ctypes.c_int), ("pass_", ctypes.c_int), ("ms", ctypes.c_float)]
 
 
-PROFILE_KINDS = {0: "init", 1: "hist", 2: "scatter", 3: "local", 4: "copy"}
+PROFILE_KINDS = {0: "init", 1: "hist", 2: "scatter", 3: "local", 4: "copy", 5: "classify"}
 
 # name -> (restype, argtypes); mirrors include/hrs.h exactly (tests check the header)
 _P = ctypes.c_void_p

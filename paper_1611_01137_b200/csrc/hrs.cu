@@ -70,14 +70,19 @@ constexpr uint32_t DEFAULT_MT_DIV = 4;
 
 // ------------------------------------------------------------------ compile-time configurations
 
-// scatter: THREADS x KPT records per tile; MINB resident CTAs per SM requested
+// scatter: THREADS x KPT records per tile (= the largest KPB); MINB resident CTAs per SM
 template <int KB, int VB>
 struct ScatterCfg {
-    static constexpr int THREADS = (KB == 4 && VB <= 4) ? 256 : 512;
-    static constexpr int KPT = (KB == 4 && VB <= 4) ? 16 : 8;
-    static constexpr int MINB = (KB == 4 && VB <= 4) ? 3 : 2;
+    static constexpr bool SMALL = (KB == 4 && VB <= 4);
+    static constexpr int THREADS = SMALL ? 256 : 512;
+    static constexpr int KPT = SMALL ? 16 : 8;
+    static constexpr int MINB = SMALL ? 2 : 1;
 };
 constexpr int HIST_THREADS = 512;
+constexpr int HIST_STAGES = 3;
+constexpr int HIST_CAP = 4096;  // >= every ScatterCfg KPB
+constexpr int CLASSIFY_THREADS = 256;
+constexpr size_t SMEM_LIMIT = 227 * 1024;
 
 template <int C>
 struct LocalCfg;
@@ -90,7 +95,32 @@ template <> struct LocalCfg<5> { static constexpr int THREADS = 256, KPT = 16; }
 template <> struct LocalCfg<6> { static constexpr int THREADS = 512, KPT = 16; };
 template <> struct LocalCfg<7> { static constexpr int THREADS = 1024, KPT = 16; };
 
-int max_class(int kb, int vb) { return (kb == 4 && vb <= 4) ? 7 : 6; }
+// two-stage TMA prefetch where it fits next to a second resident CTA, else one stage
+template <typename K, typename V, int C>
+struct LocalStages {
+    using LC = LocalCfg<C>;
+    static constexpr int NSTAGE =
+        LocalSmem<K, V, LC::THREADS, LC::KPT, 2>::bytes <= 110 * 1024 ? 2
+        : LocalSmem<K, V, LC::THREADS, LC::KPT, 2>::bytes <= SMEM_LIMIT && LC::THREADS <= 256 ? 2 : 1;
+    static constexpr size_t bytes = LocalSmem<K, V, LC::THREADS, LC::KPT, NSTAGE>::bytes;
+    static constexpr bool fits = bytes <= SMEM_LIMIT;
+};
+
+template <typename K, typename V>
+constexpr int max_class_t() {
+    return LocalStages<K, V, 7>::fits ? 7 : LocalStages<K, V, 6>::fits ? 6 : 5;
+}
+
+int max_class(int kb, int vb) {
+    if (kb == 4) {
+        if (vb == 0) return max_class_t<uint32_t, NoVal>();
+        if (vb == 4) return max_class_t<uint32_t, uint32_t>();
+        return max_class_t<uint32_t, unsigned long long>();
+    }
+    if (vb == 0) return max_class_t<unsigned long long, NoVal>();
+    if (vb == 4) return max_class_t<unsigned long long, uint32_t>();
+    return max_class_t<unsigned long long, unsigned long long>();
+}
 
 uint32_t max_kpb(int kb, int vb) {
     if (kb == 4 && vb <= 4) return ScatterCfg<4, 4>::THREADS * ScatterCfg<4, 4>::KPT;
@@ -187,8 +217,8 @@ struct Plan {
     bool wide = false;  // 64-bit look-back status words
     uint32_t tile_cap = 0, bucket_cap = 0;
     uint32_t local_cap[HRS_NUM_CLASSES] = {0};
-    size_t off_auxk = 0, off_auxv = 0, off_tiles[2] = {0, 0}, off_buckets[2] = {0, 0}, off_subrel = 0,
-           off_status[2] = {0, 0}, off_local[HRS_NUM_CLASSES] = {0}, total = 0;
+    size_t off_auxk = 0, off_auxv = 0, off_tiles[2] = {0, 0}, off_buckets[2] = {0, 0}, off_tot[2] = {0, 0},
+           off_subrel = 0, off_status = 0, off_local[HRS_NUM_CLASSES] = {0}, total = 0;
 };
 
 size_t align_up(size_t x, size_t a) { return (x + a - 1) / a * a; }
@@ -271,9 +301,11 @@ hrs_status make_plan(Plan &pl, uint64_t n, int kb, int vb, int begin, int end, c
         off = align_up(off + sizeof(Tile) * static_cast<size_t>(pl.tile_cap), 256);
         pl.off_buckets[i] = off;
         off = align_up(off + sizeof(Bucket) * static_cast<size_t>(pl.bucket_cap), 256);
-        pl.off_status[i] = off;
-        off = align_up(off + sbytes * RADIX * static_cast<size_t>(pl.tile_cap), 256);
+        pl.off_tot[i] = off;
+        off = align_up(off + sizeof(uint32_t) * RADIX * static_cast<size_t>(pl.bucket_cap), 256);
     }
+    pl.off_status = off;
+    off = align_up(off + sbytes * RADIX * static_cast<size_t>(pl.tile_cap), 256);
     pl.off_subrel = off;
     off = align_up(off + sizeof(uint32_t) * RADIX * static_cast<size_t>(pl.bucket_cap), 256);
     for (int c = 0; c < HRS_NUM_CLASSES; ++c) {
@@ -303,14 +335,12 @@ struct Runner {
     static constexpr int VB = HasVal<V>::value ? sizeof(V) : 0;
     using SC = ScatterCfg<KB, (VB == 0 ? 4 : VB)>;
 
-    static hrs_status init(const Plan &pl, void *temp, cudaStream_t st, int dev, int sms, int root_class,
-                           int counting) {
+    static hrs_status init(const Plan &pl, void *temp, cudaStream_t st, int sms, int root_class, int counting) {
         InitParams ip;
         ip.ctl = at<Ctl>(temp, 0);
         ip.tiles = at<Tile>(temp, pl.off_tiles[1]);
         ip.buckets = at<Bucket>(temp, pl.off_buckets[1]);
-        ip.status = at<void>(temp, pl.off_status[1]);
-        ip.status_bytes = sizeof(S);
+        ip.tot = at<uint32_t>(temp, pl.off_tot[1]);
         ip.root_local = root_class >= 0 ? at<LocalEntry>(temp, pl.off_local[root_class]) : nullptr;
         ip.root_class = root_class;
         ip.n = pl.n;
@@ -320,49 +350,68 @@ struct Runner {
         ip.key_bytes = pl.kb;
         ip.value_bytes = pl.vb;
         const uint64_t T1 = counting ? (pl.n + pl.kpb - 1) / pl.kpb : 0;
-        const uint64_t work = std::max<uint64_t>(T1 * RADIX * sizeof(S) / 16, 1);
-        const int grid = static_cast<int>(std::min<uint64_t>((work + 255) / 256, static_cast<uint64_t>(sms) * 8));
+        const int grid = static_cast<int>(std::min<uint64_t>(std::max<uint64_t>((T1 + 255) / 256, 1),
+                                                             static_cast<uint64_t>(sms) * 4));
         LaunchScope ls(st, 0, 0);
-        k_init<<<std::max(grid, 1), 256, 0, st>>>(ip);
+        k_init<<<grid, 256, 0, st>>>(ip);
         return last_launch();
     }
 
-    static hrs_status hist(const Plan &pl, void *temp, cudaStream_t st, int dev, int sms, int p, const void *xin,
-                           uint16_t src_code, uint64_t *out_hist, uint64_t *out_offsets, bool last) {
+    static hrs_status hist(const Plan &pl, void *temp, cudaStream_t st, int dev, int sms, int p, const void *xin) {
         HistParams hp;
-        std::memset(&hp, 0, sizeof(hp));
         hp.keys = xin;
         hp.p = p;
-        hp.last = last ? 1 : 0;
         hp.lo = pl.lo[p - 1];
-        hp.width = pl.hi[p - 1] - pl.lo[p - 1];
-        hp.mask = (1u << hp.width) - 1u;
+        hp.mask = (1u << (pl.hi[p - 1] - pl.lo[p - 1])) - 1u;
         hp.tiles = at<Tile>(temp, pl.off_tiles[p & 1]);
-        hp.buckets = at<Bucket>(temp, pl.off_buckets[p & 1]);
-        hp.next_tiles = at<Tile>(temp, pl.off_tiles[(p + 1) & 1]);
-        hp.next_buckets = at<Bucket>(temp, pl.off_buckets[(p + 1) & 1]);
-        hp.status = at<void>(temp, pl.off_status[p & 1]);
-        hp.sub_rel = at<uint32_t>(temp, pl.off_subrel);
+        hp.tot = at<uint32_t>(temp, pl.off_tot[p & 1]);
         hp.ctl = at<Ctl>(temp, 0);
-        for (int c = 0; c < HRS_NUM_CLASSES; ++c) {
-            hp.local[c] = at<LocalEntry>(temp, pl.off_local[c]);
-            hp.local_cap[c] = pl.local_cap[c];
-        }
-        hp.tile_cap = pl.tile_cap;
-        hp.bucket_cap = pl.bucket_cap;
-        hp.lt = pl.lt;
-        hp.mt = pl.mt;
-        hp.kpb = pl.kpb;
-        hp.single_class = pl.single_class;
-        hp.src_code = src_code;
-        hp.out_hist = out_hist;
-        hp.out_offsets = out_offsets;
-        auto fn = k_hist<K, S, HIST_THREADS>;
+        auto fn = k_hist<K, HIST_THREADS, HIST_STAGES, HIST_CAP>;
+        const size_t smem = HistSmem<K, HIST_THREADS, HIST_STAGES, HIST_CAP>::bytes;
         int grid = 0;
-        hrs_status s = grid_for(fn, HIST_THREADS, 0, dev, sms, &grid);
+        hrs_status s = grid_for(fn, HIST_THREADS, smem, dev, sms, &grid);
         if (s) return s;
         LaunchScope ls(st, 1, p);
-        fn<<<grid, HIST_THREADS, 0, st>>>(hp);
+        fn<<<grid, HIST_THREADS, smem, st>>>(hp);
+        return last_launch();
+    }
+
+    static hrs_status classify(const Plan &pl, void *temp, cudaStream_t st, int dev, int sms, int p,
+                               uint16_t src_code, uint64_t *out_hist, uint64_t *out_offsets, bool last) {
+        ClassifyParams cp;
+        std::memset(&cp, 0, sizeof(cp));
+        cp.p = p;
+        cp.last = last ? 1 : 0;
+        cp.lo = pl.lo[p - 1];
+        cp.width = pl.hi[p - 1] - pl.lo[p - 1];
+        cp.buckets = at<Bucket>(temp, pl.off_buckets[p & 1]);
+        cp.tot = at<uint32_t>(temp, pl.off_tot[p & 1]);
+        cp.tot_next = at<uint32_t>(temp, pl.off_tot[(p + 1) & 1]);
+        cp.next_tiles = at<Tile>(temp, pl.off_tiles[(p + 1) & 1]);
+        cp.next_buckets = at<Bucket>(temp, pl.off_buckets[(p + 1) & 1]);
+        cp.sub_rel = at<uint32_t>(temp, pl.off_subrel);
+        cp.status = at<void>(temp, pl.off_status);
+        cp.status_bytes = sizeof(S);
+        cp.ctl = at<Ctl>(temp, 0);
+        for (int c = 0; c < HRS_NUM_CLASSES; ++c) {
+            cp.local[c] = at<LocalEntry>(temp, pl.off_local[c]);
+            cp.local_cap[c] = pl.local_cap[c];
+        }
+        cp.tile_cap = pl.tile_cap;
+        cp.bucket_cap = pl.bucket_cap;
+        cp.lt = pl.lt;
+        cp.mt = pl.mt;
+        cp.kpb = pl.kpb;
+        cp.single_class = pl.single_class;
+        cp.src_code = src_code;
+        cp.out_hist = out_hist;
+        cp.out_offsets = out_offsets;
+        auto fn = k_classify<CLASSIFY_THREADS>;
+        int grid = 0;
+        hrs_status s = grid_for(fn, CLASSIFY_THREADS, 0, dev, sms, &grid);
+        if (s) return s;
+        LaunchScope ls(st, 5, p);
+        fn<<<grid, CLASSIFY_THREADS, 0, st>>>(cp);
         return last_launch();
     }
 
@@ -378,10 +427,8 @@ struct Runner {
         sp.mask = (1u << (pl.hi[p - 1] - pl.lo[p - 1])) - 1u;
         sp.tiles = at<Tile>(temp, pl.off_tiles[p & 1]);
         sp.buckets = at<Bucket>(temp, pl.off_buckets[p & 1]);
-        sp.status = at<void>(temp, pl.off_status[p & 1]);
+        sp.status = at<void>(temp, pl.off_status);
         sp.sub_rel = at<uint32_t>(temp, pl.off_subrel);
-        sp.status_next = p < pl.D ? at<void>(temp, pl.off_status[(p + 1) & 1]) : nullptr;
-        sp.status_bytes = sizeof(S);
         sp.ctl = at<Ctl>(temp, 0);
         auto fn = k_scatter<K, V, S, SC::THREADS, SC::KPT, SC::MINB>;
         const size_t smem = ScatterSmem<K, V, SC::THREADS, SC::KPT>::bytes;
@@ -396,35 +443,31 @@ struct Runner {
     template <int C>
     static hrs_status local_one(const Plan &pl, void *temp, cudaStream_t st, int dev, int sms, const void *kin,
                                 void *kout, const void *vin, void *vout) {
-        if constexpr (C > 7) {
+        using LST = LocalStages<K, V, C>;
+        if constexpr (!LST::fits) {
             return HRS_ERROR_INVALID_VALUE;
         } else {
             using LC = LocalCfg<C>;
-            using LS = LocalSmem<K, V, LC::THREADS, LC::KPT>;
-            if constexpr (LS::bytes > 220 * 1024) {
-                return HRS_ERROR_INVALID_VALUE;
-            } else {
-                LocalParams lp;
-                lp.src_keys[SRC_IN] = kin;
-                lp.src_keys[SRC_AUX] = at<void>(temp, pl.off_auxk);
-                lp.src_keys[SRC_OUT] = kout;
-                lp.src_vals[SRC_IN] = vin;
-                lp.src_vals[SRC_AUX] = VB ? at<void>(temp, pl.off_auxv) : nullptr;
-                lp.src_vals[SRC_OUT] = vout;
-                lp.keys_out = kout;
-                lp.vals_out = vout;
-                lp.list = at<LocalEntry>(temp, pl.off_local[C]);
-                lp.count = &at<Ctl>(temp, 0)->nlocal[C];
-                lp.begin_bit = pl.begin;
-                auto fn = k_local<K, V, LC::THREADS, LC::KPT, 1>;
-                int grid = 0;
-                hrs_status s = grid_for(fn, LC::THREADS, LS::bytes, dev, sms, &grid);
-                if (s) return s;
-                grid = static_cast<int>(std::min<uint64_t>(grid, std::max<uint32_t>(pl.local_cap[C], 1)));
-                LaunchScope ls(st, 3, C);
-                fn<<<grid, LC::THREADS, LS::bytes, st>>>(lp);
-                return last_launch();
-            }
+            LocalParams lp;
+            lp.src_keys[SRC_IN] = kin;
+            lp.src_keys[SRC_AUX] = at<void>(temp, pl.off_auxk);
+            lp.src_keys[SRC_OUT] = kout;
+            lp.src_vals[SRC_IN] = vin;
+            lp.src_vals[SRC_AUX] = VB ? at<void>(temp, pl.off_auxv) : nullptr;
+            lp.src_vals[SRC_OUT] = vout;
+            lp.keys_out = kout;
+            lp.vals_out = vout;
+            lp.list = at<LocalEntry>(temp, pl.off_local[C]);
+            lp.count = &at<Ctl>(temp, 0)->nlocal[C];
+            lp.begin_bit = pl.begin;
+            auto fn = k_local<K, V, LC::THREADS, LC::KPT, LST::NSTAGE, 1>;
+            int grid = 0;
+            hrs_status s = grid_for(fn, LC::THREADS, LST::bytes, dev, sms, &grid);
+            if (s) return s;
+            grid = static_cast<int>(std::min<uint64_t>(grid, std::max<uint32_t>(pl.local_cap[C], 1)));
+            LaunchScope ls(st, 3, C);
+            fn<<<grid, LC::THREADS, LST::bytes, st>>>(lp);
+            return last_launch();
         }
     }
 
@@ -446,12 +489,15 @@ struct Runner {
     static hrs_status sort(const Plan &pl, void *temp, const void *kin, void *kout, const void *vin, void *vout,
                            cudaStream_t st, int dev, int sms) {
         hrs_status s;
-        const int root_class = pl.counting ? -1 : (pl.single_class >= 0 ? pl.single_class
-                                                                        : size_class_of((uint32_t)std::max<uint64_t>(pl.n, 1)));
-        if ((s = init(pl, temp, st, dev, sms, pl.n > 0 && pl.begin < pl.end ? root_class : -1, pl.counting ? 1 : 0)))
+        const int root_class =
+            pl.counting ? -1
+                        : (pl.single_class >= 0 ? pl.single_class
+                                                : size_class_of((uint32_t)std::max<uint64_t>(pl.n, 1)));
+        if ((s = init(pl, temp, st, sms, pl.n > 0 && pl.begin < pl.end ? root_class : -1, pl.counting ? 1 : 0)))
             return s;
         if (pl.n == 0) return HRS_SUCCESS;
         if (pl.begin == pl.end) {
+            using VC = typename std::conditional<VB == 8, uint64_t, uint32_t>::type;
             const int grid = static_cast<int>(std::min<uint64_t>((pl.n + 255) / 256, static_cast<uint64_t>(sms) * 8));
             {
                 LaunchScope ls(st, 4, 0);
@@ -460,9 +506,7 @@ struct Runner {
             if ((s = last_launch())) return s;
             if (VB) {
                 LaunchScope ls(st, 4, 0);
-                k_copy<typename std::conditional<VB == 8, uint64_t, uint32_t>::type><<<grid, 256, 0, st>>>(
-                    static_cast<const typename std::conditional<VB == 8, uint64_t, uint32_t>::type *>(vin),
-                    static_cast<typename std::conditional<VB == 8, uint64_t, uint32_t>::type *>(vout), pl.n);
+                k_copy<VC><<<grid, 256, 0, st>>>(static_cast<const VC *>(vin), static_cast<VC *>(vout), pl.n);
                 if ((s = last_launch())) return s;
             }
             return HRS_SUCCESS;
@@ -475,8 +519,9 @@ struct Runner {
                 const bool to_out = ((pl.D - p) % 2) == 0;
                 void *yk = to_out ? kout : auxk;
                 void *yv = to_out ? vout : auxv;
-                if ((s = hist(pl, temp, st, dev, sms, p, xk, to_out ? SRC_OUT : SRC_AUX, nullptr, nullptr,
-                              p == pl.D)))
+                if ((s = hist(pl, temp, st, dev, sms, p, xk))) return s;
+                if ((s = classify(pl, temp, st, dev, sms, p, to_out ? SRC_OUT : SRC_AUX, nullptr, nullptr,
+                                  p == pl.D)))
                     return s;
                 if ((s = scatter(pl, temp, st, dev, sms, p, xk, yk, xv, yv))) return s;
                 xk = yk;
@@ -495,7 +540,7 @@ struct Runner {
                                      void *vout, uint64_t *out_hist, uint64_t *out_offsets, bool do_scatter,
                                      cudaStream_t st, int dev, int sms) {
         hrs_status s;
-        if ((s = init(pl, temp, st, dev, sms, -1, pl.n > 0 ? 1 : 0))) return s;
+        if ((s = init(pl, temp, st, sms, -1, pl.n > 0 ? 1 : 0))) return s;
         const int r = 1 << (pl.hi[0] - pl.lo[0]);
         if (pl.n == 0) {
             uint64_t *p = out_hist ? out_hist : out_offsets;
@@ -506,7 +551,8 @@ struct Runner {
             }
             return HRS_SUCCESS;
         }
-        if ((s = hist(pl, temp, st, dev, sms, 1, kin, SRC_OUT, out_hist, out_offsets, true))) return s;
+        if ((s = hist(pl, temp, st, dev, sms, 1, kin))) return s;
+        if ((s = classify(pl, temp, st, dev, sms, 1, SRC_OUT, out_hist, out_offsets, true))) return s;
         if (do_scatter && (s = scatter(pl, temp, st, dev, sms, 1, kin, kout, vin, vout))) return s;
         return HRS_SUCCESS;
     }

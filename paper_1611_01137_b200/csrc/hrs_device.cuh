@@ -1,27 +1,32 @@
 // hrs_device.cuh -- sm_100a kernels of the stable hybrid MSD radix sort.
 //
 // Paper: Stehle & Jacobsen, arXiv 1611.01137 (PAPER.md lines cited as P:<line>).
-// Every pass p of the MSD recursion (Fig 1) runs two kernels over a
+// Every pass p of the MSD recursion (Fig 1) runs three kernels over a
 // device-resident tile table ("key blocks"), so each pass costs a
 // constant number of launches and the host never reads device memory:
 //
-//   k_hist<p>     per tile: digit histogram with warp-aggregated shared-memory
-//                 atomics (Fig 2), then a decoupled look-back across the
-//                 tiles of the same bucket that turns tile histograms into
-//                 tile-ordered prefix sums (replaces the atomicAdd chunk
-//                 reservation of P:696-703, which is not stable).  The last tile of
-//                 every bucket owns the bucket's histogram: it computes the
-//                 sub-bucket offsets (exclusive prefix sum) and classifies
-//                 the sub-buckets (R1-R3 P:805-811, merging P:552-561), writing the
-//                 next pass's tile/bucket tables and the local-sort lists.
-//   k_scatter<p>  per tile: stable in-tile rank (warp match-any multisplit with
-//                 per-warp digit counters), staging in shared memory, and
-//                 coalesced write-combined stores of every digit run to its
-//                 sub-bucket (Fig 3); values follow their keys.
+//   k_hist<p>      streams the keys of every tile through a TMA bulk-copy ring into
+//                  shared memory and counts the digit with per-warp shared-memory
+//                  atomics (on B200 plain smem atomics run at full HBM
+//                  read rate even for a constant digit -- profiles/r01_micro_hist.txt
+//                  -- so the paper's sorting-network thread reduction, is
+//                  not needed).  Each CTA owns a contiguous run of tiles and adds the
+//                  bucket histograms to global memory once per bucket run.
+//   k_classify<p>  one CTA per bucket: exclusive prefix sum of the bucket histogram
+//                  into sub-bucket offsets and classification of the
+//                  sub-buckets (R1-R3 P:805-811, merging P:552-561) into next-pass
+//                  buckets/tiles and local-sort lists.
+//   k_scatter<p>   per tile, with the next tile already in flight through TMA: a
+//                  STABLE in-tile rank, a decoupled look-back over the preceding
+//                  tiles of the same bucket (tile order = memory order; replaces the
+//                  atomicAdd chunk reservation of P:696-703, which is not stable),
+//                  staging in shared memory and write-combined stores of every digit
+//                  run (Fig 3); values follow their keys.
 //
 // then one k_local launch per size class sorts every bucket of at most
-// ∂ˆ records on chip with a stable LSD radix sort over the remaining bits
-// (P:474-480), skipping digits that are constant across the bucket.
+// ∂ˆ records on chip: a stable LSD radix sort of (key, index) pairs over the
+// remaining bits, skipping digits that are constant across the bucket,
+// and a final gather of the values.
 //
 // Stability everywhere (ties keep input order) is the one deliberate departure
 // from the paper: the output is the unique stable sort.
@@ -36,7 +41,7 @@
 namespace hrs {
 
 constexpr int RADIX = 256;
-constexpr int NBINS = 257;            // 256 digit values + 1 bin for padding lanes
+constexpr int NBINS = 257;  // 256 digit values + 1 bin for padding lanes
 constexpr uint32_t INVALID_DIGIT = 256;
 constexpr uint64_t CTL_MAGIC = 0x4852535f31363131ull;  // "HRS_1611"
 
@@ -73,7 +78,6 @@ struct Ctl {
     uint32_t key_bytes, value_bytes;
     uint32_t ntiles[HRS_MAX_PASSES + 2];    // tiles of pass p (1-based)
     uint32_t nbuckets[HRS_MAX_PASSES + 2];  // buckets of pass p
-    uint32_t claim[HRS_MAX_PASSES + 2];     // dynamic tile claims of k_hist, pass p
     uint32_t nlocal[HRS_NUM_CLASSES];       // entries in local list c
     uint32_t overflow;
     uint32_t pad_;
@@ -125,6 +129,8 @@ template <>
 struct HasVal<NoVal> {
     static constexpr bool value = false;
 };
+template <typename V>
+using ValT = typename std::conditional<HasVal<V>::value, V, uint32_t>::type;
 
 __host__ __device__ __forceinline__ int size_class_of(uint32_t size) {
     int c = 0;
@@ -132,8 +138,9 @@ __host__ __device__ __forceinline__ int size_class_of(uint32_t size) {
     return c;
 }
 
+__host__ __device__ constexpr size_t align16(size_t x) { return (x + 15) & ~size_t(15); }
+
 // Exclusive scan of n <= 288 u32 values in shared memory, in place, by warp 0.
-// Returns nothing; caller syncs before and after.
 __device__ __forceinline__ void warp0_exclusive_scan(uint32_t *a, int n) {
     if (threadIdx.x >= 32) return;
     const int lane = threadIdx.x;
@@ -161,19 +168,159 @@ __device__ __forceinline__ void warp0_exclusive_scan(uint32_t *a, int n) {
     }
 }
 
+// ------------------------------------------------------------------ TMA bulk copies (cp.async.bulk + mbarrier)
+
+__device__ __forceinline__ uint32_t smem_u32(const void *p) {
+    return static_cast<uint32_t>(__cvta_generic_to_shared(p));
+}
+__device__ __forceinline__ void mbar_init(uint64_t *bar, uint32_t count) {
+    asm volatile("mbarrier.init.shared::cta.b64 [%0], %1;" ::"r"(smem_u32(bar)), "r"(count) : "memory");
+}
+__device__ __forceinline__ void mbar_fence_init() {
+    asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
+}
+__device__ __forceinline__ void fence_proxy_async() {
+    asm volatile("fence.proxy.async.shared::cta;" ::: "memory");
+}
+__device__ __forceinline__ void mbar_arrive_expect_tx(uint64_t *bar, uint32_t bytes) {
+    asm volatile("mbarrier.arrive.expect_tx.shared::cta.b64 _, [%0], %1;" ::"r"(smem_u32(bar)), "r"(bytes)
+                 : "memory");
+}
+__device__ __forceinline__ void mbar_wait(uint64_t *bar, uint32_t parity) {
+    asm volatile(
+        "{\n"
+        ".reg .pred P1;\n"
+        "HRS_WAIT_%=:\n"
+        "mbarrier.try_wait.parity.shared::cta.b64 P1, [%0], %1;\n"
+        "@!P1 bra HRS_WAIT_%=;\n"
+        "}\n" ::"r"(smem_u32(bar)),
+        "r"(parity)
+        : "memory");
+}
+__device__ __forceinline__ uint64_t policy_evict_first() {
+    uint64_t p;
+    asm volatile("createpolicy.fractional.L2::evict_first.b64 %0, 1.0;" : "=l"(p));
+    return p;
+}
+__device__ __forceinline__ void bulk_g2s(void *dst, const void *src, uint32_t bytes, uint64_t *bar, uint64_t pol) {
+    asm volatile(
+        "cp.async.bulk.shared::cluster.global.mbarrier::complete_tx::bytes.L2::cache_hint [%0], [%1], %2, [%3], %4;" ::
+            "r"(smem_u32(dst)),
+        "l"(src), "r"(bytes), "r"(smem_u32(bar)), "l"(pol)
+        : "memory");
+}
+
+// A staged segment of `count` elements starting at global `src`: element i lives in
+// shared memory at sbuf[pad + i] for i in [i0, i1) (the 16-byte aligned interior the
+// bulk copy moved); the unaligned head [0, i0) and tail [i1, count) stay in global.
+struct Seg {
+    uint32_t pad, i0, i1;
+};
+template <typename T>
+__device__ __forceinline__ uint32_t seg_plan(const T *src, uint32_t count, Seg &sg) {
+    const uintptr_t a = reinterpret_cast<uintptr_t>(src);
+    sg.pad = static_cast<uint32_t>((a & 15) / sizeof(T));
+    const uintptr_t lo = (a + 15) & ~uintptr_t(15);
+    const uintptr_t hi = (a + static_cast<uintptr_t>(count) * sizeof(T)) & ~uintptr_t(15);
+    if (hi > lo) {
+        sg.i0 = static_cast<uint32_t>((lo - a) / sizeof(T));
+        sg.i1 = static_cast<uint32_t>((hi - a) / sizeof(T));
+        return static_cast<uint32_t>(hi - lo);
+    }
+    sg.i0 = sg.i1 = 0;
+    return 0;
+}
+template <typename T>
+__device__ __forceinline__ void seg_issue(T *sbuf, const T *src, const Seg &sg, uint64_t *bar, uint64_t pol) {
+    if (sg.i1 > sg.i0)
+        bulk_g2s(sbuf + sg.pad + sg.i0, src + sg.i0, (sg.i1 - sg.i0) * static_cast<uint32_t>(sizeof(T)), bar, pol);
+}
+template <typename T>
+__device__ __forceinline__ T seg_get(const T *sbuf, const T *src, const Seg &sg, uint32_t i) {
+    return (i >= sg.i0 && i < sg.i1) ? sbuf[sg.pad + i] : src[i];
+}
+// copy the unaligned head/tail into the staging buffer so sbuf[pad + i] is valid for all i
+template <typename T, int THREADS>
+__device__ __forceinline__ void seg_fill_edges(T *sbuf, const T *src, const Seg &sg, uint32_t count) {
+    const uint32_t nhead = sg.i1 > sg.i0 ? sg.i0 : count;
+    const uint32_t ntail = sg.i1 > sg.i0 ? count - sg.i1 : 0;
+    for (uint32_t j = threadIdx.x; j < nhead + ntail; j += THREADS) {
+        const uint32_t i = j < nhead ? j : sg.i1 + (j - nhead);
+        sbuf[sg.pad + i] = src[i];
+    }
+}
+
+// ------------------------------------------------------------------ stable block rank
+
+// Ranks the KPT keys a warp holds in "warp-striped" order (element e of the tile =
+// warp * 32 * KPT + c * 32 + lane) by digit, stably.  Per column: the warp's running
+// digit counter is read, every lane adds 1 with a non-returning shared atomic (full
+// speed on B200 for any skew), the counter is read back: lanes whose digit occurs
+// once in the column have their rank; only lanes with duplicates run match-any among
+// themselves (its cost grows with the number of distinct values, which is small
+// there).  profiles/r01_micro_rank.txt compares this with match-only and
+// ballot-sliced ranking.
+// On entry rk[c] holds the digit (INVALID_DIGIT for padding lanes); on exit
+// (rank within the warp's run of the digit << 9) | digit.
+template <int KPT>
+__device__ __forceinline__ void rank_walk(uint32_t (&rk)[KPT], uint32_t *mycnt) {
+    const uint32_t ltm = lanemask_lt();
+#pragma unroll
+    for (int c = 0; c < KPT; ++c) {
+        const uint32_t d = rk[c];
+        const uint32_t pre = mycnt[d];
+        __syncwarp();
+        atomicAdd(&mycnt[d], 1u);
+        __syncwarp();
+        const uint32_t k = mycnt[d] - pre;
+        uint32_t r = 0;
+        const uint32_t dup = __ballot_sync(0xffffffffu, k > 1);
+        if (k > 1) {
+            const uint32_t m = __match_any_sync(dup, d);
+            r = __popc(m & ltm);
+        }
+        rk[c] = ((pre + r) << 9) | d;
+    }
+}
+
+// Column scan over warps and exclusive scan over digits: afterwards wcnt[w][d] =
+// start of warp w's run of digit d in the tile, and tot[d] = start of digit d
+// (tot[256] = number of valid elements).  Ends without a trailing barrier.
+template <int THREADS>
+__device__ __forceinline__ void block_rank_scan(uint32_t *wcnt, uint32_t *tot) {
+    constexpr int W = THREADS / 32;
+    for (int d = threadIdx.x; d < NBINS; d += THREADS) {
+        uint32_t run = 0;
+#pragma unroll
+        for (int w = 0; w < W; ++w) {
+            const uint32_t v = wcnt[w * NBINS + d];
+            wcnt[w * NBINS + d] = run;
+            run += v;
+        }
+        tot[d] = run;
+    }
+    __syncthreads();
+    warp0_exclusive_scan(tot, NBINS);
+    __syncthreads();
+    for (int d = threadIdx.x; d < NBINS; d += THREADS) {
+        const uint32_t ls = tot[d];
+#pragma unroll
+        for (int w = 0; w < W; ++w) wcnt[w * NBINS + d] += ls;
+    }
+}
+
 // ------------------------------------------------------------------ init / copy
 
 struct InitParams {
     Ctl *ctl;
-    Tile *tiles;       // pass-1 tile table
-    Bucket *buckets;   // pass-1 bucket table
-    void *status;      // pass-1 status array (to clear)
-    int status_bytes;  // sizeof(S)
+    Tile *tiles;             // pass-1 tile table
+    Bucket *buckets;         // pass-1 bucket table
+    uint32_t *tot;           // pass-1 bucket histograms (row 0 is cleared)
     LocalEntry *root_local;  // list of the root's size class (n <= ∂ˆ)
     int root_class;
     uint64_t n;
     uint32_t kpb;
-    int counting;      // 1: the root bucket is counting-sorted
+    int counting;  // 1: the root bucket is counting-sorted
     int end_bit;
     uint32_t key_bytes, value_bytes;
 };
@@ -184,6 +331,8 @@ __global__ void k_init(InitParams prm) {
     if (blockIdx.x == 0) {
         uint32_t *w = reinterpret_cast<uint32_t *>(prm.ctl);
         for (int i = threadIdx.x; i < static_cast<int>(sizeof(Ctl) / 4); i += blockDim.x) w[i] = 0;
+        if (prm.counting)
+            for (int i = threadIdx.x; i < RADIX; i += blockDim.x) prm.tot[i] = 0;
         __syncthreads();
         if (threadIdx.x == 0) {
             Ctl *c = prm.ctl;
@@ -223,10 +372,6 @@ __global__ void k_init(InitParams prm) {
         tl.bucket = 0;
         prm.tiles[t] = tl;
     }
-    // clear the pass-1 look-back status words (16-byte stores)
-    const uint64_t words16 = (static_cast<uint64_t>(T1) * RADIX * prm.status_bytes) / 16;
-    uint4 *s = reinterpret_cast<uint4 *>(prm.status);
-    for (uint64_t i = tid; i < words16; i += stride) s[i] = make_uint4(0, 0, 0, 0);
 }
 
 template <typename T>
@@ -242,43 +387,154 @@ __global__ void k_fill_u64(uint64_t *p, uint64_t n, uint64_t v) {
         p[i] = v;
 }
 
-// ------------------------------------------------------------------ histogram + look-back + classify
+// ------------------------------------------------------------------ histogram
 
 struct HistParams {
     const void *keys;  // X_{p-1}
     int p;
-    int last;          // 1: digit p is the least-significant one (no further classification)
-    int lo;            // digit bits [lo, lo + width)
-    int width;
+    int lo;
     uint32_t mask;
     const Tile *tiles;
+    uint32_t *tot;  // [bucket][256] of this pass (zeroed by the creator of the bucket)
+    Ctl *ctl;
+};
+
+template <typename K, int THREADS, int NSTAGE, int CAP>
+struct HistSmem {
+    static constexpr int W = THREADS / 32;
+    static constexpr size_t off_bar = 0;
+    static constexpr size_t off_info = align16(sizeof(uint64_t) * NSTAGE);
+    static constexpr size_t off_wh = align16(off_info + sizeof(uint32_t) * 8 * NSTAGE);
+    static constexpr size_t off_stage = align16(off_wh + sizeof(uint32_t) * W * RADIX);
+    static constexpr size_t stage_elems = CAP + 16 / sizeof(K);
+    static constexpr size_t bytes = off_stage + NSTAGE * align16(sizeof(K) * stage_elems);
+};
+
+template <typename K, int THREADS, int NSTAGE, int CAP>
+__global__ void __launch_bounds__(THREADS) k_hist(HistParams prm) {
+    using L = HistSmem<K, THREADS, NSTAGE, CAP>;
+    constexpr int W = THREADS / 32;
+    constexpr int VK = 16 / sizeof(K);
+    extern __shared__ __align__(16) unsigned char smem[];
+    uint64_t *bar = reinterpret_cast<uint64_t *>(smem + L::off_bar);
+    uint32_t *info = reinterpret_cast<uint32_t *>(smem + L::off_info);  // [s][8]: tile, count, bucket, pad, i0, i1
+    uint32_t *wh = reinterpret_cast<uint32_t *>(smem + L::off_wh);
+    auto stage = [&](int s) {
+        return reinterpret_cast<K *>(smem + L::off_stage + s * align16(sizeof(K) * L::stage_elems));
+    };
+    const K *__restrict__ keys = static_cast<const K *>(prm.keys);
+    const int tid = threadIdx.x, warp = tid >> 5;
+    const uint32_t T = prm.ctl->ntiles[prm.p];
+    // a contiguous run of tiles per CTA: bucket histograms are flushed once per run
+    const uint32_t tb = static_cast<uint32_t>((static_cast<uint64_t>(T) * blockIdx.x) / gridDim.x);
+    const uint32_t te = static_cast<uint32_t>((static_cast<uint64_t>(T) * (blockIdx.x + 1)) / gridDim.x);
+    if (tb >= te) return;
+    const uint64_t pol = policy_evict_first();
+
+    auto issue = [&](int s, uint32_t t) {
+        uint32_t *in = info + 8 * s;
+        in[0] = t;
+        if (t >= te) return;
+        const Tile tl = prm.tiles[t];
+        Seg sg;
+        const uint32_t bytes = seg_plan(keys + tl.offs, tl.count, sg);
+        in[1] = tl.count;
+        in[2] = tl.bucket;
+        in[3] = sg.pad;
+        in[4] = sg.i0;
+        in[5] = sg.i1;
+        mbar_arrive_expect_tx(&bar[s], bytes);
+        seg_issue(stage(s), keys + tl.offs, sg, &bar[s], pol);
+    };
+    if (tid == 0) {
+        for (int s = 0; s < NSTAGE; ++s) mbar_init(&bar[s], 1);
+        mbar_fence_init();
+        for (int s = 0; s < NSTAGE; ++s) issue(s, tb + s);
+    }
+    for (int i = tid; i < W * RADIX; i += THREADS) wh[i] = 0;
+    __syncthreads();
+    uint32_t *my = wh + warp * RADIX;
+    for (uint32_t t = tb, it = 0; t < te; ++t, ++it) {
+        const int s = static_cast<int>(it % NSTAGE);
+        const uint32_t par = (it / NSTAGE) & 1u;
+        const uint32_t *in = info + 8 * s;
+        const uint32_t count = in[1], bucket = in[2];
+        Seg sg;
+        sg.pad = in[3];
+        sg.i0 = in[4];
+        sg.i1 = in[5];
+        mbar_wait(&bar[s], par);
+        const K *sb = stage(s);
+        // 16-byte vectors over the staged interior
+        const uint32_t nvec = (sg.i1 - sg.i0) / VK;
+        const uint4 *vb = reinterpret_cast<const uint4 *>(sb + sg.pad + sg.i0);
+#pragma unroll 4
+        for (uint32_t v = tid; v < nvec; v += THREADS) {
+            const uint4 w = vb[v];
+            const K *kk = reinterpret_cast<const K *>(&w);
+#pragma unroll
+            for (int j = 0; j < VK; ++j) atomicAdd(&my[digit_of(kk[j], prm.lo, prm.mask)], 1u);
+        }
+        // unaligned head / tail straight from global
+        {
+            const K *src = keys + prm.tiles[t].offs;
+            const uint32_t nhead = sg.i1 > sg.i0 ? sg.i0 : count;
+            const uint32_t ntail = sg.i1 > sg.i0 ? count - sg.i1 : 0;
+            for (uint32_t j = tid; j < nhead + ntail; j += THREADS) {
+                const uint32_t i = j < nhead ? j : sg.i1 + (j - nhead);
+                atomicAdd(&my[digit_of(src[i], prm.lo, prm.mask)], 1u);
+            }
+        }
+        __syncthreads();
+        if (tid == 0) {
+            fence_proxy_async();
+            issue(s, t + NSTAGE);
+        }
+        const bool flush = (t + 1 == te) || (prm.tiles[t + 1].bucket != bucket);
+        if (flush) {
+            for (int d = tid; d < RADIX; d += THREADS) {
+                uint32_t sum = 0;
+#pragma unroll
+                for (int w = 0; w < W; ++w) {
+                    sum += wh[w * RADIX + d];
+                    wh[w * RADIX + d] = 0;
+                }
+                if (sum) atomicAdd(&prm.tot[static_cast<uint64_t>(bucket) * RADIX + d], sum);
+            }
+            __syncthreads();
+        }
+    }
+}
+
+// ------------------------------------------------------------------ classification (one CTA per bucket)
+
+struct ClassifyParams {
+    int p;
+    int last;  // 1: digit p is the least-significant one (no further classification)
+    int lo;    // digit bits [lo, lo + width)
+    int width;
     const Bucket *buckets;
+    const uint32_t *tot;  // this pass
+    uint32_t *tot_next;   // next pass (rows of created buckets are cleared)
     Tile *next_tiles;
     Bucket *next_buckets;
-    void *status;
     uint32_t *sub_rel;  // [bucket][256] sub-bucket starts relative to the bucket
+    void *status;       // look-back words of this pass: cleared for ntiles[p] tiles
+    int status_bytes;
     Ctl *ctl;
     LocalEntry *local[HRS_NUM_CLASSES];
     uint32_t local_cap[HRS_NUM_CLASSES];
     uint32_t tile_cap, bucket_cap;
     uint32_t lt, mt, kpb;
-    int single_class;  // >= 0: every local entry goes to this class (ablation)
-    uint16_t src_code; // buffer holding X_p
+    int single_class;       // >= 0: every local entry goes to this class (ablation)
+    uint16_t src_code;      // buffer holding X_p
     uint64_t *out_hist;     // building block: the root bucket's histogram
     uint64_t *out_offsets;  // building block: the root bucket's sub-bucket starts (+ n)
 };
 
-template <typename K>
-__device__ __forceinline__ void hist_add(uint32_t *hist, uint32_t d) {
-    // warp-aggregated shared-memory atomic: one atomicAdd per group of equal digits
-    const uint32_t m = __match_any_sync(0xffffffffu, d);
-    if (d != INVALID_DIGIT && (m & lanemask_lt()) == 0) atomicAdd(&hist[d], static_cast<uint32_t>(__popc(m)));
-}
-
-template <typename K, typename S, int THREADS>
-__device__ void classify_bucket(const HistParams &prm, const Bucket &bk, uint32_t bucket_id, const S *tot_in,
-                                uint32_t *sm) {
-    // sm: scratch of >= 8 * 257 u32
+template <int THREADS>
+__device__ void classify_bucket(const ClassifyParams &prm, const Bucket &bk, uint32_t bucket_id, uint32_t *sm) {
+    static_assert(THREADS >= RADIX, "one thread per digit");
     uint32_t *tot = sm;                 // 256 (+1)
     uint32_t *start = sm + 1 * NBINS;   // exclusive prefix of tot
     uint32_t *ct = sm + 2 * NBINS;      // child tiles per digit -> exclusive
@@ -287,25 +543,23 @@ __device__ void classify_bucket(const HistParams &prm, const Bucket &bk, uint32_
     uint32_t *gmulti = sm + 5 * NBINS;  // 1 if the group merged >= 2 sub-buckets
     uint32_t *misc = sm + 6 * NBINS;    // [0] base tile, [1] base bucket, [2..9] class counts, [10..17] class bases
     const int tid = threadIdx.x;
-    const S VAL = StatusBits<S>::VAL;
     for (int d = tid; d < NBINS; d += THREADS) {
-        uint32_t v = d < RADIX ? static_cast<uint32_t>(tot_in[d] & VAL) : 0u;
+        const uint32_t v = d < RADIX ? prm.tot[static_cast<uint64_t>(bucket_id) * RADIX + d] : 0u;
         tot[d] = v;
         start[d] = v;
         glead[d] = 0;
         gmulti[d] = 0;
-        bool cnt = !prm.last && v > prm.lt;
+        const bool cnt = !prm.last && v > prm.lt;
         ct[d] = cnt ? (v + prm.kpb - 1) / prm.kpb : 0u;
         cb[d] = cnt ? 1u : 0u;
     }
     if (tid < 32) misc[tid] = 0;
     __syncthreads();
-    // three exclusive scans, one per warp
-    if (tid < 32) warp0_exclusive_scan(start, NBINS);
+    warp0_exclusive_scan(start, NBINS);
     __syncthreads();
-    if (tid < 32) warp0_exclusive_scan(ct, NBINS);
+    warp0_exclusive_scan(ct, NBINS);
     __syncthreads();
-    if (tid < 32) warp0_exclusive_scan(cb, NBINS);
+    warp0_exclusive_scan(cb, NBINS);
     __syncthreads();
     const uint64_t boffs = bk.offs;
     for (int d = tid; d < RADIX; d += THREADS) prm.sub_rel[static_cast<uint64_t>(bucket_id) * RADIX + d] = start[d];
@@ -318,7 +572,7 @@ __device__ void classify_bucket(const HistParams &prm, const Bucket &bk, uint32_
     if (prm.last) return;
 
     // ---- counting children: next-pass buckets and their tiles (R2, R4)
-    const uint32_t TT = ct[RADIX];  // exclusive scan over 257 entries: ct[256] = total
+    const uint32_t TT = ct[RADIX];
     const uint32_t NC = cb[RADIX];
     if (tid == 0) {
         uint32_t bt = 0, bb = 0;
@@ -333,24 +587,27 @@ __device__ void classify_bucket(const HistParams &prm, const Bucket &bk, uint32_
     // ---- local candidates: greedy merge (R3 / reading #5)
     bool has_small = false;
     for (int d = tid; d < RADIX; d += THREADS) {
-        uint32_t s = tot[d];
+        const uint32_t s = tot[d];
         if (s > 0 && s <= prm.lt && s < prm.mt) has_small = true;
     }
     has_small = __syncthreads_or(has_small);
     if (!has_small) {
         // no sub-bucket can merge: every candidate is its own group
         for (int d = tid; d < RADIX; d += THREADS) {
-            uint32_t s = tot[d];
+            const uint32_t s = tot[d];
             if (s > 0 && s <= prm.lt) glead[d] = s;
         }
     } else if (tid == 0) {
         int gl = -1;
         uint32_t gs = 0, gc = 0;
         for (int d = 0; d < RADIX; ++d) {
-            uint32_t s = tot[d];
+            const uint32_t s = tot[d];
             if (s == 0) continue;
             if (s > prm.lt) {
-                if (gl >= 0) { glead[gl] = gs; gmulti[gl] = gc > 1; }
+                if (gl >= 0) {
+                    glead[gl] = gs;
+                    gmulti[gl] = gc > 1;
+                }
                 gl = -1;
                 continue;
             }
@@ -358,91 +615,95 @@ __device__ void classify_bucket(const HistParams &prm, const Bucket &bk, uint32_
                 gs += s;
                 ++gc;
             } else {
-                if (gl >= 0) { glead[gl] = gs; gmulti[gl] = gc > 1; }
+                if (gl >= 0) {
+                    glead[gl] = gs;
+                    gmulti[gl] = gc > 1;
+                }
                 gl = d;
                 gs = s;
                 gc = 1;
             }
         }
-        if (gl >= 0) { glead[gl] = gs; gmulti[gl] = gc > 1; }
+        if (gl >= 0) {
+            glead[gl] = gs;
+            gmulti[gl] = gc > 1;
+        }
     }
     __syncthreads();
     // per-class slot allocation
-    uint32_t my_slot[(RADIX + THREADS - 1) / THREADS];
-    int my_cls[(RADIX + THREADS - 1) / THREADS];
+    int my_cls = -1;
+    uint32_t my_slot = 0;
+    if (tid < RADIX && glead[tid]) {
+        my_cls = prm.single_class >= 0 ? prm.single_class : size_class_of(glead[tid]);
+        my_slot = atomicAdd(&misc[2 + my_cls], 1u);
+    }
+    // statistics: warp reductions of the next pass's records, local records, merged groups
+    unsigned long long recs_next = 0, lrecs = 0, merged = 0;
+    if (tid < RADIX) {
+        const uint32_t s = tot[tid];
+        if (s > prm.lt) recs_next = s;
+        lrecs = glead[tid];
+        merged = gmulti[tid];
+    }
 #pragma unroll
-    for (int i = 0; i < (RADIX + THREADS - 1) / THREADS; ++i) {
-        int d = tid + i * THREADS;
-        my_cls[i] = -1;
-        if (d < RADIX && glead[d]) {
-            int c = prm.single_class >= 0 ? prm.single_class : size_class_of(glead[d]);
-            my_cls[i] = c;
-            my_slot[i] = atomicAdd(&misc[2 + c], 1u);
-        }
+    for (int o = 16; o > 0; o >>= 1) {
+        recs_next += __shfl_xor_sync(0xffffffffu, recs_next, o);
+        lrecs += __shfl_xor_sync(0xffffffffu, lrecs, o);
+        merged += __shfl_xor_sync(0xffffffffu, merged, o);
     }
-    __syncthreads();
-    if (tid < HRS_NUM_CLASSES) {
-        uint32_t cnt = misc[2 + tid];
-        uint32_t base = cnt ? atomicAdd(&prm.ctl->nlocal[tid], cnt) : 0u;
-        if (base + cnt > prm.local_cap[tid]) atomicExch(&prm.ctl->overflow, 1u);
-        misc[10 + tid] = base;
-    }
-    if (tid == 32) {
-        // statistics: records of the next pass, local records, merged groups
-        unsigned long long recs_next = 0, lrecs = 0, merged = 0;
-        for (int d = 0; d < RADIX; ++d) {
-            uint32_t s = tot[d];
-            if (!prm.last && s > prm.lt) recs_next += s;
-            if (glead[d]) { lrecs += glead[d]; merged += gmulti[d]; }
-        }
+    if ((tid & 31) == 0 && tid < RADIX) {
         if (recs_next) atomicAdd(&prm.ctl->recs_in_pass[prm.p + 1], recs_next);
         if (lrecs) atomicAdd(&prm.ctl->local_recs, lrecs);
         if (merged) atomicAdd(&prm.ctl->merged_groups, merged);
     }
     __syncthreads();
+    if (tid < HRS_NUM_CLASSES) {
+        const uint32_t cnt = misc[2 + tid];
+        const uint32_t base = cnt ? atomicAdd(&prm.ctl->nlocal[tid], cnt) : 0u;
+        if (cnt && base + cnt > prm.local_cap[tid]) atomicExch(&prm.ctl->overflow, 1u);
+        misc[10 + tid] = base;
+    }
+    __syncthreads();
     const int hi_p = prm.lo + prm.width;
-#pragma unroll
-    for (int i = 0; i < (RADIX + THREADS - 1) / THREADS; ++i) {
-        int d = tid + i * THREADS;
-        if (my_cls[i] >= 0) {
-            int c = my_cls[i];
-            uint32_t slot = misc[10 + c] + my_slot[i];
-            if (slot < prm.local_cap[c]) {
-                LocalEntry e;
-                e.offs = boffs + start[d];
-                e.count = glead[d];
-                e.hi_bit = static_cast<uint16_t>(gmulti[d] ? hi_p : prm.lo);
-                e.src = prm.src_code;
-                prm.local[c][slot] = e;
-            }
+    if (my_cls >= 0) {
+        const uint32_t slot = misc[10 + my_cls] + my_slot;
+        if (slot < prm.local_cap[my_cls]) {
+            LocalEntry e;
+            e.offs = boffs + start[tid];
+            e.count = glead[tid];
+            e.hi_bit = static_cast<uint16_t>(gmulti[tid] ? hi_p : prm.lo);
+            e.src = prm.src_code;
+            prm.local[my_cls][slot] = e;
         }
     }
-    // child buckets
+    // child buckets (their histogram rows of the next pass are cleared here)
     const uint32_t bt = misc[0], bb = misc[1];
-    for (int d = tid; d < RADIX; d += THREADS) {
-        uint32_t s = tot[d];
-        if (!(s > prm.lt)) continue;
-        uint32_t id = bb + cb[d];
-        if (id >= prm.bucket_cap) continue;
-        Bucket nb;
-        nb.offs = boffs + start[d];
-        nb.count = s;
-        nb.first_tile = bt + ct[d];
-        nb.ntiles = (s + prm.kpb - 1) / prm.kpb;
-        nb.pad = 0;
-        prm.next_buckets[id] = nb;
+    if (tid < RADIX) {
+        const uint32_t s = tot[tid];
+        const uint32_t id = bb + cb[tid];
+        if (s > prm.lt && id < prm.bucket_cap) {
+            Bucket nb;
+            nb.offs = boffs + start[tid];
+            nb.count = s;
+            nb.first_tile = bt + ct[tid];
+            nb.ntiles = (s + prm.kpb - 1) / prm.kpb;
+            nb.pad = 0;
+            prm.next_buckets[id] = nb;
+        }
+    }
+    for (uint32_t i = tid; i < NC * RADIX; i += THREADS) {
+        const uint32_t id = bb + i / RADIX;
+        if (id < prm.bucket_cap) prm.tot_next[static_cast<uint64_t>(id) * RADIX + (i % RADIX)] = 0;
     }
     // child tiles, spread over the block (a child can own many tiles)
     for (uint32_t i = tid; i < TT; i += THREADS) {
-        // find digit d with ct[d] <= i < ct[d+1]
-        int lo = 0, hi = RADIX - 1;
+        int lo = 0, hi = RADIX - 1;  // largest d with ct[d] <= i
         while (lo < hi) {
-            int mid = (lo + hi + 1) >> 1;
-            if (ct[mid] <= i) lo = mid; else hi = mid - 1;
+            const int mid = (lo + hi + 1) >> 1;
+            if (ct[mid] <= i) lo = mid;
+            else hi = mid - 1;
         }
-        // skip digits with zero child tiles sharing the same start
-        int d = lo;
-        while (d < RADIX - 1 && ct[d + 1] <= i) ++d;
+        const int d = lo;
         const uint32_t k = i - ct[d];
         const uint32_t s = tot[d];
         if (bt + i >= prm.tile_cap) continue;
@@ -454,147 +715,22 @@ __device__ void classify_bucket(const HistParams &prm, const Bucket &bk, uint32_
     }
 }
 
-template <typename K, typename S, int THREADS>
-__global__ void __launch_bounds__(THREADS) k_hist(HistParams prm) {
-    static_assert(THREADS >= RADIX, "one thread per digit in the look-back");
-    __shared__ uint32_t hist[RADIX];
-    __shared__ uint32_t s_tile;
-    __shared__ S tot[RADIX];
-    __shared__ uint32_t scratch[8 * NBINS];
-    using SB = StatusBits<S>;
-    const K *__restrict__ keys = static_cast<const K *>(prm.keys);
-    S *status = static_cast<S *>(prm.status);
-    Ctl *ctl = prm.ctl;
-    const uint32_t T = ctl->ntiles[prm.p];
-    const int tid = threadIdx.x;
-    constexpr int VK = 16 / sizeof(K);  // keys per 16-byte vector
-    constexpr int U = 4;                // vectors in flight per thread
-
-    for (;;) {
-        if (tid == 0) s_tile = atomicAdd(&ctl->claim[prm.p], 1u);
-        for (int i = tid; i < RADIX; i += THREADS) hist[i] = 0;
-        __syncthreads();
-        const uint32_t t = s_tile;
-        if (t >= T) break;
-        const Tile tile = prm.tiles[t];
-        const K *src = keys + tile.offs;
-        const uint32_t count = tile.count;
-        // ---- histogram: scalar head up to 16-byte alignment, 16-byte vectors, scalar tail
-        const uint32_t mis = static_cast<uint32_t>((reinterpret_cast<uintptr_t>(src) & 15u) / sizeof(K));
-        const uint32_t head = min(count, mis ? static_cast<uint32_t>(VK) - mis : 0u);
-        const uint32_t nvec = (count - head) / VK;
-        const uint32_t tail0 = head + nvec * VK;
-        if (tid < 32) {
-            const uint32_t ntail = count - tail0;
-            const uint32_t u = static_cast<uint32_t>(tid);
-            uint32_t d = INVALID_DIGIT;
-            if (u < head) d = digit_of(src[u], prm.lo, prm.mask);
-            else if (u - head < ntail) d = digit_of(src[tail0 + (u - head)], prm.lo, prm.mask);
-            hist_add<K>(hist, d);
-        }
-        const uint4 *vsrc = reinterpret_cast<const uint4 *>(src + head);
-        for (uint32_t vb = 0; vb < nvec; vb += THREADS * U) {
-            uint4 w[U];
-#pragma unroll
-            for (int u = 0; u < U; ++u) {
-                uint32_t v = vb + u * THREADS + tid;
-                if (v < nvec) w[u] = __ldg(vsrc + v);
-            }
-#pragma unroll
-            for (int u = 0; u < U; ++u) {
-                const bool ok = vb + u * THREADS + tid < nvec;
-                const K *kk = reinterpret_cast<const K *>(&w[u]);
-#pragma unroll
-                for (int j = 0; j < VK; ++j) {
-                    uint32_t d = ok ? digit_of(kk[j], prm.lo, prm.mask) : INVALID_DIGIT;
-                    hist_add<K>(hist, d);
-                }
-            }
-        }
-        __syncthreads();
-        // ---- decoupled look-back over the tiles of this bucket (tile order = memory order)
-        const Bucket bk = prm.buckets[tile.bucket];
-        const bool first = t == bk.first_tile;
-        const bool lastt = t + 1 == bk.first_tile + bk.ntiles;
-        if (tid < RADIX) {
-            const S c = hist[tid];
-            S *st = status + static_cast<uint64_t>(t) * RADIX + tid;
-            S incl;
-            if (first) {
-                incl = c;
-                st_volatile(st, static_cast<S>(SB::INC | c));
-            } else {
-                st_volatile(st, static_cast<S>(SB::AGG | c));
-                S excl = 0;
-                const S *q = st - RADIX;
-                for (;;) {
-                    const S v = ld_volatile(q);
-                    if ((v & SB::FLAGS) == 0) continue;  // predecessor not published yet
-                    excl += v & SB::VAL;
-                    if (v & SB::INC) break;
-                    q -= RADIX;
-                }
-                incl = excl + c;
-                st_volatile(st, static_cast<S>(SB::INC | incl));
-            }
-            if (lastt) tot[tid] = incl;
-        }
-        if (lastt) {
-            __syncthreads();
-            classify_bucket<K, S, THREADS>(prm, bk, tile.bucket, tot, scratch);
-        }
-        __syncthreads();
-    }
-}
-
-// ------------------------------------------------------------------ stable block rank
-
-// Ranks the KPT keys a warp holds in "warp-striped" order (element e of the block
-// = warp * 32 * KPT + c * 32 + lane) by digit, stably: rank = (#elements of smaller
-// digit) + (#elements of equal digit earlier in element order).  Result per key:
-// the rank of the key within its warp's run of the digit, packed (r << 9) | digit;
-// wcnt[w][d] ends up holding the block-wide start of warp w's run of digit d.
-//   wcnt: W * NBINS u32, tot: NBINS u32 (shared)
-template <int THREADS, int KPT>
-__device__ __forceinline__ void warp_rank_walk(uint32_t (&rk)[KPT], uint32_t *mycnt) {
-    // on entry rk[c] holds the digit of key c (INVALID_DIGIT for padding lanes)
-    const uint32_t ltm = lanemask_lt();
-#pragma unroll
-    for (int c = 0; c < KPT; ++c) {
-        const uint32_t d = rk[c];
-        const uint32_t m = __match_any_sync(0xffffffffu, d);
-        const uint32_t below = m & ltm;
-        const uint32_t pre = mycnt[d];
-        __syncwarp();
-        if (below == 0) mycnt[d] = pre + __popc(m);
-        __syncwarp();
-        rk[c] = ((pre + __popc(below)) << 9) | d;
-    }
-}
-
-// Column scan over warps and exclusive scan over digits: afterwards wcnt[w][d] =
-// start of warp w's run of digit d in the block, and tot[d] = start of digit d
-// (tot[256] = number of valid elements).
 template <int THREADS>
-__device__ __forceinline__ void block_rank_scan(uint32_t *wcnt, uint32_t *tot) {
-    constexpr int W = THREADS / 32;
-    for (int d = threadIdx.x; d < NBINS; d += THREADS) {
-        uint32_t run = 0;
-#pragma unroll
-        for (int w = 0; w < W; ++w) {
-            const uint32_t v = wcnt[w * NBINS + d];
-            wcnt[w * NBINS + d] = run;
-            run += v;
-        }
-        tot[d] = run;
+__global__ void __launch_bounds__(THREADS) k_classify(ClassifyParams prm) {
+    __shared__ uint32_t scratch[7 * NBINS];
+    // clear the look-back words of this pass (the scatter that follows uses them)
+    {
+        const uint64_t words16 = (static_cast<uint64_t>(prm.ctl->ntiles[prm.p]) * RADIX * prm.status_bytes) / 16;
+        uint4 *s = static_cast<uint4 *>(prm.status);
+        for (uint64_t i = static_cast<uint64_t>(blockIdx.x) * THREADS + threadIdx.x; i < words16;
+             i += static_cast<uint64_t>(gridDim.x) * THREADS)
+            s[i] = make_uint4(0, 0, 0, 0);
     }
-    __syncthreads();
-    warp0_exclusive_scan(tot, NBINS);
-    __syncthreads();
-    for (int d = threadIdx.x; d < NBINS; d += THREADS) {
-        const uint32_t ls = tot[d];
-#pragma unroll
-        for (int w = 0; w < W; ++w) wcnt[w * NBINS + d] += ls;
+    const uint32_t nb = prm.ctl->nbuckets[prm.p];
+    for (uint32_t b = blockIdx.x; b < nb; b += gridDim.x) {
+        const Bucket bk = prm.buckets[b];
+        classify_bucket<THREADS>(prm, bk, b, scratch);
+        __syncthreads();
     }
 }
 
@@ -610,103 +746,190 @@ struct ScatterParams {
     uint32_t mask;
     const Tile *tiles;
     const Bucket *buckets;
-    const void *status;
+    void *status;
     const uint32_t *sub_rel;
-    void *status_next;  // cleared for pass p+1 (may be NULL)
-    int status_bytes;
     Ctl *ctl;
+};
+
+struct StageInfo {
+    uint32_t tile, count, bucket, kpad, k0, k1, vpad, v0, v1, pad_;
+    uint64_t offs;
 };
 
 template <typename K, typename V, int THREADS, int KPT>
 struct ScatterSmem {
     static constexpr int W = THREADS / 32;
     static constexpr int KPB = THREADS * KPT;
-    static constexpr size_t off_wcnt = 0;
-    static constexpr size_t off_tot = off_wcnt + sizeof(uint32_t) * W * NBINS;
-    static constexpr size_t off_gbase = (off_tot + sizeof(uint32_t) * NBINS + 15) & ~size_t(15);
-    static constexpr size_t off_keys = off_gbase + sizeof(unsigned long long) * RADIX;
-    static constexpr size_t off_vals = (off_keys + sizeof(K) * KPB + 15) & ~size_t(15);
-    static constexpr size_t bytes = off_vals + (HasVal<V>::value ? sizeof(V) * KPB : 0);
+    using VT = ValT<V>;
+    static constexpr bool HV = HasVal<V>::value;
+    static constexpr size_t kst_elems = KPB + 16 / sizeof(K);
+    static constexpr size_t vst_elems = KPB + 16 / sizeof(VT);
+    static constexpr size_t off_bar = 0;
+    static constexpr size_t off_info = 16;
+    static constexpr size_t off_wcnt = align16(off_info + 2 * sizeof(StageInfo));
+    static constexpr size_t off_tot = align16(off_wcnt + sizeof(uint32_t) * W * NBINS);
+    static constexpr size_t off_gbase = align16(off_tot + sizeof(uint32_t) * 288);
+    static constexpr size_t off_kst = align16(off_gbase + sizeof(unsigned long long) * RADIX);
+    static constexpr size_t kst_bytes = align16(sizeof(K) * kst_elems);
+    static constexpr size_t off_vst = off_kst + 2 * kst_bytes;
+    static constexpr size_t vst_bytes = HV ? align16(sizeof(VT) * vst_elems) : 0;
+    static constexpr size_t off_skeys = off_vst + 2 * vst_bytes;
+    static constexpr size_t off_svals = align16(off_skeys + sizeof(K) * KPB);
+    static constexpr size_t bytes = off_svals + (HV ? align16(sizeof(VT) * KPB) : 0);
 };
 
 template <typename K, typename V, typename S, int THREADS, int KPT, int MINB>
 __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
     using L = ScatterSmem<K, V, THREADS, KPT>;
+    using SB = StatusBits<S>;
     constexpr bool HV = HasVal<V>::value;
-    using VT = typename std::conditional<HV, V, uint32_t>::type;
+    using VT = ValT<V>;
     extern __shared__ __align__(16) unsigned char smem[];
+    uint64_t *bar = reinterpret_cast<uint64_t *>(smem + L::off_bar);
+    StageInfo *info = reinterpret_cast<StageInfo *>(smem + L::off_info);
     uint32_t *wcnt = reinterpret_cast<uint32_t *>(smem + L::off_wcnt);
     uint32_t *tot = reinterpret_cast<uint32_t *>(smem + L::off_tot);
     unsigned long long *gbase = reinterpret_cast<unsigned long long *>(smem + L::off_gbase);
-    K *skeys = reinterpret_cast<K *>(smem + L::off_keys);
-    VT *svals = reinterpret_cast<VT *>(smem + L::off_vals);
+    K *skeys = reinterpret_cast<K *>(smem + L::off_skeys);
+    VT *svals = reinterpret_cast<VT *>(smem + L::off_svals);
+    auto kst = [&](int s) { return reinterpret_cast<K *>(smem + L::off_kst + s * L::kst_bytes); };
+    auto vst = [&](int s) { return reinterpret_cast<VT *>(smem + L::off_vst + s * L::vst_bytes); };
 
     const K *__restrict__ kin = static_cast<const K *>(prm.keys_in);
     K *__restrict__ kout = static_cast<K *>(prm.keys_out);
     const VT *__restrict__ vin = static_cast<const VT *>(prm.vals_in);
     VT *__restrict__ vout = static_cast<VT *>(prm.vals_out);
-    const S *status = static_cast<const S *>(prm.status);
+    S *status = static_cast<S *>(prm.status);
     const int tid = threadIdx.x, lane = tid & 31, warp = tid >> 5;
     const uint32_t wbase = static_cast<uint32_t>(warp) * 32 * KPT;
     const uint32_t T = prm.ctl->ntiles[prm.p];
+    if (blockIdx.x >= T) return;
+    const uint64_t pol = policy_evict_first();
 
-    for (uint32_t t = blockIdx.x; t < T; t += gridDim.x) {
-        const Tile tile = prm.tiles[t];
-        const uint32_t count = tile.count;
-        S st = 0;
-        uint32_t srel = 0;
-        if (tid < RADIX) {
-            st = status[static_cast<uint64_t>(t) * RADIX + tid];
-            srel = prm.sub_rel[static_cast<uint64_t>(tile.bucket) * RADIX + tid];
+    // tiles blockIdx.x, blockIdx.x + gridDim.x, ...: every CTA is resident (persistent
+    // grid), so the look-back on lower-numbered tiles always makes progress
+    auto issue = [&](int s, uint32_t t) {
+        StageInfo &in = info[s];
+        in.tile = t;
+        if (t >= T) return;
+        const Tile tl = prm.tiles[t];
+        in.count = tl.count;
+        in.bucket = tl.bucket;
+        in.offs = tl.offs;
+        Seg sk, sv;
+        uint32_t bytes = seg_plan(kin + tl.offs, tl.count, sk);
+        in.kpad = sk.pad;
+        in.k0 = sk.i0;
+        in.k1 = sk.i1;
+        if (HV) {
+            bytes += seg_plan(vin + tl.offs, tl.count, sv);
+            in.vpad = sv.pad;
+            in.v0 = sv.i0;
+            in.v1 = sv.i1;
         }
-        const uint64_t boffs = prm.buckets[tile.bucket].offs;
-        // ---- load (warp-striped, coalesced)
+        mbar_arrive_expect_tx(&bar[s], bytes);
+        seg_issue(kst(s), kin + tl.offs, sk, &bar[s], pol);
+        if (HV) seg_issue(vst(s), vin + tl.offs, sv, &bar[s], pol);
+    };
+    if (tid == 0) {
+        mbar_init(&bar[0], 1);
+        mbar_init(&bar[1], 1);
+        mbar_fence_init();
+        issue(0, blockIdx.x);
+        issue(1, blockIdx.x + gridDim.x);
+    }
+    for (int i = tid; i < (THREADS / 32) * NBINS; i += THREADS) wcnt[i] = 0;
+    __syncthreads();
+
+    for (uint32_t it = 0;; ++it) {
+        const int s = static_cast<int>(it & 1u);
+        const uint32_t par = (it >> 1) & 1u;
+        const StageInfo in = info[s];
+        if (in.tile >= T) break;
+        const uint32_t t = in.tile, count = in.count;
+        // per-digit bucket data for the look-back and the destinations
+        uint32_t srel = 0;
+        uint64_t boffs = 0;
+        bool first = false;
+        if (tid < RADIX) {
+            const Bucket bk = prm.buckets[in.bucket];
+            boffs = bk.offs;
+            first = t == bk.first_tile;
+            srel = prm.sub_rel[static_cast<uint64_t>(in.bucket) * RADIX + tid];
+        }
+        Seg sk, sv;
+        sk.pad = in.kpad;
+        sk.i0 = in.k0;
+        sk.i1 = in.k1;
+        sv.pad = in.vpad;
+        sv.i0 = in.v0;
+        sv.i1 = in.v1;
+        const K *ksrc = kin + in.offs;
+        const VT *vsrc = HV ? vin + in.offs : nullptr;
+        mbar_wait(&bar[s], par);
+        // ---- keys into registers (warp-striped), stable rank
         K key[KPT];
-        VT val[KPT];
-        const K *ksrc = kin + tile.offs;
-        const VT *vsrc = HV ? vin + tile.offs : nullptr;
+        uint32_t rk[KPT];
+        const K *ks = kst(s);
 #pragma unroll
         for (int c = 0; c < KPT; ++c) {
             const uint32_t e = wbase + c * 32 + lane;
             if (e < count) {
-                key[c] = ksrc[e];
-                if (HV) val[c] = vsrc[e];
+                key[c] = seg_get(ks, ksrc, sk, e);
+                rk[c] = digit_of(key[c], prm.lo, prm.mask);
+            } else {
+                rk[c] = INVALID_DIGIT;
             }
         }
-        for (int i = tid; i < (THREADS / 32) * NBINS; i += THREADS) wcnt[i] = 0;
-        __syncthreads();
-        // ---- stable rank
-        uint32_t rk[KPT];
-        if (wbase < count) {
-#pragma unroll
-            for (int c = 0; c < KPT; ++c) {
-                const uint32_t e = wbase + c * 32 + lane;
-                rk[c] = e < count ? digit_of(key[c], prm.lo, prm.mask) : INVALID_DIGIT;
-            }
-            warp_rank_walk<THREADS, KPT>(rk, wcnt + warp * NBINS);
-        }
+        if (wbase < count) rank_walk<KPT>(rk, wcnt + warp * NBINS);
         __syncthreads();
         block_rank_scan<THREADS>(wcnt, tot);
+        // ---- publish this tile's digit counts for the successors' look-back
+        S cnt_d = 0;
         if (tid < RADIX) {
-            // destination of smem slot j holding digit d: gbase[d] + j
-            const uint64_t incl = static_cast<uint64_t>(st & StatusBits<S>::VAL);
-            gbase[tid] = boffs + srel + incl - tot[tid + 1];
+            cnt_d = tot[tid + 1] - tot[tid];
+            st_volatile(status + static_cast<uint64_t>(t) * RADIX + tid,
+                        static_cast<S>((first ? SB::INC : SB::AGG) | cnt_d));
         }
         __syncthreads();
-        // ---- stage in shared memory at the rank
-        if (wbase < count) {
+        // ---- stage in shared memory at the rank (keys from registers, values from the staging buffer)
+        {
             const uint32_t *mycnt = wcnt + warp * NBINS;
+            const VT *vs = HV ? vst(s) : nullptr;
 #pragma unroll
             for (int c = 0; c < KPT; ++c) {
                 const uint32_t d = rk[c] & 511u;
                 if (d != INVALID_DIGIT) {
                     const uint32_t r = mycnt[d] + (rk[c] >> 9);
                     skeys[r] = key[c];
-                    if (HV) svals[r] = val[c];
+                    if (HV) svals[r] = seg_get(vs, vsrc, sv, wbase + c * 32 + lane);
                 }
             }
         }
+        // ---- decoupled look-back over the preceding tiles of this bucket
+        if (tid < RADIX) {
+            S excl = 0;
+            if (!first) {
+                const S *q = status + static_cast<uint64_t>(t - 1) * RADIX + tid;
+                for (;;) {
+                    const S v = ld_volatile(q);
+                    if ((v & SB::FLAGS) == 0) continue;  // predecessor not published yet
+                    excl += v & SB::VAL;
+                    if (v & SB::INC) break;
+                    q -= RADIX;
+                }
+                st_volatile(status + static_cast<uint64_t>(t) * RADIX + tid,
+                            static_cast<S>(SB::INC | (excl + cnt_d)));
+            }
+            // destination of smem slot j holding digit d: gbase[d] + j
+            gbase[tid] = boffs + srel + static_cast<uint64_t>(excl) - tot[tid];
+        }
         __syncthreads();
+        // ---- the staging buffer is free: prefetch tile it + 2 into it
+        if (tid == 0) {
+            fence_proxy_async();
+            issue(s, blockIdx.x + (it + 2) * gridDim.x);
+        }
         // ---- write-combined stores: consecutive slots of a digit run are consecutive addresses
 #pragma unroll
         for (int c = 0; c < KPT; ++c) {
@@ -718,16 +941,8 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
                 if (HV) vout[pos] = svals[j];
             }
         }
+        for (int i = tid; i < (THREADS / 32) * NBINS; i += THREADS) wcnt[i] = 0;
         __syncthreads();
-    }
-    // clear the look-back status of pass p+1 (the array pass p-1 used)
-    if (prm.status_next) {
-        const uint64_t words16 =
-            (static_cast<uint64_t>(prm.ctl->ntiles[prm.p + 1]) * RADIX * prm.status_bytes) / 16;
-        uint4 *s = static_cast<uint4 *>(prm.status_next);
-        for (uint64_t i = static_cast<uint64_t>(blockIdx.x) * THREADS + tid; i < words16;
-             i += static_cast<uint64_t>(gridDim.x) * THREADS)
-            s[i] = make_uint4(0, 0, 0, 0);
     }
 }
 
@@ -743,16 +958,24 @@ struct LocalParams {
     int begin_bit;
 };
 
-template <typename K, typename V, int THREADS, int KPT>
+template <typename K, typename V, int THREADS, int KPT, int NSTAGE>
 struct LocalSmem {
     static constexpr int W = THREADS / 32;
     static constexpr int CAP = THREADS * KPT;
-    static constexpr size_t off_wcnt = 0;
-    static constexpr size_t off_tot = off_wcnt + sizeof(uint32_t) * W * NBINS;
-    static constexpr size_t off_red = (off_tot + sizeof(uint32_t) * NBINS + 15) & ~size_t(15);
-    static constexpr size_t off_keys = off_red + sizeof(K) * 2 * W;
-    static constexpr size_t off_vals = (off_keys + sizeof(K) * CAP + 15) & ~size_t(15);
-    static constexpr size_t bytes = off_vals + (HasVal<V>::value ? sizeof(V) * CAP : 0);
+    using VT = ValT<V>;
+    static constexpr bool HV = HasVal<V>::value;
+    static constexpr size_t off_bar = 0;
+    static constexpr size_t off_info = align16(sizeof(uint64_t) * NSTAGE);
+    static constexpr size_t off_wcnt = align16(off_info + sizeof(uint32_t) * 16 * NSTAGE);
+    static constexpr size_t off_tot = align16(off_wcnt + sizeof(uint32_t) * W * NBINS);
+    static constexpr size_t off_red = align16(off_tot + sizeof(uint32_t) * 288);
+    static constexpr size_t off_kst = align16(off_red + sizeof(K) * 2 * W);
+    static constexpr size_t kst_bytes = align16(sizeof(K) * (CAP + 16 / sizeof(K)));
+    static constexpr size_t off_vst = off_kst + NSTAGE * kst_bytes;
+    static constexpr size_t vst_bytes = HV ? align16(sizeof(VT) * (CAP + 16 / sizeof(VT))) : 0;
+    static constexpr size_t off_skeys = off_vst + NSTAGE * vst_bytes;
+    static constexpr size_t off_sidx = align16(off_skeys + sizeof(K) * CAP);
+    static constexpr size_t bytes = off_sidx + align16(sizeof(uint16_t) * CAP);
 };
 
 template <typename K>
@@ -768,43 +991,112 @@ __device__ __forceinline__ K warp_or(K x) {
     return x;
 }
 
-template <typename K, typename V, int THREADS, int KPT, int MINB>
+template <typename K, typename V, int THREADS, int KPT, int NSTAGE, int MINB>
 __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
-    using L = LocalSmem<K, V, THREADS, KPT>;
+    using L = LocalSmem<K, V, THREADS, KPT, NSTAGE>;
     constexpr int W = THREADS / 32;
     constexpr bool HV = HasVal<V>::value;
-    using VT = typename std::conditional<HV, V, uint32_t>::type;
+    using VT = ValT<V>;
     extern __shared__ __align__(16) unsigned char smem[];
+    uint64_t *bar = reinterpret_cast<uint64_t *>(smem + L::off_bar);
+    uint32_t *info = reinterpret_cast<uint32_t *>(smem + L::off_info);  // [s][16]
     uint32_t *wcnt = reinterpret_cast<uint32_t *>(smem + L::off_wcnt);
     uint32_t *tot = reinterpret_cast<uint32_t *>(smem + L::off_tot);
     K *red = reinterpret_cast<K *>(smem + L::off_red);
-    K *skeys = reinterpret_cast<K *>(smem + L::off_keys);
-    VT *svals = reinterpret_cast<VT *>(smem + L::off_vals);
+    K *skeys = reinterpret_cast<K *>(smem + L::off_skeys);
+    uint16_t *sidx = reinterpret_cast<uint16_t *>(smem + L::off_sidx);
+    auto kst = [&](int s) { return reinterpret_cast<K *>(smem + L::off_kst + s * L::kst_bytes); };
+    auto vst = [&](int s) { return reinterpret_cast<VT *>(smem + L::off_vst + s * L::vst_bytes); };
     const int tid = threadIdx.x, lane = tid & 31, warp = tid >> 5;
     const uint32_t wbase = static_cast<uint32_t>(warp) * 32 * KPT;
     const uint32_t nent = *prm.count;
+    if (blockIdx.x >= nent) return;
     K *__restrict__ kout = static_cast<K *>(prm.keys_out);
     VT *__restrict__ vout = static_cast<VT *>(prm.vals_out);
+    const uint64_t pol = policy_evict_first();
 
-    for (uint32_t ei = blockIdx.x; ei < nent; ei += gridDim.x) {
-        const LocalEntry en = prm.list[ei];
-        const uint32_t count = en.count;
-        // select without dynamic indexing of the parameter arrays (keeps them out of local memory)
-        const void *kbase = en.src == SRC_IN ? prm.src_keys[SRC_IN]
-                            : en.src == SRC_AUX ? prm.src_keys[SRC_AUX] : prm.src_keys[SRC_OUT];
-        const void *vbase = en.src == SRC_IN ? prm.src_vals[SRC_IN]
-                            : en.src == SRC_AUX ? prm.src_vals[SRC_AUX] : prm.src_vals[SRC_OUT];
-        const K *ksrc = static_cast<const K *>(kbase) + en.offs;
-        const VT *vsrc = HV ? static_cast<const VT *>(vbase) + en.offs : nullptr;
+    auto srck = [&](uint32_t code) -> const K * {
+        return static_cast<const K *>(code == SRC_IN    ? prm.src_keys[SRC_IN]
+                                      : code == SRC_AUX ? prm.src_keys[SRC_AUX]
+                                                        : prm.src_keys[SRC_OUT]);
+    };
+    auto srcv = [&](uint32_t code) -> const VT * {
+        return static_cast<const VT *>(code == SRC_IN    ? prm.src_vals[SRC_IN]
+                                       : code == SRC_AUX ? prm.src_vals[SRC_AUX]
+                                                         : prm.src_vals[SRC_OUT]);
+    };
+    // info[s]: 0 entry, 1 count, 2 hi_bit, 3 src, 4..5 offs, 6..8 key seg, 9..11 value seg
+    auto issue = [&](int s, uint32_t e) {
+        uint32_t *in = info + 16 * s;
+        in[0] = e;
+        if (e >= nent) return;
+        const LocalEntry en = prm.list[e];
+        in[1] = en.count;
+        in[2] = en.hi_bit;
+        in[3] = en.src;
+        in[4] = static_cast<uint32_t>(en.offs);
+        in[5] = static_cast<uint32_t>(en.offs >> 32);
+        Seg sk, sv;
+        const K *ks = srck(en.src) + en.offs;
+        uint32_t bytes = seg_plan(ks, en.count, sk);
+        in[6] = sk.pad;
+        in[7] = sk.i0;
+        in[8] = sk.i1;
+        const VT *vs = nullptr;
+        if (HV) {
+            vs = srcv(en.src) + en.offs;
+            bytes += seg_plan(vs, en.count, sv);
+            in[9] = sv.pad;
+            in[10] = sv.i0;
+            in[11] = sv.i1;
+        }
+        mbar_arrive_expect_tx(&bar[s], bytes);
+        seg_issue(kst(s), ks, sk, &bar[s], pol);
+        if (HV) seg_issue(vst(s), vs, sv, &bar[s], pol);
+    };
+    if (tid == 0) {
+        for (int s = 0; s < NSTAGE; ++s) mbar_init(&bar[s], 1);
+        mbar_fence_init();
+        for (int s = 0; s < NSTAGE; ++s) issue(s, blockIdx.x + s * gridDim.x);
+    }
+    __syncthreads();
+
+    for (uint32_t it = 0;; ++it) {
+        const int s = static_cast<int>(it % NSTAGE);
+        const uint32_t par = (it / NSTAGE) & 1u;
+        const uint32_t *in = info + 16 * s;
+        const uint32_t e_id = in[0];
+        if (e_id >= nent) break;
+        const uint32_t count = in[1];
+        const int hi_bit = static_cast<int>(in[2]);
+        const uint32_t src = in[3];
+        const uint64_t offs = static_cast<uint64_t>(in[4]) | (static_cast<uint64_t>(in[5]) << 32);
+        Seg sk, sv;
+        sk.pad = in[6];
+        sk.i0 = in[7];
+        sk.i1 = in[8];
+        sv.pad = in[9];
+        sv.i0 = in[10];
+        sv.i1 = in[11];
+        const K *ksrc = srck(src) + offs;
+        const VT *vsrc = HV ? srcv(src) + offs : nullptr;
+        K *ks = kst(s);
+        VT *vs = HV ? vst(s) : nullptr;
+        mbar_wait(&bar[s], par);
+        // the entry may be sorted in place: bring its unaligned edges into shared memory
+        // now, before any thread writes the output
+        seg_fill_edges<K, THREADS>(ks, ksrc, sk, count);
+        if (HV) seg_fill_edges<VT, THREADS>(vs, vsrc, sv, count);
+        __syncthreads();
         K key[KPT];
-        VT val[KPT];
+        uint32_t idx[KPT];
         K a = ~K(0), o = K(0);
 #pragma unroll
         for (int c = 0; c < KPT; ++c) {
             const uint32_t e = wbase + c * 32 + lane;
+            idx[c] = e;
             if (e < count) {
-                key[c] = ksrc[e];
-                if (HV) val[c] = vsrc[e];
+                key[c] = ks[sk.pad + e];
                 a &= key[c];
                 o |= key[c];
             }
@@ -816,6 +1108,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
             red[warp] = a;
             red[W + warp] = o;
         }
+        for (int i = tid; i < W * NBINS; i += THREADS) wcnt[i] = 0;
         __syncthreads();
         K diff = 0;
         {
@@ -828,26 +1121,20 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
             diff = aa ^ oo;
         }
         bool moved = false;
-        for (int lo = prm.begin_bit; lo < en.hi_bit; lo += 8) {
-            const int width = min(8, en.hi_bit - lo);
+        for (int lo = prm.begin_bit; lo < hi_bit; lo += 8) {
+            const int width = min(8, hi_bit - lo);
             const uint32_t mask = (1u << width) - 1u;
             if ((static_cast<uint32_t>(diff >> lo) & mask) == 0) continue;  // constant digit: identity pass
             moved = true;
-            for (int i = tid; i < W * NBINS; i += THREADS) wcnt[i] = 0;
-            __syncthreads();
             uint32_t rk[KPT];
-            if (wbase < count) {
 #pragma unroll
-                for (int c = 0; c < KPT; ++c) {
-                    const uint32_t e = wbase + c * 32 + lane;
-                    rk[c] = e < count ? digit_of(key[c], lo, mask) : INVALID_DIGIT;
-                }
-                warp_rank_walk<THREADS, KPT>(rk, wcnt + warp * NBINS);
-            }
+            for (int c = 0; c < KPT; ++c)
+                rk[c] = (wbase + c * 32 + lane) < count ? digit_of(key[c], lo, mask) : INVALID_DIGIT;
+            if (wbase < count) rank_walk<KPT>(rk, wcnt + warp * NBINS);
             __syncthreads();
             block_rank_scan<THREADS>(wcnt, tot);
             __syncthreads();
-            if (wbase < count) {
+            {
                 const uint32_t *mycnt = wcnt + warp * NBINS;
 #pragma unroll
                 for (int c = 0; c < KPT; ++c) {
@@ -855,7 +1142,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
                     if (d != INVALID_DIGIT) {
                         const uint32_t r = mycnt[d] + (rk[c] >> 9);
                         skeys[r] = key[c];
-                        if (HV) svals[r] = val[c];
+                        sidx[r] = static_cast<uint16_t>(idx[c]);
                     }
                 }
             }
@@ -865,22 +1152,28 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
                 const uint32_t e = wbase + c * 32 + lane;
                 if (e < count) {
                     key[c] = skeys[e];
-                    if (HV) val[c] = svals[e];
+                    idx[c] = sidx[e];
                 }
             }
+            for (int i = tid; i < W * NBINS; i += THREADS) wcnt[i] = 0;
             __syncthreads();
         }
-        if (moved || en.src != SRC_OUT) {
+        if (moved || src != SRC_OUT) {
 #pragma unroll
             for (int c = 0; c < KPT; ++c) {
                 const uint32_t e = wbase + c * 32 + lane;
                 if (e < count) {
-                    kout[en.offs + e] = key[c];
-                    if (HV) vout[en.offs + e] = val[c];
+                    kout[offs + e] = key[c];
+                    if (HV) vout[offs + e] = vs[sv.pad + idx[c]];
                 }
             }
         }
-        __syncthreads();  // red[] reuse
+        __syncthreads();  // staging buffer s and red[] are free
+        if (tid == 0) {
+            fence_proxy_async();
+            issue(s, blockIdx.x + (it + NSTAGE) * gridDim.x);
+        }
+        __syncthreads();
     }
 }
 
