@@ -82,6 +82,7 @@ constexpr int HIST_THREADS = 512;
 constexpr int HIST_STAGES = 3;
 constexpr int HIST_CAP = 4096;  // >= every ScatterCfg KPB
 constexpr int CLASSIFY_THREADS = 256;
+constexpr uint32_t RANGE_MAX = 1024;  // >= SMs x resident scatter CTAs per SM
 constexpr size_t SMEM_LIMIT = 227 * 1024;
 
 template <int C>
@@ -214,11 +215,11 @@ struct Plan {
     uint32_t lt = 0, mt = 0, kpb = 0;
     int single_class = -1;
     bool counting = false;
-    bool wide = false;  // 64-bit look-back status words
     uint32_t tile_cap = 0, bucket_cap = 0;
     uint32_t local_cap[HRS_NUM_CLASSES] = {0};
-    size_t off_auxk = 0, off_auxv = 0, off_tiles[2] = {0, 0}, off_buckets[2] = {0, 0}, off_tot[2] = {0, 0},
-           off_subrel = 0, off_status = 0, off_local[HRS_NUM_CLASSES] = {0}, total = 0;
+    uint32_t range_cap = 0;  // CTAs of the hist/scatter grid the temp layout allows
+    size_t off_auxk = 0, off_auxv = 0, off_buckets[2] = {0, 0}, off_tot[2] = {0, 0}, off_subrel = 0,
+           off_seg_last = 0, off_seg_meta = 0, off_carry = 0, off_local[HRS_NUM_CLASSES] = {0}, total = 0;
 };
 
 size_t align_up(size_t x, size_t a) { return (x + a - 1) / a * a; }
@@ -249,7 +250,6 @@ hrs_status make_plan(Plan &pl, uint64_t n, int kb, int vb, int begin, int end, c
     pl.mt = t.merge_threshold;
     pl.kpb = t.keys_per_tile;
     pl.single_class = t.local_classes ? size_class_of(pl.lt) : -1;
-    pl.wide = n >= (1ull << 30);
 
     // digit plan: 8-bit digits aligned to end_bit, most-significant first (reading #3)
     pl.D = 0;
@@ -295,17 +295,19 @@ hrs_status make_plan(Plan &pl, uint64_t n, int kb, int vb, int begin, int end, c
     if (need_aux) off = align_up(off + n * kb, 256);
     pl.off_auxv = off;
     if (need_aux && vb) off = align_up(off + n * vb, 256);
-    const size_t sbytes = pl.wide ? 8 : 4;
     for (int i = 0; i < 2; ++i) {
-        pl.off_tiles[i] = off;
-        off = align_up(off + sizeof(Tile) * static_cast<size_t>(pl.tile_cap), 256);
         pl.off_buckets[i] = off;
         off = align_up(off + sizeof(Bucket) * static_cast<size_t>(pl.bucket_cap), 256);
         pl.off_tot[i] = off;
         off = align_up(off + sizeof(uint32_t) * RADIX * static_cast<size_t>(pl.bucket_cap), 256);
     }
-    pl.off_status = off;
-    off = align_up(off + sbytes * RADIX * static_cast<size_t>(pl.tile_cap), 256);
+    pl.range_cap = std::min<uint32_t>(RANGE_MAX, pl.tile_cap);
+    pl.off_seg_last = off;
+    off = align_up(off + sizeof(uint32_t) * RADIX * static_cast<size_t>(pl.range_cap), 256);
+    pl.off_carry = off;
+    off = align_up(off + sizeof(uint32_t) * RADIX * static_cast<size_t>(pl.range_cap), 256);
+    pl.off_seg_meta = off;
+    off = align_up(off + sizeof(RangeMeta) * static_cast<size_t>(pl.range_cap), 256);
     pl.off_subrel = off;
     off = align_up(off + sizeof(uint32_t) * RADIX * static_cast<size_t>(pl.bucket_cap), 256);
     for (int c = 0; c < HRS_NUM_CLASSES; ++c) {
@@ -329,7 +331,7 @@ P *at(void *base, size_t off) {
 
 // ------------------------------------------------------------------ typed launch sequences
 
-template <typename K, typename V, typename S>
+template <typename K, typename V>
 struct Runner {
     static constexpr int KB = sizeof(K);
     static constexpr int VB = HasVal<V>::value ? sizeof(V) : 0;
@@ -338,7 +340,6 @@ struct Runner {
     static hrs_status init(const Plan &pl, void *temp, cudaStream_t st, int sms, int root_class, int counting) {
         InitParams ip;
         ip.ctl = at<Ctl>(temp, 0);
-        ip.tiles = at<Tile>(temp, pl.off_tiles[1]);
         ip.buckets = at<Bucket>(temp, pl.off_buckets[1]);
         ip.tot = at<uint32_t>(temp, pl.off_tot[1]);
         ip.root_local = root_class >= 0 ? at<LocalEntry>(temp, pl.off_local[root_class]) : nullptr;
@@ -349,35 +350,48 @@ struct Runner {
         ip.end_bit = pl.end;
         ip.key_bytes = pl.kb;
         ip.value_bytes = pl.vb;
-        const uint64_t T1 = counting ? (pl.n + pl.kpb - 1) / pl.kpb : 0;
-        const int grid = static_cast<int>(std::min<uint64_t>(std::max<uint64_t>((T1 + 255) / 256, 1),
-                                                             static_cast<uint64_t>(sms) * 4));
         LaunchScope ls(st, 0, 0);
-        k_init<<<grid, 256, 0, st>>>(ip);
+        k_init<<<1, 256, 0, st>>>(ip);
         return last_launch();
     }
 
-    static hrs_status hist(const Plan &pl, void *temp, cudaStream_t st, int dev, int sms, int p, const void *xin) {
+    // the hist / classify / scatter grid of a pass: the scatter's persistent grid,
+    // capped by the temp layout (range_cap >= tiles of any pass is not required)
+    static hrs_status range_grid(const Plan &pl, int dev, int sms, uint32_t *G) {
+        auto fn = k_scatter<K, V, SC::THREADS, SC::KPT, SC::MINB>;
+        const size_t smem = ScatterSmem<K, V, SC::THREADS, SC::KPT>::bytes;
+        int grid = 0;
+        hrs_status s = grid_for(fn, SC::THREADS, smem, dev, sms, &grid);
+        if (s) return s;
+        *G = std::min<uint32_t>(static_cast<uint32_t>(grid), pl.range_cap);
+        return HRS_SUCCESS;
+    }
+
+    static hrs_status hist(const Plan &pl, void *temp, cudaStream_t st, int dev, int sms, int p, const void *xin,
+                           uint32_t G) {
         HistParams hp;
         hp.keys = xin;
         hp.p = p;
         hp.lo = pl.lo[p - 1];
         hp.mask = (1u << (pl.hi[p - 1] - pl.lo[p - 1])) - 1u;
-        hp.tiles = at<Tile>(temp, pl.off_tiles[p & 1]);
+        hp.kpb = pl.kpb;
+        hp.buckets = at<Bucket>(temp, pl.off_buckets[p & 1]);
         hp.tot = at<uint32_t>(temp, pl.off_tot[p & 1]);
+        hp.seg_last = at<uint32_t>(temp, pl.off_seg_last);
+        hp.seg_meta = at<RangeMeta>(temp, pl.off_seg_meta);
         hp.ctl = at<Ctl>(temp, 0);
         auto fn = k_hist<K, HIST_THREADS, HIST_STAGES, HIST_CAP>;
         const size_t smem = HistSmem<K, HIST_THREADS, HIST_STAGES, HIST_CAP>::bytes;
         int grid = 0;
-        hrs_status s = grid_for(fn, HIST_THREADS, smem, dev, sms, &grid);
+        hrs_status s = grid_for(fn, HIST_THREADS, smem, dev, sms, &grid);  // sets the smem attribute
         if (s) return s;
         LaunchScope ls(st, 1, p);
-        fn<<<grid, HIST_THREADS, smem, st>>>(hp);
+        fn<<<G, HIST_THREADS, smem, st>>>(hp);
         return last_launch();
     }
 
     static hrs_status classify(const Plan &pl, void *temp, cudaStream_t st, int dev, int sms, int p,
-                               uint16_t src_code, uint64_t *out_hist, uint64_t *out_offsets, bool last) {
+                               uint16_t src_code, uint64_t *out_hist, uint64_t *out_offsets, bool last, uint32_t G) {
         ClassifyParams cp;
         std::memset(&cp, 0, sizeof(cp));
         cp.p = p;
@@ -387,11 +401,12 @@ struct Runner {
         cp.buckets = at<Bucket>(temp, pl.off_buckets[p & 1]);
         cp.tot = at<uint32_t>(temp, pl.off_tot[p & 1]);
         cp.tot_next = at<uint32_t>(temp, pl.off_tot[(p + 1) & 1]);
-        cp.next_tiles = at<Tile>(temp, pl.off_tiles[(p + 1) & 1]);
         cp.next_buckets = at<Bucket>(temp, pl.off_buckets[(p + 1) & 1]);
         cp.sub_rel = at<uint32_t>(temp, pl.off_subrel);
-        cp.status = at<void>(temp, pl.off_status);
-        cp.status_bytes = sizeof(S);
+        cp.seg_last = at<uint32_t>(temp, pl.off_seg_last);
+        cp.seg_meta = at<RangeMeta>(temp, pl.off_seg_meta);
+        cp.carry = at<uint32_t>(temp, pl.off_carry);
+        cp.ranges = G;
         cp.ctl = at<Ctl>(temp, 0);
         for (int c = 0; c < HRS_NUM_CLASSES; ++c) {
             cp.local[c] = at<LocalEntry>(temp, pl.off_local[c]);
@@ -410,13 +425,15 @@ struct Runner {
         int grid = 0;
         hrs_status s = grid_for(fn, CLASSIFY_THREADS, 0, dev, sms, &grid);
         if (s) return s;
+        // one block per bucket (up to the resident limit) plus the carry block
+        grid = static_cast<int>(std::min<uint64_t>(grid, std::max<uint64_t>(pl.bucket_cap, 1))) + 1;
         LaunchScope ls(st, 5, p);
         fn<<<grid, CLASSIFY_THREADS, 0, st>>>(cp);
         return last_launch();
     }
 
     static hrs_status scatter(const Plan &pl, void *temp, cudaStream_t st, int dev, int sms, int p, const void *kin,
-                              void *kout, const void *vin, void *vout) {
+                              void *kout, const void *vin, void *vout, uint32_t G) {
         ScatterParams sp;
         sp.keys_in = kin;
         sp.keys_out = kout;
@@ -425,18 +442,15 @@ struct Runner {
         sp.p = p;
         sp.lo = pl.lo[p - 1];
         sp.mask = (1u << (pl.hi[p - 1] - pl.lo[p - 1])) - 1u;
-        sp.tiles = at<Tile>(temp, pl.off_tiles[p & 1]);
+        sp.kpb = pl.kpb;
         sp.buckets = at<Bucket>(temp, pl.off_buckets[p & 1]);
-        sp.status = at<void>(temp, pl.off_status);
         sp.sub_rel = at<uint32_t>(temp, pl.off_subrel);
+        sp.carry = at<uint32_t>(temp, pl.off_carry);
         sp.ctl = at<Ctl>(temp, 0);
-        auto fn = k_scatter<K, V, S, SC::THREADS, SC::KPT, SC::MINB>;
+        auto fn = k_scatter<K, V, SC::THREADS, SC::KPT, SC::MINB>;
         const size_t smem = ScatterSmem<K, V, SC::THREADS, SC::KPT>::bytes;
-        int grid = 0;
-        hrs_status s = grid_for(fn, SC::THREADS, smem, dev, sms, &grid);
-        if (s) return s;
         LaunchScope ls(st, 2, p);
-        fn<<<grid, SC::THREADS, smem, st>>>(sp);
+        fn<<<G, SC::THREADS, smem, st>>>(sp);
         return last_launch();
     }
 
@@ -514,16 +528,18 @@ struct Runner {
         void *auxk = at<void>(temp, pl.off_auxk);
         void *auxv = VB ? at<void>(temp, pl.off_auxv) : nullptr;
         if (pl.counting) {
+            uint32_t G = 0;
+            if ((s = range_grid(pl, dev, sms, &G))) return s;
             const void *xk = kin, *xv = vin;
             for (int p = 1; p <= pl.D; ++p) {
                 const bool to_out = ((pl.D - p) % 2) == 0;
                 void *yk = to_out ? kout : auxk;
                 void *yv = to_out ? vout : auxv;
-                if ((s = hist(pl, temp, st, dev, sms, p, xk))) return s;
+                if ((s = hist(pl, temp, st, dev, sms, p, xk, G))) return s;
                 if ((s = classify(pl, temp, st, dev, sms, p, to_out ? SRC_OUT : SRC_AUX, nullptr, nullptr,
-                                  p == pl.D)))
+                                  p == pl.D, G)))
                     return s;
-                if ((s = scatter(pl, temp, st, dev, sms, p, xk, yk, xv, yv))) return s;
+                if ((s = scatter(pl, temp, st, dev, sms, p, xk, yk, xv, yv, G))) return s;
                 xk = yk;
                 xv = yv;
             }
@@ -551,9 +567,11 @@ struct Runner {
             }
             return HRS_SUCCESS;
         }
-        if ((s = hist(pl, temp, st, dev, sms, 1, kin))) return s;
-        if ((s = classify(pl, temp, st, dev, sms, 1, SRC_OUT, out_hist, out_offsets, true))) return s;
-        if (do_scatter && (s = scatter(pl, temp, st, dev, sms, 1, kin, kout, vin, vout))) return s;
+        uint32_t G = 0;
+        if ((s = range_grid(pl, dev, sms, &G))) return s;
+        if ((s = hist(pl, temp, st, dev, sms, 1, kin, G))) return s;
+        if ((s = classify(pl, temp, st, dev, sms, 1, SRC_OUT, out_hist, out_offsets, true, G))) return s;
+        if (do_scatter && (s = scatter(pl, temp, st, dev, sms, 1, kin, kout, vin, vout, G))) return s;
         return HRS_SUCCESS;
     }
 };
@@ -561,16 +579,13 @@ struct Runner {
 template <typename K, typename V>
 hrs_status run_sort(const Plan &pl, void *temp, const void *kin, void *kout, const void *vin, void *vout,
                     cudaStream_t st, int dev, int sms) {
-    if (pl.wide) return Runner<K, V, unsigned long long>::sort(pl, temp, kin, kout, vin, vout, st, dev, sms);
-    return Runner<K, V, uint32_t>::sort(pl, temp, kin, kout, vin, vout, st, dev, sms);
+    return Runner<K, V>::sort(pl, temp, kin, kout, vin, vout, st, dev, sms);
 }
 
 template <typename K, typename V>
 hrs_status run_block(const Plan &pl, void *temp, const void *kin, void *kout, const void *vin, void *vout,
                      uint64_t *h, uint64_t *o, bool sc, cudaStream_t st, int dev, int sms) {
-    if (pl.wide)
-        return Runner<K, V, unsigned long long>::building_block(pl, temp, kin, kout, vin, vout, h, o, sc, st, dev, sms);
-    return Runner<K, V, uint32_t>::building_block(pl, temp, kin, kout, vin, vout, h, o, sc, st, dev, sms);
+    return Runner<K, V>::building_block(pl, temp, kin, kout, vin, vout, h, o, sc, st, dev, sms);
 }
 
 hrs_status sort_dispatch(int kb, int vb, const Plan &pl, void *temp, const void *kin, void *kout, const void *vin,
@@ -684,11 +699,12 @@ hrs_status hrs_get_stats(const void *d_temp, hrs_stats *out, hrs_stream_t stream
     const uint64_t K = c.key_bytes, R = c.key_bytes + c.value_bytes;
     uint64_t bytes = 0;
     for (int p = 1; p <= HRS_MAX_PASSES; ++p) {
-        if (c.ntiles[p] == 0) continue;
+        const uint32_t tiles = static_cast<uint32_t>(c.alloc[p] >> 32), bks = static_cast<uint32_t>(c.alloc[p]);
+        if (tiles == 0) continue;
         out->counting_passes = p;
         out->recs_in_pass[p - 1] = c.recs_in_pass[p];
-        out->tiles_in_pass[p - 1] = c.ntiles[p];
-        out->buckets_in_pass[p - 1] = c.nbuckets[p];
+        out->tiles_in_pass[p - 1] = tiles;
+        out->buckets_in_pass[p - 1] = bks;
         bytes += c.recs_in_pass[p] * (K + 2 * R);
     }
     for (int k = 0; k < HRS_NUM_CLASSES; ++k) {

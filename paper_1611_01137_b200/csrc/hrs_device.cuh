@@ -2,8 +2,9 @@
 //
 // Paper: Stehle & Jacobsen, arXiv 1611.01137 (PAPER.md lines cited as P:<line>).
 // Every pass p of the MSD recursion (Fig 1) runs three kernels over a
-// device-resident tile table ("key blocks"), so each pass costs a
-// constant number of launches and the host never reads device memory:
+// device-resident bucket table whose buckets are cut into tiles ("key blocks",
+// P:517-541), so each pass costs a constant number of launches and the host never
+// reads device memory:
 //
 //   k_hist<p>      streams the keys of every tile through a TMA bulk-copy ring into
 //                  shared memory and counts the digit with per-warp shared-memory
@@ -17,11 +18,13 @@
 //                  sub-buckets (R1-R3 P:805-811, merging P:552-561) into next-pass
 //                  buckets/tiles and local-sort lists.
 //   k_scatter<p>   per tile, with the next tile already in flight through TMA: a
-//                  STABLE in-tile rank, a decoupled look-back over the preceding
-//                  tiles of the same bucket (tile order = memory order; replaces the
-//                  atomicAdd chunk reservation of P:696-703, which is not stable),
-//                  staging in shared memory and write-combined stores of every digit
-//                  run (Fig 3); values follow their keys.
+//                  STABLE in-tile rank, staging in shared memory and write-combined
+//                  stores of every digit run (Fig 3); values follow their
+//                  keys.  k_hist and k_scatter give every CTA the same
+//                  contiguous run of tiles, so the tile-ordered offset of each tile
+//                  inside its sub-bucket is a running sum in the CTA seeded by a
+//                  per-CTA carry (computed by k_classify): deterministic, and it
+//                  replaces the atomicAdd chunk reservation of P:696-703 (not stable).
 //
 // then one k_local launch per size class sorts every bucket of at most
 // ∂ˆ records on chip: a stable LSD radix sort of (key, index) pairs over the
@@ -47,15 +50,9 @@ constexpr uint64_t CTL_MAGIC = 0x4852535f31363131ull;  // "HRS_1611"
 
 enum SrcCode : uint16_t { SRC_IN = 0, SRC_AUX = 1, SRC_OUT = 2 };
 
-// One tile ("key block"): up to KPB consecutive records of one bucket.
-struct Tile {
-    uint64_t offs;
-    uint32_t count;
-    uint32_t bucket;
-};
-// A bucket that is counting-sorted in the current pass; its tiles are
-// first_tile .. first_tile + ntiles - 1, consecutive and in memory order (the
-// order the look-back follows, which makes the pass stable).
+// A bucket that is counting-sorted in the current pass.  Its tiles ("key blocks",
+// P:521-524; up to KPB consecutive records each) are first_tile .. first_tile +
+// ntiles - 1, consecutive and in memory order: that order makes the pass stable.
 struct Bucket {
     uint64_t offs;
     uint32_t count;
@@ -76,8 +73,9 @@ struct Ctl {
     unsigned long long magic;
     unsigned long long n;
     uint32_t key_bytes, value_bytes;
-    uint32_t ntiles[HRS_MAX_PASSES + 2];    // tiles of pass p (1-based)
-    uint32_t nbuckets[HRS_MAX_PASSES + 2];  // buckets of pass p
+    // tiles (high 32 bits) and buckets (low 32 bits) of pass p (1-based), allocated
+    // together by one 64-bit atomic so bucket order == tile order
+    unsigned long long alloc[HRS_MAX_PASSES + 2];
     uint32_t nlocal[HRS_NUM_CLASSES];       // entries in local list c
     uint32_t overflow;
     uint32_t pad_;
@@ -97,27 +95,6 @@ __device__ __forceinline__ uint32_t lanemask_lt() {
 template <typename K>
 __device__ __forceinline__ uint32_t digit_of(K key, int lo, uint32_t mask) {
     return static_cast<uint32_t>(key >> lo) & mask;
-}
-
-template <typename S>
-struct StatusBits;
-template <>
-struct StatusBits<uint32_t> {
-    static constexpr uint32_t AGG = 1u << 30, INC = 2u << 30, FLAGS = 3u << 30, VAL = (1u << 30) - 1;
-};
-template <>
-struct StatusBits<unsigned long long> {
-    static constexpr unsigned long long AGG = 1ull << 62, INC = 2ull << 62, FLAGS = 3ull << 62,
-                                        VAL = (1ull << 62) - 1;
-};
-
-template <typename T>
-__device__ __forceinline__ T ld_volatile(const T *p) {
-    return *reinterpret_cast<const volatile T *>(p);
-}
-template <typename T>
-__device__ __forceinline__ void st_volatile(T *p, T v) {
-    *reinterpret_cast<volatile T *>(p) = v;
 }
 
 struct NoVal {};
@@ -166,6 +143,67 @@ __device__ __forceinline__ void warp0_exclusive_scan(uint32_t *a, int n) {
         if (idx < n) a[idx] = run;
         run += v[i];
     }
+}
+
+// ------------------------------------------------------------------ tiles derived from the bucket table
+
+__device__ __forceinline__ uint32_t alloc_tiles(unsigned long long a) { return static_cast<uint32_t>(a >> 32); }
+__device__ __forceinline__ uint32_t alloc_buckets(unsigned long long a) { return static_cast<uint32_t>(a); }
+
+// Tile t of a pass belongs to the bucket b with first_tile <= t < first_tile + ntiles;
+// bucket ids are allocated in tile order, so a binary search finds it.
+__device__ __forceinline__ uint32_t find_bucket(const Bucket *bks, uint32_t nb, uint32_t t) {
+    uint32_t lo = 0, hi = nb - 1;
+    while (lo < hi) {
+        const uint32_t mid = (lo + hi + 1) >> 1;
+        if (bks[mid].first_tile <= t) lo = mid;
+        else hi = mid - 1;
+    }
+    return lo;
+}
+
+// Walks the tiles [tb, te) of one CTA in order (used by the producer thread).
+struct TileCursor {
+    const Bucket *bks;
+    uint32_t t, te, b, k;
+    Bucket bk;
+    uint32_t kpb;
+    __device__ __forceinline__ void start(const Bucket *bks_, uint32_t nb, uint32_t tb, uint32_t te_, uint32_t kpb_) {
+        bks = bks_;
+        t = tb;
+        te = te_;
+        kpb = kpb_;
+        if (t < te) {
+            b = find_bucket(bks, nb, t);
+            bk = bks[b];
+            k = t - bk.first_tile;
+        }
+    }
+    __device__ __forceinline__ bool valid() const { return t < te; }
+    __device__ __forceinline__ uint64_t offs() const { return bk.offs + static_cast<uint64_t>(k) * kpb; }
+    __device__ __forceinline__ uint32_t count() const { return min(kpb, bk.count - k * kpb); }
+    __device__ __forceinline__ bool last_of_bucket() const { return k + 1 == bk.ntiles; }
+    __device__ __forceinline__ void next() {
+        ++t;
+        if (t >= te) return;
+        if (++k == bk.ntiles) {
+            ++b;
+            bk = bks[b];
+            k = 0;
+        }
+    }
+};
+
+// Per-CTA range bookkeeping shared by k_hist, k_classify and k_scatter (same grid):
+// the digit counts of the CTA's last bucket segment and the bucket ids of its first
+// and last tile; k_classify turns them into the carry of each CTA's first segment.
+constexpr uint32_t EMPTY_RANGE = 0xFFFFFFFFu;
+struct RangeMeta {
+    uint32_t first_bucket, last_bucket;
+};
+
+__host__ __device__ __forceinline__ uint32_t range_begin(uint32_t T, uint32_t c, uint32_t G) {
+    return static_cast<uint32_t>((static_cast<uint64_t>(T) * c) / G);
 }
 
 // ------------------------------------------------------------------ TMA bulk copies (cp.async.bulk + mbarrier)
@@ -313,7 +351,6 @@ __device__ __forceinline__ void block_rank_scan(uint32_t *wcnt, uint32_t *tot) {
 
 struct InitParams {
     Ctl *ctl;
-    Tile *tiles;             // pass-1 tile table
     Bucket *buckets;         // pass-1 bucket table
     uint32_t *tot;           // pass-1 bucket histograms (row 0 is cleared)
     LocalEntry *root_local;  // list of the root's size class (n <= ∂ˆ)
@@ -341,8 +378,7 @@ __global__ void k_init(InitParams prm) {
             c->key_bytes = prm.key_bytes;
             c->value_bytes = prm.value_bytes;
             if (prm.counting) {
-                c->ntiles[1] = T1;
-                c->nbuckets[1] = 1;
+                c->alloc[1] = (static_cast<unsigned long long>(T1) << 32) | 1ull;
                 c->recs_in_pass[1] = n;
                 Bucket b;
                 b.offs = 0;
@@ -362,15 +398,6 @@ __global__ void k_init(InitParams prm) {
                 c->local_recs = n;
             }
         }
-    }
-    const uint64_t stride = static_cast<uint64_t>(gridDim.x) * blockDim.x;
-    const uint64_t tid = static_cast<uint64_t>(blockIdx.x) * blockDim.x + threadIdx.x;
-    for (uint64_t t = tid; t < T1; t += stride) {
-        Tile tl;
-        tl.offs = t * prm.kpb;
-        tl.count = static_cast<uint32_t>(min(static_cast<uint64_t>(prm.kpb), n - tl.offs));
-        tl.bucket = 0;
-        prm.tiles[t] = tl;
     }
 }
 
@@ -394,8 +421,11 @@ struct HistParams {
     int p;
     int lo;
     uint32_t mask;
-    const Tile *tiles;
-    uint32_t *tot;  // [bucket][256] of this pass (zeroed by the creator of the bucket)
+    uint32_t kpb;
+    const Bucket *buckets;
+    uint32_t *tot;             // [bucket][256] of this pass (zeroed by the creator of the bucket)
+    uint32_t *seg_last;        // [cta][256]: counts of the CTA's last bucket segment
+    RangeMeta *seg_meta;       // [cta]
     Ctl *ctl;
 };
 
@@ -417,39 +447,53 @@ __global__ void __launch_bounds__(THREADS) k_hist(HistParams prm) {
     constexpr int VK = 16 / sizeof(K);
     extern __shared__ __align__(16) unsigned char smem[];
     uint64_t *bar = reinterpret_cast<uint64_t *>(smem + L::off_bar);
-    uint32_t *info = reinterpret_cast<uint32_t *>(smem + L::off_info);  // [s][8]: tile, count, bucket, pad, i0, i1
+    // info[s]: 0 valid, 1 count, 2 bucket, 3 pad, 4 i0, 5 i1, 6 last tile of its bucket, 7 offs lo
+    uint32_t *info = reinterpret_cast<uint32_t *>(smem + L::off_info);
     uint32_t *wh = reinterpret_cast<uint32_t *>(smem + L::off_wh);
     auto stage = [&](int s) {
         return reinterpret_cast<K *>(smem + L::off_stage + s * align16(sizeof(K) * L::stage_elems));
     };
     const K *__restrict__ keys = static_cast<const K *>(prm.keys);
     const int tid = threadIdx.x, warp = tid >> 5;
-    const uint32_t T = prm.ctl->ntiles[prm.p];
-    // a contiguous run of tiles per CTA: bucket histograms are flushed once per run
-    const uint32_t tb = static_cast<uint32_t>((static_cast<uint64_t>(T) * blockIdx.x) / gridDim.x);
-    const uint32_t te = static_cast<uint32_t>((static_cast<uint64_t>(T) * (blockIdx.x + 1)) / gridDim.x);
-    if (tb >= te) return;
+    const unsigned long long al = prm.ctl->alloc[prm.p];
+    const uint32_t T = alloc_tiles(al), NB = alloc_buckets(al);
+    // a contiguous run of tiles per CTA (the same runs as k_scatter): bucket histograms
+    // are flushed once per bucket segment, the last segment is also kept per CTA
+    const uint32_t tb = range_begin(T, blockIdx.x, gridDim.x), te = range_begin(T, blockIdx.x + 1, gridDim.x);
+    if (tb >= te) {
+        if (tid == 0) prm.seg_meta[blockIdx.x] = RangeMeta{EMPTY_RANGE, EMPTY_RANGE};
+        return;
+    }
     const uint64_t pol = policy_evict_first();
+    __shared__ TileCursor cur;
+    __shared__ uint64_t offs_of[NSTAGE];
 
-    auto issue = [&](int s, uint32_t t) {
+    auto issue = [&](int s) {
         uint32_t *in = info + 8 * s;
-        in[0] = t;
-        if (t >= te) return;
-        const Tile tl = prm.tiles[t];
+        in[0] = cur.valid();
+        if (!cur.valid()) return;
+        const uint64_t o = cur.offs();
+        const uint32_t cnt = cur.count();
         Seg sg;
-        const uint32_t bytes = seg_plan(keys + tl.offs, tl.count, sg);
-        in[1] = tl.count;
-        in[2] = tl.bucket;
+        const uint32_t bytes = seg_plan(keys + o, cnt, sg);
+        in[1] = cnt;
+        in[2] = cur.b;
         in[3] = sg.pad;
         in[4] = sg.i0;
         in[5] = sg.i1;
+        in[6] = cur.last_of_bucket() || cur.t + 1 == te;
+        offs_of[s] = o;
         mbar_arrive_expect_tx(&bar[s], bytes);
-        seg_issue(stage(s), keys + tl.offs, sg, &bar[s], pol);
+        seg_issue(stage(s), keys + o, sg, &bar[s], pol);
+        cur.next();
     };
     if (tid == 0) {
         for (int s = 0; s < NSTAGE; ++s) mbar_init(&bar[s], 1);
         mbar_fence_init();
-        for (int s = 0; s < NSTAGE; ++s) issue(s, tb + s);
+        cur.start(prm.buckets, NB, tb, te, prm.kpb);
+        const uint32_t fb = cur.b;
+        for (int s = 0; s < NSTAGE; ++s) issue(s);
+        prm.seg_meta[blockIdx.x].first_bucket = fb;
     }
     for (int i = tid; i < W * RADIX; i += THREADS) wh[i] = 0;
     __syncthreads();
@@ -459,10 +503,12 @@ __global__ void __launch_bounds__(THREADS) k_hist(HistParams prm) {
         const uint32_t par = (it / NSTAGE) & 1u;
         const uint32_t *in = info + 8 * s;
         const uint32_t count = in[1], bucket = in[2];
+        const bool flush = in[6] != 0;
         Seg sg;
         sg.pad = in[3];
         sg.i0 = in[4];
         sg.i1 = in[5];
+        const K *src = keys + offs_of[s];
         mbar_wait(&bar[s], par);
         const K *sb = stage(s);
         // 16-byte vectors over the staged interior
@@ -477,7 +523,6 @@ __global__ void __launch_bounds__(THREADS) k_hist(HistParams prm) {
         }
         // unaligned head / tail straight from global
         {
-            const K *src = keys + prm.tiles[t].offs;
             const uint32_t nhead = sg.i1 > sg.i0 ? sg.i0 : count;
             const uint32_t ntail = sg.i1 > sg.i0 ? count - sg.i1 : 0;
             for (uint32_t j = tid; j < nhead + ntail; j += THREADS) {
@@ -488,10 +533,10 @@ __global__ void __launch_bounds__(THREADS) k_hist(HistParams prm) {
         __syncthreads();
         if (tid == 0) {
             fence_proxy_async();
-            issue(s, t + NSTAGE);
+            issue(s);
         }
-        const bool flush = (t + 1 == te) || (prm.tiles[t + 1].bucket != bucket);
         if (flush) {
+            const bool last_seg = t + 1 == te;
             for (int d = tid; d < RADIX; d += THREADS) {
                 uint32_t sum = 0;
 #pragma unroll
@@ -500,7 +545,9 @@ __global__ void __launch_bounds__(THREADS) k_hist(HistParams prm) {
                     wh[w * RADIX + d] = 0;
                 }
                 if (sum) atomicAdd(&prm.tot[static_cast<uint64_t>(bucket) * RADIX + d], sum);
+                if (last_seg) prm.seg_last[static_cast<uint64_t>(blockIdx.x) * RADIX + d] = sum;
             }
+            if (last_seg && tid == 0) prm.seg_meta[blockIdx.x].last_bucket = bucket;
             __syncthreads();
         }
     }
@@ -516,11 +563,12 @@ struct ClassifyParams {
     const Bucket *buckets;
     const uint32_t *tot;  // this pass
     uint32_t *tot_next;   // next pass (rows of created buckets are cleared)
-    Tile *next_tiles;
     Bucket *next_buckets;
     uint32_t *sub_rel;  // [bucket][256] sub-bucket starts relative to the bucket
-    void *status;       // look-back words of this pass: cleared for ntiles[p] tiles
-    int status_bytes;
+    const uint32_t *seg_last;
+    const RangeMeta *seg_meta;
+    uint32_t *carry;    // [cta][256]: tiles of the CTA's first bucket before its range
+    uint32_t ranges;    // CTAs of the hist/scatter grid
     Ctl *ctl;
     LocalEntry *local[HRS_NUM_CLASSES];
     uint32_t local_cap[HRS_NUM_CLASSES];
@@ -571,15 +619,19 @@ __device__ void classify_bucket(const ClassifyParams &prm, const Bucket &bk, uin
     }
     if (prm.last) return;
 
-    // ---- counting children: next-pass buckets and their tiles (R2, R4)
+    // ---- counting children: next-pass buckets (R2) and their tile ranges (R4); one
+    // 64-bit atomic allocates both so bucket order stays tile order
     const uint32_t TT = ct[RADIX];
     const uint32_t NC = cb[RADIX];
     if (tid == 0) {
         uint32_t bt = 0, bb = 0;
         if (NC) {
-            bt = atomicAdd(&prm.ctl->ntiles[prm.p + 1], TT);
-            bb = atomicAdd(&prm.ctl->nbuckets[prm.p + 1], NC);
-            if (bt + TT > prm.tile_cap || bb + NC > prm.bucket_cap) atomicExch(&prm.ctl->overflow, 1u);
+            const unsigned long long a = atomicAdd(&prm.ctl->alloc[prm.p + 1],
+                                                   (static_cast<unsigned long long>(TT) << 32) | NC);
+            bt = alloc_tiles(a);
+            bb = alloc_buckets(a);
+            if (static_cast<uint64_t>(bt) + TT > prm.tile_cap || static_cast<uint64_t>(bb) + NC > prm.bucket_cap)
+                atomicExch(&prm.ctl->overflow, 1u);
         }
         misc[0] = bt;
         misc[1] = bb;
@@ -695,39 +747,36 @@ __device__ void classify_bucket(const ClassifyParams &prm, const Bucket &bk, uin
         const uint32_t id = bb + i / RADIX;
         if (id < prm.bucket_cap) prm.tot_next[static_cast<uint64_t>(id) * RADIX + (i % RADIX)] = 0;
     }
-    // child tiles, spread over the block (a child can own many tiles)
-    for (uint32_t i = tid; i < TT; i += THREADS) {
-        int lo = 0, hi = RADIX - 1;  // largest d with ct[d] <= i
-        while (lo < hi) {
-            const int mid = (lo + hi + 1) >> 1;
-            if (ct[mid] <= i) lo = mid;
-            else hi = mid - 1;
+}
+
+// Carry of every hist/scatter CTA: the digit counts of the tiles of its first bucket
+// that precede its range (an exclusive scan over CTAs, segmented by bucket).
+template <int THREADS>
+__device__ void range_carries(const ClassifyParams &prm) {
+    for (int d = threadIdx.x; d < RADIX; d += THREADS) {
+        uint32_t run = 0, prev_last = EMPTY_RANGE;
+        for (uint32_t c = 0; c < prm.ranges; ++c) {
+            const RangeMeta m = prm.seg_meta[c];
+            if (m.first_bucket == EMPTY_RANGE) continue;
+            const uint32_t car = m.first_bucket == prev_last ? run : 0u;
+            prm.carry[static_cast<uint64_t>(c) * RADIX + d] = car;
+            const uint32_t sl = prm.seg_last[static_cast<uint64_t>(c) * RADIX + d];
+            run = (m.first_bucket == m.last_bucket) ? car + sl : sl;
+            prev_last = m.last_bucket;
         }
-        const int d = lo;
-        const uint32_t k = i - ct[d];
-        const uint32_t s = tot[d];
-        if (bt + i >= prm.tile_cap) continue;
-        Tile tl;
-        tl.offs = boffs + start[d] + static_cast<uint64_t>(k) * prm.kpb;
-        tl.count = min(prm.kpb, s - k * prm.kpb);
-        tl.bucket = bb + cb[d];
-        prm.next_tiles[bt + i] = tl;
     }
 }
 
 template <int THREADS>
 __global__ void __launch_bounds__(THREADS) k_classify(ClassifyParams prm) {
     __shared__ uint32_t scratch[7 * NBINS];
-    // clear the look-back words of this pass (the scatter that follows uses them)
-    {
-        const uint64_t words16 = (static_cast<uint64_t>(prm.ctl->ntiles[prm.p]) * RADIX * prm.status_bytes) / 16;
-        uint4 *s = static_cast<uint4 *>(prm.status);
-        for (uint64_t i = static_cast<uint64_t>(blockIdx.x) * THREADS + threadIdx.x; i < words16;
-             i += static_cast<uint64_t>(gridDim.x) * THREADS)
-            s[i] = make_uint4(0, 0, 0, 0);
+    if (blockIdx.x == gridDim.x - 1) {
+        range_carries<THREADS>(prm);
+        if (gridDim.x > 1) return;
     }
-    const uint32_t nb = prm.ctl->nbuckets[prm.p];
-    for (uint32_t b = blockIdx.x; b < nb; b += gridDim.x) {
+    const uint32_t nb = alloc_buckets(prm.ctl->alloc[prm.p]);
+    const uint32_t nblk = gridDim.x > 1 ? gridDim.x - 1 : 1;
+    for (uint32_t b = blockIdx.x; b < nb; b += nblk) {
         const Bucket bk = prm.buckets[b];
         classify_bucket<THREADS>(prm, bk, b, scratch);
         __syncthreads();
@@ -744,15 +793,15 @@ struct ScatterParams {
     int p;
     int lo;
     uint32_t mask;
-    const Tile *tiles;
+    uint32_t kpb;
     const Bucket *buckets;
-    void *status;
     const uint32_t *sub_rel;
+    const uint32_t *carry;
     Ctl *ctl;
 };
 
 struct StageInfo {
-    uint32_t tile, count, bucket, kpad, k0, k1, vpad, v0, v1, pad_;
+    uint32_t valid, count, bucket, first, kpad, k0, k1, vpad, v0, v1;
     uint64_t offs;
 };
 
@@ -778,10 +827,9 @@ struct ScatterSmem {
     static constexpr size_t bytes = off_svals + (HV ? align16(sizeof(VT) * KPB) : 0);
 };
 
-template <typename K, typename V, typename S, int THREADS, int KPT, int MINB>
+template <typename K, typename V, int THREADS, int KPT, int MINB>
 __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
     using L = ScatterSmem<K, V, THREADS, KPT>;
-    using SB = StatusBits<S>;
     constexpr bool HV = HasVal<V>::value;
     using VT = ValT<V>;
     extern __shared__ __align__(16) unsigned char smem[];
@@ -794,68 +842,75 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
     VT *svals = reinterpret_cast<VT *>(smem + L::off_svals);
     auto kst = [&](int s) { return reinterpret_cast<K *>(smem + L::off_kst + s * L::kst_bytes); };
     auto vst = [&](int s) { return reinterpret_cast<VT *>(smem + L::off_vst + s * L::vst_bytes); };
+    __shared__ TileCursor cur;
 
     const K *__restrict__ kin = static_cast<const K *>(prm.keys_in);
     K *__restrict__ kout = static_cast<K *>(prm.keys_out);
     const VT *__restrict__ vin = static_cast<const VT *>(prm.vals_in);
     VT *__restrict__ vout = static_cast<VT *>(prm.vals_out);
-    S *status = static_cast<S *>(prm.status);
     const int tid = threadIdx.x, lane = tid & 31, warp = tid >> 5;
     const uint32_t wbase = static_cast<uint32_t>(warp) * 32 * KPT;
-    const uint32_t T = prm.ctl->ntiles[prm.p];
-    if (blockIdx.x >= T) return;
+    const unsigned long long al = prm.ctl->alloc[prm.p];
+    const uint32_t T = alloc_tiles(al), NB = alloc_buckets(al);
+    // the contiguous tile run of this CTA (the same runs as k_hist): the tile-ordered
+    // prefix of every digit inside a bucket is a running sum, seeded with the CTA's
+    // carry from k_classify -- stable and deterministic without any look-back
+    const uint32_t tb = range_begin(T, blockIdx.x, gridDim.x), te = range_begin(T, blockIdx.x + 1, gridDim.x);
+    if (tb >= te) return;
     const uint64_t pol = policy_evict_first();
 
-    // tiles blockIdx.x, blockIdx.x + gridDim.x, ...: every CTA is resident (persistent
-    // grid), so the look-back on lower-numbered tiles always makes progress
-    auto issue = [&](int s, uint32_t t) {
+    auto issue = [&](int s) {
         StageInfo &in = info[s];
-        in.tile = t;
-        if (t >= T) return;
-        const Tile tl = prm.tiles[t];
-        in.count = tl.count;
-        in.bucket = tl.bucket;
-        in.offs = tl.offs;
+        in.valid = cur.valid();
+        if (!cur.valid()) return;
+        const uint64_t o = cur.offs();
+        const uint32_t cnt = cur.count();
+        in.count = cnt;
+        in.bucket = cur.b;
+        in.first = cur.k == 0;
+        in.offs = o;
         Seg sk, sv;
-        uint32_t bytes = seg_plan(kin + tl.offs, tl.count, sk);
+        uint32_t bytes = seg_plan(kin + o, cnt, sk);
         in.kpad = sk.pad;
         in.k0 = sk.i0;
         in.k1 = sk.i1;
         if (HV) {
-            bytes += seg_plan(vin + tl.offs, tl.count, sv);
+            bytes += seg_plan(vin + o, cnt, sv);
             in.vpad = sv.pad;
             in.v0 = sv.i0;
             in.v1 = sv.i1;
         }
         mbar_arrive_expect_tx(&bar[s], bytes);
-        seg_issue(kst(s), kin + tl.offs, sk, &bar[s], pol);
-        if (HV) seg_issue(vst(s), vin + tl.offs, sv, &bar[s], pol);
+        seg_issue(kst(s), kin + o, sk, &bar[s], pol);
+        if (HV) seg_issue(vst(s), vin + o, sv, &bar[s], pol);
+        cur.next();
     };
     if (tid == 0) {
         mbar_init(&bar[0], 1);
         mbar_init(&bar[1], 1);
         mbar_fence_init();
-        issue(0, blockIdx.x);
-        issue(1, blockIdx.x + gridDim.x);
+        cur.start(prm.buckets, NB, tb, te, prm.kpb);
+        issue(0);
+        issue(1);
     }
     for (int i = tid; i < (THREADS / 32) * NBINS; i += THREADS) wcnt[i] = 0;
+    // running tile-ordered prefix of digit tid in the current bucket
+    uint32_t running = tid < RADIX ? prm.carry[static_cast<uint64_t>(blockIdx.x) * RADIX + tid] : 0u;
     __syncthreads();
 
     for (uint32_t it = 0;; ++it) {
         const int s = static_cast<int>(it & 1u);
         const uint32_t par = (it >> 1) & 1u;
         const StageInfo in = info[s];
-        if (in.tile >= T) break;
-        const uint32_t t = in.tile, count = in.count;
-        // per-digit bucket data for the look-back and the destinations
+        if (!in.valid) break;
+        const uint32_t count = in.count;
+        // per-digit bucket data for the destinations
         uint32_t srel = 0;
         uint64_t boffs = 0;
-        bool first = false;
         if (tid < RADIX) {
-            const Bucket bk = prm.buckets[in.bucket];
-            boffs = bk.offs;
-            first = t == bk.first_tile;
+            boffs = prm.buckets[in.bucket].offs;
             srel = prm.sub_rel[static_cast<uint64_t>(in.bucket) * RADIX + tid];
+            if (in.first) running = 0;
         }
         Seg sk, sv;
         sk.pad = in.kpad;
@@ -884,12 +939,10 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
         if (wbase < count) rank_walk<KPT>(rk, wcnt + warp * NBINS);
         __syncthreads();
         block_rank_scan<THREADS>(wcnt, tot);
-        // ---- publish this tile's digit counts for the successors' look-back
-        S cnt_d = 0;
         if (tid < RADIX) {
-            cnt_d = tot[tid + 1] - tot[tid];
-            st_volatile(status + static_cast<uint64_t>(t) * RADIX + tid,
-                        static_cast<S>((first ? SB::INC : SB::AGG) | cnt_d));
+            // destination of smem slot j holding digit d: gbase[d] + j
+            gbase[tid] = boffs + srel + running - tot[tid];
+            running += tot[tid + 1] - tot[tid];
         }
         __syncthreads();
         // ---- stage in shared memory at the rank (keys from registers, values from the staging buffer)
@@ -906,29 +959,11 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
                 }
             }
         }
-        // ---- decoupled look-back over the preceding tiles of this bucket
-        if (tid < RADIX) {
-            S excl = 0;
-            if (!first) {
-                const S *q = status + static_cast<uint64_t>(t - 1) * RADIX + tid;
-                for (;;) {
-                    const S v = ld_volatile(q);
-                    if ((v & SB::FLAGS) == 0) continue;  // predecessor not published yet
-                    excl += v & SB::VAL;
-                    if (v & SB::INC) break;
-                    q -= RADIX;
-                }
-                st_volatile(status + static_cast<uint64_t>(t) * RADIX + tid,
-                            static_cast<S>(SB::INC | (excl + cnt_d)));
-            }
-            // destination of smem slot j holding digit d: gbase[d] + j
-            gbase[tid] = boffs + srel + static_cast<uint64_t>(excl) - tot[tid];
-        }
         __syncthreads();
-        // ---- the staging buffer is free: prefetch tile it + 2 into it
+        // ---- the staging buffer is free: prefetch the tile after next into it
         if (tid == 0) {
             fence_proxy_async();
-            issue(s, blockIdx.x + (it + 2) * gridDim.x);
+            issue(s);
         }
         // ---- write-combined stores: consecutive slots of a digit run are consecutive addresses
 #pragma unroll
