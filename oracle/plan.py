@@ -42,10 +42,16 @@ def digit_plan(begin_bit: int, end_bit: int):
     return out
 
 
+def class_capacity(c: int) -> int:
+    """Upper size of local-sort class c.  P:562-566 gives [1,128], (128,256], (256,512],
+    ... as an example; reading #20: powers of two up to 4096, then 6144, 8192."""
+    return (128 << c) if c < 6 else (6144 if c == 6 else 8192)
+
+
 def size_class(size: int) -> int:
-    """0 for [1,128], 1 for (128,256], 2 for (256,512], ... (P:564-566)."""
+    """Smallest class whose capacity holds `size` records (capped at class 7)."""
     c = 0
-    while (128 << c) < size:
+    while class_capacity(c) < size and c < 7:
         c += 1
     return c
 

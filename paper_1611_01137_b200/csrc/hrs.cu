@@ -93,16 +93,14 @@ template <> struct LocalCfg<2> { static constexpr int THREADS = 64, KPT = 8; };
 template <> struct LocalCfg<3> { static constexpr int THREADS = 128, KPT = 8; };
 template <> struct LocalCfg<4> { static constexpr int THREADS = 128, KPT = 16; };
 template <> struct LocalCfg<5> { static constexpr int THREADS = 256, KPT = 16; };
-template <> struct LocalCfg<6> { static constexpr int THREADS = 512, KPT = 16; };
-template <> struct LocalCfg<7> { static constexpr int THREADS = 1024, KPT = 16; };
+template <> struct LocalCfg<6> { static constexpr int THREADS = 384, KPT = 16; };
+template <> struct LocalCfg<7> { static constexpr int THREADS = 512, KPT = 16; };
 
 // two-stage TMA prefetch where it fits next to a second resident CTA, else one stage
 template <typename K, typename V, int C>
 struct LocalStages {
     using LC = LocalCfg<C>;
-    static constexpr int NSTAGE =
-        LocalSmem<K, V, LC::THREADS, LC::KPT, 2>::bytes <= 110 * 1024 ? 2
-        : LocalSmem<K, V, LC::THREADS, LC::KPT, 2>::bytes <= SMEM_LIMIT && LC::THREADS <= 256 ? 2 : 1;
+    static constexpr int NSTAGE = LocalSmem<K, V, LC::THREADS, LC::KPT, 2>::bytes <= 110 * 1024 ? 2 : 1;
     static constexpr size_t bytes = LocalSmem<K, V, LC::THREADS, LC::KPT, NSTAGE>::bytes;
     static constexpr bool fits = bytes <= SMEM_LIMIT;
 };
@@ -127,7 +125,7 @@ uint32_t max_kpb(int kb, int vb) {
     if (kb == 4 && vb <= 4) return ScatterCfg<4, 4>::THREADS * ScatterCfg<4, 4>::KPT;
     return ScatterCfg<8, 8>::THREADS * ScatterCfg<8, 8>::KPT;
 }
-uint32_t max_lt(int kb, int vb) { return 128u << max_class(kb, vb); }
+uint32_t max_lt(int kb, int vb) { return class_capacity(max_class(kb, vb)); }
 
 // ------------------------------------------------------------------ launch helpers
 
@@ -280,8 +278,8 @@ hrs_status make_plan(Plan &pl, uint64_t n, int kb, int vb, int begin, int end, c
                 cap = c == pl.single_class ? std::min<uint64_t>(n, 2 * n / pl.mt + 2 * pl.D * (n / lt + 1)) + 2 : 0;
             } else if (c == 0) {
                 cap = std::min<uint64_t>(n, 2 * n / pl.mt + 2 * pl.D * (n / lt + 1)) + 2;
-            } else if ((64u << c) < pl.lt) {
-                cap = n / (64ull << c) + 2;  // entries of class c hold > 64 * 2^c records
+            } else if (class_capacity(c - 1) < pl.lt) {
+                cap = n / (class_capacity(c - 1) + 1ull) + 2;  // entries of class c hold > capacity(c - 1)
             }
             if (!pl.counting) cap = (c == (pl.single_class >= 0 ? pl.single_class : size_class_of((uint32_t)std::max<uint64_t>(n, 1)))) ? 1 : 0;
         }
@@ -474,7 +472,7 @@ struct Runner {
             lp.list = at<LocalEntry>(temp, pl.off_local[C]);
             lp.count = &at<Ctl>(temp, 0)->nlocal[C];
             lp.begin_bit = pl.begin;
-            auto fn = k_local<K, V, LC::THREADS, LC::KPT, LST::NSTAGE, 1>;
+            auto fn = k_local<K, V, LC::THREADS, LC::KPT, LST::NSTAGE, (LC::THREADS >= 256 ? 2 : 1)>;
             int grid = 0;
             hrs_status s = grid_for(fn, LC::THREADS, LST::bytes, dev, sms, &grid);
             if (s) return s;

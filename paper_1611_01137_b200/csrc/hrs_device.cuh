@@ -109,9 +109,15 @@ struct HasVal<NoVal> {
 template <typename V>
 using ValT = typename std::conditional<HasVal<V>::value, V, uint32_t>::type;
 
+// Local-sort size classes (P:562-566 gives [1,128], (128,256], (256,512], ... as an
+// example): powers of two up to 4096, then (4096, 6144] and (6144, 8192] so that the
+// ~4096-record buckets a uniform input leaves after two passes fill their CTA.
+__host__ __device__ __forceinline__ uint32_t class_capacity(int c) {
+    return c < 6 ? (128u << c) : (c == 6 ? 6144u : 8192u);
+}
 __host__ __device__ __forceinline__ int size_class_of(uint32_t size) {
     int c = 0;
-    while ((128u << c) < size && c < HRS_NUM_CLASSES - 1) ++c;
+    while (class_capacity(c) < size && c < HRS_NUM_CLASSES - 1) ++c;
     return c;
 }
 
@@ -289,35 +295,45 @@ __device__ __forceinline__ void seg_fill_edges(T *sbuf, const T *src, const Seg 
 }
 
 // ------------------------------------------------------------------ stable block rank
+//
+// The KPT keys a warp holds are in "warp-striped" order: element e of the tile is
+// warp * 32 * KPT + c * 32 + lane.  A stable rank (position among all keys of the
+// tile, ties in element order) is computed in three steps:
+//   1. count_digits: per-warp digit histogram with non-returning shared atomics
+//      (full speed on B200 whatever the skew; profiles/r01_micro_hist.txt);
+//   2. block_rank_scan: wcnt[w][d] = first slot of warp w's run of digit d;
+//   3. rank_in_place: column by column, every lane reads the warp's next free slot
+//      of its digit, adds 1 with a non-returning atomic and reads the counter back:
+//      the difference is the number of lanes of the column with that digit.  Lanes
+//      with duplicates take their order from one match-any over the column where
+//      all other lanes share one dummy value, so its cost depends only on the few
+//      distinct duplicated digits (match-any over 32 distinct values is what makes a
+//      pure match-based multisplit slow on B200; profiles/r01_micro_rank.txt).
 
-// Ranks the KPT keys a warp holds in "warp-striped" order (element e of the tile =
-// warp * 32 * KPT + c * 32 + lane) by digit, stably.  Per column: the warp's running
-// digit counter is read, every lane adds 1 with a non-returning shared atomic (full
-// speed on B200 for any skew), the counter is read back: lanes whose digit occurs
-// once in the column have their rank; only lanes with duplicates run match-any among
-// themselves (its cost grows with the number of distinct values, which is small
-// there).  profiles/r01_micro_rank.txt compares this with match-only and
-// ballot-sliced ranking.
-// On entry rk[c] holds the digit (INVALID_DIGIT for padding lanes); on exit
-// (rank within the warp's run of the digit << 9) | digit.
 template <int KPT>
-__device__ __forceinline__ void rank_walk(uint32_t (&rk)[KPT], uint32_t *mycnt) {
+__device__ __forceinline__ void count_digits(const uint32_t (&dg)[KPT], uint32_t *mycnt) {
+#pragma unroll
+    for (int c = 0; c < KPT; ++c) atomicAdd(&mycnt[dg[c]], 1u);
+}
+
+// On entry dg[c] holds the digit (INVALID_DIGIT for padding); on exit the slot.
+template <int KPT>
+__device__ __forceinline__ void rank_in_place(uint32_t (&dg)[KPT], uint32_t *mycnt) {
     const uint32_t ltm = lanemask_lt();
 #pragma unroll
     for (int c = 0; c < KPT; ++c) {
-        const uint32_t d = rk[c];
+        const uint32_t d = dg[c];
         const uint32_t pre = mycnt[d];
         __syncwarp();
         atomicAdd(&mycnt[d], 1u);
         __syncwarp();
         const uint32_t k = mycnt[d] - pre;
         uint32_t r = 0;
-        const uint32_t dup = __ballot_sync(0xffffffffu, k > 1);
-        if (k > 1) {
-            const uint32_t m = __match_any_sync(dup, d);
-            r = __popc(m & ltm);
+        if (__any_sync(0xffffffffu, k > 1)) {
+            const uint32_t m = __match_any_sync(0xffffffffu, k > 1 ? d : 0xFFFFFFFFu);
+            r = k > 1 ? __popc(m & ltm) : 0u;
         }
-        rk[c] = ((pre + r) << 9) | d;
+        dg[c] = pre + r;
     }
 }
 
@@ -898,6 +914,9 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
     uint32_t running = tid < RADIX ? prm.carry[static_cast<uint64_t>(blockIdx.x) * RADIX + tid] : 0u;
     __syncthreads();
 
+    const int lo = prm.lo;
+    const uint32_t mask = prm.mask;
+    uint32_t *mycnt = wcnt + warp * NBINS;
     for (uint32_t it = 0;; ++it) {
         const int s = static_cast<int>(it & 1u);
         const uint32_t par = (it >> 1) & 1u;
@@ -922,43 +941,49 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
         const K *ksrc = kin + in.offs;
         const VT *vsrc = HV ? vin + in.offs : nullptr;
         mbar_wait(&bar[s], par);
-        // ---- keys into registers (warp-striped), stable rank
-        K key[KPT];
-        uint32_t rk[KPT];
         const K *ks = kst(s);
-#pragma unroll
-        for (int c = 0; c < KPT; ++c) {
-            const uint32_t e = wbase + c * 32 + lane;
-            if (e < count) {
-                key[c] = seg_get(ks, ksrc, sk, e);
-                rk[c] = digit_of(key[c], prm.lo, prm.mask);
-            } else {
-                rk[c] = INVALID_DIGIT;
-            }
-        }
-        if (wbase < count) rank_walk<KPT>(rk, wcnt + warp * NBINS);
-        __syncthreads();
-        block_rank_scan<THREADS>(wcnt, tot);
-        if (tid < RADIX) {
-            // destination of smem slot j holding digit d: gbase[d] + j
-            gbase[tid] = boffs + srel + running - tot[tid];
-            running += tot[tid + 1] - tot[tid];
-        }
-        __syncthreads();
-        // ---- stage in shared memory at the rank (keys from registers, values from the staging buffer)
-        {
-            const uint32_t *mycnt = wcnt + warp * NBINS;
-            const VT *vs = HV ? vst(s) : nullptr;
+        const VT *vs = HV ? vst(s) : nullptr;
+        // full tiles with an aligned interior take the predicate-free path
+        const bool full = count == static_cast<uint32_t>(L::KPB) && sk.i0 == 0 && sk.i1 == count &&
+                          (!HV || (sv.i0 == 0 && sv.i1 == count));
+        auto body = [&](auto full_tag) {
+            constexpr bool FULL = decltype(full_tag)::value;
+            // ---- keys into registers (warp-striped) and digits
+            K key[KPT];
+            uint32_t dg[KPT];
 #pragma unroll
             for (int c = 0; c < KPT; ++c) {
-                const uint32_t d = rk[c] & 511u;
-                if (d != INVALID_DIGIT) {
-                    const uint32_t r = mycnt[d] + (rk[c] >> 9);
-                    skeys[r] = key[c];
-                    if (HV) svals[r] = seg_get(vs, vsrc, sv, wbase + c * 32 + lane);
+                const uint32_t e = wbase + c * 32 + lane;
+                if (FULL || e < count) {
+                    key[c] = FULL ? ks[sk.pad + e] : seg_get(ks, ksrc, sk, e);
+                    dg[c] = digit_of(key[c], lo, mask);
+                } else {
+                    dg[c] = INVALID_DIGIT;
                 }
             }
-        }
+            // ---- stable rank
+            if (FULL || wbase < count) count_digits<KPT>(dg, mycnt);
+            __syncthreads();
+            block_rank_scan<THREADS>(wcnt, tot);
+            if (tid < RADIX) {
+                // destination of smem slot j holding digit d: gbase[d] + j
+                gbase[tid] = boffs + srel + running - tot[tid];
+                running += tot[tid + 1] - tot[tid];
+            }
+            __syncthreads();
+            if (FULL || wbase < count) rank_in_place<KPT>(dg, mycnt);
+            // ---- stage in shared memory at the rank
+#pragma unroll
+            for (int c = 0; c < KPT; ++c) {
+                const uint32_t e = wbase + c * 32 + lane;
+                if (FULL || e < count) {
+                    skeys[dg[c]] = key[c];
+                    if (HV) svals[dg[c]] = FULL ? vs[sv.pad + e] : seg_get(vs, vsrc, sv, e);
+                }
+            }
+        };
+        if (full) body(std::true_type{});
+        else body(std::false_type{});
         __syncthreads();
         // ---- the staging buffer is free: prefetch the tile after next into it
         if (tid == 0) {
@@ -966,14 +991,25 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
             issue(s);
         }
         // ---- write-combined stores: consecutive slots of a digit run are consecutive addresses
+        if (count == static_cast<uint32_t>(L::KPB)) {
 #pragma unroll
-        for (int c = 0; c < KPT; ++c) {
-            const uint32_t j = c * THREADS + tid;
-            if (j < count) {
+            for (int c = 0; c < KPT; ++c) {
+                const uint32_t j = c * THREADS + tid;
                 const K k = skeys[j];
-                const uint64_t pos = gbase[digit_of(k, prm.lo, prm.mask)] + j;
+                const uint64_t pos = gbase[digit_of(k, lo, mask)] + j;
                 kout[pos] = k;
                 if (HV) vout[pos] = svals[j];
+            }
+        } else {
+#pragma unroll
+            for (int c = 0; c < KPT; ++c) {
+                const uint32_t j = c * THREADS + tid;
+                if (j < count) {
+                    const K k = skeys[j];
+                    const uint64_t pos = gbase[digit_of(k, lo, mask)] + j;
+                    kout[pos] = k;
+                    if (HV) vout[pos] = svals[j];
+                }
             }
         }
         for (int i = tid; i < (THREADS / 32) * NBINS; i += THREADS) wcnt[i] = 0;
@@ -993,6 +1029,10 @@ struct LocalParams {
     int begin_bit;
 };
 
+// Shared memory of one local-sort CTA: NSTAGE staging buffers {keys, values}; after
+// the keys have been read into registers the key buffer doubles as the buffer of
+// the LSD passes, which move (key, 16-bit index) pairs; the values are gathered from
+// their staging buffer once, at the end.
 template <typename K, typename V, int THREADS, int KPT, int NSTAGE>
 struct LocalSmem {
     static constexpr int W = THREADS / 32;
@@ -1004,13 +1044,12 @@ struct LocalSmem {
     static constexpr size_t off_wcnt = align16(off_info + sizeof(uint32_t) * 16 * NSTAGE);
     static constexpr size_t off_tot = align16(off_wcnt + sizeof(uint32_t) * W * NBINS);
     static constexpr size_t off_red = align16(off_tot + sizeof(uint32_t) * 288);
-    static constexpr size_t off_kst = align16(off_red + sizeof(K) * 2 * W);
+    static constexpr size_t off_sidx = align16(off_red + sizeof(K) * 2 * W);
+    static constexpr size_t off_kst = align16(off_sidx + sizeof(uint16_t) * CAP);
     static constexpr size_t kst_bytes = align16(sizeof(K) * (CAP + 16 / sizeof(K)));
     static constexpr size_t off_vst = off_kst + NSTAGE * kst_bytes;
     static constexpr size_t vst_bytes = HV ? align16(sizeof(VT) * (CAP + 16 / sizeof(VT))) : 0;
-    static constexpr size_t off_skeys = off_vst + NSTAGE * vst_bytes;
-    static constexpr size_t off_sidx = align16(off_skeys + sizeof(K) * CAP);
-    static constexpr size_t bytes = off_sidx + align16(sizeof(uint16_t) * CAP);
+    static constexpr size_t bytes = off_vst + NSTAGE * vst_bytes;
 };
 
 template <typename K>
@@ -1038,7 +1077,6 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
     uint32_t *wcnt = reinterpret_cast<uint32_t *>(smem + L::off_wcnt);
     uint32_t *tot = reinterpret_cast<uint32_t *>(smem + L::off_tot);
     K *red = reinterpret_cast<K *>(smem + L::off_red);
-    K *skeys = reinterpret_cast<K *>(smem + L::off_skeys);
     uint16_t *sidx = reinterpret_cast<uint16_t *>(smem + L::off_sidx);
     auto kst = [&](int s) { return reinterpret_cast<K *>(smem + L::off_kst + s * L::kst_bytes); };
     auto vst = [&](int s) { return reinterpret_cast<VT *>(smem + L::off_vst + s * L::vst_bytes); };
@@ -1049,6 +1087,8 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
     K *__restrict__ kout = static_cast<K *>(prm.keys_out);
     VT *__restrict__ vout = static_cast<VT *>(prm.vals_out);
     const uint64_t pol = policy_evict_first();
+    const int begin_bit = prm.begin_bit;
+    uint32_t *mycnt = wcnt + warp * NBINS;
 
     auto srck = [&](uint32_t code) -> const K * {
         return static_cast<const K *>(code == SRC_IN    ? prm.src_keys[SRC_IN]
@@ -1094,6 +1134,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
         mbar_fence_init();
         for (int s = 0; s < NSTAGE; ++s) issue(s, blockIdx.x + s * gridDim.x);
     }
+    for (int i = tid; i < W * NBINS; i += THREADS) wcnt[i] = 0;
     __syncthreads();
 
     for (uint32_t it = 0;; ++it) {
@@ -1143,7 +1184,6 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
             red[warp] = a;
             red[W + warp] = o;
         }
-        for (int i = tid; i < W * NBINS; i += THREADS) wcnt[i] = 0;
         __syncthreads();
         K diff = 0;
         {
@@ -1155,30 +1195,28 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
             }
             diff = aa ^ oo;
         }
+        K *skeys = ks;  // the keys are in registers: their staging buffer sorts them
+        const bool active = wbase < count;
         bool moved = false;
-        for (int lo = prm.begin_bit; lo < hi_bit; lo += 8) {
+        for (int lo = begin_bit; lo < hi_bit; lo += 8) {
             const int width = min(8, hi_bit - lo);
             const uint32_t mask = (1u << width) - 1u;
             if ((static_cast<uint32_t>(diff >> lo) & mask) == 0) continue;  // constant digit: identity pass
             moved = true;
-            uint32_t rk[KPT];
+            uint32_t dg[KPT];
 #pragma unroll
             for (int c = 0; c < KPT; ++c)
-                rk[c] = (wbase + c * 32 + lane) < count ? digit_of(key[c], lo, mask) : INVALID_DIGIT;
-            if (wbase < count) rank_walk<KPT>(rk, wcnt + warp * NBINS);
+                dg[c] = (wbase + c * 32 + lane) < count ? digit_of(key[c], lo, mask) : INVALID_DIGIT;
+            if (active) count_digits<KPT>(dg, mycnt);
             __syncthreads();
             block_rank_scan<THREADS>(wcnt, tot);
             __syncthreads();
-            {
-                const uint32_t *mycnt = wcnt + warp * NBINS;
+            if (active) rank_in_place<KPT>(dg, mycnt);
 #pragma unroll
-                for (int c = 0; c < KPT; ++c) {
-                    const uint32_t d = rk[c] & 511u;
-                    if (d != INVALID_DIGIT) {
-                        const uint32_t r = mycnt[d] + (rk[c] >> 9);
-                        skeys[r] = key[c];
-                        sidx[r] = static_cast<uint16_t>(idx[c]);
-                    }
+            for (int c = 0; c < KPT; ++c) {
+                if ((wbase + c * 32 + lane) < count) {
+                    skeys[dg[c]] = key[c];
+                    sidx[dg[c]] = static_cast<uint16_t>(idx[c]);
                 }
             }
             __syncthreads();
@@ -1208,7 +1246,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
             fence_proxy_async();
             issue(s, blockIdx.x + (it + NSTAGE) * gridDim.x);
         }
-        __syncthreads();
+        __syncthreads();  // info[s] is rewritten above
     }
 }
 
