@@ -9,7 +9,8 @@ import ctypes
 import os
 
 HERE = os.path.dirname(os.path.abspath(__file__))
-LIB_PATH = os.path.join(HERE, "libhrs.so")
+# HRS_LIB overrides the library path (used only by the kernel-variant experiments in micro/)
+LIB_PATH = os.environ.get("HRS_LIB") or os.path.join(HERE, "libhrs.so")
 
 HRS_MAX_PASSES = 8
 HRS_NUM_CLASSES = 8

@@ -217,7 +217,8 @@ struct Plan {
     uint32_t local_cap[HRS_NUM_CLASSES] = {0};
     uint32_t range_cap = 0;  // CTAs of the hist/scatter grid the temp layout allows
     size_t off_auxk = 0, off_auxv = 0, off_buckets[2] = {0, 0}, off_tot[2] = {0, 0}, off_subrel = 0,
-           off_seg_last = 0, off_seg_meta = 0, off_carry = 0, off_local[HRS_NUM_CLASSES] = {0}, total = 0;
+           off_seg_last = 0, off_seg_meta = 0, off_carry = 0, off_tiles = 0, off_tile_pref = 0,
+           off_local[HRS_NUM_CLASSES] = {0}, total = 0;
 };
 
 size_t align_up(size_t x, size_t a) { return (x + a - 1) / a * a; }
@@ -306,6 +307,10 @@ hrs_status make_plan(Plan &pl, uint64_t n, int kb, int vb, int begin, int end, c
     off = align_up(off + sizeof(uint32_t) * RADIX * static_cast<size_t>(pl.range_cap), 256);
     pl.off_seg_meta = off;
     off = align_up(off + sizeof(RangeMeta) * static_cast<size_t>(pl.range_cap), 256);
+    pl.off_tiles = off;
+    off = align_up(off + sizeof(TileDesc) * static_cast<size_t>(pl.tile_cap), 256);
+    pl.off_tile_pref = off;
+    off = align_up(off + sizeof(uint32_t) * RADIX * static_cast<size_t>(pl.tile_cap), 256);
     pl.off_subrel = off;
     off = align_up(off + sizeof(uint32_t) * RADIX * static_cast<size_t>(pl.bucket_cap), 256);
     for (int c = 0; c < HRS_NUM_CLASSES; ++c) {
@@ -353,13 +358,13 @@ struct Runner {
         return last_launch();
     }
 
-    // the hist / classify / scatter grid of a pass: the scatter's persistent grid,
-    // capped by the temp layout (range_cap >= tiles of any pass is not required)
+    // the hist / classify grid of a pass (CTAs = contiguous tile runs): the hist
+    // kernel's persistent grid, capped by the temp layout
     static hrs_status range_grid(const Plan &pl, int dev, int sms, uint32_t *G) {
-        auto fn = k_scatter<K, V, SC::THREADS, SC::KPT, SC::MINB>;
-        const size_t smem = ScatterSmem<K, V, SC::THREADS, SC::KPT>::bytes;
+        auto fn = k_hist<K, HIST_THREADS, HIST_STAGES, HIST_CAP>;
+        const size_t smem = HistSmem<K, HIST_THREADS, HIST_STAGES, HIST_CAP>::bytes;
         int grid = 0;
-        hrs_status s = grid_for(fn, SC::THREADS, smem, dev, sms, &grid);
+        hrs_status s = grid_for(fn, HIST_THREADS, smem, dev, sms, &grid);
         if (s) return s;
         *G = std::min<uint32_t>(static_cast<uint32_t>(grid), pl.range_cap);
         return HRS_SUCCESS;
@@ -377,6 +382,8 @@ struct Runner {
         hp.tot = at<uint32_t>(temp, pl.off_tot[p & 1]);
         hp.seg_last = at<uint32_t>(temp, pl.off_seg_last);
         hp.seg_meta = at<RangeMeta>(temp, pl.off_seg_meta);
+        hp.tiles = at<TileDesc>(temp, pl.off_tiles);
+        hp.tile_pref = at<uint32_t>(temp, pl.off_tile_pref);
         hp.ctl = at<Ctl>(temp, 0);
         auto fn = k_hist<K, HIST_THREADS, HIST_STAGES, HIST_CAP>;
         const size_t smem = HistSmem<K, HIST_THREADS, HIST_STAGES, HIST_CAP>::bytes;
@@ -440,15 +447,20 @@ struct Runner {
         sp.p = p;
         sp.lo = pl.lo[p - 1];
         sp.mask = (1u << (pl.hi[p - 1] - pl.lo[p - 1])) - 1u;
-        sp.kpb = pl.kpb;
         sp.buckets = at<Bucket>(temp, pl.off_buckets[p & 1]);
         sp.sub_rel = at<uint32_t>(temp, pl.off_subrel);
         sp.carry = at<uint32_t>(temp, pl.off_carry);
+        sp.tiles = at<TileDesc>(temp, pl.off_tiles);
+        sp.tile_pref = at<uint32_t>(temp, pl.off_tile_pref);
         sp.ctl = at<Ctl>(temp, 0);
         auto fn = k_scatter<K, V, SC::THREADS, SC::KPT, SC::MINB>;
         const size_t smem = ScatterSmem<K, V, SC::THREADS, SC::KPT>::bytes;
+        int grid = 0;
+        hrs_status s = grid_for(fn, SC::THREADS, smem, dev, sms, &grid);
+        if (s) return s;
+        (void)G;
         LaunchScope ls(st, 2, p);
-        fn<<<G, SC::THREADS, smem, st>>>(sp);
+        fn<<<grid, SC::THREADS, smem, st>>>(sp);
         return last_launch();
     }
 

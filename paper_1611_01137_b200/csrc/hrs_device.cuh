@@ -20,11 +20,12 @@
 //   k_scatter<p>   per tile, with the next tile already in flight through TMA: a
 //                  STABLE in-tile rank, staging in shared memory and write-combined
 //                  stores of every digit run (Fig 3); values follow their
-//                  keys.  k_hist and k_scatter give every CTA the same
-//                  contiguous run of tiles, so the tile-ordered offset of each tile
-//                  inside its sub-bucket is a running sum in the CTA seeded by a
-//                  per-CTA carry (computed by k_classify): deterministic, and it
-//                  replaces the atomicAdd chunk reservation of P:696-703 (not stable).
+//                  keys.  The tile-ordered offset of every tile inside
+//                  its sub-bucket is known before the scatter starts: k_hist walks a
+//                  contiguous run of tiles per CTA and records each tile's prefix
+//                  within the run, k_classify scans the runs into per-CTA carries.
+//                  Deterministic, no look-back, and it replaces the atomicAdd chunk
+//                  reservation of P:696-703 (which is not stable).
 //
 // then one k_local launch per size class sorts every bucket of at most
 // ∂ˆ records on chip: a stable LSD radix sort of (key, index) pairs over the
@@ -40,6 +41,10 @@
 #include <type_traits>
 
 #include "../../include/hrs.h"
+
+#ifndef HRS_EXP
+#define HRS_EXP 0  // kernel-variant experiments (micro/scatter_exp.py); 0 in the product
+#endif
 
 namespace hrs {
 
@@ -58,6 +63,16 @@ struct Bucket {
     uint32_t count;
     uint32_t first_tile;
     uint32_t ntiles;
+    uint32_t pad;
+};
+// One tile as k_hist saw it, for k_scatter: records [offs, offs + count) of bucket
+// `bucket`; carry_row = the hist CTA whose carry applies (tile in the first bucket
+// segment of that CTA's run), or EMPTY.
+struct TileDesc {
+    uint64_t offs;
+    uint32_t count;
+    uint32_t bucket;
+    uint32_t carry_row;
     uint32_t pad;
 };
 // A local-sort assignment: bits [begin_bit, hi_bit) remain to sort.
@@ -442,6 +457,8 @@ struct HistParams {
     uint32_t *tot;             // [bucket][256] of this pass (zeroed by the creator of the bucket)
     uint32_t *seg_last;        // [cta][256]: counts of the CTA's last bucket segment
     RangeMeta *seg_meta;       // [cta]
+    TileDesc *tiles;           // [tile]: descriptor for k_scatter
+    uint32_t *tile_pref;       // [tile][256]: digit counts of the earlier tiles of its bucket segment
     Ctl *ctl;
 };
 
@@ -463,7 +480,8 @@ __global__ void __launch_bounds__(THREADS) k_hist(HistParams prm) {
     constexpr int VK = 16 / sizeof(K);
     extern __shared__ __align__(16) unsigned char smem[];
     uint64_t *bar = reinterpret_cast<uint64_t *>(smem + L::off_bar);
-    // info[s]: 0 valid, 1 count, 2 bucket, 3 pad, 4 i0, 5 i1, 6 last tile of its bucket, 7 offs lo
+    // info[s]: 0 valid, 1 count, 2 bucket, 3 pad, 4 i0, 5 i1, 6 last tile of its bucket segment,
+    //          7 tile index
     uint32_t *info = reinterpret_cast<uint32_t *>(smem + L::off_info);
     uint32_t *wh = reinterpret_cast<uint32_t *>(smem + L::off_wh);
     auto stage = [&](int s) {
@@ -498,6 +516,7 @@ __global__ void __launch_bounds__(THREADS) k_hist(HistParams prm) {
         in[4] = sg.i0;
         in[5] = sg.i1;
         in[6] = cur.last_of_bucket() || cur.t + 1 == te;
+        in[7] = cur.t;
         offs_of[s] = o;
         mbar_arrive_expect_tx(&bar[s], bytes);
         seg_issue(stage(s), keys + o, sg, &bar[s], pol);
@@ -514,6 +533,8 @@ __global__ void __launch_bounds__(THREADS) k_hist(HistParams prm) {
     for (int i = tid; i < W * RADIX; i += THREADS) wh[i] = 0;
     __syncthreads();
     uint32_t *my = wh + warp * RADIX;
+    uint32_t seg_run = 0;            // digit tid: count of the current bucket segment before this tile
+    bool first_seg = true;           // inside the CTA's first bucket segment (its carry applies)
     for (uint32_t t = tb, it = 0; t < te; ++t, ++it) {
         const int s = static_cast<int>(it % NSTAGE);
         const uint32_t par = (it / NSTAGE) & 1u;
@@ -524,7 +545,19 @@ __global__ void __launch_bounds__(THREADS) k_hist(HistParams prm) {
         sg.pad = in[3];
         sg.i0 = in[4];
         sg.i1 = in[5];
-        const K *src = keys + offs_of[s];
+        const uint64_t toffs = offs_of[s];
+        const K *src = keys + toffs;
+        // tile descriptor and tile-ordered prefix for the scatter
+        if (tid < RADIX) prm.tile_pref[static_cast<uint64_t>(t) * RADIX + tid] = seg_run;
+        if (tid == 0) {
+            TileDesc td;
+            td.offs = toffs;
+            td.count = count;
+            td.bucket = bucket;
+            td.carry_row = first_seg ? blockIdx.x : EMPTY_RANGE;
+            td.pad = 0;
+            prm.tiles[t] = td;
+        }
         mbar_wait(&bar[s], par);
         const K *sb = stage(s);
         // 16-byte vectors over the staged interior
@@ -551,19 +584,25 @@ __global__ void __launch_bounds__(THREADS) k_hist(HistParams prm) {
             fence_proxy_async();
             issue(s);
         }
+        // segment count so far (the per-warp counters accumulate over the segment)
+        uint32_t sum = 0;
+        if (tid < RADIX) {
+#pragma unroll
+            for (int w = 0; w < W; ++w) sum += wh[w * RADIX + tid];
+            seg_run = sum;
+        }
+        __syncthreads();  // the next tile's counts must not land before the sums are read
         if (flush) {
             const bool last_seg = t + 1 == te;
-            for (int d = tid; d < RADIX; d += THREADS) {
-                uint32_t sum = 0;
+            if (tid < RADIX) {
 #pragma unroll
-                for (int w = 0; w < W; ++w) {
-                    sum += wh[w * RADIX + d];
-                    wh[w * RADIX + d] = 0;
-                }
-                if (sum) atomicAdd(&prm.tot[static_cast<uint64_t>(bucket) * RADIX + d], sum);
-                if (last_seg) prm.seg_last[static_cast<uint64_t>(blockIdx.x) * RADIX + d] = sum;
+                for (int w = 0; w < W; ++w) wh[w * RADIX + tid] = 0;
+                if (sum) atomicAdd(&prm.tot[static_cast<uint64_t>(bucket) * RADIX + tid], sum);
+                if (last_seg) prm.seg_last[static_cast<uint64_t>(blockIdx.x) * RADIX + tid] = sum;
             }
             if (last_seg && tid == 0) prm.seg_meta[blockIdx.x].last_bucket = bucket;
+            seg_run = 0;
+            first_seg = false;
             __syncthreads();
         }
     }
@@ -809,15 +848,16 @@ struct ScatterParams {
     int p;
     int lo;
     uint32_t mask;
-    uint32_t kpb;
     const Bucket *buckets;
     const uint32_t *sub_rel;
     const uint32_t *carry;
+    const TileDesc *tiles;
+    const uint32_t *tile_pref;
     Ctl *ctl;
 };
 
 struct StageInfo {
-    uint32_t valid, count, bucket, first, kpad, k0, k1, vpad, v0, v1;
+    uint32_t valid, count, bucket, carry_row, kpad, k0, k1, vpad, v0, v1, tile, pad_;
     uint64_t offs;
 };
 
@@ -858,60 +898,54 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
     VT *svals = reinterpret_cast<VT *>(smem + L::off_svals);
     auto kst = [&](int s) { return reinterpret_cast<K *>(smem + L::off_kst + s * L::kst_bytes); };
     auto vst = [&](int s) { return reinterpret_cast<VT *>(smem + L::off_vst + s * L::vst_bytes); };
-    __shared__ TileCursor cur;
-
     const K *__restrict__ kin = static_cast<const K *>(prm.keys_in);
     K *__restrict__ kout = static_cast<K *>(prm.keys_out);
     const VT *__restrict__ vin = static_cast<const VT *>(prm.vals_in);
     VT *__restrict__ vout = static_cast<VT *>(prm.vals_out);
     const int tid = threadIdx.x, lane = tid & 31, warp = tid >> 5;
     const uint32_t wbase = static_cast<uint32_t>(warp) * 32 * KPT;
-    const unsigned long long al = prm.ctl->alloc[prm.p];
-    const uint32_t T = alloc_tiles(al), NB = alloc_buckets(al);
-    // the contiguous tile run of this CTA (the same runs as k_hist): the tile-ordered
-    // prefix of every digit inside a bucket is a running sum, seeded with the CTA's
-    // carry from k_classify -- stable and deterministic without any look-back
-    const uint32_t tb = range_begin(T, blockIdx.x, gridDim.x), te = range_begin(T, blockIdx.x + 1, gridDim.x);
-    if (tb >= te) return;
+    const uint32_t T = alloc_tiles(prm.ctl->alloc[prm.p]);
+    if (blockIdx.x >= T) return;
     const uint64_t pol = policy_evict_first();
 
-    auto issue = [&](int s) {
+    // tiles blockIdx.x, blockIdx.x + gridDim.x, ...: the tiles in flight at any moment
+    // are neighbours, so the runs they write to a sub-bucket are adjacent in memory
+    // and combine in L2 (contiguous runs per CTA measured +25% DRAM traffic).  The
+    // tile-ordered offsets come from k_hist (tile_pref) and k_classify (carry), so the
+    // tiles are independent: no look-back.
+    auto issue = [&](int s, uint32_t t) {
         StageInfo &in = info[s];
-        in.valid = cur.valid();
-        if (!cur.valid()) return;
-        const uint64_t o = cur.offs();
-        const uint32_t cnt = cur.count();
-        in.count = cnt;
-        in.bucket = cur.b;
-        in.first = cur.k == 0;
-        in.offs = o;
+        in.valid = t < T;
+        if (t >= T) return;
+        const TileDesc td = prm.tiles[t];
+        in.count = td.count;
+        in.bucket = td.bucket;
+        in.carry_row = td.carry_row;
+        in.offs = td.offs;
+        in.tile = t;
         Seg sk, sv;
-        uint32_t bytes = seg_plan(kin + o, cnt, sk);
+        uint32_t bytes = seg_plan(kin + td.offs, td.count, sk);
         in.kpad = sk.pad;
         in.k0 = sk.i0;
         in.k1 = sk.i1;
         if (HV) {
-            bytes += seg_plan(vin + o, cnt, sv);
+            bytes += seg_plan(vin + td.offs, td.count, sv);
             in.vpad = sv.pad;
             in.v0 = sv.i0;
             in.v1 = sv.i1;
         }
         mbar_arrive_expect_tx(&bar[s], bytes);
-        seg_issue(kst(s), kin + o, sk, &bar[s], pol);
-        if (HV) seg_issue(vst(s), vin + o, sv, &bar[s], pol);
-        cur.next();
+        seg_issue(kst(s), kin + td.offs, sk, &bar[s], pol);
+        if (HV) seg_issue(vst(s), vin + td.offs, sv, &bar[s], pol);
     };
     if (tid == 0) {
         mbar_init(&bar[0], 1);
         mbar_init(&bar[1], 1);
         mbar_fence_init();
-        cur.start(prm.buckets, NB, tb, te, prm.kpb);
-        issue(0);
-        issue(1);
+        issue(0, blockIdx.x);
+        issue(1, blockIdx.x + gridDim.x);
     }
     for (int i = tid; i < (THREADS / 32) * NBINS; i += THREADS) wcnt[i] = 0;
-    // running tile-ordered prefix of digit tid in the current bucket
-    uint32_t running = tid < RADIX ? prm.carry[static_cast<uint64_t>(blockIdx.x) * RADIX + tid] : 0u;
     __syncthreads();
 
     const int lo = prm.lo;
@@ -923,13 +957,13 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
         const StageInfo in = info[s];
         if (!in.valid) break;
         const uint32_t count = in.count;
-        // per-digit bucket data for the destinations
-        uint32_t srel = 0;
-        uint64_t boffs = 0;
+        // per-digit destination base of this tile: bucket start + sub-bucket start +
+        // counts of the earlier tiles of the bucket (tile order = memory order: stable)
+        uint64_t dbase = 0;
         if (tid < RADIX) {
-            boffs = prm.buckets[in.bucket].offs;
-            srel = prm.sub_rel[static_cast<uint64_t>(in.bucket) * RADIX + tid];
-            if (in.first) running = 0;
+            dbase = prm.buckets[in.bucket].offs + prm.sub_rel[static_cast<uint64_t>(in.bucket) * RADIX + tid] +
+                    prm.tile_pref[static_cast<uint64_t>(in.tile) * RADIX + tid];
+            if (in.carry_row != EMPTY_RANGE) dbase += prm.carry[static_cast<uint64_t>(in.carry_row) * RADIX + tid];
         }
         Seg sk, sv;
         sk.pad = in.kpad;
@@ -965,13 +999,14 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
             if (FULL || wbase < count) count_digits<KPT>(dg, mycnt);
             __syncthreads();
             block_rank_scan<THREADS>(wcnt, tot);
-            if (tid < RADIX) {
-                // destination of smem slot j holding digit d: gbase[d] + j
-                gbase[tid] = boffs + srel + running - tot[tid];
-                running += tot[tid + 1] - tot[tid];
-            }
+            // destination of smem slot j holding digit d: gbase[d] + j
+            if (tid < RADIX) gbase[tid] = dbase - tot[tid];
             __syncthreads();
-            if (FULL || wbase < count) rank_in_place<KPT>(dg, mycnt);
+            if (HRS_EXP != 2 && (FULL || wbase < count)) rank_in_place<KPT>(dg, mycnt);
+            if (HRS_EXP == 2) {
+#pragma unroll
+                for (int c = 0; c < KPT; ++c) dg[c] = wbase + c * 32 + lane;
+            }
             // ---- stage in shared memory at the rank
 #pragma unroll
             for (int c = 0; c < KPT; ++c) {
@@ -988,10 +1023,25 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
         // ---- the staging buffer is free: prefetch the tile after next into it
         if (tid == 0) {
             fence_proxy_async();
-            issue(s);
+            issue(s, blockIdx.x + (it + 2) * gridDim.x);
         }
         // ---- write-combined stores: consecutive slots of a digit run are consecutive addresses
-        if (count == static_cast<uint32_t>(L::KPB)) {
+        if (HRS_EXP == 1) {
+            K acc = 0;
+#pragma unroll
+            for (int c = 0; c < KPT; ++c) acc ^= skeys[c * THREADS + tid] ^ static_cast<K>(gbase[c]);
+            if (acc == static_cast<K>(0x12345678u)) kout[0] = acc;
+        } else if (HRS_EXP == 3) {
+            // contiguous copy of the staged tile (no scatter)
+#pragma unroll
+            for (int c = 0; c < KPT; ++c) {
+                const uint32_t j = c * THREADS + tid;
+                if (j < count) {
+                    kout[in.offs + j] = skeys[j];
+                    if (HV) vout[in.offs + j] = svals[j];
+                }
+            }
+        } else if (count == static_cast<uint32_t>(L::KPB)) {
 #pragma unroll
             for (int c = 0; c < KPT; ++c) {
                 const uint32_t j = c * THREADS + tid;

@@ -64,8 +64,8 @@ def test_size_query_and_validation_without_gpu():
     st, size = _sz(lib.hrs_sort_ex, None, None, None, None, 1 << 20, 4, 4, 0, 32, None, None)
     assert st == 0 and size > (1 << 20) * 8  # aux buffers for the double buffering (M1)
     # M2..M5 (metadata) stay a small fraction of M1 = input + aux (the paper's 5 %
-    # is for its 16-byte tables, ours keep two look-back status arrays): < 10 % of M1
-    assert size - (1 << 20) * 8 < 0.10 * 2 * (1 << 20) * 8
+    # is for its 16-byte tables; ours add per-tile prefixes and per-CTA carries): < 15 % of M1
+    assert size - (1 << 20) * 8 < 0.15 * 2 * (1 << 20) * 8
     assert _sz(lib.hrs_sort_ex, None, None, None, None, 10, 4, 0, 0, 33, None, None)[0] == 2   # bits
     assert _sz(lib.hrs_sort_ex, None, None, None, None, 10, 4, 0, 5, 4, None, None)[0] == 2
     assert _sz(lib.hrs_sort_ex, None, None, None, None, 10, 3, 0, 0, 24, None, None)[0] == 1   # key bytes
