@@ -75,8 +75,8 @@ template <int KB, int VB>
 struct ScatterCfg {
     static constexpr bool SMALL = (KB == 4 && VB <= 4);
     static constexpr int THREADS = SMALL ? 256 : 512;
-    static constexpr int KPT = SMALL ? 16 : 8;
-    static constexpr int MINB = SMALL ? 2 : 1;
+    static constexpr int KPT = SMALL ? 15 : 8;  // 256 x 15: two staging buffers for three CTAs per SM
+    static constexpr int MINB = SMALL ? 3 : 1;
 };
 constexpr int HIST_THREADS = 512;
 constexpr int HIST_STAGES = 3;

@@ -92,6 +92,7 @@ struct Ctl {
     // together by one 64-bit atomic so bucket order == tile order
     unsigned long long alloc[HRS_MAX_PASSES + 2];
     uint32_t nlocal[HRS_NUM_CLASSES];       // entries in local list c
+    uint32_t claim[HRS_MAX_PASSES + 2];     // k_scatter tile claims of pass p
     uint32_t overflow;
     uint32_t pad_;
     unsigned long long recs_in_pass[HRS_MAX_PASSES + 2];
@@ -333,8 +334,7 @@ __device__ __forceinline__ void count_digits(const uint32_t (&dg)[KPT], uint32_t
 
 // On entry dg[c] holds the digit (INVALID_DIGIT for padding); on exit the slot.
 template <int KPT>
-__device__ __forceinline__ void rank_in_place(uint32_t (&dg)[KPT], uint32_t *mycnt) {
-    const uint32_t ltm = lanemask_lt();
+__device__ __forceinline__ void rank_in_place(uint32_t (&dg)[KPT], uint32_t *mycnt, uint32_t ltm) {
 #pragma unroll
     for (int c = 0; c < KPT; ++c) {
         const uint32_t d = dg[c];
@@ -874,15 +874,16 @@ struct ScatterSmem {
     static constexpr size_t off_wcnt = align16(off_info + 2 * sizeof(StageInfo));
     static constexpr size_t off_tot = align16(off_wcnt + sizeof(uint32_t) * W * NBINS);
     static constexpr size_t off_gbase = align16(off_tot + sizeof(uint32_t) * 288);
-    static constexpr size_t off_kst = align16(off_gbase + sizeof(unsigned long long) * RADIX);
+    static constexpr size_t off_kst = align16(off_gbase + sizeof(uint32_t) * RADIX);
     static constexpr size_t kst_bytes = align16(sizeof(K) * kst_elems);
     static constexpr size_t off_vst = off_kst + 2 * kst_bytes;
     static constexpr size_t vst_bytes = HV ? align16(sizeof(VT) * vst_elems) : 0;
-    static constexpr size_t off_skeys = off_vst + 2 * vst_bytes;
-    static constexpr size_t off_svals = align16(off_skeys + sizeof(K) * KPB);
-    static constexpr size_t bytes = off_svals + (HV ? align16(sizeof(VT) * KPB) : 0);
+    static constexpr size_t bytes = off_vst + 2 * vst_bytes;
 };
 
+// Two staging buffers: while tile i is ranked, staged back into its own buffer in
+// sorted order (keys and values pass through registers) and stored, tile i + 1 is in
+// flight into the other buffer.
 template <typename K, typename V, int THREADS, int KPT, int MINB>
 __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
     using L = ScatterSmem<K, V, THREADS, KPT>;
@@ -893,11 +894,10 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
     StageInfo *info = reinterpret_cast<StageInfo *>(smem + L::off_info);
     uint32_t *wcnt = reinterpret_cast<uint32_t *>(smem + L::off_wcnt);
     uint32_t *tot = reinterpret_cast<uint32_t *>(smem + L::off_tot);
-    unsigned long long *gbase = reinterpret_cast<unsigned long long *>(smem + L::off_gbase);
-    K *skeys = reinterpret_cast<K *>(smem + L::off_skeys);
-    VT *svals = reinterpret_cast<VT *>(smem + L::off_svals);
+    uint32_t *gbase = reinterpret_cast<uint32_t *>(smem + L::off_gbase);
     auto kst = [&](int s) { return reinterpret_cast<K *>(smem + L::off_kst + s * L::kst_bytes); };
     auto vst = [&](int s) { return reinterpret_cast<VT *>(smem + L::off_vst + s * L::vst_bytes); };
+
     const K *__restrict__ kin = static_cast<const K *>(prm.keys_in);
     K *__restrict__ kout = static_cast<K *>(prm.keys_out);
     const VT *__restrict__ vin = static_cast<const VT *>(prm.vals_in);
@@ -908,7 +908,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
     if (blockIdx.x >= T) return;
     const uint64_t pol = policy_evict_first();
 
-    // tiles blockIdx.x, blockIdx.x + gridDim.x, ...: the tiles in flight at any moment
+    // tiles are claimed in order from a counter: the tiles in flight at any moment
     // are neighbours, so the runs they write to a sub-bucket are adjacent in memory
     // and combine in L2 (contiguous runs per CTA measured +25% DRAM traffic).  The
     // tile-ordered offsets come from k_hist (tile_pref) and k_classify (carry), so the
@@ -942,29 +942,39 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
         mbar_init(&bar[0], 1);
         mbar_init(&bar[1], 1);
         mbar_fence_init();
-        issue(0, blockIdx.x);
-        issue(1, blockIdx.x + gridDim.x);
+        issue(0, atomicAdd(&prm.ctl->claim[prm.p], 1u));
+        issue(1, atomicAdd(&prm.ctl->claim[prm.p], 1u));
     }
     for (int i = tid; i < (THREADS / 32) * NBINS; i += THREADS) wcnt[i] = 0;
     __syncthreads();
 
     const int lo = prm.lo;
     const uint32_t mask = prm.mask;
+    const uint32_t ltm = lanemask_lt();
     uint32_t *mycnt = wcnt + warp * NBINS;
+    // per-digit destination base of a tile, relative to its bucket: sub-bucket start
+    // + counts of the earlier tiles of the bucket (tile order = memory order: stable).
+    // Loaded one tile ahead so the global loads overlap the previous tile.
+    auto tile_base = [&](const StageInfo &in) -> uint32_t {
+        uint32_t b = prm.sub_rel[static_cast<uint64_t>(in.bucket) * RADIX + tid] +
+                     prm.tile_pref[static_cast<uint64_t>(in.tile) * RADIX + tid];
+        if (in.carry_row != EMPTY_RANGE) b += prm.carry[static_cast<uint64_t>(in.carry_row) * RADIX + tid];
+        return b;
+    };
+    uint32_t rbase = 0;
+    uint64_t boffs = 0;
+    if (tid < RADIX && info[0].valid) {
+        rbase = tile_base(info[0]);
+        boffs = prm.buckets[info[0].bucket].offs;
+    }
     for (uint32_t it = 0;; ++it) {
         const int s = static_cast<int>(it & 1u);
         const uint32_t par = (it >> 1) & 1u;
         const StageInfo in = info[s];
         if (!in.valid) break;
         const uint32_t count = in.count;
-        // per-digit destination base of this tile: bucket start + sub-bucket start +
-        // counts of the earlier tiles of the bucket (tile order = memory order: stable)
-        uint64_t dbase = 0;
-        if (tid < RADIX) {
-            dbase = prm.buckets[in.bucket].offs + prm.sub_rel[static_cast<uint64_t>(in.bucket) * RADIX + tid] +
-                    prm.tile_pref[static_cast<uint64_t>(in.tile) * RADIX + tid];
-            if (in.carry_row != EMPTY_RANGE) dbase += prm.carry[static_cast<uint64_t>(in.carry_row) * RADIX + tid];
-        }
+        const uint32_t dbase = rbase;
+        const uint64_t tboffs = tid < RADIX ? boffs : prm.buckets[in.bucket].offs;
         Seg sk, sv;
         sk.pad = in.kpad;
         sk.i0 = in.k0;
@@ -974,9 +984,9 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
         sv.i1 = in.v1;
         const K *ksrc = kin + in.offs;
         const VT *vsrc = HV ? vin + in.offs : nullptr;
+        K *ks = kst(s);
+        VT *vs = HV ? vst(s) : nullptr;
         mbar_wait(&bar[s], par);
-        const K *ks = kst(s);
-        const VT *vs = HV ? vst(s) : nullptr;
         // full tiles with an aligned interior take the predicate-free path
         const bool full = count == static_cast<uint32_t>(L::KPB) && sk.i0 == 0 && sk.i1 == count &&
                           (!HV || (sv.i0 == 0 && sv.i1 == count));
@@ -989,7 +999,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
             for (int c = 0; c < KPT; ++c) {
                 const uint32_t e = wbase + c * 32 + lane;
                 if (FULL || e < count) {
-                    key[c] = FULL ? ks[sk.pad + e] : seg_get(ks, ksrc, sk, e);
+                    key[c] = FULL ? ks[e] : seg_get(ks, ksrc, sk, e);
                     dg[c] = digit_of(key[c], lo, mask);
                 } else {
                     dg[c] = INVALID_DIGIT;
@@ -999,37 +1009,54 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
             if (FULL || wbase < count) count_digits<KPT>(dg, mycnt);
             __syncthreads();
             block_rank_scan<THREADS>(wcnt, tot);
-            // destination of smem slot j holding digit d: gbase[d] + j
+            // destination of slot j holding digit d: bucket offset + gbase[d] + j
             if (tid < RADIX) gbase[tid] = dbase - tot[tid];
             __syncthreads();
-            if (HRS_EXP != 2 && (FULL || wbase < count)) rank_in_place<KPT>(dg, mycnt);
-            if (HRS_EXP == 2) {
+            if (FULL || wbase < count) rank_in_place<KPT>(dg, mycnt, ltm);
+            // ---- values into registers, then everything back into the staging buffer
+            //      in slot order (slot j at index j, the pad is no longer needed)
+            if (HV) {
+                VT val[KPT];
 #pragma unroll
-                for (int c = 0; c < KPT; ++c) dg[c] = wbase + c * 32 + lane;
-            }
-            // ---- stage in shared memory at the rank
+                for (int c = 0; c < KPT; ++c) {
+                    const uint32_t e = wbase + c * 32 + lane;
+                    if (FULL || e < count) val[c] = FULL ? vs[e] : seg_get(vs, vsrc, sv, e);
+                }
+                __syncthreads();
 #pragma unroll
-            for (int c = 0; c < KPT; ++c) {
-                const uint32_t e = wbase + c * 32 + lane;
-                if (FULL || e < count) {
-                    skeys[dg[c]] = key[c];
-                    if (HV) svals[dg[c]] = FULL ? vs[sv.pad + e] : seg_get(vs, vsrc, sv, e);
+                for (int c = 0; c < KPT; ++c) {
+                    const uint32_t e = wbase + c * 32 + lane;
+                    if (FULL || e < count) {
+                        ks[dg[c]] = key[c];
+                        vs[dg[c]] = val[c];
+                    }
+                }
+            } else {
+                __syncthreads();
+#pragma unroll
+                for (int c = 0; c < KPT; ++c) {
+                    const uint32_t e = wbase + c * 32 + lane;
+                    if (FULL || e < count) ks[dg[c]] = key[c];
                 }
             }
         };
         if (full) body(std::true_type{});
         else body(std::false_type{});
-        __syncthreads();
-        // ---- the staging buffer is free: prefetch the tile after next into it
-        if (tid == 0) {
-            fence_proxy_async();
-            issue(s, blockIdx.x + (it + 2) * gridDim.x);
+        {
+            // the next tile's metadata (info[s ^ 1] was published before the barriers above)
+            const StageInfo nx = info[s ^ 1];
+            if (tid < RADIX && nx.valid) {
+                rbase = tile_base(nx);
+                boffs = prm.buckets[nx.bucket].offs;
+            }
         }
+        for (int i = tid; i < (THREADS / 32) * NBINS; i += THREADS) wcnt[i] = 0;
+        __syncthreads();
         // ---- write-combined stores: consecutive slots of a digit run are consecutive addresses
         if (HRS_EXP == 1) {
             K acc = 0;
 #pragma unroll
-            for (int c = 0; c < KPT; ++c) acc ^= skeys[c * THREADS + tid] ^ static_cast<K>(gbase[c]);
+            for (int c = 0; c < KPT; ++c) acc ^= ks[c * THREADS + tid] ^ static_cast<K>(gbase[c] + tboffs);
             if (acc == static_cast<K>(0x12345678u)) kout[0] = acc;
         } else if (HRS_EXP == 3) {
             // contiguous copy of the staged tile (no scatter)
@@ -1037,33 +1064,41 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
             for (int c = 0; c < KPT; ++c) {
                 const uint32_t j = c * THREADS + tid;
                 if (j < count) {
-                    kout[in.offs + j] = skeys[j];
-                    if (HV) vout[in.offs + j] = svals[j];
+                    kout[in.offs + j] = ks[j];
+                    if (HV) vout[in.offs + j] = vs[j];
                 }
             }
-        } else if (count == static_cast<uint32_t>(L::KPB)) {
-#pragma unroll
-            for (int c = 0; c < KPT; ++c) {
-                const uint32_t j = c * THREADS + tid;
-                const K k = skeys[j];
-                const uint64_t pos = gbase[digit_of(k, lo, mask)] + j;
-                kout[pos] = k;
-                if (HV) vout[pos] = svals[j];
-            }
         } else {
+            K *const kdst = kout + tboffs;
+            VT *const vdst = HV ? vout + tboffs : nullptr;
+            if (count == static_cast<uint32_t>(L::KPB)) {
 #pragma unroll
-            for (int c = 0; c < KPT; ++c) {
-                const uint32_t j = c * THREADS + tid;
-                if (j < count) {
-                    const K k = skeys[j];
-                    const uint64_t pos = gbase[digit_of(k, lo, mask)] + j;
-                    kout[pos] = k;
-                    if (HV) vout[pos] = svals[j];
+                for (int c = 0; c < KPT; ++c) {
+                    const uint32_t j = c * THREADS + tid;
+                    const K k = ks[j];
+                    const uint32_t pos = gbase[digit_of(k, lo, mask)] + j;
+                    kdst[pos] = k;
+                    if (HV) vdst[pos] = vs[j];
+                }
+            } else {
+#pragma unroll
+                for (int c = 0; c < KPT; ++c) {
+                    const uint32_t j = c * THREADS + tid;
+                    if (j < count) {
+                        const K k = ks[j];
+                        const uint32_t pos = gbase[digit_of(k, lo, mask)] + j;
+                        kdst[pos] = k;
+                        if (HV) vdst[pos] = vs[j];
+                    }
                 }
             }
         }
-        for (int i = tid; i < (THREADS / 32) * NBINS; i += THREADS) wcnt[i] = 0;
         __syncthreads();
+        // ---- the staging buffer is free again: claim the next tile into it
+        if (tid == 0) {
+            fence_proxy_async();
+            issue(s, atomicAdd(&prm.ctl->claim[prm.p], 1u));
+        }
     }
 }
 
@@ -1138,6 +1173,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
     VT *__restrict__ vout = static_cast<VT *>(prm.vals_out);
     const uint64_t pol = policy_evict_first();
     const int begin_bit = prm.begin_bit;
+    const uint32_t ltm = lanemask_lt();
     uint32_t *mycnt = wcnt + warp * NBINS;
 
     auto srck = [&](uint32_t code) -> const K * {
@@ -1221,8 +1257,8 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
         for (int c = 0; c < KPT; ++c) {
             const uint32_t e = wbase + c * 32 + lane;
             idx[c] = e;
+            key[c] = ks[sk.pad + e];  // slots past count hold stale data and are never written out
             if (e < count) {
-                key[c] = ks[sk.pad + e];
                 a &= key[c];
                 o |= key[c];
             }
@@ -1246,40 +1282,47 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
             diff = aa ^ oo;
         }
         K *skeys = ks;  // the keys are in registers: their staging buffer sorts them
-        const bool active = wbase < count;
+        const bool active = wbase < count;  // warps past the end of the bucket idle
         bool moved = false;
         for (int lo = begin_bit; lo < hi_bit; lo += 8) {
             const int width = min(8, hi_bit - lo);
             const uint32_t mask = (1u << width) - 1u;
             if ((static_cast<uint32_t>(diff >> lo) & mask) == 0) continue;  // constant digit: identity pass
             moved = true;
-            uint32_t dg[KPT];
+            if (active) {
+                // padding slots (e >= count) carry digit 256: they rank after every record
+                // and end up in slots >= count again, so no per-element guards are needed
+                uint32_t dg[KPT];
 #pragma unroll
-            for (int c = 0; c < KPT; ++c)
-                dg[c] = (wbase + c * 32 + lane) < count ? digit_of(key[c], lo, mask) : INVALID_DIGIT;
-            if (active) count_digits<KPT>(dg, mycnt);
-            __syncthreads();
-            block_rank_scan<THREADS>(wcnt, tot);
-            __syncthreads();
-            if (active) rank_in_place<KPT>(dg, mycnt);
+                for (int c = 0; c < KPT; ++c)
+                    dg[c] = (wbase + c * 32 + lane) < count ? digit_of(key[c], lo, mask) : INVALID_DIGIT;
+                count_digits<KPT>(dg, mycnt);
+                __syncthreads();
+                block_rank_scan<THREADS>(wcnt, tot);
+                __syncthreads();
+                rank_in_place<KPT>(dg, mycnt, ltm);
 #pragma unroll
-            for (int c = 0; c < KPT; ++c) {
-                if ((wbase + c * 32 + lane) < count) {
+                for (int c = 0; c < KPT; ++c) {
                     skeys[dg[c]] = key[c];
                     sidx[dg[c]] = static_cast<uint16_t>(idx[c]);
                 }
-            }
-            __syncthreads();
+                __syncthreads();
 #pragma unroll
-            for (int c = 0; c < KPT; ++c) {
-                const uint32_t e = wbase + c * 32 + lane;
-                if (e < count) {
+                for (int c = 0; c < KPT; ++c) {
+                    const uint32_t e = wbase + c * 32 + lane;
                     key[c] = skeys[e];
                     idx[c] = sidx[e];
                 }
+                for (int i = tid; i < W * NBINS; i += THREADS) wcnt[i] = 0;
+                __syncthreads();
+            } else {
+                __syncthreads();
+                block_rank_scan<THREADS>(wcnt, tot);
+                __syncthreads();
+                __syncthreads();
+                for (int i = tid; i < W * NBINS; i += THREADS) wcnt[i] = 0;
+                __syncthreads();
             }
-            for (int i = tid; i < W * NBINS; i += THREADS) wcnt[i] = 0;
-            __syncthreads();
         }
         if (moved || src != SRC_OUT) {
 #pragma unroll
