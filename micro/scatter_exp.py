@@ -5,7 +5,9 @@ import subprocess
 import sys
 
 ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
-VARIANTS = {0: "product", 1: "no global stores", 2: "no rank (identity slots)", 3: "contiguous stores (no scatter)"}
+VARIANTS = {0: "product", 1: "no global stores", 3: "contiguous stores (no scatter)",
+            10: "local: balanced kpt", 11: "local: 2 chains/warp", 12: "local: balanced + 2 chains",
+            13: "rank: always match"}
 
 
 def build():

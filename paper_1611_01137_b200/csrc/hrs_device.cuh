@@ -312,71 +312,120 @@ __device__ __forceinline__ void seg_fill_edges(T *sbuf, const T *src, const Seg 
 
 // ------------------------------------------------------------------ stable block rank
 //
-// The KPT keys a warp holds are in "warp-striped" order: element e of the tile is
-// warp * 32 * KPT + c * 32 + lane.  A stable rank (position among all keys of the
+// The keys a warp holds are in "warp-striped" order (element e of the tile is
+// warp * 32 * kpt + c * 32 + lane).  A stable rank (position among all keys of the
 // tile, ties in element order) is computed in three steps:
-//   1. count_digits: per-warp digit histogram with non-returning shared atomics
+//   1. count: per-(virtual-)warp digit histogram with non-returning shared atomics
 //      (full speed on B200 whatever the skew; profiles/r01_micro_hist.txt);
-//   2. block_rank_scan: wcnt[w][d] = first slot of warp w's run of digit d;
-//   3. rank_in_place: column by column, every lane reads the warp's next free slot
-//      of its digit, adds 1 with a non-returning atomic and reads the counter back:
-//      the difference is the number of lanes of the column with that digit.  Lanes
-//      with duplicates take their order from one match-any over the column where
-//      all other lanes share one dummy value, so its cost depends only on the few
+//   2. scan: exclusive prefix over the warps per digit and over the digits, folded
+//      into each warp's counters = first slot of the warp's run of each digit;
+//   3. rank: column by column, every lane reads the warp's next free slot of its
+//      digit, adds 1 with a non-returning atomic and reads the counter back: the
+//      difference is the number of lanes of the column with that digit.  Lanes with
+//      duplicates take their order from one match-any over the column where all
+//      other lanes share one dummy value, so its cost depends only on the few
 //      distinct duplicated digits (match-any over 32 distinct values is what makes a
 //      pure match-based multisplit slow on B200; profiles/r01_micro_rank.txt).
 
-template <int KPT>
-__device__ __forceinline__ void count_digits(const uint32_t (&dg)[KPT], uint32_t *mycnt) {
-#pragma unroll
-    for (int c = 0; c < KPT; ++c) atomicAdd(&mycnt[dg[c]], 1u);
-}
+// Block-wide stable ranking of the keys of a tile, shared by k_scatter and k_local.
+// Each warp owns `kpt` columns (runtime, <= KPT) of 32 consecutive elements:
+// element e = warp * 32 * kpt + c * 32 + lane.  With VWPW = 2 the warp's columns are
+// split into two halves with separate counters ("virtual warps"), so the two
+// column-by-column counter chains of the rank are independent (ILP 2).  Each warp
+// clears its own counters right after its rank, so the next tile / pass needs no
+// extra barrier.
+template <int THREADS, int KPT, int VWPW>
+struct Ranker {
+    static constexpr int W = THREADS / 32;
+    static constexpr int VW = VWPW * W;
+    static constexpr int KH = VWPW == 2 ? (KPT + 1) / 2 : KPT;  // columns of the first half
+    static constexpr size_t cnt_words = static_cast<size_t>(VW) * NBINS;
+    static constexpr size_t smem_bytes = sizeof(uint32_t) * (cnt_words + 288);
+    uint32_t *cnt;  // [VW][NBINS]
+    uint32_t *tot;  // [288]
 
-// On entry dg[c] holds the digit (INVALID_DIGIT for padding); on exit the slot.
-template <int KPT>
-__device__ __forceinline__ void rank_in_place(uint32_t (&dg)[KPT], uint32_t *mycnt, uint32_t ltm) {
-#pragma unroll
-    for (int c = 0; c < KPT; ++c) {
-        const uint32_t d = dg[c];
-        const uint32_t pre = mycnt[d];
-        __syncwarp();
-        atomicAdd(&mycnt[d], 1u);
-        __syncwarp();
-        const uint32_t k = mycnt[d] - pre;
-        uint32_t r = 0;
-        if (__any_sync(0xffffffffu, k > 1)) {
-            const uint32_t m = __match_any_sync(0xffffffffu, k > 1 ? d : 0xFFFFFFFFu);
-            r = k > 1 ? __popc(m & ltm) : 0u;
-        }
-        dg[c] = pre + r;
-    }
-}
+    __device__ __forceinline__ uint32_t *vcnt(int vw) const { return cnt + vw * NBINS; }
 
-// Column scan over warps and exclusive scan over digits: afterwards wcnt[w][d] =
-// start of warp w's run of digit d in the tile, and tot[d] = start of digit d
-// (tot[256] = number of valid elements).  Ends without a trailing barrier.
-template <int THREADS>
-__device__ __forceinline__ void block_rank_scan(uint32_t *wcnt, uint32_t *tot) {
-    constexpr int W = THREADS / 32;
-    for (int d = threadIdx.x; d < NBINS; d += THREADS) {
-        uint32_t run = 0;
+    __device__ __forceinline__ void init(uint32_t *base) {
+        cnt = base;
+        tot = base + cnt_words;
+        for (int i = threadIdx.x; i < static_cast<int>(cnt_words); i += THREADS) cnt[i] = 0;
+    }
+
+    // dg: digits on entry (INVALID_DIGIT for padding), slots on exit.  kpt: active
+    // columns (the same for all warps); active: this warp holds elements.  Contains
+    // three block barriers; the caller needs one more before reading the slots' data.
+    // Afterwards tot[d] = first slot of digit d (tot[256] = valid elements).
+    __device__ __forceinline__ void rank(uint32_t (&dg)[KPT], int kpt, bool active, uint32_t ltm) {
+        const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+        uint32_t *ca = vcnt(VWPW * warp);
+        uint32_t *cb = vcnt(VWPW * warp + (VWPW - 1));
+        if (active) {
 #pragma unroll
-        for (int w = 0; w < W; ++w) {
-            const uint32_t v = wcnt[w * NBINS + d];
-            wcnt[w * NBINS + d] = run;
-            run += v;
+            for (int c = 0; c < KPT; ++c)
+                if (c < kpt) atomicAdd(&(c < KH ? ca : cb)[dg[c]], 1u);
         }
-        tot[d] = run;
-    }
-    __syncthreads();
-    warp0_exclusive_scan(tot, NBINS);
-    __syncthreads();
-    for (int d = threadIdx.x; d < NBINS; d += THREADS) {
-        const uint32_t ls = tot[d];
+        __syncthreads();
+        // exclusive prefix over the virtual warps per digit, digit totals
+        for (int d = threadIdx.x; d < NBINS; d += THREADS) {
+            uint32_t v[VW];
 #pragma unroll
-        for (int w = 0; w < W; ++w) wcnt[w * NBINS + d] += ls;
+            for (int w = 0; w < VW; ++w) v[w] = vcnt(w)[d];
+            uint32_t run = 0;
+#pragma unroll
+            for (int w = 0; w < VW; ++w) {
+                vcnt(w)[d] = run;
+                run += v[w];
+            }
+            tot[d] = run;
+        }
+        __syncthreads();
+        warp0_exclusive_scan(tot, NBINS);
+        __syncthreads();
+        // each warp folds the digit starts into its own counters
+        for (int d = lane; d < NBINS; d += 32) {
+            const uint32_t t = tot[d];
+            ca[d] += t;
+            if (VWPW == 2) cb[d] += t;
+        }
+        __syncwarp();
+        if (active) {
+#pragma unroll
+            for (int i = 0; i < KH; ++i) {
+                // column i of half A and column KH + i of half B: independent chains
+                const int c1 = KH + i < KPT ? KH + i : KPT - 1;
+                const bool v0 = i < kpt, v1 = VWPW == 2 && (KH + i < KPT) && (KH + i < kpt);
+                const uint32_t d0 = v0 ? dg[i] : 0u;
+                const uint32_t d1 = v1 ? dg[c1] : 0u;
+                const uint32_t p0 = v0 ? ca[d0] : 0u;
+                const uint32_t p1 = v1 ? cb[d1] : 0u;
+                __syncwarp();
+                if (v0) atomicAdd(&ca[d0], 1u);
+                if (v1) atomicAdd(&cb[d1], 1u);
+                __syncwarp();
+                const uint32_t k0 = v0 ? ca[d0] - p0 : 0u;
+                const uint32_t k1 = v1 ? cb[d1] - p1 : 0u;
+                uint32_t r0 = 0, r1 = 0;
+                {
+                    const uint32_t m = __match_any_sync(0xffffffffu, k0 > 1 ? d0 : 0xFFFFFFFFu);
+                    r0 = k0 > 1 ? __popc(m & ltm) : 0u;
+                }
+                if (VWPW == 2) {
+                    const uint32_t m = __match_any_sync(0xffffffffu, k1 > 1 ? d1 : 0xFFFFFFFFu);
+                    r1 = k1 > 1 ? __popc(m & ltm) : 0u;
+                }
+                if (v0) dg[i] = p0 + r0;
+                if (v1) dg[c1] = p1 + r1;
+            }
+        }
+        __syncwarp();
+        // clear this warp's counters for the next tile / pass
+        for (int d = lane; d < NBINS; d += 32) {
+            ca[d] = 0;
+            if (VWPW == 2) cb[d] = 0;
+        }
     }
-}
+};
 
 // ------------------------------------------------------------------ init / copy
 
@@ -805,19 +854,38 @@ __device__ void classify_bucket(const ClassifyParams &prm, const Bucket &bk, uin
 }
 
 // Carry of every hist/scatter CTA: the digit counts of the tiles of its first bucket
-// that precede its range (an exclusive scan over CTAs, segmented by bucket).
+// that precede its range (an exclusive scan over CTAs, segmented by bucket).  One
+// thread per digit walks the CTAs; the loads are batched so their latencies overlap.
 template <int THREADS>
 __device__ void range_carries(const ClassifyParams &prm) {
+    constexpr int B = 32;
+    const RangeMeta *__restrict__ meta = prm.seg_meta;
+    const uint32_t *__restrict__ segl = prm.seg_last;
+    uint32_t *__restrict__ carry = prm.carry;
     for (int d = threadIdx.x; d < RADIX; d += THREADS) {
         uint32_t run = 0, prev_last = EMPTY_RANGE;
-        for (uint32_t c = 0; c < prm.ranges; ++c) {
-            const RangeMeta m = prm.seg_meta[c];
-            if (m.first_bucket == EMPTY_RANGE) continue;
-            const uint32_t car = m.first_bucket == prev_last ? run : 0u;
-            prm.carry[static_cast<uint64_t>(c) * RADIX + d] = car;
-            const uint32_t sl = prm.seg_last[static_cast<uint64_t>(c) * RADIX + d];
-            run = (m.first_bucket == m.last_bucket) ? car + sl : sl;
-            prev_last = m.last_bucket;
+        for (uint32_t c0 = 0; c0 < prm.ranges; c0 += B) {
+            RangeMeta m[B];
+            uint32_t sl[B];
+#pragma unroll
+            for (int i = 0; i < B; ++i) {
+                if (c0 + i < prm.ranges) {
+                    m[i] = meta[c0 + i];
+                    sl[i] = segl[static_cast<uint64_t>(c0 + i) * RADIX + d];
+                } else {
+                    m[i].first_bucket = EMPTY_RANGE;
+                    m[i].last_bucket = EMPTY_RANGE;
+                    sl[i] = 0;
+                }
+            }
+#pragma unroll
+            for (int i = 0; i < B; ++i) {
+                if (m[i].first_bucket == EMPTY_RANGE) continue;
+                const uint32_t car = m[i].first_bucket == prev_last ? run : 0u;
+                carry[static_cast<uint64_t>(c0 + i) * RADIX + d] = car;
+                run = (m[i].first_bucket == m[i].last_bucket) ? car + sl[i] : sl[i];
+                prev_last = m[i].last_bucket;
+            }
         }
     }
 }
@@ -825,11 +893,12 @@ __device__ void range_carries(const ClassifyParams &prm) {
 template <int THREADS>
 __global__ void __launch_bounds__(THREADS) k_classify(ClassifyParams prm) {
     __shared__ uint32_t scratch[7 * NBINS];
+    const uint32_t nb = alloc_buckets(prm.ctl->alloc[prm.p]);
+    if (nb == 0) return;  // nothing reached this pass
     if (blockIdx.x == gridDim.x - 1) {
         range_carries<THREADS>(prm);
         if (gridDim.x > 1) return;
     }
-    const uint32_t nb = alloc_buckets(prm.ctl->alloc[prm.p]);
     const uint32_t nblk = gridDim.x > 1 ? gridDim.x - 1 : 1;
     for (uint32_t b = blockIdx.x; b < nb; b += nblk) {
         const Bucket bk = prm.buckets[b];
@@ -871,9 +940,9 @@ struct ScatterSmem {
     static constexpr size_t vst_elems = KPB + 16 / sizeof(VT);
     static constexpr size_t off_bar = 0;
     static constexpr size_t off_info = 16;
-    static constexpr size_t off_wcnt = align16(off_info + 2 * sizeof(StageInfo));
-    static constexpr size_t off_tot = align16(off_wcnt + sizeof(uint32_t) * W * NBINS);
-    static constexpr size_t off_gbase = align16(off_tot + sizeof(uint32_t) * 288);
+    using RK = Ranker<THREADS, KPT, 1>;
+    static constexpr size_t off_rank = align16(off_info + 2 * sizeof(StageInfo));
+    static constexpr size_t off_gbase = align16(off_rank + RK::smem_bytes);
     static constexpr size_t off_kst = align16(off_gbase + sizeof(uint32_t) * RADIX);
     static constexpr size_t kst_bytes = align16(sizeof(K) * kst_elems);
     static constexpr size_t off_vst = off_kst + 2 * kst_bytes;
@@ -892,8 +961,8 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
     extern __shared__ __align__(16) unsigned char smem[];
     uint64_t *bar = reinterpret_cast<uint64_t *>(smem + L::off_bar);
     StageInfo *info = reinterpret_cast<StageInfo *>(smem + L::off_info);
-    uint32_t *wcnt = reinterpret_cast<uint32_t *>(smem + L::off_wcnt);
-    uint32_t *tot = reinterpret_cast<uint32_t *>(smem + L::off_tot);
+    typename L::RK ranker;
+    ranker.init(reinterpret_cast<uint32_t *>(smem + L::off_rank));
     uint32_t *gbase = reinterpret_cast<uint32_t *>(smem + L::off_gbase);
     auto kst = [&](int s) { return reinterpret_cast<K *>(smem + L::off_kst + s * L::kst_bytes); };
     auto vst = [&](int s) { return reinterpret_cast<VT *>(smem + L::off_vst + s * L::vst_bytes); };
@@ -945,13 +1014,11 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
         issue(0, atomicAdd(&prm.ctl->claim[prm.p], 1u));
         issue(1, atomicAdd(&prm.ctl->claim[prm.p], 1u));
     }
-    for (int i = tid; i < (THREADS / 32) * NBINS; i += THREADS) wcnt[i] = 0;
     __syncthreads();
 
     const int lo = prm.lo;
     const uint32_t mask = prm.mask;
     const uint32_t ltm = lanemask_lt();
-    uint32_t *mycnt = wcnt + warp * NBINS;
     // per-digit destination base of a tile, relative to its bucket: sub-bucket start
     // + counts of the earlier tiles of the bucket (tile order = memory order: stable).
     // Loaded one tile ahead so the global loads overlap the previous tile.
@@ -1006,13 +1073,9 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
                 }
             }
             // ---- stable rank
-            if (FULL || wbase < count) count_digits<KPT>(dg, mycnt);
-            __syncthreads();
-            block_rank_scan<THREADS>(wcnt, tot);
+            ranker.rank(dg, KPT, FULL || wbase < count, ltm);
             // destination of slot j holding digit d: bucket offset + gbase[d] + j
-            if (tid < RADIX) gbase[tid] = dbase - tot[tid];
-            __syncthreads();
-            if (FULL || wbase < count) rank_in_place<KPT>(dg, mycnt, ltm);
+            if (tid < RADIX) gbase[tid] = dbase - ranker.tot[tid];
             // ---- values into registers, then everything back into the staging buffer
             //      in slot order (slot j at index j, the pad is no longer needed)
             if (HV) {
@@ -1050,7 +1113,6 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
                 boffs = prm.buckets[nx.bucket].offs;
             }
         }
-        for (int i = tid; i < (THREADS / 32) * NBINS; i += THREADS) wcnt[i] = 0;
         __syncthreads();
         // ---- write-combined stores: consecutive slots of a digit run are consecutive addresses
         if (HRS_EXP == 1) {
@@ -1126,9 +1188,10 @@ struct LocalSmem {
     static constexpr bool HV = HasVal<V>::value;
     static constexpr size_t off_bar = 0;
     static constexpr size_t off_info = align16(sizeof(uint64_t) * NSTAGE);
-    static constexpr size_t off_wcnt = align16(off_info + sizeof(uint32_t) * 16 * NSTAGE);
-    static constexpr size_t off_tot = align16(off_wcnt + sizeof(uint32_t) * W * NBINS);
-    static constexpr size_t off_red = align16(off_tot + sizeof(uint32_t) * 288);
+    static constexpr int VWPW = (HRS_EXP == 11 || HRS_EXP == 12) ? 2 : 1;
+    using RK = Ranker<THREADS, KPT, VWPW>;
+    static constexpr size_t off_rank = align16(off_info + sizeof(uint32_t) * 16 * NSTAGE);
+    static constexpr size_t off_red = align16(off_rank + RK::smem_bytes);
     static constexpr size_t off_sidx = align16(off_red + sizeof(K) * 2 * W);
     static constexpr size_t off_kst = align16(off_sidx + sizeof(uint16_t) * CAP);
     static constexpr size_t kst_bytes = align16(sizeof(K) * (CAP + 16 / sizeof(K)));
@@ -1137,17 +1200,17 @@ struct LocalSmem {
     static constexpr size_t bytes = off_vst + NSTAGE * vst_bytes;
 };
 
-template <typename K>
-__device__ __forceinline__ K warp_and(K x) {
-#pragma unroll
-    for (int o = 16; o > 0; o >>= 1) x &= __shfl_xor_sync(0xffffffffu, x, o);
-    return x;
+__device__ __forceinline__ uint32_t warp_and(uint32_t x) { return __reduce_and_sync(0xffffffffu, x); }
+__device__ __forceinline__ uint32_t warp_or(uint32_t x) { return __reduce_or_sync(0xffffffffu, x); }
+__device__ __forceinline__ unsigned long long warp_and(unsigned long long x) {
+    const uint32_t lo = __reduce_and_sync(0xffffffffu, static_cast<uint32_t>(x));
+    const uint32_t hi = __reduce_and_sync(0xffffffffu, static_cast<uint32_t>(x >> 32));
+    return (static_cast<unsigned long long>(hi) << 32) | lo;
 }
-template <typename K>
-__device__ __forceinline__ K warp_or(K x) {
-#pragma unroll
-    for (int o = 16; o > 0; o >>= 1) x |= __shfl_xor_sync(0xffffffffu, x, o);
-    return x;
+__device__ __forceinline__ unsigned long long warp_or(unsigned long long x) {
+    const uint32_t lo = __reduce_or_sync(0xffffffffu, static_cast<uint32_t>(x));
+    const uint32_t hi = __reduce_or_sync(0xffffffffu, static_cast<uint32_t>(x >> 32));
+    return (static_cast<unsigned long long>(hi) << 32) | lo;
 }
 
 template <typename K, typename V, int THREADS, int KPT, int NSTAGE, int MINB>
@@ -1159,14 +1222,13 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
     extern __shared__ __align__(16) unsigned char smem[];
     uint64_t *bar = reinterpret_cast<uint64_t *>(smem + L::off_bar);
     uint32_t *info = reinterpret_cast<uint32_t *>(smem + L::off_info);  // [s][16]
-    uint32_t *wcnt = reinterpret_cast<uint32_t *>(smem + L::off_wcnt);
-    uint32_t *tot = reinterpret_cast<uint32_t *>(smem + L::off_tot);
+    typename L::RK ranker;
+    ranker.init(reinterpret_cast<uint32_t *>(smem + L::off_rank));
     K *red = reinterpret_cast<K *>(smem + L::off_red);
     uint16_t *sidx = reinterpret_cast<uint16_t *>(smem + L::off_sidx);
     auto kst = [&](int s) { return reinterpret_cast<K *>(smem + L::off_kst + s * L::kst_bytes); };
     auto vst = [&](int s) { return reinterpret_cast<VT *>(smem + L::off_vst + s * L::vst_bytes); };
     const int tid = threadIdx.x, lane = tid & 31, warp = tid >> 5;
-    const uint32_t wbase = static_cast<uint32_t>(warp) * 32 * KPT;
     const uint32_t nent = *prm.count;
     if (blockIdx.x >= nent) return;
     K *__restrict__ kout = static_cast<K *>(prm.keys_out);
@@ -1174,7 +1236,6 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
     const uint64_t pol = policy_evict_first();
     const int begin_bit = prm.begin_bit;
     const uint32_t ltm = lanemask_lt();
-    uint32_t *mycnt = wcnt + warp * NBINS;
 
     auto srck = [&](uint32_t code) -> const K * {
         return static_cast<const K *>(code == SRC_IN    ? prm.src_keys[SRC_IN]
@@ -1220,7 +1281,6 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
         mbar_fence_init();
         for (int s = 0; s < NSTAGE; ++s) issue(s, blockIdx.x + s * gridDim.x);
     }
-    for (int i = tid; i < W * NBINS; i += THREADS) wcnt[i] = 0;
     __syncthreads();
 
     for (uint32_t it = 0;; ++it) {
@@ -1250,6 +1310,12 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
         seg_fill_edges<K, THREADS>(ks, ksrc, sk, count);
         if (HV) seg_fill_edges<VT, THREADS>(vs, vsrc, sv, count);
         __syncthreads();
+        // BAL: every warp takes kpt = ceil(count / THREADS) columns, so the work is spread
+        // over all warps whatever the bucket size (element e = warp*32*kpt + c*32 + lane);
+        // otherwise kpt = KPT and warps past the end of the bucket idle
+        constexpr bool BAL = HRS_EXP == 10 || HRS_EXP == 12;
+        const int kpt = BAL ? static_cast<int>(min((count + THREADS - 1) / THREADS, static_cast<uint32_t>(KPT))) : KPT;
+        const uint32_t wbase = static_cast<uint32_t>(warp) * 32u * kpt;
         K key[KPT];
         uint32_t idx[KPT];
         K a = ~K(0), o = K(0);
@@ -1257,11 +1323,10 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
         for (int c = 0; c < KPT; ++c) {
             const uint32_t e = wbase + c * 32 + lane;
             idx[c] = e;
-            key[c] = ks[sk.pad + e];  // slots past count hold stale data and are never written out
-            if (e < count) {
-                a &= key[c];
-                o |= key[c];
-            }
+            key[c] = (!BAL || c < kpt) ? ks[sk.pad + e] : K(0);  // slots past count: stale, never written out
+            const bool v = (!BAL || c < kpt) && e < count;
+            a &= v ? key[c] : ~K(0);
+            o |= v ? key[c] : K(0);
         }
         // bits that vary across the bucket: digits where they are all equal are skipped
         a = warp_and(a);
@@ -1282,55 +1347,51 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
             diff = aa ^ oo;
         }
         K *skeys = ks;  // the keys are in registers: their staging buffer sorts them
-        const bool active = wbase < count;  // warps past the end of the bucket idle
+        const bool active = wbase < count;
         bool moved = false;
         for (int lo = begin_bit; lo < hi_bit; lo += 8) {
             const int width = min(8, hi_bit - lo);
             const uint32_t mask = (1u << width) - 1u;
             if ((static_cast<uint32_t>(diff >> lo) & mask) == 0) continue;  // constant digit: identity pass
             moved = true;
+            // padding slots (e >= count) carry digit 256: they rank after every record
+            // and end up in slots >= count again, so no per-element guards are needed
+            uint32_t dg[KPT];
+#pragma unroll
+            for (int c = 0; c < KPT; ++c)
+                dg[c] = (wbase + c * 32 + lane) < count ? digit_of(key[c], lo, mask) : INVALID_DIGIT;
+            ranker.rank(dg, kpt, active, ltm);
             if (active) {
-                // padding slots (e >= count) carry digit 256: they rank after every record
-                // and end up in slots >= count again, so no per-element guards are needed
-                uint32_t dg[KPT];
-#pragma unroll
-                for (int c = 0; c < KPT; ++c)
-                    dg[c] = (wbase + c * 32 + lane) < count ? digit_of(key[c], lo, mask) : INVALID_DIGIT;
-                count_digits<KPT>(dg, mycnt);
-                __syncthreads();
-                block_rank_scan<THREADS>(wcnt, tot);
-                __syncthreads();
-                rank_in_place<KPT>(dg, mycnt, ltm);
 #pragma unroll
                 for (int c = 0; c < KPT; ++c) {
-                    skeys[dg[c]] = key[c];
-                    sidx[dg[c]] = static_cast<uint16_t>(idx[c]);
+                    if (!BAL || c < kpt) {
+                        skeys[dg[c]] = key[c];
+                        sidx[dg[c]] = static_cast<uint16_t>(idx[c]);
+                    }
                 }
-                __syncthreads();
+            }
+            __syncthreads();
+            if (active) {
 #pragma unroll
                 for (int c = 0; c < KPT; ++c) {
-                    const uint32_t e = wbase + c * 32 + lane;
-                    key[c] = skeys[e];
-                    idx[c] = sidx[e];
+                    if (!BAL || c < kpt) {
+                        const uint32_t e = wbase + c * 32 + lane;
+                        key[c] = skeys[e];
+                        idx[c] = sidx[e];
+                    }
                 }
-                for (int i = tid; i < W * NBINS; i += THREADS) wcnt[i] = 0;
-                __syncthreads();
-            } else {
-                __syncthreads();
-                block_rank_scan<THREADS>(wcnt, tot);
-                __syncthreads();
-                __syncthreads();
-                for (int i = tid; i < W * NBINS; i += THREADS) wcnt[i] = 0;
-                __syncthreads();
             }
         }
         if (moved || src != SRC_OUT) {
+            K *const kd = kout + offs;
+            VT *const vd = HV ? vout + offs : nullptr;
+            const VT *const vsp = HV ? vs + sv.pad : nullptr;
 #pragma unroll
             for (int c = 0; c < KPT; ++c) {
                 const uint32_t e = wbase + c * 32 + lane;
-                if (e < count) {
-                    kout[offs + e] = key[c];
-                    if (HV) vout[offs + e] = vs[sv.pad + idx[c]];
+                if ((!BAL || c < kpt) && e < count) {
+                    kd[e] = key[c];
+                    if (HV) vd[e] = vsp[idx[c]];
                 }
             }
         }
