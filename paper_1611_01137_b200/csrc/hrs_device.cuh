@@ -1192,8 +1192,10 @@ struct LocalSmem {
     using RK = Ranker<THREADS, KPT, VWPW>;
     static constexpr size_t off_rank = align16(off_info + sizeof(uint32_t) * 16 * NSTAGE);
     static constexpr size_t off_red = align16(off_rank + RK::smem_bytes);
+    // composite buffer: CAP x K words ((sort bits << 13) | index); the wide path uses
+    // its first CAP x 2 bytes as the 16-bit index buffer
     static constexpr size_t off_sidx = align16(off_red + sizeof(K) * 2 * W);
-    static constexpr size_t off_kst = align16(off_sidx + sizeof(uint16_t) * CAP);
+    static constexpr size_t off_kst = align16(off_sidx + sizeof(K) * CAP);
     static constexpr size_t kst_bytes = align16(sizeof(K) * (CAP + 16 / sizeof(K)));
     static constexpr size_t off_vst = off_kst + NSTAGE * kst_bytes;
     static constexpr size_t vst_bytes = HV ? align16(sizeof(VT) * (CAP + 16 / sizeof(VT))) : 0;
@@ -1346,52 +1348,107 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
             }
             diff = aa ^ oo;
         }
-        K *skeys = ks;  // the keys are in registers: their staging buffer sorts them
         const bool active = wbase < count;
         bool moved = false;
-        for (int lo = begin_bit; lo < hi_bit; lo += 8) {
-            const int width = min(8, hi_bit - lo);
-            const uint32_t mask = (1u << width) - 1u;
-            if ((static_cast<uint32_t>(diff >> lo) & mask) == 0) continue;  // constant digit: identity pass
-            moved = true;
-            // padding slots (e >= count) carry digit 256: they rank after every record
-            // and end up in slots >= count again, so no per-element guards are needed
-            uint32_t dg[KPT];
+        constexpr int IB = 13;  // index bits: CAP <= 8192
+        static_assert(L::CAP <= (1 << IB), "local-sort capacity exceeds the composite index");
+        const int sb = hi_bit - begin_bit;
+        if (sb + IB <= static_cast<int>(8 * sizeof(K))) {
+            // ---- narrow path: one word per record, composite = (sort bits << IB) | index.
+            // The LSD passes move composites only; keys and values are gathered from the
+            // staging buffers through the index at the end (the key bits outside the
+            // sorted range are carried that way too).
+            K *comp = reinterpret_cast<K *>(sidx);
+            const K smask = sb >= static_cast<int>(8 * sizeof(K)) ? ~K(0) : ((K(1) << sb) - 1);
+            K cv[KPT];
 #pragma unroll
-            for (int c = 0; c < KPT; ++c)
-                dg[c] = (wbase + c * 32 + lane) < count ? digit_of(key[c], lo, mask) : INVALID_DIGIT;
-            ranker.rank(dg, kpt, active, ltm);
-            if (active) {
+            for (int c = 0; c < KPT; ++c) cv[c] = (((key[c] >> begin_bit) & smask) << IB) | static_cast<K>(idx[c]);
+            const K cdiff = ((diff >> begin_bit) & smask) << IB;
+            for (int lo = IB; lo < IB + sb; lo += 8) {
+                const int width = min(8, IB + sb - lo);
+                const uint32_t mask = (1u << width) - 1u;
+                if ((static_cast<uint32_t>(cdiff >> lo) & mask) == 0) continue;  // constant digit: identity pass
+                moved = true;
+                // padding slots (e >= count) carry digit 256: they rank after every record
+                // and end up in slots >= count again, so no per-element guards are needed
+                uint32_t dg[KPT];
+#pragma unroll
+                for (int c = 0; c < KPT; ++c)
+                    dg[c] = (wbase + c * 32 + lane) < count ? digit_of(cv[c], lo, mask) : INVALID_DIGIT;
+                ranker.rank(dg, kpt, active, ltm);
+                if (active) {
+#pragma unroll
+                    for (int c = 0; c < KPT; ++c)
+                        if (!BAL || c < kpt) comp[dg[c]] = cv[c];
+                }
+                __syncthreads();
+                if (active) {
+#pragma unroll
+                    for (int c = 0; c < KPT; ++c)
+                        if (!BAL || c < kpt) cv[c] = comp[wbase + c * 32 + lane];
+                }
+            }
+            if (moved || src != SRC_OUT) {
+                K *const kd = kout + offs;
+                VT *const vd = HV ? vout + offs : nullptr;
+                const K *const ksp = ks + sk.pad;
+                const VT *const vsp = HV ? vs + sv.pad : nullptr;
 #pragma unroll
                 for (int c = 0; c < KPT; ++c) {
-                    if (!BAL || c < kpt) {
-                        skeys[dg[c]] = key[c];
-                        sidx[dg[c]] = static_cast<uint16_t>(idx[c]);
+                    const uint32_t e = wbase + c * 32 + lane;
+                    if ((!BAL || c < kpt) && e < count) {
+                        const uint32_t ix = static_cast<uint32_t>(cv[c]) & ((1u << IB) - 1u);
+                        kd[e] = ksp[ix];
+                        if (HV) vd[e] = vsp[ix];
                     }
                 }
             }
-            __syncthreads();
-            if (active) {
+        } else {
+            // ---- wide path (more than 8*sizeof(K) - 13 bits to sort): (key, index) pairs,
+            // the key staging buffer doubles as the sort buffer
+            K *skeys = ks;
+            for (int lo = begin_bit; lo < hi_bit; lo += 8) {
+                const int width = min(8, hi_bit - lo);
+                const uint32_t mask = (1u << width) - 1u;
+                if ((static_cast<uint32_t>(diff >> lo) & mask) == 0) continue;  // constant digit: identity pass
+                moved = true;
+                uint32_t dg[KPT];
 #pragma unroll
-                for (int c = 0; c < KPT; ++c) {
-                    if (!BAL || c < kpt) {
-                        const uint32_t e = wbase + c * 32 + lane;
-                        key[c] = skeys[e];
-                        idx[c] = sidx[e];
+                for (int c = 0; c < KPT; ++c)
+                    dg[c] = (wbase + c * 32 + lane) < count ? digit_of(key[c], lo, mask) : INVALID_DIGIT;
+                ranker.rank(dg, kpt, active, ltm);
+                if (active) {
+#pragma unroll
+                    for (int c = 0; c < KPT; ++c) {
+                        if (!BAL || c < kpt) {
+                            skeys[dg[c]] = key[c];
+                            sidx[dg[c]] = static_cast<uint16_t>(idx[c]);
+                        }
+                    }
+                }
+                __syncthreads();
+                if (active) {
+#pragma unroll
+                    for (int c = 0; c < KPT; ++c) {
+                        if (!BAL || c < kpt) {
+                            const uint32_t e = wbase + c * 32 + lane;
+                            key[c] = skeys[e];
+                            idx[c] = sidx[e];
+                        }
                     }
                 }
             }
-        }
-        if (moved || src != SRC_OUT) {
-            K *const kd = kout + offs;
-            VT *const vd = HV ? vout + offs : nullptr;
-            const VT *const vsp = HV ? vs + sv.pad : nullptr;
+            if (moved || src != SRC_OUT) {
+                K *const kd = kout + offs;
+                VT *const vd = HV ? vout + offs : nullptr;
+                const VT *const vsp = HV ? vs + sv.pad : nullptr;
 #pragma unroll
-            for (int c = 0; c < KPT; ++c) {
-                const uint32_t e = wbase + c * 32 + lane;
-                if ((!BAL || c < kpt) && e < count) {
-                    kd[e] = key[c];
-                    if (HV) vd[e] = vsp[idx[c]];
+                for (int c = 0; c < KPT; ++c) {
+                    const uint32_t e = wbase + c * 32 + lane;
+                    if ((!BAL || c < kpt) && e < count) {
+                        kd[e] = key[c];
+                        if (HV) vd[e] = vsp[idx[c]];
+                    }
                 }
             }
         }
