@@ -97,12 +97,19 @@ template <> struct LocalCfg<6> { static constexpr int THREADS = 384, KPT = 16; }
 template <> struct LocalCfg<7> { static constexpr int THREADS = 512, KPT = 16; };
 
 // two-stage TMA prefetch where it fits next to a second resident CTA, else one stage
-template <typename K, typename V, int C>
+// two-stage TMA prefetch when three CTAs still fit per SM, else one stage; the
+// register cap (launch bounds) is set for the occupancy the shared memory allows
+template <typename K, typename V, int C, int WIDE = 0>
 struct LocalStages {
     using LC = LocalCfg<C>;
-    static constexpr int NSTAGE = LocalSmem<K, V, LC::THREADS, LC::KPT, 2>::bytes <= 110 * 1024 ? 2 : 1;
-    static constexpr size_t bytes = LocalSmem<K, V, LC::THREADS, LC::KPT, NSTAGE>::bytes;
-    static constexpr bool fits = bytes <= SMEM_LIMIT;
+    static constexpr size_t SM_BUDGET = 224 * 1024;
+    static constexpr int NSTAGE = 3 * LocalSmem<K, V, LC::THREADS, LC::KPT, 2, WIDE>::bytes <= SM_BUDGET ? 2 : 1;
+    static constexpr size_t bytes = LocalSmem<K, V, LC::THREADS, LC::KPT, NSTAGE, WIDE>::bytes;
+    static constexpr bool fits = bytes <= SMEM_LIMIT && LocalSmem<K, V, LC::THREADS, LC::KPT, 1, 1>::bytes <= SMEM_LIMIT;
+    static constexpr int by_smem = static_cast<int>(SM_BUDGET / (bytes + 1024));
+    static constexpr int by_threads = 2048 / LC::THREADS;
+    static constexpr int OCC0 = by_smem < by_threads ? by_smem : by_threads;
+    static constexpr int OCC = OCC0 < 1 ? 1 : (OCC0 > 4 ? 4 : OCC0);
 };
 
 template <typename K, typename V>
@@ -464,10 +471,10 @@ struct Runner {
         return last_launch();
     }
 
-    template <int C>
-    static hrs_status local_one(const Plan &pl, void *temp, cudaStream_t st, int dev, int sms, const void *kin,
-                                void *kout, const void *vin, void *vout) {
-        using LST = LocalStages<K, V, C>;
+    template <int C, int WIDE>
+    static hrs_status local_variant(const Plan &pl, void *temp, cudaStream_t st, int dev, int sms, const void *kin,
+                                    void *kout, const void *vin, void *vout) {
+        using LST = LocalStages<K, V, C, WIDE>;
         if constexpr (!LST::fits) {
             return HRS_ERROR_INVALID_VALUE;
         } else {
@@ -484,7 +491,7 @@ struct Runner {
             lp.list = at<LocalEntry>(temp, pl.off_local[C]);
             lp.count = &at<Ctl>(temp, 0)->nlocal[C];
             lp.begin_bit = pl.begin;
-            auto fn = k_local<K, V, LC::THREADS, LC::KPT, LST::NSTAGE, (LC::THREADS >= 256 ? 2 : 1)>;
+            auto fn = k_local<K, V, LC::THREADS, LC::KPT, LST::NSTAGE, LST::OCC, WIDE>;
             int grid = 0;
             hrs_status s = grid_for(fn, LC::THREADS, LST::bytes, dev, sms, &grid);
             if (s) return s;
@@ -493,6 +500,19 @@ struct Runner {
             fn<<<grid, LC::THREADS, LST::bytes, st>>>(lp);
             return last_launch();
         }
+    }
+
+    // the entries of one size class: most take the narrow variant; the wide one only
+    // runs when some entry sorts more bits than a key-width composite holds
+    template <int C>
+    static hrs_status local_one(const Plan &pl, void *temp, cudaStream_t st, int dev, int sms, const void *kin,
+                                void *kout, const void *vin, void *vout) {
+        hrs_status s = local_variant<C, 0>(pl, temp, st, dev, sms, kin, kout, vin, vout);
+        if (s) return s;
+        // a key-width composite holds (end - begin) + 13 bits: otherwise some entries
+        // (those partitioned on few digits) need the wide variant
+        if (pl.end - pl.begin + 13 > 8 * KB) s = local_variant<C, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout);
+        return s;
     }
 
     static hrs_status local(const Plan &pl, void *temp, cudaStream_t st, int dev, int sms, int c, const void *kin,

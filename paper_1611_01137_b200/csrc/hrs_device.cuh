@@ -1180,7 +1180,17 @@ struct LocalParams {
 // the keys have been read into registers the key buffer doubles as the buffer of
 // the LSD passes, which move (key, 16-bit index) pairs; the values are gathered from
 // their staging buffer once, at the end.
-template <typename K, typename V, int THREADS, int KPT, int NSTAGE>
+// Composite word of the local sort: the narrow variant ranks (sort bits << 13 | index)
+// in a word of the key's width; the wide variant in 64 bits for 32-bit keys and as
+// (key, 16-bit index) pairs for 64-bit keys (more than 51 bits to sort).
+template <typename K, int WIDE>
+struct LocalWord {
+    using CT = typename std::conditional<(WIDE && sizeof(K) == 4), unsigned long long, K>::type;
+    static constexpr bool PAIRS = WIDE && sizeof(K) == 8;
+    static constexpr size_t buf_bytes = PAIRS ? sizeof(uint16_t) : sizeof(CT);
+};
+
+template <typename K, typename V, int THREADS, int KPT, int NSTAGE, int WIDE = 0>
 struct LocalSmem {
     static constexpr int W = THREADS / 32;
     static constexpr int CAP = THREADS * KPT;
@@ -1190,12 +1200,11 @@ struct LocalSmem {
     static constexpr size_t off_info = align16(sizeof(uint64_t) * NSTAGE);
     static constexpr int VWPW = (HRS_EXP == 11 || HRS_EXP == 12) ? 2 : 1;
     using RK = Ranker<THREADS, KPT, VWPW>;
-    static constexpr size_t off_rank = align16(off_info + sizeof(uint32_t) * 16 * NSTAGE);
+    static constexpr size_t off_rank = align16(off_info + sizeof(uint32_t) * 16 * (NSTAGE + 1));
     static constexpr size_t off_red = align16(off_rank + RK::smem_bytes);
-    // composite buffer: CAP x K words ((sort bits << 13) | index); the wide path uses
-    // its first CAP x 2 bytes as the 16-bit index buffer
+    // composite buffer (or the 16-bit index buffer of the pair path)
     static constexpr size_t off_sidx = align16(off_red + sizeof(K) * 2 * W);
-    static constexpr size_t off_kst = align16(off_sidx + sizeof(K) * CAP);
+    static constexpr size_t off_kst = align16(off_sidx + LocalWord<K, WIDE>::buf_bytes * CAP);
     static constexpr size_t kst_bytes = align16(sizeof(K) * (CAP + 16 / sizeof(K)));
     static constexpr size_t off_vst = off_kst + NSTAGE * kst_bytes;
     static constexpr size_t vst_bytes = HV ? align16(sizeof(VT) * (CAP + 16 / sizeof(VT))) : 0;
@@ -1215,9 +1224,13 @@ __device__ __forceinline__ unsigned long long warp_or(unsigned long long x) {
     return (static_cast<unsigned long long>(hi) << 32) | lo;
 }
 
-template <typename K, typename V, int THREADS, int KPT, int NSTAGE, int MINB>
+template <typename K, typename V, int THREADS, int KPT, int NSTAGE, int MINB, int WIDE>
 __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
-    using L = LocalSmem<K, V, THREADS, KPT, NSTAGE>;
+    using L = LocalSmem<K, V, THREADS, KPT, NSTAGE, WIDE>;
+    using LW = LocalWord<K, WIDE>;
+    using CT = typename LW::CT;
+    constexpr int IB = 13;  // index bits: CAP <= 8192
+    static_assert(L::CAP <= (1 << IB), "local-sort capacity exceeds the composite index");
     constexpr int W = THREADS / 32;
     constexpr bool HV = HasVal<V>::value;
     using VT = ValT<V>;
@@ -1249,12 +1262,23 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
                                        : code == SRC_AUX ? prm.src_vals[SRC_AUX]
                                                          : prm.src_vals[SRC_OUT]);
     };
-    // info[s]: 0 entry, 1 count, 2 hi_bit, 3 src, 4..5 offs, 6..8 key seg, 9..11 value seg
+    // an entry belongs to the narrow variant iff its sort bits and the index fit in one
+    // key-width word
+    auto mine = [&](const LocalEntry &en) {
+        const bool narrow = static_cast<int>(en.hi_bit) - prm.begin_bit + IB <= static_cast<int>(8 * sizeof(K));
+        return narrow == (WIDE == 0);
+    };
+    // info[s]: 0 entry, 1 count, 2 hi_bit, 3 src, 4..5 offs, 6..8 key seg, 9..11 value seg, 12 next stride
     auto issue = [&](int s, uint32_t e) {
         uint32_t *in = info + 16 * s;
+        LocalEntry en;
+        while (e < nent) {  // grid-stride over the entries of this variant
+            en = prm.list[e];
+            if (mine(en)) break;
+            e += gridDim.x;
+        }
         in[0] = e;
         if (e >= nent) return;
-        const LocalEntry en = prm.list[e];
         in[1] = en.count;
         in[2] = en.hi_bit;
         in[3] = en.src;
@@ -1281,7 +1305,12 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
     if (tid == 0) {
         for (int s = 0; s < NSTAGE; ++s) mbar_init(&bar[s], 1);
         mbar_fence_init();
-        for (int s = 0; s < NSTAGE; ++s) issue(s, blockIdx.x + s * gridDim.x);
+        uint32_t e = blockIdx.x;
+        for (int s = 0; s < NSTAGE; ++s) {
+            issue(s, e);
+            e = info[16 * s] + gridDim.x;
+        }
+        info[16 * NSTAGE] = e;  // next entry to look at
     }
     __syncthreads();
 
@@ -1350,20 +1379,19 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
         }
         const bool active = wbase < count;
         bool moved = false;
-        constexpr int IB = 13;  // index bits: CAP <= 8192
-        static_assert(L::CAP <= (1 << IB), "local-sort capacity exceeds the composite index");
         const int sb = hi_bit - begin_bit;
-        if (sb + IB <= static_cast<int>(8 * sizeof(K))) {
-            // ---- narrow path: one word per record, composite = (sort bits << IB) | index.
+        if constexpr (!LW::PAIRS) {
+            // ---- composite path: one word per record, composite = (sort bits << IB) | index.
             // The LSD passes move composites only; keys and values are gathered from the
             // staging buffers through the index at the end (the key bits outside the
             // sorted range are carried that way too).
-            K *comp = reinterpret_cast<K *>(sidx);
-            const K smask = sb >= static_cast<int>(8 * sizeof(K)) ? ~K(0) : ((K(1) << sb) - 1);
-            K cv[KPT];
+            CT *comp = reinterpret_cast<CT *>(sidx);
+            const CT smask = sb >= static_cast<int>(8 * sizeof(CT)) ? ~CT(0) : ((CT(1) << sb) - 1);
+            CT cv[KPT];
 #pragma unroll
-            for (int c = 0; c < KPT; ++c) cv[c] = (((key[c] >> begin_bit) & smask) << IB) | static_cast<K>(idx[c]);
-            const K cdiff = ((diff >> begin_bit) & smask) << IB;
+            for (int c = 0; c < KPT; ++c)
+                cv[c] = ((static_cast<CT>(key[c] >> begin_bit) & smask) << IB) | static_cast<CT>(idx[c]);
+            const CT cdiff = (static_cast<CT>(diff >> begin_bit) & smask) << IB;
             for (int lo = IB; lo < IB + sb; lo += 8) {
                 const int width = min(8, IB + sb - lo);
                 const uint32_t mask = (1u << width) - 1u;
@@ -1393,6 +1421,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
                 VT *const vd = HV ? vout + offs : nullptr;
                 const K *const ksp = ks + sk.pad;
                 const VT *const vsp = HV ? vs + sv.pad : nullptr;
+                static_assert(sizeof(CT) >= sizeof(K), "composite narrower than the key");
 #pragma unroll
                 for (int c = 0; c < KPT; ++c) {
                     const uint32_t e = wbase + c * 32 + lane;
@@ -1404,8 +1433,8 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
                 }
             }
         } else {
-            // ---- wide path (more than 8*sizeof(K) - 13 bits to sort): (key, index) pairs,
-            // the key staging buffer doubles as the sort buffer
+            // ---- pair path (64-bit keys with more than 51 bits to sort): (key, index)
+            // pairs, the key staging buffer doubles as the sort buffer
             K *skeys = ks;
             for (int lo = begin_bit; lo < hi_bit; lo += 8) {
                 const int width = min(8, hi_bit - lo);
@@ -1455,7 +1484,8 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
         __syncthreads();  // staging buffer s and red[] are free
         if (tid == 0) {
             fence_proxy_async();
-            issue(s, blockIdx.x + (it + NSTAGE) * gridDim.x);
+            issue(s, info[16 * NSTAGE]);
+            info[16 * NSTAGE] = info[16 * s] + gridDim.x;
         }
         __syncthreads();  // info[s] is rewritten above
     }
