@@ -225,7 +225,8 @@ struct Plan {
     uint32_t range_cap = 0;  // CTAs of the hist/scatter grid the temp layout allows
     size_t off_auxk = 0, off_auxv = 0, off_buckets[2] = {0, 0}, off_tot[2] = {0, 0}, off_subrel = 0,
            off_seg_last = 0, off_seg_meta = 0, off_carry = 0, off_tiles = 0, off_tile_pref = 0,
-           off_local[HRS_NUM_CLASSES] = {0}, total = 0;
+           off_local[HRS_NUM_CLASSES] = {0}, off_local_fb = 0, total = 0;
+    uint32_t local_fb_cap = 0;
 };
 
 size_t align_up(size_t x, size_t a) { return (x + a - 1) / a * a; }
@@ -320,10 +321,17 @@ hrs_status make_plan(Plan &pl, uint64_t n, int kb, int vb, int begin, int end, c
     off = align_up(off + sizeof(uint32_t) * RADIX * static_cast<size_t>(pl.tile_cap), 256);
     pl.off_subrel = off;
     off = align_up(off + sizeof(uint32_t) * RADIX * static_cast<size_t>(pl.bucket_cap), 256);
+    uint64_t fb = 0;
     for (int c = 0; c < HRS_NUM_CLASSES; ++c) {
         pl.off_local[c] = off;
         off = align_up(off + sizeof(LocalEntry) * static_cast<size_t>(pl.local_cap[c]), 256);
+        fb += pl.local_cap[c];
     }
+    // entries of more than 19 sort bits whose top bits tie in long runs go to the wide
+    // local sort: at most every entry
+    pl.local_fb_cap = static_cast<uint32_t>(std::min<uint64_t>(fb, 0xFFFFFFFFull));
+    pl.off_local_fb = off;
+    off = align_up(off + sizeof(LocalEntry) * static_cast<size_t>(pl.local_fb_cap), 256);
     pl.total = off;
     return HRS_SUCCESS;
 }
@@ -488,31 +496,44 @@ struct Runner {
             lp.src_vals[SRC_OUT] = vout;
             lp.keys_out = kout;
             lp.vals_out = vout;
-            lp.list = at<LocalEntry>(temp, pl.off_local[C]);
-            lp.count = &at<Ctl>(temp, 0)->nlocal[C];
+            Ctl *ctl = at<Ctl>(temp, 0);
+            lp.fb_list = at<LocalEntry>(temp, pl.off_local_fb);
+            lp.fb_count = &ctl->nlocal_fb;
+            lp.fb_cap = pl.local_fb_cap;
+            if (WIDE) {  // the wide variant sorts what the narrow ones handed over
+                lp.list = lp.fb_list;
+                lp.count = &ctl->nlocal_fb;
+            } else {
+                lp.list = at<LocalEntry>(temp, pl.off_local[C]);
+                lp.count = &ctl->nlocal[C];
+            }
             lp.begin_bit = pl.begin;
             auto fn = k_local<K, V, LC::THREADS, LC::KPT, LST::NSTAGE, LST::OCC, WIDE>;
             int grid = 0;
             hrs_status s = grid_for(fn, LC::THREADS, LST::bytes, dev, sms, &grid);
             if (s) return s;
-            grid = static_cast<int>(std::min<uint64_t>(grid, std::max<uint32_t>(pl.local_cap[C], 1)));
-            LaunchScope ls(st, 3, C);
+            const uint32_t cap = WIDE ? pl.local_fb_cap : pl.local_cap[C];
+            grid = static_cast<int>(std::min<uint64_t>(grid, std::max<uint32_t>(cap, 1)));
+            LaunchScope ls(st, 3, WIDE ? 8 : C);
             fn<<<grid, LC::THREADS, LST::bytes, st>>>(lp);
             return last_launch();
         }
     }
 
-    // the entries of one size class: most take the narrow variant; the wide one only
-    // runs when some entry sorts more bits than a key-width composite holds
     template <int C>
     static hrs_status local_one(const Plan &pl, void *temp, cudaStream_t st, int dev, int sms, const void *kin,
                                 void *kout, const void *vin, void *vout) {
-        hrs_status s = local_variant<C, 0>(pl, temp, st, dev, sms, kin, kout, vin, vout);
-        if (s) return s;
-        // a key-width composite holds (end - begin) + 13 bits: otherwise some entries
-        // (those partitioned on few digits) need the wide variant
-        if (pl.end - pl.begin + 13 > 8 * KB) s = local_variant<C, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout);
-        return s;
+        return local_variant<C, 0>(pl, temp, st, dev, sms, kin, kout, vin, vout);
+    }
+
+    // one wide launch (largest configuration) for whatever the narrow ones handed over;
+    // only needed when more than 19 bits can remain to sort
+    static hrs_status local_wide(const Plan &pl, void *temp, cudaStream_t st, int dev, int sms, const void *kin,
+                                 void *kout, const void *vin, void *vout) {
+        if (pl.end - pl.begin <= 19) return HRS_SUCCESS;
+        if (max_class_t<K, V>() == 7)
+            return local_variant<7, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout);
+        return local_variant<6, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout);
     }
 
     static hrs_status local(const Plan &pl, void *temp, cudaStream_t st, int dev, int sms, int c, const void *kin,
@@ -579,6 +600,7 @@ struct Runner {
         } else {
             if ((s = local(pl, temp, st, dev, sms, root_class, kin, kout, vin, vout))) return s;
         }
+        if ((s = local_wide(pl, temp, st, dev, sms, kin, kout, vin, vout))) return s;
         return HRS_SUCCESS;
     }
 

@@ -93,6 +93,8 @@ struct Ctl {
     unsigned long long alloc[HRS_MAX_PASSES + 2];
     uint32_t nlocal[HRS_NUM_CLASSES];       // entries in local list c
     uint32_t claim[HRS_MAX_PASSES + 2];     // k_scatter tile claims of pass p
+    uint32_t nlocal_fb;                     // entries the narrow local sort handed to the wide one
+    uint32_t pad2_;
     uint32_t overflow;
     uint32_t pad_;
     unsigned long long recs_in_pass[HRS_MAX_PASSES + 2];
@@ -1173,6 +1175,9 @@ struct LocalParams {
     void *vals_out;
     const LocalEntry *list;
     const uint32_t *count;  // entries in the list
+    LocalEntry *fb_list;    // narrow variant: entries handed to the wide variant
+    uint32_t *fb_count;
+    uint32_t fb_cap;
     int begin_bit;
 };
 
@@ -1180,12 +1185,13 @@ struct LocalParams {
 // the keys have been read into registers the key buffer doubles as the buffer of
 // the LSD passes, which move (key, 16-bit index) pairs; the values are gathered from
 // their staging buffer once, at the end.
-// Composite word of the local sort: the narrow variant ranks (sort bits << 13 | index)
-// in a word of the key's width; the wide variant in 64 bits for 32-bit keys and as
-// (key, 16-bit index) pairs for 64-bit keys (more than 51 bits to sort).
+// Composite word of the local sort.  The narrow variant ranks 32-bit composites
+// (top <= 19 sort bits << 13 | index) and resolves ties of the top bits afterwards;
+// the wide variant (entries the narrow one hands over) ranks 64-bit composites for
+// 32-bit keys and (key, 16-bit index) pairs for 64-bit keys.
 template <typename K, int WIDE>
 struct LocalWord {
-    using CT = typename std::conditional<(WIDE && sizeof(K) == 4), unsigned long long, K>::type;
+    using CT = typename std::conditional<WIDE, unsigned long long, uint32_t>::type;
     static constexpr bool PAIRS = WIDE && sizeof(K) == 8;
     static constexpr size_t buf_bytes = PAIRS ? sizeof(uint16_t) : sizeof(CT);
 };
@@ -1262,12 +1268,8 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
                                        : code == SRC_AUX ? prm.src_vals[SRC_AUX]
                                                          : prm.src_vals[SRC_OUT]);
     };
-    // an entry belongs to the narrow variant iff its sort bits and the index fit in one
-    // key-width word
-    auto mine = [&](const LocalEntry &en) {
-        const bool narrow = static_cast<int>(en.hi_bit) - prm.begin_bit + IB <= static_cast<int>(8 * sizeof(K));
-        return narrow == (WIDE == 0);
-    };
+    auto mine = [&](const LocalEntry &) { return true; };
+    __shared__ uint32_t s_fallback;
     // info[s]: 0 entry, 1 count, 2 hi_bit, 3 src, 4..5 offs, 6..8 key seg, 9..11 value seg, 12 next stride
     auto issue = [&](int s, uint32_t e) {
         uint32_t *in = info + 16 * s;
@@ -1381,19 +1383,26 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
         bool moved = false;
         const int sb = hi_bit - begin_bit;
         if constexpr (!LW::PAIRS) {
-            // ---- composite path: one word per record, composite = (sort bits << IB) | index.
+            // ---- composite path: one word per record, composite = (top sort bits << IB) | index.
             // The LSD passes move composites only; keys and values are gathered from the
             // staging buffers through the index at the end (the key bits outside the
-            // sorted range are carried that way too).
+            // sorted range are carried that way too).  The narrow variant keeps the top
+            // TB <= 19 sort bits and then orders the runs of records that tie on them by
+            // the remaining bits (insertion sort; a bucket with a run longer than RUN_MAX
+            // is handed to the wide variant).
+            constexpr int CB = static_cast<int>(8 * sizeof(CT)) - IB;  // sort bits a composite holds
+            constexpr uint32_t RUN_MAX = 16;
+            const int tb = sb < CB ? sb : CB;
+            const int tlo = hi_bit - tb;  // composite field = key bits [tlo, hi_bit)
             CT *comp = reinterpret_cast<CT *>(sidx);
-            const CT smask = sb >= static_cast<int>(8 * sizeof(CT)) ? ~CT(0) : ((CT(1) << sb) - 1);
+            const CT tmask = tb >= static_cast<int>(8 * sizeof(CT)) ? ~CT(0) : ((CT(1) << tb) - 1);
             CT cv[KPT];
 #pragma unroll
             for (int c = 0; c < KPT; ++c)
-                cv[c] = ((static_cast<CT>(key[c] >> begin_bit) & smask) << IB) | static_cast<CT>(idx[c]);
-            const CT cdiff = (static_cast<CT>(diff >> begin_bit) & smask) << IB;
-            for (int lo = IB; lo < IB + sb; lo += 8) {
-                const int width = min(8, IB + sb - lo);
+                cv[c] = ((static_cast<CT>(key[c] >> tlo) & tmask) << IB) | static_cast<CT>(idx[c]);
+            const CT cdiff = (static_cast<CT>(diff >> tlo) & tmask) << IB;
+            for (int lo = IB; lo < IB + tb; lo += 8) {
+                const int width = min(8, IB + tb - lo);
                 const uint32_t mask = (1u << width) - 1u;
                 if ((static_cast<uint32_t>(cdiff >> lo) & mask) == 0) continue;  // constant digit: identity pass
                 moved = true;
@@ -1416,12 +1425,73 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
                         if (!BAL || c < kpt) cv[c] = comp[wbase + c * 32 + lane];
                 }
             }
-            if (moved || src != SRC_OUT) {
+            const K *const ksp = ks + sk.pad;
+            bool fallback = false;
+            if (sb > tb) {
+                // ---- runs that tie on the top bits: insertion sort by (low bits, index);
+                // inside a run the records are in index order (the passes are stable), so
+                // shifting only past strictly greater low bits keeps the sort stable
+                if (!moved) {
+                    // comp was not written: store the (unsorted) composites
+#pragma unroll
+                    for (int c = 0; c < KPT; ++c)
+                        if ((!BAL || c < kpt) && active) comp[wbase + c * 32 + lane] = cv[c];
+                }
+                if (tid == 0) s_fallback = 0;
+                __syncthreads();
+                const int lb = sb - tb;
+                const K lmask = lb >= static_cast<int>(8 * sizeof(K)) ? ~K(0) : ((K(1) << lb) - 1);
+                auto low = [&](CT x) -> K {
+                    return (ksp[static_cast<uint32_t>(x) & ((1u << IB) - 1u)] >> begin_bit) & lmask;
+                };
+                for (uint32_t e = tid; e + 1 < count; e += THREADS) {
+                    const CT t = comp[e] >> IB;
+                    if ((comp[e + 1] >> IB) != t) continue;
+                    if (e > 0 && (comp[e - 1] >> IB) == t) continue;  // not the start of the run
+                    uint32_t r = 2;
+                    while (e + r < count && (comp[e + r] >> IB) == t) ++r;
+                    if (r > RUN_MAX) {
+                        s_fallback = 1;
+                        continue;
+                    }
+                    for (uint32_t i = 1; i < r; ++i) {
+                        const CT x = comp[e + i];
+                        const K lx = low(x);
+                        int j = static_cast<int>(i) - 1;
+                        while (j >= 0) {
+                            const CT y = comp[e + j];
+                            if (low(y) <= lx) break;
+                            comp[e + j + 1] = y;
+                            --j;
+                        }
+                        comp[e + j + 1] = x;
+                    }
+                }
+                __syncthreads();
+                fallback = s_fallback != 0;
+                moved = true;
+                if (!fallback && active) {
+#pragma unroll
+                    for (int c = 0; c < KPT; ++c)
+                        if (!BAL || c < kpt) cv[c] = comp[wbase + c * 32 + lane];
+                }
+            }
+            if (fallback) {
+                if (tid == 0) {
+                    const uint32_t slot = atomicAdd(prm.fb_count, 1u);
+                    if (slot < prm.fb_cap) {
+                        LocalEntry en;
+                        en.offs = offs;
+                        en.count = count;
+                        en.hi_bit = static_cast<uint16_t>(hi_bit);
+                        en.src = static_cast<uint16_t>(src);
+                        prm.fb_list[slot] = en;
+                    }
+                }
+            } else if (moved || src != SRC_OUT) {
                 K *const kd = kout + offs;
                 VT *const vd = HV ? vout + offs : nullptr;
-                const K *const ksp = ks + sk.pad;
                 const VT *const vsp = HV ? vs + sv.pad : nullptr;
-                static_assert(sizeof(CT) >= sizeof(K), "composite narrower than the key");
 #pragma unroll
                 for (int c = 0; c < KPT; ++c) {
                     const uint32_t e = wbase + c * 32 + lane;
