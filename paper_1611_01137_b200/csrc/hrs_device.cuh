@@ -342,22 +342,24 @@ struct Ranker {
     static constexpr int VW = VWPW * W;
     static constexpr int KH = VWPW == 2 ? (KPT + 1) / 2 : KPT;  // columns of the first half
     static constexpr size_t cnt_words = static_cast<size_t>(VW) * NBINS;
-    static constexpr size_t smem_bytes = sizeof(uint32_t) * (cnt_words + 288);
-    uint32_t *cnt;  // [VW][NBINS]
-    uint32_t *tot;  // [288]
+    static constexpr size_t smem_bytes = sizeof(uint32_t) * (cnt_words + 2 * 288);
+    uint32_t *cnt;    // [VW][NBINS]
+    uint32_t *tot;    // [288] digit totals of the tile
+    uint32_t *start;  // [288] first slot of each digit (valid after the caller's next barrier)
 
     __device__ __forceinline__ uint32_t *vcnt(int vw) const { return cnt + vw * NBINS; }
 
     __device__ __forceinline__ void init(uint32_t *base) {
         cnt = base;
         tot = base + cnt_words;
+        start = tot + 288;
         for (int i = threadIdx.x; i < static_cast<int>(cnt_words); i += THREADS) cnt[i] = 0;
     }
 
     // dg: digits on entry (INVALID_DIGIT for padding), slots on exit.  kpt: active
     // columns (the same for all warps); active: this warp holds elements.  Contains
-    // three block barriers; the caller needs one more before reading the slots' data.
-    // Afterwards tot[d] = first slot of digit d (tot[256] = valid elements).
+    // two block barriers; the caller needs one more before reading the slots' data
+    // and before reading start[d] = first slot of digit d.
     __device__ __forceinline__ void rank(uint32_t (&dg)[KPT], int kpt, bool active, uint32_t ltm) {
         const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
         uint32_t *ca = vcnt(VWPW * warp);
@@ -382,13 +384,36 @@ struct Ranker {
             tot[d] = run;
         }
         __syncthreads();
-        warp0_exclusive_scan(tot, NBINS);
-        __syncthreads();
-        // each warp folds the digit starts into its own counters
-        for (int d = lane; d < NBINS; d += 32) {
-            const uint32_t t = tot[d];
-            ca[d] += t;
-            if (VWPW == 2) cb[d] += t;
+        // every warp scans the 257 digit totals itself (lane l: digits 9l .. 9l+8) and
+        // folds the digit starts into its own counters -- no barrier for a single-warp
+        // scan; warp 0 also publishes the starts (read by the caller after its next barrier)
+        {
+            constexpr int PER = 9;
+            uint32_t v[PER];
+            uint32_t sum = 0;
+#pragma unroll
+            for (int i = 0; i < PER; ++i) {
+                const int d = lane * PER + i;
+                v[i] = d < NBINS ? tot[d] : 0u;
+                sum += v[i];
+            }
+            uint32_t incl = sum;
+#pragma unroll
+            for (int o = 1; o < 32; o <<= 1) {
+                const uint32_t y = __shfl_up_sync(0xffffffffu, incl, o);
+                if (lane >= o) incl += y;
+            }
+            uint32_t run = incl - sum;
+#pragma unroll
+            for (int i = 0; i < PER; ++i) {
+                const int d = lane * PER + i;
+                if (d < NBINS) {
+                    ca[d] += run;
+                    if (VWPW == 2) cb[d] += run;
+                    if (warp == 0) start[d] = run;
+                }
+                run += v[i];
+            }
         }
         __syncwarp();
         if (active) {
@@ -1076,8 +1101,6 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
             }
             // ---- stable rank
             ranker.rank(dg, KPT, FULL || wbase < count, ltm);
-            // destination of slot j holding digit d: bucket offset + gbase[d] + j
-            if (tid < RADIX) gbase[tid] = dbase - ranker.tot[tid];
             // ---- values into registers, then everything back into the staging buffer
             //      in slot order (slot j at index j, the pad is no longer needed)
             if (HV) {
@@ -1088,6 +1111,8 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
                     if (FULL || e < count) val[c] = FULL ? vs[e] : seg_get(vs, vsrc, sv, e);
                 }
                 __syncthreads();
+                // destination of slot j holding digit d: bucket offset + gbase[d] + j
+                if (tid < RADIX) gbase[tid] = dbase - ranker.start[tid];
 #pragma unroll
                 for (int c = 0; c < KPT; ++c) {
                     const uint32_t e = wbase + c * 32 + lane;
@@ -1098,6 +1123,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
                 }
             } else {
                 __syncthreads();
+                if (tid < RADIX) gbase[tid] = dbase - ranker.start[tid];
 #pragma unroll
                 for (int c = 0; c < KPT; ++c) {
                     const uint32_t e = wbase + c * 32 + lane;
