@@ -102,10 +102,12 @@ template <> struct LocalCfg<7> { static constexpr int THREADS = 512, KPT = 16; }
 template <typename K, typename V, int C, int WIDE = 0>
 struct LocalStages {
     using LC = LocalCfg<C>;
-    static constexpr size_t SM_BUDGET = 224 * 1024;
-    static constexpr int NSTAGE = 3 * LocalSmem<K, V, LC::THREADS, LC::KPT, 2, WIDE>::bytes <= SM_BUDGET ? 2 : 1;
+    static constexpr size_t SM_BUDGET = 228 * 1024;  // shared memory per SM; 1 KB reserved per CTA
+    static constexpr int NSTAGE =
+        3 * (LocalSmem<K, V, LC::THREADS, LC::KPT, 2, WIDE>::bytes + 1024) <= SM_BUDGET ? 2 : 1;
     static constexpr size_t bytes = LocalSmem<K, V, LC::THREADS, LC::KPT, NSTAGE, WIDE>::bytes;
-    static constexpr bool fits = bytes <= SMEM_LIMIT && LocalSmem<K, V, LC::THREADS, LC::KPT, 1, 1>::bytes <= SMEM_LIMIT;
+    static constexpr bool fits = bytes <= SMEM_LIMIT && LocalSmem<K, V, LC::THREADS, LC::KPT, 1, 1>::bytes <= SMEM_LIMIT &&
+                                 LocalSmem<K, V, LC::THREADS, LC::KPT, 1, 0>::bytes <= SMEM_LIMIT;
     static constexpr int by_smem = static_cast<int>(SM_BUDGET / (bytes + 1024));
     static constexpr int by_threads = 2048 / LC::THREADS;
     static constexpr int OCC0 = by_smem < by_threads ? by_smem : by_threads;
@@ -500,7 +502,7 @@ struct Runner {
             lp.fb_list = at<LocalEntry>(temp, pl.off_local_fb);
             lp.fb_count = &ctl->nlocal_fb;
             lp.fb_cap = pl.local_fb_cap;
-            if (WIDE) {  // the wide variant sorts what the narrow ones handed over
+            if (WIDE == 1) {  // the wide variant sorts what the narrow ones handed over
                 lp.list = lp.fb_list;
                 lp.count = &ctl->nlocal_fb;
             } else {
@@ -512,9 +514,9 @@ struct Runner {
             int grid = 0;
             hrs_status s = grid_for(fn, LC::THREADS, LST::bytes, dev, sms, &grid);
             if (s) return s;
-            const uint32_t cap = WIDE ? pl.local_fb_cap : pl.local_cap[C];
+            const uint32_t cap = WIDE == 1 ? pl.local_fb_cap : pl.local_cap[C];
             grid = static_cast<int>(std::min<uint64_t>(grid, std::max<uint32_t>(cap, 1)));
-            LaunchScope ls(st, 3, WIDE ? 8 : C);
+            LaunchScope ls(st, 3, WIDE == 1 ? 8 : C);
             fn<<<grid, LC::THREADS, LST::bytes, st>>>(lp);
             return last_launch();
         }
@@ -523,6 +525,8 @@ struct Runner {
     template <int C>
     static hrs_status local_one(const Plan &pl, void *temp, cudaStream_t st, int dev, int sms, const void *kin,
                                 void *kout, const void *vin, void *vout) {
+        // full-range sorts of 32-bit keys rebuild the keys from the composites
+        if (KB == 4 && pl.begin == 0) return local_variant<C, 2>(pl, temp, st, dev, sms, kin, kout, vin, vout);
         return local_variant<C, 0>(pl, temp, st, dev, sms, kin, kout, vin, vout);
     }
 
@@ -530,7 +534,7 @@ struct Runner {
     // only needed when more than 19 bits can remain to sort
     static hrs_status local_wide(const Plan &pl, void *temp, cudaStream_t st, int dev, int sms, const void *kin,
                                  void *kout, const void *vin, void *vout) {
-        if (pl.end - pl.begin <= 19) return HRS_SUCCESS;
+        if (pl.end - pl.begin <= 19) return HRS_SUCCESS;  // every entry fits a narrow composite
         if (max_class_t<K, V>() == 7)
             return local_variant<7, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout);
         return local_variant<6, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout);

@@ -544,7 +544,7 @@ struct HistSmem {
     static constexpr size_t off_bar = 0;
     static constexpr size_t off_info = align16(sizeof(uint64_t) * NSTAGE);
     static constexpr size_t off_wh = align16(off_info + sizeof(uint32_t) * 8 * NSTAGE);
-    static constexpr size_t off_stage = align16(off_wh + sizeof(uint32_t) * W * RADIX);
+    static constexpr size_t off_stage = align16(off_wh + sizeof(uint32_t) * 2 * RADIX);
     static constexpr size_t stage_elems = CAP + 16 / sizeof(K);
     static constexpr size_t bytes = off_stage + NSTAGE * align16(sizeof(K) * stage_elems);
 };
@@ -606,9 +606,8 @@ __global__ void __launch_bounds__(THREADS) k_hist(HistParams prm) {
         for (int s = 0; s < NSTAGE; ++s) issue(s);
         prm.seg_meta[blockIdx.x].first_bucket = fb;
     }
-    for (int i = tid; i < W * RADIX; i += THREADS) wh[i] = 0;
+    for (int i = tid; i < 2 * RADIX; i += THREADS) wh[i] = 0;
     __syncthreads();
-    uint32_t *my = wh + warp * RADIX;
     uint32_t seg_run = 0;            // digit tid: count of the current bucket segment before this tile
     bool first_seg = true;           // inside the CTA's first bucket segment (its carry applies)
     for (uint32_t t = tb, it = 0; t < te; ++t, ++it) {
@@ -623,6 +622,9 @@ __global__ void __launch_bounds__(THREADS) k_hist(HistParams prm) {
         sg.i1 = in[5];
         const uint64_t toffs = offs_of[s];
         const K *src = keys + toffs;
+        // one block histogram per tile, double-buffered: the counts of tile i are read
+        // and cleared while tile i + 1 is counted into the other buffer
+        uint32_t *my = wh + (it & 1u) * RADIX;
         // tile descriptor and tile-ordered prefix for the scatter
         if (tid < RADIX) prm.tile_pref[static_cast<uint64_t>(t) * RADIX + tid] = seg_run;
         if (tid == 0) {
@@ -660,26 +662,20 @@ __global__ void __launch_bounds__(THREADS) k_hist(HistParams prm) {
             fence_proxy_async();
             issue(s);
         }
-        // segment count so far (the per-warp counters accumulate over the segment)
-        uint32_t sum = 0;
+        // segment count so far
         if (tid < RADIX) {
-#pragma unroll
-            for (int w = 0; w < W; ++w) sum += wh[w * RADIX + tid];
-            seg_run = sum;
+            seg_run += my[tid];
+            my[tid] = 0;
         }
-        __syncthreads();  // the next tile's counts must not land before the sums are read
         if (flush) {
             const bool last_seg = t + 1 == te;
             if (tid < RADIX) {
-#pragma unroll
-                for (int w = 0; w < W; ++w) wh[w * RADIX + tid] = 0;
-                if (sum) atomicAdd(&prm.tot[static_cast<uint64_t>(bucket) * RADIX + tid], sum);
-                if (last_seg) prm.seg_last[static_cast<uint64_t>(blockIdx.x) * RADIX + tid] = sum;
+                if (seg_run) atomicAdd(&prm.tot[static_cast<uint64_t>(bucket) * RADIX + tid], seg_run);
+                if (last_seg) prm.seg_last[static_cast<uint64_t>(blockIdx.x) * RADIX + tid] = seg_run;
             }
             if (last_seg && tid == 0) prm.seg_meta[blockIdx.x].last_bucket = bucket;
             seg_run = 0;
             first_seg = false;
-            __syncthreads();
         }
     }
 }
@@ -1215,11 +1211,16 @@ struct LocalParams {
 // (top <= 19 sort bits << 13 | index) and resolves ties of the top bits afterwards;
 // the wide variant (entries the narrow one hands over) ranks 64-bit composites for
 // 32-bit keys and (key, 16-bit index) pairs for 64-bit keys.
+// WIDE = 2 is the narrow variant for begin_bit == 0: entries of at most 19 sort bits
+// rank their composites inside the key staging buffer and rebuild the keys from the
+// composite and the bucket's common high bits (no key gather, no composite buffer);
+// entries with more sort bits go straight to the wide variant.
 template <typename K, int WIDE>
 struct LocalWord {
-    using CT = typename std::conditional<WIDE, unsigned long long, uint32_t>::type;
-    static constexpr bool PAIRS = WIDE && sizeof(K) == 8;
-    static constexpr size_t buf_bytes = PAIRS ? sizeof(uint16_t) : sizeof(CT);
+    using CT = typename std::conditional<WIDE == 1, unsigned long long, uint32_t>::type;
+    static constexpr bool PAIRS = WIDE == 1 && sizeof(K) == 8;
+    static constexpr bool RECON = WIDE == 2;
+    static constexpr size_t buf_bytes = RECON ? 0 : (PAIRS ? sizeof(uint16_t) : sizeof(CT));
 };
 
 template <typename K, typename V, int THREADS, int KPT, int NSTAGE, int WIDE = 0>
@@ -1294,7 +1295,13 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
                                        : code == SRC_AUX ? prm.src_vals[SRC_AUX]
                                                          : prm.src_vals[SRC_OUT]);
     };
-    auto mine = [&](const LocalEntry &) { return true; };
+    // the recon variant hands entries of more than 19 sort bits to the wide variant
+    auto mine = [&](const LocalEntry &en) {
+        if (!LW::RECON || static_cast<int>(en.hi_bit) - prm.begin_bit <= 32 - IB) return true;
+        const uint32_t slot = atomicAdd(prm.fb_count, 1u);
+        if (slot < prm.fb_cap) prm.fb_list[slot] = en;
+        return false;
+    };
     __shared__ uint32_t s_fallback;
     // info[s]: 0 entry, 1 count, 2 hi_bit, 3 src, 4..5 offs, 6..8 key seg, 9..11 value seg, 12 next stride
     auto issue = [&](int s, uint32_t e) {
@@ -1395,7 +1402,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
             red[W + warp] = o;
         }
         __syncthreads();
-        K diff = 0;
+        K diff = 0, kconst = 0;
         {
             K aa = ~K(0), oo = K(0);
 #pragma unroll
@@ -1404,6 +1411,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
                 oo |= red[W + w];
             }
             diff = aa ^ oo;
+            kconst = aa;  // the bits of positions where diff == 0 are common to all keys
         }
         const bool active = wbase < count;
         bool moved = false;
@@ -1420,7 +1428,8 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
             constexpr uint32_t RUN_MAX = 16;
             const int tb = sb < CB ? sb : CB;
             const int tlo = hi_bit - tb;  // composite field = key bits [tlo, hi_bit)
-            CT *comp = reinterpret_cast<CT *>(sidx);
+            // recon: the keys are in registers, their staging buffer holds the composites
+            CT *comp = LW::RECON ? reinterpret_cast<CT *>(ks) : reinterpret_cast<CT *>(sidx);
             const CT tmask = tb >= static_cast<int>(8 * sizeof(CT)) ? ~CT(0) : ((CT(1) << tb) - 1);
             CT cv[KPT];
 #pragma unroll
@@ -1453,7 +1462,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
             }
             const K *const ksp = ks + sk.pad;
             bool fallback = false;
-            if (sb > tb) {
+            if (!LW::RECON && sb > tb) {
                 // ---- runs that tie on the top bits: insertion sort by (low bits, index);
                 // inside a run the records are in index order (the passes are stable), so
                 // shifting only past strictly greater low bits keeps the sort stable
@@ -1518,12 +1527,15 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
                 K *const kd = kout + offs;
                 VT *const vd = HV ? vout + offs : nullptr;
                 const VT *const vsp = HV ? vs + sv.pad : nullptr;
+                // recon (begin_bit == 0, all sort bits in the composite): key = common bits
+                // above hi_bit | the composite's sort field
+                const K khigh = hi_bit >= static_cast<int>(8 * sizeof(K)) ? K(0) : (kconst & ~((K(1) << hi_bit) - 1));
 #pragma unroll
                 for (int c = 0; c < KPT; ++c) {
                     const uint32_t e = wbase + c * 32 + lane;
                     if ((!BAL || c < kpt) && e < count) {
                         const uint32_t ix = static_cast<uint32_t>(cv[c]) & ((1u << IB) - 1u);
-                        kd[e] = ksp[ix];
+                        kd[e] = LW::RECON ? (khigh | static_cast<K>(static_cast<uint32_t>(cv[c]) >> IB)) : ksp[ix];
                         if (HV) vd[e] = vsp[ix];
                     }
                 }
