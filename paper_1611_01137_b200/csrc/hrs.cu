@@ -203,6 +203,22 @@ hrs_status grid_for(F *fn, int threads, size_t smem, int dev, int sms, int *grid
     return HRS_SUCCESS;
 }
 
+// launch with programmatic stream serialization (PDL); kernels call pdl_wait() first
+template <typename... KArgs, typename... Args>
+void launch_pdl(void (*fn)(KArgs...), dim3 grid, dim3 block, size_t smem, cudaStream_t st, Args &&...args) {
+    cudaLaunchConfig_t cfg = {};
+    cfg.gridDim = grid;
+    cfg.blockDim = block;
+    cfg.dynamicSmemBytes = smem;
+    cfg.stream = st;
+    cudaLaunchAttribute attr[1];
+    attr[0].id = cudaLaunchAttributeProgrammaticStreamSerialization;
+    attr[0].val.programmaticStreamSerializationAllowed = 1;
+    cfg.attrs = attr;
+    cfg.numAttrs = 1;
+    cudaLaunchKernelEx(&cfg, fn, std::forward<Args>(args)...);
+}
+
 hrs_status last_launch() {
     cudaError_t e = cudaGetLastError();
     if (e != cudaSuccess) return cuda_fail(e);
@@ -371,7 +387,7 @@ struct Runner {
         ip.key_bytes = pl.kb;
         ip.value_bytes = pl.vb;
         LaunchScope ls(st, 0, 0);
-        k_init<<<1, 256, 0, st>>>(ip);
+        launch_pdl(k_init, dim3(1), dim3(256), 0, st, ip);
         return last_launch();
     }
 
@@ -408,7 +424,7 @@ struct Runner {
         hrs_status s = grid_for(fn, HIST_THREADS, smem, dev, sms, &grid);  // sets the smem attribute
         if (s) return s;
         LaunchScope ls(st, 1, p);
-        fn<<<G, HIST_THREADS, smem, st>>>(hp);
+        launch_pdl(fn, dim3(G), dim3(HIST_THREADS), smem, st, hp);
         return last_launch();
     }
 
@@ -450,7 +466,7 @@ struct Runner {
         // one block per bucket (up to the resident limit) plus the carry block
         grid = static_cast<int>(std::min<uint64_t>(grid, std::max<uint64_t>(pl.bucket_cap, 1))) + 1;
         LaunchScope ls(st, 5, p);
-        fn<<<grid, CLASSIFY_THREADS, 0, st>>>(cp);
+        launch_pdl(fn, dim3(grid), dim3(CLASSIFY_THREADS), 0, st, cp);
         return last_launch();
     }
 
@@ -477,7 +493,7 @@ struct Runner {
         if (s) return s;
         (void)G;
         LaunchScope ls(st, 2, p);
-        fn<<<grid, SC::THREADS, smem, st>>>(sp);
+        launch_pdl(fn, dim3(grid), dim3(SC::THREADS), smem, st, sp);
         return last_launch();
     }
 
@@ -517,7 +533,7 @@ struct Runner {
             const uint32_t cap = WIDE == 1 ? pl.local_fb_cap : pl.local_cap[C];
             grid = static_cast<int>(std::min<uint64_t>(grid, std::max<uint32_t>(cap, 1)));
             LaunchScope ls(st, 3, WIDE == 1 ? 8 : C);
-            fn<<<grid, LC::THREADS, LST::bytes, st>>>(lp);
+            launch_pdl(fn, dim3(grid), dim3(LC::THREADS), LST::bytes, st, lp);
             return last_launch();
         }
     }

@@ -230,6 +230,11 @@ __host__ __device__ __forceinline__ uint32_t range_begin(uint32_t T, uint32_t c,
     return static_cast<uint32_t>((static_cast<uint64_t>(T) * c) / G);
 }
 
+// Programmatic dependent launch: every kernel of a sort is launched with PDL, so its
+// launch and prologue overlap the previous kernel's tail; it waits here before it
+// touches memory the previous kernels wrote.
+__device__ __forceinline__ void pdl_wait() { asm volatile("griddepcontrol.wait;" ::: "memory"); }
+
 // ------------------------------------------------------------------ TMA bulk copies (cp.async.bulk + mbarrier)
 
 __device__ __forceinline__ uint32_t smem_u32(const void *p) {
@@ -470,6 +475,7 @@ struct InitParams {
 };
 
 __global__ void k_init(InitParams prm) {
+    pdl_wait();
     const uint64_t n = prm.n;
     const uint32_t T1 = prm.counting ? static_cast<uint32_t>((n + prm.kpb - 1) / prm.kpb) : 0u;
     if (blockIdx.x == 0) {
@@ -551,6 +557,7 @@ struct HistSmem {
 
 template <typename K, int THREADS, int NSTAGE, int CAP>
 __global__ void __launch_bounds__(THREADS) k_hist(HistParams prm) {
+    pdl_wait();
     using L = HistSmem<K, THREADS, NSTAGE, CAP>;
     constexpr int W = THREADS / 32;
     constexpr int VK = 16 / sizeof(K);
@@ -915,6 +922,7 @@ __device__ void range_carries(const ClassifyParams &prm) {
 
 template <int THREADS>
 __global__ void __launch_bounds__(THREADS) k_classify(ClassifyParams prm) {
+    pdl_wait();
     __shared__ uint32_t scratch[7 * NBINS];
     const uint32_t nb = alloc_buckets(prm.ctl->alloc[prm.p]);
     if (nb == 0) return;  // nothing reached this pass
@@ -978,6 +986,7 @@ struct ScatterSmem {
 // flight into the other buffer.
 template <typename K, typename V, int THREADS, int KPT, int MINB>
 __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
+    pdl_wait();
     using L = ScatterSmem<K, V, THREADS, KPT>;
     constexpr bool HV = HasVal<V>::value;
     using VT = ValT<V>;
@@ -1259,6 +1268,7 @@ __device__ __forceinline__ unsigned long long warp_or(unsigned long long x) {
 
 template <typename K, typename V, int THREADS, int KPT, int NSTAGE, int MINB, int WIDE>
 __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
+    pdl_wait();
     using L = LocalSmem<K, V, THREADS, KPT, NSTAGE, WIDE>;
     using LW = LocalWord<K, WIDE>;
     using CT = typename LW::CT;
