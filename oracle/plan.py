@@ -44,8 +44,8 @@ def digit_plan(begin_bit: int, end_bit: int):
 
 def class_capacity(c: int) -> int:
     """Upper size of local-sort class c.  P:562-566 gives [1,128], (128,256], (256,512],
-    ... as an example; reading #20: powers of two up to 4096, then 6144, 8192."""
-    return (128 << c) if c < 6 else (6144 if c == 6 else 8192)
+    ... as an example; reading #20: powers of two up to 4096, then 4608, 8192."""
+    return (128 << c) if c < 6 else (4608 if c == 6 else 8192)
 
 
 def size_class(size: int) -> int:

@@ -93,7 +93,7 @@ template <> struct LocalCfg<2> { static constexpr int THREADS = 64, KPT = 8; };
 template <> struct LocalCfg<3> { static constexpr int THREADS = 128, KPT = 8; };
 template <> struct LocalCfg<4> { static constexpr int THREADS = 128, KPT = 16; };
 template <> struct LocalCfg<5> { static constexpr int THREADS = 256, KPT = 16; };
-template <> struct LocalCfg<6> { static constexpr int THREADS = 384, KPT = 16; };
+template <> struct LocalCfg<6> { static constexpr int THREADS = 288, KPT = 16; };
 template <> struct LocalCfg<7> { static constexpr int THREADS = 512, KPT = 16; };
 
 // two-stage TMA prefetch where it fits next to a second resident CTA, else one stage

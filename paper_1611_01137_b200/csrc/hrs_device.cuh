@@ -128,10 +128,10 @@ template <typename V>
 using ValT = typename std::conditional<HasVal<V>::value, V, uint32_t>::type;
 
 // Local-sort size classes (P:562-566 gives [1,128], (128,256], (256,512], ... as an
-// example): powers of two up to 4096, then (4096, 6144] and (6144, 8192] so that the
-// ~4096-record buckets a uniform input leaves after two passes fill their CTA.
+// example): powers of two up to 4096, then (4096, 4608] and (4608, 8192] so that the
+// ~4096-record buckets a uniform input leaves after two passes keep every warp busy.
 __host__ __device__ __forceinline__ uint32_t class_capacity(int c) {
-    return c < 6 ? (128u << c) : (c == 6 ? 6144u : 8192u);
+    return c < 6 ? (128u << c) : (c == 6 ? 4608u : 8192u);
 }
 __host__ __device__ __forceinline__ int size_class_of(uint32_t size) {
     int c = 0;

@@ -201,8 +201,8 @@ def test_merge_rule_worked_vector():
 
 def test_size_classes():
     # [1,128] -> 0, (128,256] -> 1, (256,512] -> 2, ..., (2048,4096] -> 5,
-    # then (4096,6144] -> 6 and (6144,8192] -> 7 (reading #20)
-    assert [plan.size_class(s) for s in (1, 128, 129, 256, 257, 512, 513, 4096, 4097, 6144, 6145, 8192)] == \
+    # then (4096,4608] -> 6 and (4608,8192] -> 7 (reading #20)
+    assert [plan.size_class(s) for s in (1, 128, 129, 256, 257, 512, 513, 4096, 4097, 4608, 4609, 8192)] == \
         [0, 0, 1, 1, 2, 2, 3, 5, 6, 6, 7, 7]
 
 
