@@ -209,6 +209,38 @@ __global__ void __launch_bounds__(THREADS) k_rank(const uint32_t* __restrict__ i
         }
         rk[c] = ((pre + r) << 9) | d;
       }
+    } else if (MODE == 8) {  // bit-sliced ballots, leader returning atomicAdd + shfl
+#pragma unroll
+      for (int c = 0; c < KPT; ++c) {
+        uint32_t d = (key[c] >> shift) & 255;
+        uint32_t m = 0xffffffffu;
+#pragma unroll
+        for (int b = 0; b < 8; ++b) {
+          uint32_t bal = __ballot_sync(0xffffffffu, (d >> b) & 1);
+          m &= ((d >> b) & 1) ? bal : ~bal;
+        }
+        const int leader = __ffs(m) - 1;
+        uint32_t pre = 0;
+        if (lane == leader) pre = atomicAdd(&my[d], (uint32_t)__popc(m));
+        pre = __shfl_sync(0xffffffffu, pre, leader);
+        rk[c] = ((pre + __popc(m & ltm)) << 9) | d;
+      }
+    } else if (MODE == 9) {  // ballots with xor-trick mask, leader returning atomicAdd + shfl
+#pragma unroll
+      for (int c = 0; c < KPT; ++c) {
+        uint32_t d = (key[c] >> shift) & 255;
+        uint32_t m = 0xffffffffu;
+#pragma unroll
+        for (int b = 0; b < 8; ++b) {
+          uint32_t bal = __ballot_sync(0xffffffffu, (d >> b) & 1);
+          m &= bal ^ (((d >> b) & 1) - 1u);
+        }
+        const int leader = __ffs(m) - 1;
+        uint32_t pre = 0;
+        if (lane == leader) pre = atomicAdd(&my[d], (uint32_t)__popc(m));
+        pre = __shfl_sync(0xffffffffu, pre, leader);
+        rk[c] = ((pre + __popc(m & ltm)) << 9) | d;
+      }
     } else {  // MODE 2: unstable reference: atomicAdd returning old (NOT stable; cost reference only)
 #pragma unroll
       for (int c = 0; c < KPT; ++c) {
@@ -261,6 +293,12 @@ __global__ void k_gen(uint32_t* k, size_t n, int m) {
   }
 }
 
+__global__ void k_cmp(const uint32_t* a, const uint32_t* b, size_t n, unsigned long long* bad) {
+  unsigned long long c = 0;
+  for (size_t i = blockIdx.x * (size_t)blockDim.x + threadIdx.x; i < n; i += (size_t)gridDim.x * blockDim.x) c += a[i] != b[i];
+  if (c) atomicAdd(bad, c);
+}
+
 template <typename F>
 float timeit(F f, int reps = 5) {
   cudaEvent_t a, b; cudaEventCreate(&a); cudaEventCreate(&b);
@@ -302,13 +340,33 @@ int main() {
         float t = timeit([&] { kern<<<sms * per, threads, smem>>>(keys, out, n, 24); });
         printf("rank %-7s %-22s occ%d: %.3f ms  %.0f GB/s (r+w keys)\n", dname[di], name, per, t, 2.0 * n * 4 / t / 1e6);
       };
+      {
+        uint32_t* ref; unsigned long long* bad;
+        CK(cudaMalloc(&ref, n * 4)); CK(cudaMalloc(&bad, 8));
+        for (int shift : {0, 8, 16, 24}) {
+          auto go = [&](auto kern, uint32_t* o) {
+            size_t smem = (256 / 32 * 257 + 288 + 256 * 16 + 256 / 32 * 512) * 4;
+            cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+            kern<<<sms * 3, 256, smem>>>(keys, o, n, shift);
+          };
+          go(k_rank<256, 16, 7>, ref);
+          go(k_rank<256, 16, 2>, out);
+          cudaMemset(bad, 0, 8);
+          k_cmp<<<sms * 4, 512>>>(ref, out, n, bad);
+          unsigned long long hb = 0; CK(cudaMemcpy(&hb, bad, 8, cudaMemcpyDeviceToHost));
+          printf("order check %-7s shift %2d: returning-atomic rank differs from stable rank at %llu of %zu\n", dname[di], shift, hb, n);
+        }
+        cudaFree(ref); cudaFree(bad);
+      }
+      continue;
       run(k_rank<256, 16, 0>, 256, 16, "match 256x16");
       run(k_rank<256, 16, 2>, 256, 16, "atomic(unstable) 256x16");
       run(k_rank<256, 16, 7>, 256, 16, "cnt+dupmatch 256x16");
-      run(k_rank<512, 16, 7>, 512, 16, "cnt+dupmatch 512x16");
-      run(k_rank<256, 32, 7>, 256, 32, "cnt+dupmatch 256x32");
-      run(k_rank<128, 16, 7>, 128, 16, "cnt+dupmatch 128x16");
-      run(k_rank<256, 8, 7>, 256, 8, "cnt+dupmatch 256x8");
+      run(k_rank<256, 16, 1>, 256, 16, "ballot+lds 256x16");
+      run(k_rank<256, 16, 8>, 256, 16, "ballot+ratom 256x16");
+      run(k_rank<256, 16, 9>, 256, 16, "ballotx+ratom 256x16");
+      run(k_rank<256, 8, 9>, 256, 8, "ballotx+ratom 256x8");
+      run(k_rank<512, 8, 9>, 512, 8, "ballotx+ratom 512x8");
     }
   }
   return 0;

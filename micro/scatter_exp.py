@@ -7,7 +7,7 @@ import sys
 ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
 VARIANTS = {0: "product", 1: "no global stores", 3: "contiguous stores (no scatter)",
             10: "local: balanced kpt", 11: "local: 2 chains/warp", 12: "local: balanced + 2 chains",
-            13: "rank: always match"}
+            }
 
 
 def build():
@@ -15,7 +15,7 @@ def build():
     spec = importlib.util.spec_from_file_location("b", os.path.join(ROOT, "paper_1611_01137_b200", "build.py"))
     b = importlib.util.module_from_spec(spec)
     spec.loader.exec_module(b)
-    for v in VARIANTS:
+    for v in (sys.argv[2:] and map(int, sys.argv[2:])) or VARIANTS:
         b.build(force=True, out=os.path.join(ROOT, "micro", f"libhrs_exp{v}.so"), defines=[f"HRS_EXP={v}"])
 
 
@@ -39,7 +39,11 @@ def run(v):
     per = {}
     for kind, p, ms in recs:
         per.setdefault(f"{kind}{p}", []).append(ms)
-    print(f"exp{v} {VARIANTS[v]:32s} " + " ".join(f"{k2}={sum(x)/len(x):.3f}" for k2, x in sorted(per.items())
+    k64 = k.view(torch.int32).to(torch.int64) & 0xFFFFFFFF
+    sk, si = torch.sort(k64, stable=True)
+    ok = bool(torch.equal(ko.view(torch.int32).to(torch.int64) & 0xFFFFFFFF, sk)) and \
+        bool(torch.equal(vo.view(torch.int32).to(torch.int64), si))
+    print(f"exp{v} {'OK ' if ok else 'BAD'} {VARIANTS[v]:32s} " + " ".join(f"{k2}={sum(x)/len(x):.3f}" for k2, x in sorted(per.items())
                                                  if sum(x) / len(x) > 0.02))
 
 

@@ -46,7 +46,7 @@ def build(force: bool = False, verbose: bool = False, out: str | None = None, de
         return LIB
     cmd = [NVCC, *NVCC_FLAGS, *[f"-D{d}" for d in defines], "-shared", "-o", lib + ".tmp", *sources()]
     res = subprocess.run(cmd, capture_output=True, text=True)
-    log = os.path.join(HERE, "build.log")
+    log = os.path.join(HERE, "build.log") if out is None else lib + ".log"
     with open(log, "w") as f:
         f.write(" ".join(cmd) + "\n" + res.stdout + res.stderr)
     if res.returncode != 0:
