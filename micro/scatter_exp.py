@@ -1,37 +1,40 @@
-"""Time k_scatter variants (HRS_EXP compile flag) on 2^28 u32/u32 uniform pairs.
-Builds are made on the CPU box: python micro/scatter_exp.py build; run on the GPU box."""
+"""Time libhrs variants built with different compile-time defines on 2^28 u32/u32 pairs.
+Builds are made on the CPU box:  python micro/scatter_exp.py build NAME "DEF=1 DEF2=3" ...
+then on the GPU box:             python micro/scatter_exp.py run NAME [dist]"""
 import os
-import subprocess
 import sys
 
 ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
-VARIANTS = {0: "product", 1: "no global stores", 3: "contiguous stores (no scatter)",
-            10: "local: balanced kpt", 11: "local: 2 chains/warp", 12: "local: balanced + 2 chains",
-            }
 
 
-def build():
+def build(name, defs):
     import importlib.util
     spec = importlib.util.spec_from_file_location("b", os.path.join(ROOT, "paper_1611_01137_b200", "build.py"))
     b = importlib.util.module_from_spec(spec)
     spec.loader.exec_module(b)
-    for v in (sys.argv[2:] and map(int, sys.argv[2:])) or VARIANTS:
-        b.build(force=True, out=os.path.join(ROOT, "micro", f"libhrs_exp{v}.so"), defines=[f"HRS_EXP={v}"])
+    b.build(force=True, out=os.path.join(ROOT, "micro", f"libhrs_{name}.so"), defines=defs.split())
 
 
-def run(v):
-    os.environ["HRS_LIB"] = os.path.join(ROOT, "micro", f"libhrs_exp{v}.so")
+def run(name, dist="uniform"):
+    os.environ["HRS_LIB"] = os.path.join(ROOT, "micro", f"libhrs_{name}.so")
     sys.path.insert(0, ROOT)
     import torch
     import gen
     import paper_1611_01137_b200 as hrs
     n = 1 << 28
-    k = gen.keys(n, 32, sys.argv[3] if len(sys.argv) > 3 else "uniform", device="cuda")
+    k = gen.keys(n, 32, dist, device="cuda")
     val = gen.values(n, 32, "index", device="cuda")
     ko, vo = torch.empty_like(k), torch.empty_like(val)
     temp = torch.empty(hrs.temp_bytes(n, 4, 4), dtype=torch.uint8, device="cuda")
     for _ in range(3):
         hrs.sort(k, val, keys_out=ko, values_out=vo, temp=temp)
+    st, en = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+    st.record()
+    for _ in range(10):
+        hrs.sort(k, val, keys_out=ko, values_out=vo, temp=temp)
+    en.record()
+    torch.cuda.synchronize()
+    tot = st.elapsed_time(en) / 10
     hrs.profile_enable(True)
     for _ in range(5):
         hrs.sort(k, val, keys_out=ko, values_out=vo, temp=temp)
@@ -43,12 +46,13 @@ def run(v):
     sk, si = torch.sort(k64, stable=True)
     ok = bool(torch.equal(ko.view(torch.int32).to(torch.int64) & 0xFFFFFFFF, sk)) and \
         bool(torch.equal(vo.view(torch.int32).to(torch.int64), si))
-    print(f"exp{v} {'OK ' if ok else 'BAD'} {VARIANTS[v]:32s} " + " ".join(f"{k2}={sum(x)/len(x):.3f}" for k2, x in sorted(per.items())
-                                                 if sum(x) / len(x) > 0.02))
+    print(f"{name:12s} {dist:8s} {'OK ' if ok else 'BAD'} step={tot:.3f} ms " + " ".join(
+        f"{k2}={sum(x) / len(x):.3f}" for k2, x in sorted(per.items()) if sum(x) / len(x) > 0.02), flush=True)
 
 
 if __name__ == "__main__":
     if sys.argv[1] == "build":
-        build()
+        for i in range(2, len(sys.argv), 2):
+            build(sys.argv[i], sys.argv[i + 1])
     else:
-        run(int(sys.argv[2]))
+        run(sys.argv[2], *(sys.argv[3:4]))

@@ -68,6 +68,17 @@ struct LaunchScope {
 
 constexpr uint32_t DEFAULT_MT_DIV = 4;
 
+// 32-bit-key scatter shape (overridable for experiments, micro/scatter_exp.py)
+#ifndef HRS_SC_KPT
+#define HRS_SC_KPT 13
+#endif
+#ifndef HRS_SC_NBUF
+#define HRS_SC_NBUF 2
+#endif
+#ifndef HRS_SC_MINB
+#define HRS_SC_MINB 3
+#endif
+
 // ------------------------------------------------------------------ compile-time configurations
 
 // scatter: THREADS x KPT records per tile (= the largest KPB); MINB resident CTAs per SM
@@ -75,8 +86,9 @@ template <int KB, int VB>
 struct ScatterCfg {
     static constexpr bool SMALL = (KB == 4 && VB <= 4);
     static constexpr int THREADS = SMALL ? 256 : 512;
-    static constexpr int KPT = SMALL ? 15 : 8;  // 256 x 15: two staging buffers for three CTAs per SM
-    static constexpr int MINB = SMALL ? 3 : 1;
+    static constexpr int KPT = SMALL ? HRS_SC_KPT : 8;  // 256 x 13: two staging buffers + the slot index for three CTAs per SM
+    static constexpr int MINB = SMALL ? HRS_SC_MINB : 1;
+    static constexpr int NBUF = SMALL ? HRS_SC_NBUF : 2;
 };
 constexpr int HIST_THREADS = 512;
 constexpr int HIST_STAGES = 3;
@@ -486,8 +498,8 @@ struct Runner {
         sp.tiles = at<TileDesc>(temp, pl.off_tiles);
         sp.tile_pref = at<uint32_t>(temp, pl.off_tile_pref);
         sp.ctl = at<Ctl>(temp, 0);
-        auto fn = k_scatter<K, V, SC::THREADS, SC::KPT, SC::MINB>;
-        const size_t smem = ScatterSmem<K, V, SC::THREADS, SC::KPT>::bytes;
+        auto fn = k_scatter<K, V, SC::THREADS, SC::KPT, SC::MINB, SC::NBUF>;
+        const size_t smem = ScatterSmem<K, V, SC::THREADS, SC::KPT, SC::NBUF>::bytes;
         int grid = 0;
         hrs_status s = grid_for(fn, SC::THREADS, smem, dev, sms, &grid);
         if (s) return s;

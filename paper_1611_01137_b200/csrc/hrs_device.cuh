@@ -320,39 +320,43 @@ __device__ __forceinline__ void seg_fill_edges(T *sbuf, const T *src, const Seg 
 // ------------------------------------------------------------------ stable block rank
 //
 // The keys a warp holds are in "warp-striped" order (element e of the tile is
-// warp * 32 * kpt + c * 32 + lane).  A stable rank (position among all keys of the
-// tile, ties in element order) is computed in three steps:
-//   1. count: per-(virtual-)warp digit histogram with non-returning shared atomics
-//      (full speed on B200 whatever the skew; profiles/r01_micro_hist.txt);
+// warp * 32 * kpt + c * 32 + lane).  The stable rank of a key (its slot among all
+// keys of the tile, ties in element order) is
+//     start[d] + (keys of digit d in earlier warps) + (keys of digit d before it in its warp),
+// computed in three steps:
+//   1. count: per-warp digit counters in shared memory, one atomic per key;
 //   2. scan: exclusive prefix over the warps per digit and over the digits, folded
 //      into each warp's counters = first slot of the warp's run of each digit;
-//   3. rank: column by column, every lane reads the warp's next free slot of its
-//      digit, adds 1 with a non-returning atomic and reads the counter back: the
-//      difference is the number of lanes of the column with that digit.  Lanes with
-//      duplicates take their order from one match-any over the column where all
-//      other lanes share one dummy value, so its cost depends only on the few
-//      distinct duplicated digits (match-any over 32 distinct values is what makes a
-//      pure match-based multisplit slow on B200; profiles/r01_micro_rank.txt).
-
-// Block-wide stable ranking of the keys of a tile, shared by k_scatter and k_local.
-// Each warp owns `kpt` columns (runtime, <= KPT) of 32 consecutive elements:
-// element e = warp * 32 * kpt + c * 32 + lane.  With VWPW = 2 the warp's columns are
-// split into two halves with separate counters ("virtual warps"), so the two
-// column-by-column counter chains of the rank are independent (ILP 2).  Each warp
-// clears its own counters right after its rank, so the next tile / pass needs no
-// extra barrier.
-template <int THREADS, int KPT, int VWPW>
+//   3. in-warp rank, one of two ways, chosen per warp:
+//      fast  -- the count atomics of step 1 RETURN the old counter value, and that is
+//               taken as the in-warp rank.  It is the stable rank exactly when the
+//               same-address lanes of one atomic instruction are served in lane order
+//               (and a warp's instructions in program order), which B200 does
+//               (profiles/r01_micro_rank_ballot.txt) but PTX leaves unspecified, so
+//               every caller checks the order it produced and redoes the tile with
+//               the exact path if it is not the stable one.  One shared operation
+//               per key besides the count.
+//      exact -- stable by construction: column by column, every lane reads the warp's
+//               next free slot of its digit, adds 1 with a non-returning atomic and
+//               reads the counter back; the difference is the number of lanes of the
+//               column with that digit, and lanes with duplicates take their order
+//               from one match-any over the column where all other lanes share one
+//               dummy value (match-any over 32 distinct values is what makes a pure
+//               match-based multisplit slow on B200; profiles/r01_micro_rank.txt).
+//   Returning atomics serialise same-address lanes, so a warp whose first column shows
+//   heavy digit contention (skewed keys) takes the exact path, where same-address
+//   lanes are cheap.
+template <int THREADS, int KPT>
 struct Ranker {
     static constexpr int W = THREADS / 32;
-    static constexpr int VW = VWPW * W;
-    static constexpr int KH = VWPW == 2 ? (KPT + 1) / 2 : KPT;  // columns of the first half
-    static constexpr size_t cnt_words = static_cast<size_t>(VW) * NBINS;
+    static constexpr size_t cnt_words = static_cast<size_t>(W) * NBINS;
     static constexpr size_t smem_bytes = sizeof(uint32_t) * (cnt_words + 2 * 288);
-    uint32_t *cnt;    // [VW][NBINS]
+    static_assert(32 * KPT < (1 << 16), "the in-warp rank is packed above the digit");
+    uint32_t *cnt;    // [W][NBINS]
     uint32_t *tot;    // [288] digit totals of the tile
     uint32_t *start;  // [288] first slot of each digit (valid after the caller's next barrier)
 
-    __device__ __forceinline__ uint32_t *vcnt(int vw) const { return cnt + vw * NBINS; }
+    __device__ __forceinline__ uint32_t *vcnt(int w) const { return cnt + w * NBINS; }
 
     __device__ __forceinline__ void init(uint32_t *base) {
         cnt = base;
@@ -362,27 +366,46 @@ struct Ranker {
     }
 
     // dg: digits on entry (INVALID_DIGIT for padding), slots on exit.  kpt: active
-    // columns (the same for all warps); active: this warp holds elements.  Contains
-    // two block barriers; the caller needs one more before reading the slots' data
-    // and before reading start[d] = first slot of digit d.
-    __device__ __forceinline__ void rank(uint32_t (&dg)[KPT], int kpt, bool active, uint32_t ltm) {
+    // columns (the same for all warps); active: this warp holds elements.  allow_fast:
+    // the fast in-warp rank may be used (the caller checks the result).  gs (optional,
+    // [RADIX]): gs[d].x holds a per-digit base on entry, {base - start[d], start[d]} on
+    // exit.  Contains two block barriers; start[] and gs are valid after the caller's
+    // next barrier.  Each warp clears its own counters at the end, so the next tile /
+    // pass needs no extra barrier.
+    __device__ __forceinline__ void rank(uint32_t (&dg)[KPT], int kpt, bool active, uint32_t ltm, bool allow_fast,
+                                         uint2 *gs = nullptr) {
         const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
-        uint32_t *ca = vcnt(VWPW * warp);
-        uint32_t *cb = vcnt(VWPW * warp + (VWPW - 1));
-        if (active) {
+        uint32_t *ca = vcnt(warp);
+        bool fast = false;
+        if (active && allow_fast) {
+            // contention probe: equal digits among the 5 butterfly partners of column 0
+            // (a uniform digit gives 0.6 on average over the warp)
+            const uint32_t d0 = dg[0];
+            uint32_t eq = 0;
 #pragma unroll
-            for (int c = 0; c < KPT; ++c)
-                if (c < kpt) atomicAdd(&(c < KH ? ca : cb)[dg[c]], 1u);
+            for (int k = 1; k < 32; k <<= 1) eq += __shfl_xor_sync(0xffffffffu, d0, k) == d0;
+            fast = __reduce_add_sync(0xffffffffu, eq) < 8;
+        }
+        if (active) {
+            if (fast) {
+#pragma unroll
+                for (int c = 0; c < KPT; ++c)
+                    if (c < kpt) dg[c] |= atomicAdd(&ca[dg[c]], 1u) << 16;
+            } else {
+#pragma unroll
+                for (int c = 0; c < KPT; ++c)
+                    if (c < kpt) atomicAdd(&ca[dg[c]], 1u);
+            }
         }
         __syncthreads();
-        // exclusive prefix over the virtual warps per digit, digit totals
+        // exclusive prefix over the warps per digit, digit totals
         for (int d = threadIdx.x; d < NBINS; d += THREADS) {
-            uint32_t v[VW];
+            uint32_t v[W];
 #pragma unroll
-            for (int w = 0; w < VW; ++w) v[w] = vcnt(w)[d];
+            for (int w = 0; w < W; ++w) v[w] = vcnt(w)[d];
             uint32_t run = 0;
 #pragma unroll
-            for (int w = 0; w < VW; ++w) {
+            for (int w = 0; w < W; ++w) {
                 vcnt(w)[d] = run;
                 run += v[w];
             }
@@ -414,48 +437,37 @@ struct Ranker {
                 const int d = lane * PER + i;
                 if (d < NBINS) {
                     ca[d] += run;
-                    if (VWPW == 2) cb[d] += run;
-                    if (warp == 0) start[d] = run;
+                    if (warp == 0) {
+                        start[d] = run;
+                        if (gs != nullptr && d < RADIX) gs[d] = make_uint2(gs[d].x - run, run);
+                    }
                 }
                 run += v[i];
             }
         }
         __syncwarp();
         if (active) {
+            if (fast) {
 #pragma unroll
-            for (int i = 0; i < KH; ++i) {
-                // column i of half A and column KH + i of half B: independent chains
-                const int c1 = KH + i < KPT ? KH + i : KPT - 1;
-                const bool v0 = i < kpt, v1 = VWPW == 2 && (KH + i < KPT) && (KH + i < kpt);
-                const uint32_t d0 = v0 ? dg[i] : 0u;
-                const uint32_t d1 = v1 ? dg[c1] : 0u;
-                const uint32_t p0 = v0 ? ca[d0] : 0u;
-                const uint32_t p1 = v1 ? cb[d1] : 0u;
-                __syncwarp();
-                if (v0) atomicAdd(&ca[d0], 1u);
-                if (v1) atomicAdd(&cb[d1], 1u);
-                __syncwarp();
-                const uint32_t k0 = v0 ? ca[d0] - p0 : 0u;
-                const uint32_t k1 = v1 ? cb[d1] - p1 : 0u;
-                uint32_t r0 = 0, r1 = 0;
-                {
+                for (int c = 0; c < KPT; ++c)
+                    if (c < kpt) dg[c] = ca[dg[c] & 0xFFFFu] + (dg[c] >> 16);
+            } else {
+#pragma unroll
+                for (int c = 0; c < KPT; ++c) {
+                    const bool v0 = c < kpt;
+                    const uint32_t d0 = v0 ? dg[c] : 0u;
+                    const uint32_t p0 = v0 ? ca[d0] : 0u;
+                    __syncwarp();
+                    if (v0) atomicAdd(&ca[d0], 1u);
+                    __syncwarp();
+                    const uint32_t k0 = v0 ? ca[d0] - p0 : 0u;
                     const uint32_t m = __match_any_sync(0xffffffffu, k0 > 1 ? d0 : 0xFFFFFFFFu);
-                    r0 = k0 > 1 ? __popc(m & ltm) : 0u;
+                    if (v0) dg[c] = p0 + (k0 > 1 ? __popc(m & ltm) : 0u);
                 }
-                if (VWPW == 2) {
-                    const uint32_t m = __match_any_sync(0xffffffffu, k1 > 1 ? d1 : 0xFFFFFFFFu);
-                    r1 = k1 > 1 ? __popc(m & ltm) : 0u;
-                }
-                if (v0) dg[i] = p0 + r0;
-                if (v1) dg[c1] = p1 + r1;
             }
         }
         __syncwarp();
-        // clear this warp's counters for the next tile / pass
-        for (int d = lane; d < NBINS; d += 32) {
-            ca[d] = 0;
-            if (VWPW == 2) cb[d] = 0;
-        }
+        for (int d = lane; d < NBINS; d += 32) ca[d] = 0;
     }
 };
 
@@ -961,7 +973,7 @@ struct StageInfo {
     uint64_t offs;
 };
 
-template <typename K, typename V, int THREADS, int KPT>
+template <typename K, typename V, int THREADS, int KPT, int NBUF>
 struct ScatterSmem {
     static constexpr int W = THREADS / 32;
     static constexpr int KPB = THREADS * KPT;
@@ -971,23 +983,26 @@ struct ScatterSmem {
     static constexpr size_t vst_elems = KPB + 16 / sizeof(VT);
     static constexpr size_t off_bar = 0;
     static constexpr size_t off_info = 16;
-    using RK = Ranker<THREADS, KPT, 1>;
-    static constexpr size_t off_rank = align16(off_info + 2 * sizeof(StageInfo));
-    static constexpr size_t off_gbase = align16(off_rank + RK::smem_bytes);
-    static constexpr size_t off_kst = align16(off_gbase + sizeof(uint32_t) * RADIX);
+    using RK = Ranker<THREADS, KPT>;
+    static constexpr size_t off_rank = align16(off_info + NBUF * sizeof(StageInfo));
+    static constexpr size_t off_gs = align16(off_rank + RK::smem_bytes);
+    static constexpr size_t off_sidx = align16(off_gs + sizeof(uint2) * RADIX);
+    static constexpr size_t off_kst = align16(off_sidx + sizeof(uint16_t) * KPB);
     static constexpr size_t kst_bytes = align16(sizeof(K) * kst_elems);
-    static constexpr size_t off_vst = off_kst + 2 * kst_bytes;
+    static constexpr size_t off_vst = off_kst + NBUF * kst_bytes;
     static constexpr size_t vst_bytes = HV ? align16(sizeof(VT) * vst_elems) : 0;
-    static constexpr size_t bytes = off_vst + 2 * vst_bytes;
+    static constexpr size_t bytes = off_vst + NBUF * vst_bytes;
 };
 
-// Two staging buffers: while tile i is ranked, staged back into its own buffer in
-// sorted order (keys and values pass through registers) and stored, tile i + 1 is in
-// flight into the other buffer.
-template <typename K, typename V, int THREADS, int KPT, int MINB>
+// NBUF staging buffers: with two, tile i + 1 is in flight into the other buffer while
+// tile i is ranked and written out; with one, the other resident CTAs cover the load.  The staged keys and values are never moved inside shared
+// memory: the rank produces, for every slot of the sorted tile, the index of the
+// element that goes there (sidx), and the write-out gathers key and value through it.
+template <typename K, typename V, int THREADS, int KPT, int MINB, int NBUF>
 __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
     pdl_wait();
-    using L = ScatterSmem<K, V, THREADS, KPT>;
+    static_assert(NBUF == 1 || NBUF == 2, "one or two staging buffers");
+    using L = ScatterSmem<K, V, THREADS, KPT, NBUF>;
     constexpr bool HV = HasVal<V>::value;
     using VT = ValT<V>;
     extern __shared__ __align__(16) unsigned char smem[];
@@ -995,7 +1010,9 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
     StageInfo *info = reinterpret_cast<StageInfo *>(smem + L::off_info);
     typename L::RK ranker;
     ranker.init(reinterpret_cast<uint32_t *>(smem + L::off_rank));
-    uint32_t *gbase = reinterpret_cast<uint32_t *>(smem + L::off_gbase);
+    // gs[d] = {destination of slot 0 of digit d relative to the bucket, first slot of d}
+    uint2 *gs = reinterpret_cast<uint2 *>(smem + L::off_gs);
+    uint16_t *sidx = reinterpret_cast<uint16_t *>(smem + L::off_sidx);
     auto kst = [&](int s) { return reinterpret_cast<K *>(smem + L::off_kst + s * L::kst_bytes); };
     auto vst = [&](int s) { return reinterpret_cast<VT *>(smem + L::off_vst + s * L::vst_bytes); };
 
@@ -1040,11 +1057,9 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
         if (HV) seg_issue(vst(s), vin + td.offs, sv, &bar[s], pol);
     };
     if (tid == 0) {
-        mbar_init(&bar[0], 1);
-        mbar_init(&bar[1], 1);
+        for (int b = 0; b < NBUF; ++b) mbar_init(&bar[b], 1);
         mbar_fence_init();
-        issue(0, atomicAdd(&prm.ctl->claim[prm.p], 1u));
-        issue(1, atomicAdd(&prm.ctl->claim[prm.p], 1u));
+        for (int b = 0; b < NBUF; ++b) issue(b, atomicAdd(&prm.ctl->claim[prm.p], 1u));
     }
     __syncthreads();
 
@@ -1054,26 +1069,28 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
     // per-digit destination base of a tile, relative to its bucket: sub-bucket start
     // + counts of the earlier tiles of the bucket (tile order = memory order: stable).
     // Loaded one tile ahead so the global loads overlap the previous tile.
-    auto tile_base = [&](const StageInfo &in) -> uint32_t {
-        uint32_t b = prm.sub_rel[static_cast<uint64_t>(in.bucket) * RADIX + tid] +
-                     prm.tile_pref[static_cast<uint64_t>(in.tile) * RADIX + tid];
-        if (in.carry_row != EMPTY_RANGE) b += prm.carry[static_cast<uint64_t>(in.carry_row) * RADIX + tid];
-        return b;
-    };
-    uint32_t rbase = 0;
+    // The three terms are loaded a whole tile ahead (two buffers) or before the wait
+    // for the tile's data (one buffer) and added only when needed.
+    uint32_t m0 = 0, m1 = 0, m2 = 0;
     uint64_t boffs = 0;
-    if (tid < RADIX && info[0].valid) {
-        rbase = tile_base(info[0]);
-        boffs = prm.buckets[info[0].bucket].offs;
-    }
+    auto meta_load = [&](const StageInfo &in) {
+        if (tid < RADIX && in.valid) {
+            m0 = prm.sub_rel[static_cast<uint64_t>(in.bucket) * RADIX + tid];
+            m1 = prm.tile_pref[static_cast<uint64_t>(in.tile) * RADIX + tid];
+            m2 = in.carry_row != EMPTY_RANGE ? prm.carry[static_cast<uint64_t>(in.carry_row) * RADIX + tid] : 0u;
+            boffs = prm.buckets[in.bucket].offs;
+        }
+    };
+    meta_load(info[0]);
     for (uint32_t it = 0;; ++it) {
-        const int s = static_cast<int>(it & 1u);
-        const uint32_t par = (it >> 1) & 1u;
+        const int s = static_cast<int>(it % NBUF);
+        const uint32_t par = (it / NBUF) & 1u;
         const StageInfo in = info[s];
         if (!in.valid) break;
         const uint32_t count = in.count;
-        const uint32_t dbase = rbase;
+        const uint32_t rbase = m0 + m1 + m2;
         const uint64_t tboffs = tid < RADIX ? boffs : prm.buckets[in.bucket].offs;
+        if (tid < RADIX) gs[tid].x = rbase;     // rank() turns it into {base - start, start}
         Seg sk, sv;
         sk.pad = in.kpad;
         sk.i0 = in.k0;
@@ -1089,110 +1106,85 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
         // full tiles with an aligned interior take the predicate-free path
         const bool full = count == static_cast<uint32_t>(L::KPB) && sk.i0 == 0 && sk.i1 == count &&
                           (!HV || (sv.i0 == 0 && sv.i1 == count));
+        const K *const kb = ks + sk.pad;  // element i of the tile (after the edges are filled)
+        const VT *const vb = HV ? vs + sv.pad : nullptr;
         auto body = [&](auto full_tag) {
             constexpr bool FULL = decltype(full_tag)::value;
-            // ---- keys into registers (warp-striped) and digits
-            K key[KPT];
+            if (!FULL) {
+                // unaligned head / tail into shared memory (read by the gathers, after barriers)
+                seg_fill_edges<K, THREADS>(ks, ksrc, sk, count);
+                if (HV) seg_fill_edges<VT, THREADS>(vs, vsrc, sv, count);
+            }
+            K *const kdst = kout + tboffs;
+            VT *const vdst = HV ? vout + tboffs : nullptr;
+            // slot j of the sorted tile holds element sidx[j]: gather, store at its
+            // destination, and (check) test that slot j - 1, when it holds the same digit,
+            // holds an earlier element -- the complete stability condition
+            auto write_out = [&](bool check) -> bool {
+                bool bad = false;
+#pragma unroll
+                for (int c = 0; c < KPT; ++c) {
+                    const uint32_t j = c * THREADS + tid;
+                    if (FULL || j < count) {
+                        const uint32_t i = sidx[j];
+                        const K k = kb[i];
+                        const uint2 g = gs[digit_of(k, lo, mask)];
+                        const uint32_t pos = g.x + j;
+                        kdst[pos] = k;
+                        if (HV) vdst[pos] = vb[i];
+                        if (check && j > g.y) bad |= sidx[j - 1] > i;
+                    }
+                }
+                return bad;
+            };
+            // ---- digits (warp-striped: element e = warp * 32 * KPT + c * 32 + lane)
             uint32_t dg[KPT];
 #pragma unroll
             for (int c = 0; c < KPT; ++c) {
                 const uint32_t e = wbase + c * 32 + lane;
-                if (FULL || e < count) {
-                    key[c] = FULL ? ks[e] : seg_get(ks, ksrc, sk, e);
-                    dg[c] = digit_of(key[c], lo, mask);
-                } else {
-                    dg[c] = INVALID_DIGIT;
-                }
+                if (FULL || e < count) dg[c] = digit_of(FULL ? ks[e] : seg_get(ks, ksrc, sk, e), lo, mask);
+                else dg[c] = INVALID_DIGIT;
             }
-            // ---- stable rank
-            ranker.rank(dg, KPT, FULL || wbase < count, ltm);
-            // ---- values into registers, then everything back into the staging buffer
-            //      in slot order (slot j at index j, the pad is no longer needed)
-            if (HV) {
-                VT val[KPT];
+            const bool active = FULL || wbase < count;
+            ranker.rank(dg, KPT, active, ltm, true, gs);
+            // the next tile's metadata (info[s ^ 1], published before the rank's barriers)
+            if (NBUF == 2) meta_load(info[s ^ 1]);
+#pragma unroll
+            for (int c = 0; c < KPT; ++c) {
+                const uint32_t e = wbase + c * 32 + lane;
+                if (FULL || e < count) sidx[dg[c]] = static_cast<uint16_t>(e);
+            }
+            __syncthreads();
+            const bool bad = write_out(true);
+            if (__syncthreads_or(bad)) {
+                // the atomics did not serve the lanes in order: redo the tile with the
+                // rank that is stable by construction (same digit starts, so gs holds)
 #pragma unroll
                 for (int c = 0; c < KPT; ++c) {
                     const uint32_t e = wbase + c * 32 + lane;
-                    if (FULL || e < count) val[c] = FULL ? vs[e] : seg_get(vs, vsrc, sv, e);
+                    dg[c] = (FULL || e < count) ? digit_of(kb[e], lo, mask) : INVALID_DIGIT;
+                }
+                ranker.rank(dg, KPT, active, ltm, false);
+#pragma unroll
+                for (int c = 0; c < KPT; ++c) {
+                    const uint32_t e = wbase + c * 32 + lane;
+                    if (FULL || e < count) sidx[dg[c]] = static_cast<uint16_t>(e);
                 }
                 __syncthreads();
-                // destination of slot j holding digit d: bucket offset + gbase[d] + j
-                if (tid < RADIX) gbase[tid] = dbase - ranker.start[tid];
-#pragma unroll
-                for (int c = 0; c < KPT; ++c) {
-                    const uint32_t e = wbase + c * 32 + lane;
-                    if (FULL || e < count) {
-                        ks[dg[c]] = key[c];
-                        vs[dg[c]] = val[c];
-                    }
-                }
-            } else {
+                write_out(false);
                 __syncthreads();
-                if (tid < RADIX) gbase[tid] = dbase - ranker.start[tid];
-#pragma unroll
-                for (int c = 0; c < KPT; ++c) {
-                    const uint32_t e = wbase + c * 32 + lane;
-                    if (FULL || e < count) ks[dg[c]] = key[c];
-                }
             }
         };
         if (full) body(std::true_type{});
         else body(std::false_type{});
-        {
-            // the next tile's metadata (info[s ^ 1] was published before the barriers above)
-            const StageInfo nx = info[s ^ 1];
-            if (tid < RADIX && nx.valid) {
-                rbase = tile_base(nx);
-                boffs = prm.buckets[nx.bucket].offs;
-            }
-        }
-        __syncthreads();
-        // ---- write-combined stores: consecutive slots of a digit run are consecutive addresses
-        if (HRS_EXP == 1) {
-            K acc = 0;
-#pragma unroll
-            for (int c = 0; c < KPT; ++c) acc ^= ks[c * THREADS + tid] ^ static_cast<K>(gbase[c] + tboffs);
-            if (acc == static_cast<K>(0x12345678u)) kout[0] = acc;
-        } else if (HRS_EXP == 3) {
-            // contiguous copy of the staged tile (no scatter)
-#pragma unroll
-            for (int c = 0; c < KPT; ++c) {
-                const uint32_t j = c * THREADS + tid;
-                if (j < count) {
-                    kout[in.offs + j] = ks[j];
-                    if (HV) vout[in.offs + j] = vs[j];
-                }
-            }
-        } else {
-            K *const kdst = kout + tboffs;
-            VT *const vdst = HV ? vout + tboffs : nullptr;
-            if (count == static_cast<uint32_t>(L::KPB)) {
-#pragma unroll
-                for (int c = 0; c < KPT; ++c) {
-                    const uint32_t j = c * THREADS + tid;
-                    const K k = ks[j];
-                    const uint32_t pos = gbase[digit_of(k, lo, mask)] + j;
-                    kdst[pos] = k;
-                    if (HV) vdst[pos] = vs[j];
-                }
-            } else {
-#pragma unroll
-                for (int c = 0; c < KPT; ++c) {
-                    const uint32_t j = c * THREADS + tid;
-                    if (j < count) {
-                        const K k = ks[j];
-                        const uint32_t pos = gbase[digit_of(k, lo, mask)] + j;
-                        kdst[pos] = k;
-                        if (HV) vdst[pos] = vs[j];
-                    }
-                }
-            }
-        }
-        __syncthreads();
-        // ---- the staging buffer is free again: claim the next tile into it
+        // ---- the staging buffer is free again (barrier above): claim the next tile into it
         if (tid == 0) {
             fence_proxy_async();
             issue(s, atomicAdd(&prm.ctl->claim[prm.p], 1u));
+        }
+        if (NBUF == 1) {
+            __syncthreads();  // info[0] of the next tile
+            meta_load(info[0]);
         }
     }
 }
@@ -1240,8 +1232,7 @@ struct LocalSmem {
     static constexpr bool HV = HasVal<V>::value;
     static constexpr size_t off_bar = 0;
     static constexpr size_t off_info = align16(sizeof(uint64_t) * NSTAGE);
-    static constexpr int VWPW = (HRS_EXP == 11 || HRS_EXP == 12) ? 2 : 1;
-    using RK = Ranker<THREADS, KPT, VWPW>;
+    using RK = Ranker<THREADS, KPT>;
     static constexpr size_t off_rank = align16(off_info + sizeof(uint32_t) * 16 * (NSTAGE + 1));
     static constexpr size_t off_red = align16(off_rank + RK::smem_bytes);
     // composite buffer (or the 16-bit index buffer of the pair path)
@@ -1446,28 +1437,59 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
             for (int c = 0; c < KPT; ++c)
                 cv[c] = ((static_cast<CT>(key[c] >> tlo) & tmask) << IB) | static_cast<CT>(idx[c]);
             const CT cdiff = (static_cast<CT>(diff >> tlo) & tmask) << IB;
-            for (int lo = IB; lo < IB + tb; lo += 8) {
-                const int width = min(8, IB + tb - lo);
-                const uint32_t mask = (1u << width) - 1u;
-                if ((static_cast<uint32_t>(cdiff >> lo) & mask) == 0) continue;  // constant digit: identity pass
-                moved = true;
-                // padding slots (e >= count) carry digit 256: they rank after every record
-                // and end up in slots >= count again, so no per-element guards are needed
-                uint32_t dg[KPT];
-#pragma unroll
-                for (int c = 0; c < KPT; ++c)
-                    dg[c] = (wbase + c * 32 + lane) < count ? digit_of(cv[c], lo, mask) : INVALID_DIGIT;
-                ranker.rank(dg, kpt, active, ltm);
-                if (active) {
+            // LSD passes over the composites, with the fast rank first (fast = true)
+            auto passes = [&](bool fast) {
+                for (int lo = IB; lo < IB + tb; lo += 8) {
+                    const int width = min(8, IB + tb - lo);
+                    const uint32_t mask = (1u << width) - 1u;
+                    if ((static_cast<uint32_t>(cdiff >> lo) & mask) == 0) continue;  // constant digit: identity pass
+                    moved = true;
+                    // padding slots (e >= count) carry digit 256: they rank after every record
+                    // and end up in slots >= count again, so no per-element guards are needed
+                    uint32_t dg[KPT];
 #pragma unroll
                     for (int c = 0; c < KPT; ++c)
-                        if (!BAL || c < kpt) comp[dg[c]] = cv[c];
+                        dg[c] = (wbase + c * 32 + lane) < count ? digit_of(cv[c], lo, mask) : INVALID_DIGIT;
+                    ranker.rank(dg, kpt, active, ltm, fast);
+                    if (active) {
+#pragma unroll
+                        for (int c = 0; c < KPT; ++c)
+                            if (!BAL || c < kpt) comp[dg[c]] = cv[c];
+                    }
+                    __syncthreads();
+                    if (active) {
+#pragma unroll
+                        for (int c = 0; c < KPT; ++c)
+                            if (!BAL || c < kpt) cv[c] = comp[wbase + c * 32 + lane];
+                    }
                 }
-                __syncthreads();
+            };
+            passes(true);
+            if (moved) {
+                // the composites are distinct (index field), so the passes were all stable
+                // iff they end strictly increasing; otherwise put every composite back at
+                // its index and redo the passes with the rank that is stable by construction
+                bool bad = false;
                 if (active) {
 #pragma unroll
-                    for (int c = 0; c < KPT; ++c)
-                        if (!BAL || c < kpt) cv[c] = comp[wbase + c * 32 + lane];
+                    for (int c = 0; c < KPT; ++c) {
+                        const uint32_t e = wbase + c * 32 + lane;
+                        if ((!BAL || c < kpt) && e > 0 && e < count) bad |= comp[e - 1] >= cv[c];
+                    }
+                }
+                if (__syncthreads_or(bad)) {
+                    if (active) {
+#pragma unroll
+                        for (int c = 0; c < KPT; ++c)
+                            if (!BAL || c < kpt) comp[static_cast<uint32_t>(cv[c]) & ((1u << IB) - 1u)] = cv[c];
+                    }
+                    __syncthreads();
+                    if (active) {
+#pragma unroll
+                        for (int c = 0; c < KPT; ++c)
+                            if (!BAL || c < kpt) cv[c] = comp[wbase + c * 32 + lane];
+                    }
+                    passes(false);
                 }
             }
             const K *const ksp = ks + sk.pad;
@@ -1563,7 +1585,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
 #pragma unroll
                 for (int c = 0; c < KPT; ++c)
                     dg[c] = (wbase + c * 32 + lane) < count ? digit_of(key[c], lo, mask) : INVALID_DIGIT;
-                ranker.rank(dg, kpt, active, ltm);
+                ranker.rank(dg, kpt, active, ltm, false);
                 if (active) {
 #pragma unroll
                     for (int c = 0; c < KPT; ++c) {
