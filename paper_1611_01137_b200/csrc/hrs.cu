@@ -90,9 +90,14 @@ struct ScatterCfg {
     static constexpr int MINB = SMALL ? HRS_SC_MINB : 1;
     static constexpr int NBUF = SMALL ? HRS_SC_NBUF : 2;
 };
-constexpr int HIST_THREADS = 512;
-constexpr int HIST_STAGES = 3;
-constexpr int HIST_CAP = 4096;  // >= every ScatterCfg KPB
+#ifndef HRS_HIST_THREADS
+#define HRS_HIST_THREADS 256
+#endif
+#ifndef HRS_HIST_STAGES
+#define HRS_HIST_STAGES 3
+#endif
+constexpr int HIST_THREADS = HRS_HIST_THREADS;
+constexpr int HIST_STAGES = HRS_HIST_STAGES;
 constexpr int CLASSIFY_THREADS = 256;
 constexpr uint32_t RANGE_MAX = 1024;  // >= SMs x resident scatter CTAs per SM
 constexpr size_t SMEM_LIMIT = 227 * 1024;
@@ -383,6 +388,8 @@ template <typename K, typename V>
 struct Runner {
     static constexpr int KB = sizeof(K);
     static constexpr int VB = HasVal<V>::value ? sizeof(V) : 0;
+    // histogram staging = one scatter tile (the largest KPB of this key/value type)
+    static constexpr int HIST_CAP = ScatterCfg<KB, VB>::THREADS * ScatterCfg<KB, VB>::KPT;
     using SC = ScatterCfg<KB, (VB == 0 ? 4 : VB)>;
 
     static hrs_status init(const Plan &pl, void *temp, cudaStream_t st, int sms, int root_class, int counting) {
@@ -418,6 +425,7 @@ struct Runner {
     static hrs_status hist(const Plan &pl, void *temp, cudaStream_t st, int dev, int sms, int p, const void *xin,
                            uint32_t G) {
         HistParams hp;
+        hp.n = pl.n;
         hp.keys = xin;
         hp.p = p;
         hp.lo = pl.lo[p - 1];
@@ -485,6 +493,7 @@ struct Runner {
     static hrs_status scatter(const Plan &pl, void *temp, cudaStream_t st, int dev, int sms, int p, const void *kin,
                               void *kout, const void *vin, void *vout, uint32_t G) {
         ScatterParams sp;
+        sp.n = pl.n;
         sp.keys_in = kin;
         sp.keys_out = kout;
         sp.vals_in = vin;
@@ -518,6 +527,7 @@ struct Runner {
         } else {
             using LC = LocalCfg<C>;
             LocalParams lp;
+            lp.n = pl.n;
             lp.src_keys[SRC_IN] = kin;
             lp.src_keys[SRC_AUX] = at<void>(temp, pl.off_auxk);
             lp.src_keys[SRC_OUT] = kout;

@@ -277,21 +277,30 @@ __device__ __forceinline__ void bulk_g2s(void *dst, const void *src, uint32_t by
         : "memory");
 }
 
-// A staged segment of `count` elements starting at global `src`: element i lives in
-// shared memory at sbuf[pad + i] for i in [i0, i1) (the 16-byte aligned interior the
-// bulk copy moved); the unaligned head [0, i0) and tail [i1, count) stay in global.
+// A staged segment of `count` elements starting at global `src`, inside a buffer
+// [base, limit): one bulk copy moves the 16-byte aligned SUPERSET of the segment (up to
+// 12 bytes of the neighbouring segments on each side, which are never used), clipped
+// to the buffer, so the unaligned head and tail need no separate global loads.  Element
+// i lives in shared memory at sbuf[pad + i] for i in [i0, i1) (i0 <= 0 and i1 >= count
+// unless the clip to the buffer cut the copy); elements outside stay in global memory.
+// The staging buffer needs room for count + 2 * 16 / sizeof(T) elements.
 struct Seg {
-    uint32_t pad, i0, i1;
+    uint32_t pad;
+    int32_t i0, i1;
 };
 template <typename T>
-__device__ __forceinline__ uint32_t seg_plan(const T *src, uint32_t count, Seg &sg) {
+__device__ __forceinline__ uint32_t seg_plan(const T *src, uint32_t count, const T *base, const T *limit, Seg &sg) {
     const uintptr_t a = reinterpret_cast<uintptr_t>(src);
     sg.pad = static_cast<uint32_t>((a & 15) / sizeof(T));
-    const uintptr_t lo = (a + 15) & ~uintptr_t(15);
-    const uintptr_t hi = (a + static_cast<uintptr_t>(count) * sizeof(T)) & ~uintptr_t(15);
-    if (hi > lo) {
-        sg.i0 = static_cast<uint32_t>((lo - a) / sizeof(T));
-        sg.i1 = static_cast<uint32_t>((hi - a) / sizeof(T));
+    uintptr_t lo = a & ~uintptr_t(15);
+    const uintptr_t b16 = (reinterpret_cast<uintptr_t>(base) + 15) & ~uintptr_t(15);
+    if (lo < b16) lo = b16;
+    uintptr_t hi = (a + static_cast<uintptr_t>(count) * sizeof(T) + 15) & ~uintptr_t(15);
+    const uintptr_t l16 = reinterpret_cast<uintptr_t>(limit) & ~uintptr_t(15);
+    if (hi > l16) hi = l16;
+    if (count > 0 && hi > lo) {
+        sg.i0 = static_cast<int32_t>((static_cast<intptr_t>(lo) - static_cast<intptr_t>(a)) / static_cast<intptr_t>(sizeof(T)));
+        sg.i1 = static_cast<int32_t>((static_cast<intptr_t>(hi) - static_cast<intptr_t>(a)) / static_cast<intptr_t>(sizeof(T)));
         return static_cast<uint32_t>(hi - lo);
     }
     sg.i0 = sg.i1 = 0;
@@ -300,19 +309,26 @@ __device__ __forceinline__ uint32_t seg_plan(const T *src, uint32_t count, Seg &
 template <typename T>
 __device__ __forceinline__ void seg_issue(T *sbuf, const T *src, const Seg &sg, uint64_t *bar, uint64_t pol) {
     if (sg.i1 > sg.i0)
-        bulk_g2s(sbuf + sg.pad + sg.i0, src + sg.i0, (sg.i1 - sg.i0) * static_cast<uint32_t>(sizeof(T)), bar, pol);
+        bulk_g2s(sbuf + (static_cast<int32_t>(sg.pad) + sg.i0), src + sg.i0,
+                 static_cast<uint32_t>(sg.i1 - sg.i0) * static_cast<uint32_t>(sizeof(T)), bar, pol);
+}
+// every element of the segment is in shared memory
+__device__ __forceinline__ bool seg_full(const Seg &sg, uint32_t count) {
+    return sg.i0 <= 0 && sg.i1 >= static_cast<int32_t>(count);
 }
 template <typename T>
 __device__ __forceinline__ T seg_get(const T *sbuf, const T *src, const Seg &sg, uint32_t i) {
-    return (i >= sg.i0 && i < sg.i1) ? sbuf[sg.pad + i] : src[i];
+    return (static_cast<int32_t>(i) >= sg.i0 && static_cast<int32_t>(i) < sg.i1) ? sbuf[sg.pad + i] : src[i];
 }
-// copy the unaligned head/tail into the staging buffer so sbuf[pad + i] is valid for all i
+// copy the elements the bulk copy did not cover into the staging buffer, so
+// sbuf[pad + i] is valid for all i < count (only segments at the ends of the buffer)
 template <typename T, int THREADS>
 __device__ __forceinline__ void seg_fill_edges(T *sbuf, const T *src, const Seg &sg, uint32_t count) {
-    const uint32_t nhead = sg.i1 > sg.i0 ? sg.i0 : count;
-    const uint32_t ntail = sg.i1 > sg.i0 ? count - sg.i1 : 0;
-    for (uint32_t j = threadIdx.x; j < nhead + ntail; j += THREADS) {
-        const uint32_t i = j < nhead ? j : sg.i1 + (j - nhead);
+    if (seg_full(sg, count)) return;
+    const uint32_t h = sg.i1 > sg.i0 ? static_cast<uint32_t>(max(sg.i0, 0)) : count;     // head [0, h)
+    const uint32_t t = sg.i1 > sg.i0 ? static_cast<uint32_t>(min(sg.i1, static_cast<int32_t>(count))) : count;  // tail [t, count)
+    for (uint32_t j = threadIdx.x; j < h + (count - t); j += THREADS) {
+        const uint32_t i = j < h ? j : t + (j - h);
         sbuf[sg.pad + i] = src[i];
     }
 }
@@ -543,6 +559,7 @@ __global__ void k_fill_u64(uint64_t *p, uint64_t n, uint64_t v) {
 
 struct HistParams {
     const void *keys;  // X_{p-1}
+    uint64_t n;        // elements of the buffer
     int p;
     int lo;
     uint32_t mask;
@@ -563,7 +580,7 @@ struct HistSmem {
     static constexpr size_t off_info = align16(sizeof(uint64_t) * NSTAGE);
     static constexpr size_t off_wh = align16(off_info + sizeof(uint32_t) * 8 * NSTAGE);
     static constexpr size_t off_stage = align16(off_wh + sizeof(uint32_t) * 2 * RADIX);
-    static constexpr size_t stage_elems = CAP + 16 / sizeof(K);
+    static constexpr size_t stage_elems = CAP + 32 / sizeof(K);
     static constexpr size_t bytes = off_stage + NSTAGE * align16(sizeof(K) * stage_elems);
 };
 
@@ -571,7 +588,7 @@ template <typename K, int THREADS, int NSTAGE, int CAP>
 __global__ void __launch_bounds__(THREADS) k_hist(HistParams prm) {
     pdl_wait();
     using L = HistSmem<K, THREADS, NSTAGE, CAP>;
-    constexpr int W = THREADS / 32;
+    static_assert(THREADS >= RADIX, "one thread per digit for the tile prefixes");
     constexpr int VK = 16 / sizeof(K);
     extern __shared__ __align__(16) unsigned char smem[];
     uint64_t *bar = reinterpret_cast<uint64_t *>(smem + L::off_bar);
@@ -604,12 +621,12 @@ __global__ void __launch_bounds__(THREADS) k_hist(HistParams prm) {
         const uint64_t o = cur.offs();
         const uint32_t cnt = cur.count();
         Seg sg;
-        const uint32_t bytes = seg_plan(keys + o, cnt, sg);
+        const uint32_t bytes = seg_plan(keys + o, cnt, keys, keys + prm.n, sg);
         in[1] = cnt;
         in[2] = cur.b;
         in[3] = sg.pad;
-        in[4] = sg.i0;
-        in[5] = sg.i1;
+        in[4] = static_cast<uint32_t>(sg.i0);
+        in[5] = static_cast<uint32_t>(sg.i1);
         in[6] = cur.last_of_bucket() || cur.t + 1 == te;
         in[7] = cur.t;
         offs_of[s] = o;
@@ -637,8 +654,8 @@ __global__ void __launch_bounds__(THREADS) k_hist(HistParams prm) {
         const bool flush = in[6] != 0;
         Seg sg;
         sg.pad = in[3];
-        sg.i0 = in[4];
-        sg.i1 = in[5];
+        sg.i0 = static_cast<int32_t>(in[4]);
+        sg.i1 = static_cast<int32_t>(in[5]);
         const uint64_t toffs = offs_of[s];
         const K *src = keys + toffs;
         // one block histogram per tile, double-buffered: the counts of tile i are read
@@ -657,22 +674,41 @@ __global__ void __launch_bounds__(THREADS) k_hist(HistParams prm) {
         }
         mbar_wait(&bar[s], par);
         const K *sb = stage(s);
-        // 16-byte vectors over the staged interior
-        const uint32_t nvec = (sg.i1 - sg.i0) / VK;
-        const uint4 *vb = reinterpret_cast<const uint4 *>(sb + sg.pad + sg.i0);
+        // 16-byte vectors over the staged superset: vector v holds elements ibase + v*VK
+        // .. + VK - 1 (element i = position - pad); the vectors wholly inside [0, count)
+        // are counted without checks, the (at most two) partial edge vectors per element
+        if (sg.i1 > sg.i0) {
+            const int32_t q0 = (static_cast<int32_t>(sg.pad) + sg.i0) / VK;
+            const int32_t nq = (sg.i1 - sg.i0) / VK;
+            const uint4 *vb = reinterpret_cast<const uint4 *>(sb) + q0;
+            const int32_t ibase = q0 * VK - static_cast<int32_t>(sg.pad);
+            const int32_t vlo = ibase < 0 ? 1 : 0;
+            const int32_t vhi = min(nq, (static_cast<int32_t>(count) - ibase) / VK);
 #pragma unroll 4
-        for (uint32_t v = tid; v < nvec; v += THREADS) {
-            const uint4 w = vb[v];
-            const K *kk = reinterpret_cast<const K *>(&w);
+            for (int32_t v = vlo + tid; v < vhi; v += THREADS) {
+                const uint4 w = vb[v];
+                const K *kk = reinterpret_cast<const K *>(&w);
 #pragma unroll
-            for (int j = 0; j < VK; ++j) atomicAdd(&my[digit_of(kk[j], prm.lo, prm.mask)], 1u);
+                for (int j = 0; j < VK; ++j) atomicAdd(&my[digit_of(kk[j], prm.lo, prm.mask)], 1u);
+            }
+            // edge vectors: v = 0 when it starts before element 0, v = vhi when partial
+            const int32_t ve = tid == 0 ? (vlo ? 0 : -1) : (tid == 1 && vhi < nq && vhi >= vlo ? vhi : -1);
+            if (ve >= 0) {
+                const uint4 w = vb[ve];
+                const K *kk = reinterpret_cast<const K *>(&w);
+                const int32_t i = ibase + ve * VK;
+#pragma unroll
+                for (int j = 0; j < VK; ++j)
+                    if (i + j >= 0 && i + j < static_cast<int32_t>(count))
+                        atomicAdd(&my[digit_of(kk[j], prm.lo, prm.mask)], 1u);
+            }
         }
-        // unaligned head / tail straight from global
-        {
-            const uint32_t nhead = sg.i1 > sg.i0 ? sg.i0 : count;
-            const uint32_t ntail = sg.i1 > sg.i0 ? count - sg.i1 : 0;
-            for (uint32_t j = tid; j < nhead + ntail; j += THREADS) {
-                const uint32_t i = j < nhead ? j : sg.i1 + (j - nhead);
+        // elements the copy did not cover (segments at the ends of the buffer) from global
+        if (!seg_full(sg, count)) {
+            const uint32_t h = sg.i1 > sg.i0 ? static_cast<uint32_t>(max(sg.i0, 0)) : count;
+            const uint32_t tl = sg.i1 > sg.i0 ? static_cast<uint32_t>(min(sg.i1, static_cast<int32_t>(count))) : count;
+            for (uint32_t j = tid; j < h + (count - tl); j += THREADS) {
+                const uint32_t i = j < h ? j : tl + (j - h);
                 atomicAdd(&my[digit_of(src[i], prm.lo, prm.mask)], 1u);
             }
         }
@@ -953,6 +989,7 @@ __global__ void __launch_bounds__(THREADS) k_classify(ClassifyParams prm) {
 // ------------------------------------------------------------------ scatter
 
 struct ScatterParams {
+    uint64_t n;  // elements of the buffers
     const void *keys_in;
     void *keys_out;
     const void *vals_in;
@@ -979,8 +1016,8 @@ struct ScatterSmem {
     static constexpr int KPB = THREADS * KPT;
     using VT = ValT<V>;
     static constexpr bool HV = HasVal<V>::value;
-    static constexpr size_t kst_elems = KPB + 16 / sizeof(K);
-    static constexpr size_t vst_elems = KPB + 16 / sizeof(VT);
+    static constexpr size_t kst_elems = KPB + 32 / sizeof(K);
+    static constexpr size_t vst_elems = KPB + 32 / sizeof(VT);
     static constexpr size_t off_bar = 0;
     static constexpr size_t off_info = 16;
     using RK = Ranker<THREADS, KPT>;
@@ -1042,15 +1079,15 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
         in.offs = td.offs;
         in.tile = t;
         Seg sk, sv;
-        uint32_t bytes = seg_plan(kin + td.offs, td.count, sk);
+        uint32_t bytes = seg_plan(kin + td.offs, td.count, kin, kin + prm.n, sk);
         in.kpad = sk.pad;
-        in.k0 = sk.i0;
-        in.k1 = sk.i1;
+        in.k0 = static_cast<uint32_t>(sk.i0);
+        in.k1 = static_cast<uint32_t>(sk.i1);
         if (HV) {
-            bytes += seg_plan(vin + td.offs, td.count, sv);
+            bytes += seg_plan(vin + td.offs, td.count, vin, vin + prm.n, sv);
             in.vpad = sv.pad;
-            in.v0 = sv.i0;
-            in.v1 = sv.i1;
+            in.v0 = static_cast<uint32_t>(sv.i0);
+            in.v1 = static_cast<uint32_t>(sv.i1);
         }
         mbar_arrive_expect_tx(&bar[s], bytes);
         seg_issue(kst(s), kin + td.offs, sk, &bar[s], pol);
@@ -1093,19 +1130,18 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
         if (tid < RADIX) gs[tid].x = rbase;     // rank() turns it into {base - start, start}
         Seg sk, sv;
         sk.pad = in.kpad;
-        sk.i0 = in.k0;
-        sk.i1 = in.k1;
+        sk.i0 = static_cast<int32_t>(in.k0);
+        sk.i1 = static_cast<int32_t>(in.k1);
         sv.pad = in.vpad;
-        sv.i0 = in.v0;
-        sv.i1 = in.v1;
+        sv.i0 = static_cast<int32_t>(in.v0);
+        sv.i1 = static_cast<int32_t>(in.v1);
         const K *ksrc = kin + in.offs;
         const VT *vsrc = HV ? vin + in.offs : nullptr;
         K *ks = kst(s);
         VT *vs = HV ? vst(s) : nullptr;
         mbar_wait(&bar[s], par);
         // full tiles with an aligned interior take the predicate-free path
-        const bool full = count == static_cast<uint32_t>(L::KPB) && sk.i0 == 0 && sk.i1 == count &&
-                          (!HV || (sv.i0 == 0 && sv.i1 == count));
+        const bool full = count == static_cast<uint32_t>(L::KPB) && seg_full(sk, count) && (!HV || seg_full(sv, count));
         const K *const kb = ks + sk.pad;  // element i of the tile (after the edges are filled)
         const VT *const vb = HV ? vs + sv.pad : nullptr;
         auto body = [&](auto full_tag) {
@@ -1142,7 +1178,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
 #pragma unroll
             for (int c = 0; c < KPT; ++c) {
                 const uint32_t e = wbase + c * 32 + lane;
-                if (FULL || e < count) dg[c] = digit_of(FULL ? ks[e] : seg_get(ks, ksrc, sk, e), lo, mask);
+                if (FULL || e < count) dg[c] = digit_of(FULL ? kb[e] : seg_get(ks, ksrc, sk, e), lo, mask);
                 else dg[c] = INVALID_DIGIT;
             }
             const bool active = FULL || wbase < count;
@@ -1192,6 +1228,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
 // ------------------------------------------------------------------ local sort
 
 struct LocalParams {
+    uint64_t n;  // elements of the buffers
     const void *src_keys[3];  // indexed by SrcCode
     const void *src_vals[3];
     void *keys_out;
@@ -1238,9 +1275,9 @@ struct LocalSmem {
     // composite buffer (or the 16-bit index buffer of the pair path)
     static constexpr size_t off_sidx = align16(off_red + sizeof(K) * 2 * W);
     static constexpr size_t off_kst = align16(off_sidx + LocalWord<K, WIDE>::buf_bytes * CAP);
-    static constexpr size_t kst_bytes = align16(sizeof(K) * (CAP + 16 / sizeof(K)));
+    static constexpr size_t kst_bytes = align16(sizeof(K) * (CAP + 32 / sizeof(K)));
     static constexpr size_t off_vst = off_kst + NSTAGE * kst_bytes;
-    static constexpr size_t vst_bytes = HV ? align16(sizeof(VT) * (CAP + 16 / sizeof(VT))) : 0;
+    static constexpr size_t vst_bytes = HV ? align16(sizeof(VT) * (CAP + 32 / sizeof(VT))) : 0;
     static constexpr size_t bytes = off_vst + NSTAGE * vst_bytes;
 };
 
@@ -1314,25 +1351,30 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
             e += gridDim.x;
         }
         in[0] = e;
-        if (e >= nent) return;
+        if (e >= nent) {
+            mbar_arrive_expect_tx(&bar[s], 0);  // completes the phase: the waiters see the end
+            return;
+        }
         in[1] = en.count;
         in[2] = en.hi_bit;
         in[3] = en.src;
         in[4] = static_cast<uint32_t>(en.offs);
         in[5] = static_cast<uint32_t>(en.offs >> 32);
         Seg sk, sv;
-        const K *ks = srck(en.src) + en.offs;
-        uint32_t bytes = seg_plan(ks, en.count, sk);
+        const K *kbuf = srck(en.src);
+        const K *ks = kbuf + en.offs;
+        uint32_t bytes = seg_plan(ks, en.count, kbuf, kbuf + prm.n, sk);
         in[6] = sk.pad;
-        in[7] = sk.i0;
-        in[8] = sk.i1;
+        in[7] = static_cast<uint32_t>(sk.i0);
+        in[8] = static_cast<uint32_t>(sk.i1);
         const VT *vs = nullptr;
         if (HV) {
-            vs = srcv(en.src) + en.offs;
-            bytes += seg_plan(vs, en.count, sv);
+            const VT *vbuf = srcv(en.src);
+            vs = vbuf + en.offs;
+            bytes += seg_plan(vs, en.count, vbuf, vbuf + prm.n, sv);
             in[9] = sv.pad;
-            in[10] = sv.i0;
-            in[11] = sv.i1;
+            in[10] = static_cast<uint32_t>(sv.i0);
+            in[11] = static_cast<uint32_t>(sv.i1);
         }
         mbar_arrive_expect_tx(&bar[s], bytes);
         seg_issue(kst(s), ks, sk, &bar[s], pol);
@@ -1354,6 +1396,8 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
         const int s = static_cast<int>(it % NSTAGE);
         const uint32_t par = (it / NSTAGE) & 1u;
         const uint32_t *in = info + 16 * s;
+        // the producer wrote info[s] before its arrive on bar[s]: the wait acquires it
+        mbar_wait(&bar[s], par);
         const uint32_t e_id = in[0];
         if (e_id >= nent) break;
         const uint32_t count = in[1];
@@ -1362,21 +1406,20 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
         const uint64_t offs = static_cast<uint64_t>(in[4]) | (static_cast<uint64_t>(in[5]) << 32);
         Seg sk, sv;
         sk.pad = in[6];
-        sk.i0 = in[7];
-        sk.i1 = in[8];
+        sk.i0 = static_cast<int32_t>(in[7]);
+        sk.i1 = static_cast<int32_t>(in[8]);
         sv.pad = in[9];
-        sv.i0 = in[10];
-        sv.i1 = in[11];
+        sv.i0 = static_cast<int32_t>(in[10]);
+        sv.i1 = static_cast<int32_t>(in[11]);
         const K *ksrc = srck(src) + offs;
         const VT *vsrc = HV ? srcv(src) + offs : nullptr;
         K *ks = kst(s);
         VT *vs = HV ? vst(s) : nullptr;
-        mbar_wait(&bar[s], par);
-        // the entry may be sorted in place: bring its unaligned edges into shared memory
-        // now, before any thread writes the output
+        // the entry may be sorted in place: elements the bulk copy did not cover (entries
+        // at the ends of the buffer) go into shared memory now, before any thread writes
+        // the output; they are read through seg_get until the next barrier
         seg_fill_edges<K, THREADS>(ks, ksrc, sk, count);
         if (HV) seg_fill_edges<VT, THREADS>(vs, vsrc, sv, count);
-        __syncthreads();
         // BAL: every warp takes kpt = ceil(count / THREADS) columns, so the work is spread
         // over all warps whatever the bucket size (element e = warp*32*kpt + c*32 + lane);
         // otherwise kpt = KPT and warps past the end of the bucket idle
@@ -1390,7 +1433,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
         for (int c = 0; c < KPT; ++c) {
             const uint32_t e = wbase + c * 32 + lane;
             idx[c] = e;
-            key[c] = (!BAL || c < kpt) ? ks[sk.pad + e] : K(0);  // slots past count: stale, never written out
+            key[c] = (!BAL || c < kpt) ? (e < count ? seg_get(ks, ksrc, sk, e) : ks[sk.pad + e]) : K(0);  // past count: stale, never written out
             const bool v = (!BAL || c < kpt) && e < count;
             a &= v ? key[c] : ~K(0);
             o |= v ? key[c] : K(0);
@@ -1621,13 +1664,12 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
                 }
             }
         }
-        __syncthreads();  // staging buffer s and red[] are free
+        __syncthreads();  // staging buffer s, info[s] and red[] are free
         if (tid == 0) {
             fence_proxy_async();
             issue(s, info[16 * NSTAGE]);
             info[16 * NSTAGE] = info[16 * s] + gridDim.x;
         }
-        __syncthreads();  // info[s] is rewritten above
     }
 }
 
