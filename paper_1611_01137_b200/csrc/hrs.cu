@@ -131,6 +131,31 @@ struct LocalStages {
     static constexpr int OCC = OCC0 < 1 ? 1 : (OCC0 > 4 ? 4 : OCC0);
 };
 
+// counting local sort (k_local_cnt) for the large classes: 2^15 counted values for 8-byte
+// records, 2^14 for larger ones (shared memory for two or three CTAs per SM)
+#ifndef HRS_LOCAL_CNT
+#define HRS_LOCAL_CNT 1
+#endif
+#ifndef HRS_LC_CB8
+#define HRS_LC_CB8 14
+#endif
+constexpr int CNT_LO = 5, CNT_HI = 6;
+template <typename K, typename V, int C, bool RECON>
+struct LocalCntStages {
+    using LC = LocalCfg<C>;
+    static constexpr int VBYTES = HasVal<V>::value ? static_cast<int>(sizeof(V)) : 0;
+    static constexpr int CB = static_cast<int>(sizeof(K)) + VBYTES <= 8 ? HRS_LC_CB8 : 14;
+    static constexpr size_t SM_BUDGET = 228 * 1024;
+    static constexpr int NSTAGE =
+        3 * (LocalCntSmem<K, V, LC::THREADS, LC::KPT, 2, CB, RECON>::bytes + 1024) <= SM_BUDGET ? 2 : 1;
+    static constexpr size_t bytes = LocalCntSmem<K, V, LC::THREADS, LC::KPT, NSTAGE, CB, RECON>::bytes;
+    static constexpr bool fits = HRS_LOCAL_CNT && LC::THREADS >= LC_SCAN && bytes <= SMEM_LIMIT;
+    static constexpr int by_smem = static_cast<int>(SM_BUDGET / (bytes + 1024));
+    static constexpr int by_threads = 2048 / LC::THREADS;
+    static constexpr int OCC0 = by_smem < by_threads ? by_smem : by_threads;
+    static constexpr int OCC = OCC0 < 1 ? 1 : (OCC0 > 4 ? 4 : OCC0);
+};
+
 template <typename K, typename V>
 constexpr int max_class_t() {
     return LocalStages<K, V, 7>::fits ? 7 : LocalStages<K, V, 6>::fits ? 6 : 5;
@@ -260,8 +285,8 @@ struct Plan {
     uint32_t range_cap = 0;  // CTAs of the hist/scatter grid the temp layout allows
     size_t off_auxk = 0, off_auxv = 0, off_buckets[2] = {0, 0}, off_tot[2] = {0, 0}, off_subrel = 0,
            off_seg_last = 0, off_seg_meta = 0, off_carry = 0, off_tiles = 0, off_tile_pref = 0,
-           off_local[HRS_NUM_CLASSES] = {0}, off_local_fb = 0, total = 0;
-    uint32_t local_fb_cap = 0;
+           off_local[HRS_NUM_CLASSES] = {0}, off_local_fb = 0, off_local_fb2 = 0, total = 0;
+    uint32_t local_fb_cap = 0, local_fb2_cap = 0;
 };
 
 size_t align_up(size_t x, size_t a) { return (x + a - 1) / a * a; }
@@ -367,6 +392,12 @@ hrs_status make_plan(Plan &pl, uint64_t n, int kb, int vb, int begin, int end, c
     pl.local_fb_cap = static_cast<uint32_t>(std::min<uint64_t>(fb, 0xFFFFFFFFull));
     pl.off_local_fb = off;
     off = align_up(off + sizeof(LocalEntry) * static_cast<size_t>(pl.local_fb_cap), 256);
+    // entries the counting local sort (classes CNT_LO..CNT_HI) hands to the narrow one
+    uint64_t fb2 = 0;
+    for (int c = CNT_LO; c <= CNT_HI; ++c) fb2 += pl.local_cap[c];
+    pl.local_fb2_cap = static_cast<uint32_t>(std::min<uint64_t>(fb2, 0xFFFFFFFFull));
+    pl.off_local_fb2 = off;
+    off = align_up(off + sizeof(LocalEntry) * static_cast<size_t>(pl.local_fb2_cap), 256);
     pl.total = off;
     return HRS_SUCCESS;
 }
@@ -518,43 +549,92 @@ struct Runner {
         return last_launch();
     }
 
+    // which list a local launch sorts: its class list, or a hand-off list
+    enum LocalList { LIST_CLASS = 0, LIST_FB = 1, LIST_FB2 = 2 };
+
+    static void local_params(LocalParams &lp, const Plan &pl, void *temp, const void *kin, void *kout,
+                             const void *vin, void *vout) {
+        lp.n = pl.n;
+        lp.src_keys[SRC_IN] = kin;
+        lp.src_keys[SRC_AUX] = at<void>(temp, pl.off_auxk);
+        lp.src_keys[SRC_OUT] = kout;
+        lp.src_vals[SRC_IN] = vin;
+        lp.src_vals[SRC_AUX] = VB ? at<void>(temp, pl.off_auxv) : nullptr;
+        lp.src_vals[SRC_OUT] = vout;
+        lp.keys_out = kout;
+        lp.vals_out = vout;
+        lp.begin_bit = pl.begin;
+    }
+
+    // the counting local sort of class C; hands what it does not take to LIST_FB2
+    template <int C, bool RECON>
+    static hrs_status local_cnt_variant(const Plan &pl, void *temp, cudaStream_t st, int dev, int sms,
+                                        const void *kin, void *kout, const void *vin, void *vout) {
+        using LST = LocalCntStages<K, V, C, RECON>;
+        if constexpr (!LST::fits) {
+            return HRS_ERROR_INVALID_VALUE;
+        } else {
+            using LC = LocalCfg<C>;
+            LocalParams lp;
+            local_params(lp, pl, temp, kin, kout, vin, vout);
+            Ctl *ctl = at<Ctl>(temp, 0);
+            lp.list = at<LocalEntry>(temp, pl.off_local[C]);
+            lp.count = &ctl->nlocal[C];
+            lp.fb_list = at<LocalEntry>(temp, pl.off_local_fb2);
+            lp.fb_count = &ctl->nlocal_fb2;
+            lp.fb_cap = pl.local_fb2_cap;
+            auto fn = k_local_cnt<K, V, LC::THREADS, LC::KPT, LST::NSTAGE, LST::OCC, LST::CB, RECON>;
+            int grid = 0;
+            hrs_status s = grid_for(fn, LC::THREADS, LST::bytes, dev, sms, &grid);
+            if (s) return s;
+            grid = static_cast<int>(std::min<uint64_t>(grid, std::max<uint32_t>(pl.local_cap[C], 1)));
+            LaunchScope ls(st, 3, C);
+            launch_pdl(fn, dim3(grid), dim3(LC::THREADS), LST::bytes, st, lp);
+            return last_launch();
+        }
+    }
+
+    // the counting variant serves classes CNT_LO..CNT_HI when it fits this key/value type
+    static constexpr bool cnt_ok(int c) {
+        return c >= CNT_LO && c <= CNT_HI && c <= max_class_t<K, V>() &&
+               (c == 5 ? LocalCntStages<K, V, 5, false>::fits && (KB != 4 || LocalCntStages<K, V, 5, true>::fits)
+                       : LocalCntStages<K, V, 6, false>::fits && (KB != 4 || LocalCntStages<K, V, 6, true>::fits));
+    }
+    static bool recon(const Plan &pl) { return KB == 4 && pl.begin == 0 && pl.end == 32; }
+
     template <int C, int WIDE>
     static hrs_status local_variant(const Plan &pl, void *temp, cudaStream_t st, int dev, int sms, const void *kin,
-                                    void *kout, const void *vin, void *vout) {
+                                    void *kout, const void *vin, void *vout, int which = LIST_CLASS) {
         using LST = LocalStages<K, V, C, WIDE>;
         if constexpr (!LST::fits) {
             return HRS_ERROR_INVALID_VALUE;
         } else {
             using LC = LocalCfg<C>;
             LocalParams lp;
-            lp.n = pl.n;
-            lp.src_keys[SRC_IN] = kin;
-            lp.src_keys[SRC_AUX] = at<void>(temp, pl.off_auxk);
-            lp.src_keys[SRC_OUT] = kout;
-            lp.src_vals[SRC_IN] = vin;
-            lp.src_vals[SRC_AUX] = VB ? at<void>(temp, pl.off_auxv) : nullptr;
-            lp.src_vals[SRC_OUT] = vout;
-            lp.keys_out = kout;
-            lp.vals_out = vout;
+            local_params(lp, pl, temp, kin, kout, vin, vout);
             Ctl *ctl = at<Ctl>(temp, 0);
             lp.fb_list = at<LocalEntry>(temp, pl.off_local_fb);
             lp.fb_count = &ctl->nlocal_fb;
             lp.fb_cap = pl.local_fb_cap;
-            if (WIDE == 1) {  // the wide variant sorts what the narrow ones handed over
+            uint32_t cap = pl.local_cap[C];
+            if (which == LIST_FB) {  // the wide variant sorts what the narrow ones handed over
                 lp.list = lp.fb_list;
                 lp.count = &ctl->nlocal_fb;
+                cap = pl.local_fb_cap;
+            } else if (which == LIST_FB2) {  // what the counting variant handed over
+                lp.list = at<LocalEntry>(temp, pl.off_local_fb2);
+                lp.count = &ctl->nlocal_fb2;
+                cap = pl.local_fb2_cap;
             } else {
                 lp.list = at<LocalEntry>(temp, pl.off_local[C]);
                 lp.count = &ctl->nlocal[C];
             }
-            lp.begin_bit = pl.begin;
             auto fn = k_local<K, V, LC::THREADS, LC::KPT, LST::NSTAGE, LST::OCC, WIDE>;
             int grid = 0;
             hrs_status s = grid_for(fn, LC::THREADS, LST::bytes, dev, sms, &grid);
             if (s) return s;
-            const uint32_t cap = WIDE == 1 ? pl.local_fb_cap : pl.local_cap[C];
             grid = static_cast<int>(std::min<uint64_t>(grid, std::max<uint32_t>(cap, 1)));
-            LaunchScope ls(st, 3, WIDE == 1 ? 8 : C);
+            LaunchScope ls(st, 3, which == LIST_FB ? 8 : which == LIST_FB2 ? 9 : C);
             launch_pdl(fn, dim3(grid), dim3(LC::THREADS), LST::bytes, st, lp);
             return last_launch();
         }
@@ -563,8 +643,18 @@ struct Runner {
     template <int C>
     static hrs_status local_one(const Plan &pl, void *temp, cudaStream_t st, int dev, int sms, const void *kin,
                                 void *kout, const void *vin, void *vout) {
-        // full-range sorts of 32-bit keys rebuild the keys from the composites
-        if (KB == 4 && pl.begin == 0) return local_variant<C, 2>(pl, temp, st, dev, sms, kin, kout, vin, vout);
+        if constexpr (cnt_ok(C)) {
+            if (pl.single_class < 0) {  // (the single-configuration ablation keeps k_local)
+                if constexpr (KB == 4)
+                    if (recon(pl)) return local_cnt_variant<C, true>(pl, temp, st, dev, sms, kin, kout, vin, vout);
+                return local_cnt_variant<C, false>(pl, temp, st, dev, sms, kin, kout, vin, vout);
+            }
+        }
+        // full-range sorts of 32-bit keys rebuild the keys from the composites: every key
+        // bit above a bucket's sorted bits is then a digit it was partitioned on, common
+        // to the bucket (with end_bit < 32 the bits above end_bit vary and are carried)
+        if (KB == 4 && pl.begin == 0 && pl.end == 32)
+            return local_variant<C, 2>(pl, temp, st, dev, sms, kin, kout, vin, vout);
         return local_variant<C, 0>(pl, temp, st, dev, sms, kin, kout, vin, vout);
     }
 
@@ -574,8 +664,17 @@ struct Runner {
                                  void *kout, const void *vin, void *vout) {
         if (pl.end - pl.begin <= 19) return HRS_SUCCESS;  // every entry fits a narrow composite
         if (max_class_t<K, V>() == 7)
-            return local_variant<7, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout);
-        return local_variant<6, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout);
+            return local_variant<7, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout, LIST_FB);
+        return local_variant<6, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout, LIST_FB);
+    }
+
+    // the narrow k_local over the entries the counting variant handed over (sizes up to
+    // the capacity of class CNT_HI); launched whenever a counting launch was
+    static hrs_status local_fb2(const Plan &pl, void *temp, cudaStream_t st, int dev, int sms, const void *kin,
+                                void *kout, const void *vin, void *vout) {
+        constexpr int CF = max_class_t<K, V>() < CNT_HI ? max_class_t<K, V>() : CNT_HI;
+        if (recon(pl)) return local_variant<CF, 2>(pl, temp, st, dev, sms, kin, kout, vin, vout, LIST_FB2);
+        return local_variant<CF, 0>(pl, temp, st, dev, sms, kin, kout, vin, vout, LIST_FB2);
     }
 
     static hrs_status local(const Plan &pl, void *temp, cudaStream_t st, int dev, int sms, int c, const void *kin,
@@ -637,10 +736,17 @@ struct Runner {
                 xv = yv;
             }
             const int cmax = pl.single_class >= 0 ? pl.single_class : size_class_of(pl.lt);
-            for (int c = (pl.single_class >= 0 ? pl.single_class : 0); c <= cmax; ++c)
+            bool cnt = false;
+            for (int c = (pl.single_class >= 0 ? pl.single_class : 0); c <= cmax; ++c) {
                 if ((s = local(pl, temp, st, dev, sms, c, kin, kout, vin, vout))) return s;
+                cnt = cnt || (pl.single_class < 0 && cnt_ok(c));
+            }
+            if (cnt && (s = local_fb2(pl, temp, st, dev, sms, kin, kout, vin, vout))) return s;
         } else {
             if ((s = local(pl, temp, st, dev, sms, root_class, kin, kout, vin, vout))) return s;
+            if (pl.single_class < 0 && cnt_ok(root_class) &&
+                (s = local_fb2(pl, temp, st, dev, sms, kin, kout, vin, vout)))
+                return s;
         }
         if ((s = local_wide(pl, temp, st, dev, sms, kin, kout, vin, vout))) return s;
         return HRS_SUCCESS;

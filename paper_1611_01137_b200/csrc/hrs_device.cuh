@@ -94,7 +94,7 @@ struct Ctl {
     uint32_t nlocal[HRS_NUM_CLASSES];       // entries in local list c
     uint32_t claim[HRS_MAX_PASSES + 2];     // k_scatter tile claims of pass p
     uint32_t nlocal_fb;                     // entries the narrow local sort handed to the wide one
-    uint32_t pad2_;
+    uint32_t nlocal_fb2;                    // entries the counting local sort handed to the narrow one
     uint32_t overflow;
     uint32_t pad_;
     unsigned long long recs_in_pass[HRS_MAX_PASSES + 2];
@@ -1669,6 +1669,375 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
             fence_proxy_async();
             issue(s, info[16 * NSTAGE]);
             info[16 * NSTAGE] = info[16 * s] + gridDim.x;
+        }
+    }
+}
+
+// ------------------------------------------------------------------ counting local sort
+//
+// The local sort of a bucket as ONE counting pass instead of
+// ceil(bits / 8) LSD passes: a counting sort (histogram -> exclusive prefix -> placement,
+// the same three steps as a counting pass) on the top CB <= 15 sort bits that
+// vary across the bucket, with 2^CB four-bit counters packed eight to a word.  2^CB is
+// many times the bucket size (<= 4608), so the counted values are nearly distinct; the
+// records that tie on them (about one in eight for uniform keys) are put in order by a
+// short insertion sort of each tie run, on the remaining sort bits and then the input
+// index -- so the result is the stable sort.  The placement slot of a record is
+// prefix(word) + counts of the smaller values in its word + the count returned by its
+// own counter increment (any order among the ties: the fix-up orders them).
+//
+// Buckets it does not take go to a hand-off list sorted afterwards by k_local:
+//   * at most 8 varying sort bits (one LSD pass is cheaper);
+//   * a counted value held by more than 15 records (four-bit counter overflow: skewed keys);
+//   * RECON: more than 19 varying sort bits (the keys are rebuilt from the composites).
+// Per record: one shared atomic, two lookups, one composite store and the value gather
+// -- about 30 shared-memory wavefronts per 32 records against about 42 for two LSD passes
+// (profiles/).
+constexpr int LC_SCAN = 256;  // threads that scan the counters
+
+template <int CB>
+struct CntGeom {
+    static constexpr int NW = (1 << CB) / 8;      // counter words
+    static constexpr int PW = NW / LC_SCAN;       // words per scanning thread
+    static_assert(PW >= 1 && PW <= 32 && (PW & (PW - 1)) == 0, "scan geometry");
+    // word w lives at t*PW + (k ^ swz(t)) (t = w / PW, k = w % PW): the scanning threads
+    // t = 0..31 of a warp reading their k-th words hit 32 different banks
+    __device__ __forceinline__ static uint32_t swz(uint32_t t) { return ((t & 31u) * PW / 32u) & (PW - 1u); }
+    // = t*PW + (k ^ swz(t)): swz(t) < PW only touches the bits of k
+    __device__ __forceinline__ static uint32_t phys(uint32_t w) { return w ^ ((w >> 5) & (PW - 1u)); }
+};
+
+// sum of the eight 4-bit fields of x
+__device__ __forceinline__ uint32_t nib_sum(uint32_t x) {
+    x = (x & 0x0F0F0F0Fu) + ((x >> 4) & 0x0F0F0F0Fu);
+    return (x * 0x01010101u) >> 24;
+}
+
+template <typename K, typename V, int THREADS, int KPT, int NSTAGE, int CB, bool RECON>
+struct LocalCntSmem {
+    static constexpr int W = THREADS / 32;
+    static constexpr int CAP = THREADS * KPT;
+    using VT = ValT<V>;
+    static constexpr bool HV = HasVal<V>::value;
+    using G = CntGeom<CB>;
+    static constexpr size_t off_bar = 0;
+    static constexpr size_t off_info = align16(sizeof(uint64_t) * NSTAGE);
+    static constexpr size_t off_red = align16(off_info + sizeof(uint32_t) * 16 * (NSTAGE + 1));
+    static constexpr size_t off_wsum = align16(off_red + sizeof(K) * 2 * W);
+    static constexpr size_t off_cnt = align16(off_wsum + sizeof(uint32_t) * 16);
+    static constexpr size_t off_pref = off_cnt + sizeof(uint32_t) * G::NW;
+    static constexpr size_t off_comp = align16(off_pref + sizeof(uint16_t) * G::NW);
+    // RECON: the composites overwrite the key staging buffer (the keys are in registers)
+    static constexpr size_t off_kst = align16(off_comp + (RECON ? 0 : sizeof(uint32_t) * CAP));
+    static constexpr size_t kst_bytes = align16(sizeof(K) * (CAP + 32 / sizeof(K)));
+    static constexpr size_t off_vst = off_kst + NSTAGE * kst_bytes;
+    static constexpr size_t vst_bytes = HV ? align16(sizeof(VT) * (CAP + 32 / sizeof(VT))) : 0;
+    static constexpr size_t bytes = off_vst + NSTAGE * vst_bytes;
+};
+
+template <typename K, typename V, int THREADS, int KPT, int NSTAGE, int MINB, int CB, bool RECON>
+__global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
+    pdl_wait();
+    using L = LocalCntSmem<K, V, THREADS, KPT, NSTAGE, CB, RECON>;
+    using G = CntGeom<CB>;
+    constexpr int IB = 13;     // index bits of a composite
+    constexpr int CBITS = 19;  // sort bits of a composite
+    constexpr uint32_t IMASK = (1u << IB) - 1u;
+    constexpr int W = THREADS / 32;
+    constexpr int KBITS = 8 * static_cast<int>(sizeof(K));
+    constexpr bool HV = HasVal<V>::value;
+    using VT = ValT<V>;
+    static_assert(THREADS >= LC_SCAN, "the counter scan needs 256 threads");
+    static_assert(L::CAP <= (1 << IB), "bucket capacity exceeds the composite index");
+    static_assert(!RECON || sizeof(K) == 4, "keys are rebuilt from 32-bit composites only");
+    extern __shared__ __align__(16) unsigned char smem[];
+    uint64_t *bar = reinterpret_cast<uint64_t *>(smem + L::off_bar);
+    uint32_t *info = reinterpret_cast<uint32_t *>(smem + L::off_info);
+    K *red = reinterpret_cast<K *>(smem + L::off_red);
+    uint32_t *wsum = reinterpret_cast<uint32_t *>(smem + L::off_wsum);
+    uint32_t *cnt = reinterpret_cast<uint32_t *>(smem + L::off_cnt);
+    uint16_t *pref = reinterpret_cast<uint16_t *>(smem + L::off_pref);
+    auto kst = [&](int s) { return reinterpret_cast<K *>(smem + L::off_kst + s * L::kst_bytes); };
+    auto vst = [&](int s) { return reinterpret_cast<VT *>(smem + L::off_vst + s * L::vst_bytes); };
+    const int tid = threadIdx.x, lane = tid & 31, warp = tid >> 5;
+    const uint32_t nent = *prm.count;
+    if (blockIdx.x >= nent) return;
+    K *__restrict__ kout = static_cast<K *>(prm.keys_out);
+    VT *__restrict__ vout = static_cast<VT *>(prm.vals_out);
+    const uint64_t pol = policy_evict_first();
+    const int begin_bit = prm.begin_bit;
+
+    auto srck = [&](uint32_t code) -> const K * {
+        return static_cast<const K *>(code == SRC_IN    ? prm.src_keys[SRC_IN]
+                                      : code == SRC_AUX ? prm.src_keys[SRC_AUX]
+                                                        : prm.src_keys[SRC_OUT]);
+    };
+    auto srcv = [&](uint32_t code) -> const VT * {
+        return static_cast<const VT *>(code == SRC_IN    ? prm.src_vals[SRC_IN]
+                                       : code == SRC_AUX ? prm.src_vals[SRC_AUX]
+                                                         : prm.src_vals[SRC_OUT]);
+    };
+    // info[s]: 0 entry, 1 count, 2 hi_bit, 3 src, 4..5 offs, 6..8 key seg, 9..11 value seg
+    auto issue = [&](int s, uint32_t e) {
+        uint32_t *in = info + 16 * s;
+        in[0] = e;
+        if (e >= nent) {
+            mbar_arrive_expect_tx(&bar[s], 0);  // completes the phase: the waiters see the end
+            return;
+        }
+        const LocalEntry en = prm.list[e];
+        in[1] = en.count;
+        in[2] = en.hi_bit;
+        in[3] = en.src;
+        in[4] = static_cast<uint32_t>(en.offs);
+        in[5] = static_cast<uint32_t>(en.offs >> 32);
+        Seg sk, sv;
+        const K *kbuf = srck(en.src);
+        uint32_t bytes = seg_plan(kbuf + en.offs, en.count, kbuf, kbuf + prm.n, sk);
+        in[6] = sk.pad;
+        in[7] = static_cast<uint32_t>(sk.i0);
+        in[8] = static_cast<uint32_t>(sk.i1);
+        if (HV) {
+            const VT *vbuf = srcv(en.src);
+            bytes += seg_plan(vbuf + en.offs, en.count, vbuf, vbuf + prm.n, sv);
+            in[9] = sv.pad;
+            in[10] = static_cast<uint32_t>(sv.i0);
+            in[11] = static_cast<uint32_t>(sv.i1);
+        }
+        mbar_arrive_expect_tx(&bar[s], bytes);
+        seg_issue(kst(s), kbuf + en.offs, sk, &bar[s], pol);
+        if (HV) seg_issue(vst(s), srcv(en.src) + en.offs, sv, &bar[s], pol);
+    };
+    auto hand_off = [&](uint64_t offs, uint32_t count, int hi_bit, uint32_t src) {
+        const uint32_t slot = atomicAdd(prm.fb_count, 1u);
+        if (slot < prm.fb_cap) {
+            LocalEntry en;
+            en.offs = offs;
+            en.count = count;
+            en.hi_bit = static_cast<uint16_t>(hi_bit);
+            en.src = static_cast<uint16_t>(src);
+            prm.fb_list[slot] = en;
+        }
+    };
+    for (int i = tid; i < G::NW; i += THREADS) cnt[i] = 0;  // cleared again after every bucket
+    if (tid == 0) {
+        for (int s = 0; s < NSTAGE; ++s) mbar_init(&bar[s], 1);
+        mbar_fence_init();
+        for (int s = 0; s < NSTAGE; ++s) issue(s, blockIdx.x + s * gridDim.x);
+        info[16 * NSTAGE] = blockIdx.x + NSTAGE * gridDim.x;  // next entry to issue
+    }
+    __syncthreads();
+
+    for (uint32_t it = 0;; ++it) {
+        const int s = static_cast<int>(it % NSTAGE);
+        const uint32_t par = (it / NSTAGE) & 1u;
+        const uint32_t *in = info + 16 * s;
+        mbar_wait(&bar[s], par);  // the producer wrote info[s] before its arrive: the wait acquires it
+        const uint32_t e_id = in[0];
+        if (e_id >= nent) break;
+        const uint32_t count = in[1];
+        const int hi_bit = static_cast<int>(in[2]);
+        const uint32_t src = in[3];
+        const uint64_t offs = static_cast<uint64_t>(in[4]) | (static_cast<uint64_t>(in[5]) << 32);
+        Seg sk, sv;
+        sk.pad = in[6];
+        sk.i0 = static_cast<int32_t>(in[7]);
+        sk.i1 = static_cast<int32_t>(in[8]);
+        sv.pad = in[9];
+        sv.i0 = static_cast<int32_t>(in[10]);
+        sv.i1 = static_cast<int32_t>(in[11]);
+        const K *ksrc = srck(src) + offs;
+        const VT *vsrc = HV ? srcv(src) + offs : nullptr;
+        K *ks = kst(s);
+        VT *vs = HV ? vst(s) : nullptr;
+        // elements the bulk copy did not cover (entries at the ends of a buffer): into
+        // shared memory before anything is written (the entry may be sorted in place)
+        if (!seg_full(sk, count) || (HV && !seg_full(sv, count))) {
+            seg_fill_edges<K, THREADS>(ks, ksrc, sk, count);
+            if (HV) seg_fill_edges<VT, THREADS>(vs, vsrc, sv, count);
+            __syncthreads();
+        }
+        const K *const ksp = ks + sk.pad;
+        K key[KPT];
+        K a = ~K(0), o = K(0);
+#pragma unroll
+        for (int c = 0; c < KPT; ++c) {
+            const uint32_t e = c * THREADS + tid;
+            key[c] = e < count ? ksp[e] : K(0);
+            a &= e < count ? key[c] : ~K(0);
+            o |= e < count ? key[c] : K(0);
+        }
+        a = warp_and(a);
+        o = warp_or(o);
+        if (lane == 0) {
+            red[warp] = a;
+            red[W + warp] = o;
+        }
+        __syncthreads();  // B1: red[], filled edges
+        K aa = ~K(0), oo = K(0);
+#pragma unroll
+        for (int w = 0; w < W; ++w) {
+            aa &= red[w];
+            oo |= red[W + w];
+        }
+        const K diff = aa ^ oo;
+        const K rmask = (hi_bit >= KBITS ? ~K(0) : ((K(1) << hi_bit) - 1)) & ~((K(1) << begin_bit) - 1);
+        const K dv = diff & rmask;  // sort bits that vary across the bucket
+        int thi = 0;
+        if (dv != 0) thi = KBITS - (sizeof(K) == 8 ? __clzll(static_cast<long long>(dv)) : __clz(static_cast<int>(dv)));
+        const int clo = max(begin_bit, thi - CBITS);  // composite: key bits [clo, thi)
+        const int flo = max(clo, thi - CB);           // counted: key bits [flo, thi)
+        const bool nosort = dv == 0;
+        bool take = !nosort && thi - begin_bit > 8;
+        if (RECON) take = take && begin_bit == 0 && clo == 0 && (thi >= KBITS || (diff >> thi) == 0);
+        K *const kd = kout + offs;
+        VT *const vd = HV ? vout + offs : nullptr;
+        const VT *const vsp = HV ? vs + sv.pad : nullptr;
+        if (nosort) {
+            // every record has the same sort bits: the stable order is the input order
+            if (src != SRC_OUT) {
+#pragma unroll
+                for (int c = 0; c < KPT; ++c) {
+                    const uint32_t e = c * THREADS + tid;
+                    if (e < count) {
+                        kd[e] = key[c];
+                        if (HV) vd[e] = vsp[e];
+                    }
+                }
+            }
+        } else if (!take) {
+            if (tid == 0) hand_off(offs, count, hi_bit, src);
+        } else {
+            const int FS = IB + (flo - clo);  // composite >> FS = counted value
+            const uint32_t cmask = (1u << (thi - clo)) - 1u;
+            uint32_t cv[KPT], rec[KPT];
+            bool ovf = false;
+#pragma unroll
+            for (int c = 0; c < KPT; ++c) {
+                const uint32_t e = c * THREADS + tid;
+                cv[c] = ((static_cast<uint32_t>(key[c] >> clo) & cmask) << IB) | e;
+                if (e < count) {
+                    const uint32_t v = cv[c] >> FS;
+                    const uint32_t ph = G::phys(v >> 3), sh = (v & 7u) * 4u;
+                    const uint32_t on = (atomicAdd(&cnt[ph], 1u << sh) >> sh) & 15u;
+                    ovf |= on == 15u;
+                    rec[c] = ph | (sh << 16) | (on << 24);
+                }
+            }
+            if (__syncthreads_or(ovf)) {  // B2 (counts complete)
+                for (int i = tid; i < G::NW; i += THREADS) cnt[i] = 0;
+                if (tid == 0) hand_off(offs, count, hi_bit, src);
+            } else {
+                // exclusive prefix of the word totals: 256 threads own PW consecutive words
+                uint32_t ws[G::PW];
+                uint32_t tsum = 0, incl = 0;
+                const uint32_t sw = G::swz(static_cast<uint32_t>(tid));
+                if (tid < LC_SCAN) {
+#pragma unroll
+                    for (int k = 0; k < G::PW; ++k) {
+                        ws[k] = nib_sum(cnt[tid * G::PW + (k ^ sw)]);
+                        tsum += ws[k];
+                    }
+                    incl = tsum;
+#pragma unroll
+                    for (int d = 1; d < 32; d <<= 1) {
+                        const uint32_t y = __shfl_up_sync(0xffffffffu, incl, d);
+                        if (lane >= d) incl += y;
+                    }
+                    if (lane == 31) wsum[warp] = incl;
+                }
+                __syncthreads();  // B3
+                if (tid < LC_SCAN) {
+                    uint32_t base = incl - tsum;
+#pragma unroll
+                    for (int w = 0; w < LC_SCAN / 32; ++w) base += w < warp ? wsum[w] : 0u;
+#pragma unroll
+                    for (int k = 0; k < G::PW; ++k) {
+                        pref[tid * G::PW + (k ^ sw)] = static_cast<uint16_t>(base);
+                        base += ws[k];
+                    }
+                }
+                __syncthreads();  // B4
+                uint32_t *comp = RECON ? reinterpret_cast<uint32_t *>(ks)
+                                       : reinterpret_cast<uint32_t *>(smem + L::off_comp);
+                // slot = prefix of the word + counts of the smaller values in the word + the
+                // record's own rank among the ties; the record that counted first (on == 0)
+                // of a value held by r > 1 records owns that tie run: run[c] = start | r << 16
+                uint32_t run[KPT];
+#pragma unroll
+                for (int c = 0; c < KPT; ++c) {
+                    const uint32_t e = c * THREADS + tid;
+                    run[c] = 0;
+                    if (e < count) {
+                        const uint32_t ph = rec[c] & 0xFFFFu, sh = (rec[c] >> 16) & 31u, on = rec[c] >> 24;
+                        const uint32_t w = cnt[ph];
+                        const uint32_t slot = pref[ph] + nib_sum(w & ((1u << sh) - 1u)) + on;
+                        comp[slot] = cv[c];
+                        const uint32_t r = (w >> sh) & 15u;
+                        if (on == 0 && r > 1) run[c] = slot | (r << 16);
+                    }
+                }
+                __syncthreads();  // B5
+                for (int i = tid; i < G::NW; i += THREADS) cnt[i] = 0;
+                // tie runs (equal counted value, at most 15 records): insertion sort by the
+                // rest of the composite, then the key bits below it, then the index
+                const bool low = clo > begin_bit;
+                const int lb = clo - begin_bit;
+                const K lmask = lb >= KBITS ? ~K(0) : ((K(1) << lb) - 1);
+                auto less = [&](uint32_t x, uint32_t y) -> bool {
+                    if ((x >> IB) != (y >> IB)) return x < y;
+                    if (low) {
+                        const K lx = (ksp[x & IMASK] >> begin_bit) & lmask, ly = (ksp[y & IMASK] >> begin_bit) & lmask;
+                        if (lx != ly) return lx < ly;
+                    }
+                    return x < y;
+                };
+#pragma unroll
+                for (int c = 0; c < KPT; ++c) {
+                    if (run[c]) {
+                        uint32_t *rb = comp + (run[c] & 0xFFFFu);
+                        const uint32_t r = run[c] >> 16;
+                        if (r == 2) {  // most tie runs are pairs
+                            const uint32_t x = rb[0], y = rb[1];
+                            if (low ? less(y, x) : y < x) {
+                                rb[0] = y;
+                                rb[1] = x;
+                            }
+                            continue;
+                        }
+                        for (uint32_t i = 1; i < r; ++i) {
+                            const uint32_t x = rb[i];
+                            int j = static_cast<int>(i) - 1;
+                            while (j >= 0) {
+                                const uint32_t y = rb[j];
+                                if (low ? !less(x, y) : !(x < y)) break;
+                                rb[j + 1] = y;
+                                --j;
+                            }
+                            rb[j + 1] = x;
+                        }
+                    }
+                }
+                __syncthreads();  // B6
+                // write-out: RECON rebuilds the key from the bits above thi (common to
+                // the bucket) and the composite's sort field; otherwise it is gathered
+                const K khigh = thi >= KBITS ? K(0) : (aa & ~((K(1) << thi) - 1));
+#pragma unroll
+                for (int c = 0; c < KPT; ++c) {
+                    const uint32_t e = c * THREADS + tid;
+                    if (e < count) {
+                        const uint32_t x = comp[e], ix = x & IMASK;
+                        kd[e] = RECON ? (khigh | static_cast<K>(x >> IB)) : ksp[ix];
+                        if (HV) vd[e] = vsp[ix];
+                    }
+                }
+            }
+        }
+        __syncthreads();  // staging buffer s, info[s], red[], comp are free
+        if (tid == 0) {
+            fence_proxy_async();
+            issue(s, info[16 * NSTAGE]);
+            info[16 * NSTAGE] += gridDim.x;
         }
     }
 }

@@ -71,6 +71,16 @@ def test_bit_ranges(kbits, vbits):
         _run_and_check(k, v, b, e)
 
 
+@pytest.mark.parametrize("kbits,vbits", [(32, 32), (32, 0), (64, 64)])
+def test_partial_ranges_deep_buckets(kbits, vbits):
+    """begin = 0 with end < key bits at a size where local sorts run after two counting
+    passes: the key bits above end_bit vary inside a bucket and must be carried (not
+    rebuilt from the bucket's common bits)."""
+    k, v = _inputs((1 << 22) + 5, kbits, vbits, "uniform", seed=21)
+    for b, e in ((0, kbits - 3), (0, 24), (0, 20), (2, kbits - 1)):
+        _run_and_check(k, v, b, e)
+
+
 def test_tie_heavy_stability():
     """Constant and two-valued keys: only stability decides the value order."""
     n = 200000
