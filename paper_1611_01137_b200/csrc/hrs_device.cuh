@@ -45,6 +45,9 @@
 #ifndef HRS_EXP
 #define HRS_EXP 0  // kernel-variant experiments (micro/scatter_exp.py); 0 in the product
 #endif
+#ifndef HRS_RANK2
+#define HRS_RANK2 1  // Ranker::rank2 for blocks of >= 256 threads
+#endif
 
 namespace hrs {
 
@@ -374,6 +377,10 @@ struct Ranker {
 
     __device__ __forceinline__ uint32_t *vcnt(int w) const { return cnt + w * NBINS; }
 
+    // THREADS >= 256: the per-digit fold is done by one thread per digit (see rank2)
+    static constexpr bool FOLD = THREADS >= RADIX && HRS_RANK2;
+    static constexpr int BOWN = THREADS > RADIX ? RADIX : 0;  // thread that folds bin 256
+
     __device__ __forceinline__ void init(uint32_t *base) {
         cnt = base;
         tot = base + cnt_words;
@@ -381,13 +388,81 @@ struct Ranker {
         for (int i = threadIdx.x; i < static_cast<int>(cnt_words); i += THREADS) cnt[i] = 0;
     }
 
-    // dg: digits on entry (INVALID_DIGIT for padding), slots on exit.  kpt: active
-    // columns (the same for all warps); active: this warp holds elements.  allow_fast:
-    // the fast in-warp rank may be used (the caller checks the result).  gs (optional,
-    // [RADIX]): gs[d].x holds a per-digit base on entry, {base - start[d], start[d]} on
-    // exit.  Contains two block barriers; start[] and gs are valid after the caller's
-    // next barrier.  Each warp clears its own counters at the end, so the next tile /
-    // pass needs no extra barrier.
+    // the fold for THREADS >= 256 after the count phase and its barrier: thread d (< 256)
+    // reads the W warp counters of digit d, scans the digit totals with shuffles and
+    // writes every warp's first slot of digit d back (rank() instead has every warp
+    // re-read the 257 totals and fold them into its own counters).  About 60 % of the
+    // per-digit shared-memory traffic of rank(), one more barrier.
+    __device__ __forceinline__ void fold2(uint2 *gs) {
+        const int tid = threadIdx.x, warp = tid >> 5, lane = tid & 31;
+        uint32_t *wsum = tot;  // [8] digit totals of warps 0..7
+        uint32_t t = 0;
+        if (tid < RADIX) {
+#pragma unroll
+            for (int w = 0; w < W; ++w) t += vcnt(w)[tid];
+            uint32_t incl = t;
+#pragma unroll
+            for (int o = 1; o < 32; o <<= 1) {
+                const uint32_t y = __shfl_up_sync(0xffffffffu, incl, o);
+                if (lane >= o) incl += y;
+            }
+            if (lane == 31) wsum[warp] = incl;
+            t = incl - t;  // exclusive within the warp's 32 digits
+        }
+        __syncthreads();
+        if (tid < RADIX) {
+            uint32_t run = t;
+#pragma unroll
+            for (int w = 0; w < RADIX / 32; ++w) run += w < warp ? wsum[w] : 0u;
+            if (gs != nullptr) gs[tid] = make_uint2(gs[tid].x - run, run);
+#pragma unroll
+            for (int w = 0; w < W; ++w) {  // (counts re-read: fewer live registers across the barrier)
+                const uint32_t nw = vcnt(w)[tid];
+                vcnt(w)[tid] = run;
+                run += nw;
+            }
+        }
+        if (tid == BOWN) {  // bin 256 (padding lanes): after every digit
+            uint32_t run = 0;
+#pragma unroll
+            for (int w = 0; w < RADIX / 32; ++w) run += wsum[w];
+            for (int w = 0; w < W; ++w) {
+                const uint32_t nw = vcnt(w)[RADIX];
+                vcnt(w)[RADIX] = run;
+                run += nw;
+            }
+        }
+        __syncthreads();
+    }
+
+    // in-warp ranks from the folded counters (warp-local; clears the warp's counters)
+    __device__ __forceinline__ void lookup(uint32_t (&dg)[KPT], int kpt, bool active, uint32_t ltm, bool fast) {
+        const int lane = threadIdx.x & 31;
+        uint32_t *ca = vcnt(threadIdx.x >> 5);
+        if (active) {
+            if (fast) {
+#pragma unroll
+                for (int c = 0; c < KPT; ++c)
+                    if (c < kpt) dg[c] = ca[dg[c] & 0xFFFFu] + (dg[c] >> 16);
+            } else {
+#pragma unroll
+                for (int c = 0; c < KPT; ++c) {
+                    const bool v0 = c < kpt;
+                    const uint32_t d0 = v0 ? dg[c] : 0u;
+                    const uint32_t p0 = v0 ? ca[d0] : 0u;
+                    __syncwarp();
+                    if (v0) atomicAdd(&ca[d0], 1u);
+                    __syncwarp();
+                    const uint32_t k0 = v0 ? ca[d0] - p0 : 0u;
+                    const uint32_t m = __match_any_sync(0xffffffffu, k0 > 1 ? d0 : 0xFFFFFFFFu);
+                    if (v0) dg[c] = p0 + (k0 > 1 ? __popc(m & ltm) : 0u);
+                }
+            }
+        }
+        __syncwarp();
+        for (int d = lane; d < NBINS; d += 32) ca[d] = 0;
+    }
+
     __device__ __forceinline__ void rank(uint32_t (&dg)[KPT], int kpt, bool active, uint32_t ltm, bool allow_fast,
                                          uint2 *gs = nullptr) {
         const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
@@ -413,7 +488,17 @@ struct Ranker {
                     if (c < kpt) atomicAdd(&ca[dg[c]], 1u);
             }
         }
-        __syncthreads();
+        if constexpr (FOLD) {
+            // a block where some warp takes the exact rank (skewed digits) folds with one
+            // thread per digit (measured faster there); otherwise every warp folds its own
+            if (__syncthreads_or(active && !fast)) {
+                fold2(gs);
+                lookup(dg, kpt, active, ltm, fast);
+                return;
+            }
+        } else {
+            __syncthreads();
+        }
         // exclusive prefix over the warps per digit, digit totals
         for (int d = threadIdx.x; d < NBINS; d += THREADS) {
             uint32_t v[W];
@@ -462,28 +547,7 @@ struct Ranker {
             }
         }
         __syncwarp();
-        if (active) {
-            if (fast) {
-#pragma unroll
-                for (int c = 0; c < KPT; ++c)
-                    if (c < kpt) dg[c] = ca[dg[c] & 0xFFFFu] + (dg[c] >> 16);
-            } else {
-#pragma unroll
-                for (int c = 0; c < KPT; ++c) {
-                    const bool v0 = c < kpt;
-                    const uint32_t d0 = v0 ? dg[c] : 0u;
-                    const uint32_t p0 = v0 ? ca[d0] : 0u;
-                    __syncwarp();
-                    if (v0) atomicAdd(&ca[d0], 1u);
-                    __syncwarp();
-                    const uint32_t k0 = v0 ? ca[d0] - p0 : 0u;
-                    const uint32_t m = __match_any_sync(0xffffffffu, k0 > 1 ? d0 : 0xFFFFFFFFu);
-                    if (v0) dg[c] = p0 + (k0 > 1 ? __popc(m & ltm) : 0u);
-                }
-            }
-        }
-        __syncwarp();
-        for (int d = lane; d < NBINS; d += 32) ca[d] = 0;
+        lookup(dg, kpt, active, ltm, fast);
     }
 };
 
