@@ -136,6 +136,9 @@ struct LocalStages {
 #ifndef HRS_LOCAL_CNT
 #define HRS_LOCAL_CNT 1
 #endif
+#ifndef HRS_LC_NSTAGE
+#define HRS_LC_NSTAGE 0  // 0: two stages when three CTAs still fit per SM
+#endif
 #ifndef HRS_LC_CB8
 #define HRS_LC_CB8 14
 #endif
@@ -147,7 +150,8 @@ struct LocalCntStages {
     static constexpr int CB = static_cast<int>(sizeof(K)) + VBYTES <= 8 ? HRS_LC_CB8 : 14;
     static constexpr size_t SM_BUDGET = 228 * 1024;
     static constexpr int NSTAGE =
-        3 * (LocalCntSmem<K, V, LC::THREADS, LC::KPT, 2, CB, RECON>::bytes + 1024) <= SM_BUDGET ? 2 : 1;
+        HRS_LC_NSTAGE ? HRS_LC_NSTAGE
+                      : (3 * (LocalCntSmem<K, V, LC::THREADS, LC::KPT, 2, CB, RECON>::bytes + 1024) <= SM_BUDGET ? 2 : 1);
     static constexpr size_t bytes = LocalCntSmem<K, V, LC::THREADS, LC::KPT, NSTAGE, CB, RECON>::bytes;
     static constexpr bool fits = HRS_LOCAL_CNT && LC::THREADS >= LC_SCAN && bytes <= SMEM_LIMIT;
     static constexpr int by_smem = static_cast<int>(SM_BUDGET / (bytes + 1024));

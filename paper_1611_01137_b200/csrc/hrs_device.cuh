@@ -45,6 +45,9 @@
 #ifndef HRS_EXP
 #define HRS_EXP 0  // kernel-variant experiments (micro/scatter_exp.py); 0 in the product
 #endif
+#ifndef HRS_WAIT1
+#define HRS_WAIT1 0  // (measured slower when 1) k_hist / k_scatter: one warp waits on the TMA mbarrier, a CTA barrier releases the others
+#endif
 #ifndef HRS_RANK2
 #define HRS_RANK2 1  // Ranker::rank2 for blocks of >= 256 threads
 #endif
@@ -736,7 +739,8 @@ __global__ void __launch_bounds__(THREADS) k_hist(HistParams prm) {
             td.pad = 0;
             prm.tiles[t] = td;
         }
-        mbar_wait(&bar[s], par);
+        if (!HRS_WAIT1 || warp == 0) mbar_wait(&bar[s], par);  // one warp waits, the barrier releases the rest
+        if (HRS_WAIT1) __syncthreads();
         const K *sb = stage(s);
         // 16-byte vectors over the staged superset: vector v holds elements ibase + v*VK
         // .. + VK - 1 (element i = position - pad); the vectors wholly inside [0, count)
@@ -1203,7 +1207,8 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
         const VT *vsrc = HV ? vin + in.offs : nullptr;
         K *ks = kst(s);
         VT *vs = HV ? vst(s) : nullptr;
-        mbar_wait(&bar[s], par);
+        if (!HRS_WAIT1 || warp == 0) mbar_wait(&bar[s], par);  // one warp waits, the barrier releases the rest
+        if (HRS_WAIT1) __syncthreads();
         // full tiles with an aligned interior take the predicate-free path
         const bool full = count == static_cast<uint32_t>(L::KPB) && seg_full(sk, count) && (!HV || seg_full(sv, count));
         const K *const kb = ks + sk.pad;  // element i of the tile (after the edges are filled)
@@ -1896,7 +1901,11 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
         const int s = static_cast<int>(it % NSTAGE);
         const uint32_t par = (it / NSTAGE) & 1u;
         const uint32_t *in = info + 16 * s;
-        mbar_wait(&bar[s], par);  // the producer wrote info[s] before its arrive: the wait acquires it
+        // one warp waits for the bulk copies (the producer wrote info[s] before its arrive:
+        // the wait acquires it); the barrier passes both on to the other warps, which
+        // meanwhile do not take issue slots from the other resident CTAs
+        if (warp == 0) mbar_wait(&bar[s], par);
+        __syncthreads();
         const uint32_t e_id = in[0];
         if (e_id >= nent) break;
         const uint32_t count = in[1];
@@ -1927,9 +1936,9 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
 #pragma unroll
         for (int c = 0; c < KPT; ++c) {
             const uint32_t e = c * THREADS + tid;
-            key[c] = e < count ? ksp[e] : K(0);
-            a &= e < count ? key[c] : ~K(0);
-            o |= e < count ? key[c] : K(0);
+            key[c] = ksp[e < count ? e : 0u];  // past the end: a copy of key 0 (neutral for and/or)
+            a &= key[c];
+            o |= key[c];
         }
         a = warp_and(a);
         o = warp_or(o);
@@ -1975,7 +1984,6 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
             const int FS = IB + (flo - clo);  // composite >> FS = counted value
             const uint32_t cmask = (1u << (thi - clo)) - 1u;
             uint32_t cv[KPT], rec[KPT];
-            bool ovf = false;
 #pragma unroll
             for (int c = 0; c < KPT; ++c) {
                 const uint32_t e = c * THREADS + tid;
@@ -1984,15 +1992,14 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
                     const uint32_t v = cv[c] >> FS;
                     const uint32_t ph = G::phys(v >> 3), sh = (v & 7u) * 4u;
                     const uint32_t on = (atomicAdd(&cnt[ph], 1u << sh) >> sh) & 15u;
-                    ovf |= on == 15u;
                     rec[c] = ph | (sh << 16) | (on << 24);
                 }
             }
-            if (__syncthreads_or(ovf)) {  // B2 (counts complete)
-                for (int i = tid; i < G::NW; i += THREADS) cnt[i] = 0;
-                if (tid == 0) hand_off(offs, count, hi_bit, src);
-            } else {
-                // exclusive prefix of the word totals: 256 threads own PW consecutive words
+            __syncthreads();  // B2 (counts complete)
+            {
+                // exclusive prefix of the word totals: 256 threads own PW consecutive words.
+                // A counter that passed 15 wrapped (-16, +1 carried into its neighbour or
+                // lost): the nibble total then falls short of count, checked after B3.
                 uint32_t ws[G::PW];
                 uint32_t tsum = 0, incl = 0;
                 const uint32_t sw = G::swz(static_cast<uint32_t>(tid));
@@ -2011,6 +2018,14 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
                     if (lane == 31) wsum[warp] = incl;
                 }
                 __syncthreads();  // B3
+                uint32_t total = 0;
+#pragma unroll
+                for (int w = 0; w < LC_SCAN / 32; ++w) total += wsum[w];
+                if (total != count) {  // four-bit counter overflow: k_local takes the bucket
+                    for (int i = tid; i < G::NW; i += THREADS) cnt[i] = 0;
+                    if (tid == 0) hand_off(offs, count, hi_bit, src);
+                    goto next_entry;
+                }
                 if (tid < LC_SCAN) {
                     uint32_t base = incl - tsum;
 #pragma unroll
@@ -2097,6 +2112,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
                 }
             }
         }
+    next_entry:
         __syncthreads();  // staging buffer s, info[s], red[], comp are free
         if (tid == 0) {
             fence_proxy_async();
