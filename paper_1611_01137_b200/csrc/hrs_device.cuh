@@ -830,6 +830,94 @@ struct ClassifyParams {
     uint64_t *out_offsets;  // building block: the root bucket's sub-bucket starts (+ n)
 };
 
+// Block-wide suffix minimum of one value per thread (THREADS == 256 = RADIX threads,
+// thread d holds digit d): returns min(v[d .. 255]).  wbuf: 8 words.
+__device__ __forceinline__ uint32_t block_suffix_min256(uint32_t v, uint32_t *wbuf) {
+    const int tid = threadIdx.x, lane = tid & 31, warp = tid >> 5;
+#pragma unroll
+    for (int o = 1; o < 32; o <<= 1) {
+        const uint32_t y = __shfl_down_sync(0xffffffffu, v, o);
+        if (lane + o < 32) v = min(v, y);
+    }
+    if (lane == 0) wbuf[warp] = v;  // the minimum of the warp's 32 digits
+    __syncthreads();
+#pragma unroll
+    for (int w = 0; w < RADIX / 32; ++w) v = w > warp ? min(v, wbuf[w]) : v;
+    __syncthreads();  // wbuf is reused by the next call
+    return v;
+}
+
+// The greedy merge of the local candidates of one bucket (reading #5 of DESIGN.md: in
+// digit order, a candidate joins the open group while the group stays below ∂, a
+// sibling > ∂ˆ closes it, empty sub-buckets are skipped), computed by one thread per
+// digit instead of one thread walking 256 digits.  With P = exclusive prefix of the
+// sub-bucket sizes, the group that starts at candidate i ends at
+//     gend(i) = min(first sibling > ∂ˆ after i,  first k > i with P[k+1] >= P[i] + ∂)
+// (it holds the candidates of [i, gend), size P[gend] - P[i]) and the next group
+// starts at the first candidate >= gend.  The groups are the chain of starts from the
+// first candidate, marked by pointer doubling (8 rounds for 256 digits).
+// Writes glead[i] = group size and gmulti[i] = (>= 2 members) at every group start i.
+template <int THREADS>
+__device__ void merge_groups(const ClassifyParams &prm, const uint32_t *tot, const uint32_t *P, uint32_t *glead,
+                             uint32_t *gmulti, uint32_t *ws) {
+    static_assert(THREADS == RADIX, "one thread per digit");
+    uint32_t *jmp = ws;               // [2][NBINS] successor tables (double-buffered)
+    uint32_t *flag = ws + 2 * NBINS;  // [NBINS] group start
+    uint32_t *wbuf = ws + 3 * NBINS;  // [8]
+    const uint32_t d = threadIdx.x;
+    const uint32_t s = tot[d];
+    const bool cand = s > 0 && s <= prm.lt, big = s > prm.lt;
+    // first big sibling after d, first candidate at or after d (256 = none)
+    const uint32_t nb_incl = block_suffix_min256(big ? d : RADIX, wbuf);
+    const uint32_t nc = block_suffix_min256(cand ? d : RADIX, wbuf);
+    flag[d] = nc;  // (temporary: NC table, read below)
+    jmp[d] = nb_incl;
+    if (d == 0) {
+        flag[RADIX] = RADIX;
+        jmp[RADIX] = RADIX;
+    }
+    __syncthreads();
+    uint32_t succ = RADIX, gend = RADIX, size = 0;
+    bool multi = false;
+    if (cand) {
+        const uint32_t b = jmp[d + 1];  // first big after d
+        // first q in [d + 2, 256] with P[q] >= P[d] + ∂ (k = q - 1), else k = 256
+        const uint32_t target = P[d] + prm.mt;
+        uint32_t lo = d + 2, hi = RADIX + 1;  // answer in [lo, hi); hi = none
+        while (lo < hi) {
+            const uint32_t mid = (lo + hi) >> 1;
+            if (P[mid] >= target) hi = mid;
+            else lo = mid + 1;
+        }
+        const uint32_t k1 = lo <= RADIX ? lo - 1 : RADIX;
+        gend = min(k1, b);
+        size = P[gend] - P[d];
+        succ = flag[gend];           // first candidate >= gend
+        multi = flag[d + 1] < gend;  // a second candidate inside the group
+    }
+    const uint32_t first = flag[0];
+    __syncthreads();  // NC / NB tables consumed
+    jmp[d] = succ;
+    flag[d] = d == first ? 1u : 0u;
+    if (d == 0) jmp[RADIX] = RADIX;
+    __syncthreads();
+    uint32_t *ja = jmp, *jb = jmp + NBINS;
+    for (int round = 0; round < 8; ++round) {
+        const uint32_t j = ja[d];
+        if (flag[d] && j < RADIX) flag[j] = 1u;  // (flags only ever go 0 -> 1)
+        jb[d] = j < RADIX ? ja[j] : RADIX;
+        if (d == 0) jb[RADIX] = RADIX;
+        __syncthreads();
+        uint32_t *t = ja;
+        ja = jb;
+        jb = t;
+    }
+    if (cand && flag[d]) {
+        glead[d] = size;
+        gmulti[d] = multi ? 1u : 0u;
+    }
+}
+
 template <int THREADS>
 __device__ void classify_bucket(const ClassifyParams &prm, const Bucket &bk, uint32_t bucket_id, uint32_t *sm) {
     static_assert(THREADS >= RADIX, "one thread per digit");
@@ -899,37 +987,8 @@ __device__ void classify_bucket(const ClassifyParams &prm, const Bucket &bk, uin
             const uint32_t s = tot[d];
             if (s > 0 && s <= prm.lt) glead[d] = s;
         }
-    } else if (tid == 0) {
-        int gl = -1;
-        uint32_t gs = 0, gc = 0;
-        for (int d = 0; d < RADIX; ++d) {
-            const uint32_t s = tot[d];
-            if (s == 0) continue;
-            if (s > prm.lt) {
-                if (gl >= 0) {
-                    glead[gl] = gs;
-                    gmulti[gl] = gc > 1;
-                }
-                gl = -1;
-                continue;
-            }
-            if (gl >= 0 && gs + s < prm.mt) {
-                gs += s;
-                ++gc;
-            } else {
-                if (gl >= 0) {
-                    glead[gl] = gs;
-                    gmulti[gl] = gc > 1;
-                }
-                gl = d;
-                gs = s;
-                gc = 1;
-            }
-        }
-        if (gl >= 0) {
-            glead[gl] = gs;
-            gmulti[gl] = gc > 1;
-        }
+    } else {
+        merge_groups<THREADS>(prm, tot, start, glead, gmulti, sm + 7 * NBINS);
     }
     __syncthreads();
     // per-class slot allocation
@@ -1039,7 +1098,7 @@ __device__ void range_carries(const ClassifyParams &prm) {
 template <int THREADS>
 __global__ void __launch_bounds__(THREADS) k_classify(ClassifyParams prm) {
     pdl_wait();
-    __shared__ uint32_t scratch[7 * NBINS];
+    __shared__ uint32_t scratch[11 * NBINS];  // classify_bucket: 7 rows, merge_groups: 3 rows + 8 words
     const uint32_t nb = alloc_buckets(prm.ctl->alloc[prm.p]);
     if (nb == 0) return;  // nothing reached this pass
     if (blockIdx.x == gridDim.x - 1) {
