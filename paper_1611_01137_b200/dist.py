@@ -6,10 +6,15 @@ host merge, which this replaces):
 
   1. every rank histograms the most-significant digit of its shard (libhrs kernel);
   2. all_gather of the 256-bin histograms (2 KiB per rank);
-  3. a deterministic bucket -> rank assignment, identical on every rank: rank j owns
-     the contiguous digit range whose global prefix starts in [j N/G, (j+1) N/G);
-  4. one stable counting pass on that digit (libhrs kernel) groups the shard by
-     destination, and all_to_all_single exchanges keys and values over NVLink;
+  3. one stable counting pass on that digit (libhrs kernel) groups the shard by bucket;
+     rank j receives exactly the global sorted positions [j N/G, (j+1) N/G) (SURVEY
+     §8(f) N1, skew-robust splitting): only the buckets that contain a boundary j N/G
+     are refined, digit by digit, with the same stable counting pass on their local
+     sub-ranges and an all_gather of their sub-bucket histograms; at full key
+     resolution a boundary lies inside a run of equal keys, which is split by global
+     index (rank-major, reading #17).  Every rank then knows every rank's split
+     positions, so the send/receive counts need no further exchange;
+  4. all_to_all_single exchanges keys and values over NVLink;
   5. every rank sorts what it received with the single-GPU hybrid sort.  The
      received segments arrive in source-rank order, i.e. global input order, so the
      concatenation of the rank outputs is the unique stable sort of the global input
@@ -17,7 +22,7 @@ host merge, which this replaces):
 
 The local operations are injected (`ops`): the product uses the CUDA library
 (`CudaOps`); the CPU gloo tests inject an oracle-backed implementation to check the
-host-side plumbing (assignment, split sizes, exchange order) without a GPU.
+host-side plumbing (split positions, split sizes, exchange order) without a GPU.
 """
 from __future__ import annotations
 
@@ -30,6 +35,30 @@ _SIGNED = {torch.uint32: torch.int32, torch.uint64: torch.int64}
 def _bits(t: torch.Tensor) -> torch.Tensor:
     """Signed view with the same bits (collectives do not take unsigned dtypes)."""
     return t.view(_SIGNED[t.dtype]) if t.dtype in _SIGNED else t
+
+
+def _host_staged(group, t: torch.Tensor) -> bool:
+    """gloo cannot run these collectives on CUDA tensors: stage them through host memory
+    (used by the single-GPU multi-process tests; NCCL takes device tensors directly)."""
+    return t.is_cuda and dist.get_backend(group) == "gloo"
+
+
+def _all_gather(out: torch.Tensor, inp: torch.Tensor, group) -> None:
+    if _host_staged(group, inp):
+        o = out.cpu()
+        dist.all_gather_into_tensor(o, inp.cpu(), group=group)
+        out.copy_(o)
+    else:
+        dist.all_gather_into_tensor(out, inp, group=group)
+
+
+def _all_to_all(out: torch.Tensor, inp: torch.Tensor, out_splits, in_splits, group) -> None:
+    if _host_staged(group, inp):
+        o = out.cpu()
+        dist.all_to_all_single(o, inp.cpu(), output_split_sizes=out_splits, input_split_sizes=in_splits, group=group)
+        out.copy_(o)
+    else:
+        dist.all_to_all_single(out, inp, output_split_sizes=out_splits, input_split_sizes=in_splits, group=group)
 
 
 class CudaOps:
@@ -45,32 +74,14 @@ class CudaOps:
     def partition_pass(self, keys, vals, lo, hi):
         return self.hrs.partition_pass(keys, vals, lo, hi)
 
+    def partition_into(self, keys, vals, lo, hi, keys_out, vals_out):
+        """Stable counting pass of keys (vals) into keys_out (vals_out); returns the
+        sub-bucket offsets (r + 1 entries) on the host."""
+        _, _, offs = self.hrs.partition_pass(keys, vals, lo, hi, keys_out=keys_out, values_out=vals_out)
+        return offs.cpu().tolist()
+
     def sort(self, keys, vals, begin_bit, end_bit):
         return self.hrs.sort(keys, vals, begin_bit, end_bit)
-
-
-def assign_buckets(global_hist: list[int], world: int) -> list[int]:
-    """owner[b] for the 256 top-digit buckets: rank j owns the buckets whose global
-    exclusive prefix lies in [j N / G, (j + 1) N / G) -- contiguous, monotone,
-    deterministic (every rank computes the same list)."""
-    n = sum(global_hist)
-    owner = []
-    run = 0
-    for c in global_hist:
-        owner.append(min(world - 1, (run * world) // n) if n else 0)
-        run += c
-    return owner
-
-
-def split_counts(hists: list[list[int]], owner: list[int], world: int):
-    """send[r][j] = records rank r sends to rank j (hists[r] = rank r's histogram)."""
-    out = []
-    for h in hists:
-        row = [0] * world
-        for b, c in enumerate(h):
-            row[owner[b]] += c
-        out.append(row)
-    return out
 
 
 class DistributedSorter:
@@ -89,46 +100,124 @@ class DistributedSorter:
         self.rank = dist.get_rank(group)
         self.last = {}
 
+    def digits(self):
+        """The (lo, hi) bit ranges of the 8-bit digits, most significant first."""
+        out, hi = [], self.end
+        while hi > self.begin:
+            lo = max(self.begin, hi - 8)
+            out.append((lo, hi))
+            hi = lo
+        return out
+
     def step(self):
         keys, vals = self.keys, self.vals
-        world = self.world
-        hi = self.end
-        lo = max(self.begin, hi - 8)
-        if hi == lo:  # empty bit range: the stable sort is the identity
+        world, me = self.world, self.rank
+        if self.end == self.begin:  # empty bit range: the stable sort is the identity
             return keys.clone(), (vals.clone() if vals is not None else None), self._offset_identity()
-        r = 1 << (hi - lo)
-        # 1-2. first-digit histograms, gathered on every rank
-        h = self.ops.digit_histogram(keys, lo, hi)
-        gathered = torch.empty(world * r, dtype=torch.int64, device=h.device)
-        dist.all_gather_into_tensor(gathered, _bits(h).contiguous(), group=self.group)
-        hists = gathered.view(world, r).cpu().tolist()
-        glob = [sum(col) for col in zip(*hists)]
-        # 3. deterministic assignment of buckets to ranks
-        owner = assign_buckets(glob, world)
-        send = split_counts(hists, owner, world)
-        recv = [send[src][self.rank] for src in range(world)]
-        # 4. stable partition by destination (bucket order = destination order) + exchange
-        kp, vp, _ = self.ops.partition_pass(keys, vals, lo, hi)
+        digits = self.digits()
+        # 1-3a. first-digit partition of the whole shard; its histogram, gathered
+        kp = torch.empty_like(keys)
+        vp = torch.empty_like(vals) if vals is not None else None
+        lo, hi = digits[0]
+        offs = self.ops.partition_into(keys, vals, lo, hi, kp, vp)
+        hists = self._gather([[offs[b + 1] - offs[b] for b in range(len(offs) - 1)]])[0]  # [rank][bucket]
+        N = sum(sum(h) for h in hists)
+        # split[j][r]: local position on rank r of global sorted position t_j = j N / G
+        split = [[0] * world for _ in range(world + 1)]
+        split[world] = [sum(h) for h in hists]
+        todo = []  # boundaries inside a segment: (j, t_j, level, g0, starts[r], counts[r])
+        for j in range(1, world):
+            self._place(j, j * N // world, 0, 0, [0] * world, hists, split, todo)
+        # 3b. refine the segments that contain a boundary, one digit at a time
+        scratch_k = scratch_v = None
+        levels = 0  # digits below the first that some boundary needed
+        for level in range(1, len(digits)):
+            if not todo:
+                break
+            levels = level
+            if scratch_k is None:
+                scratch_k = torch.empty_like(kp)
+                scratch_v = torch.empty_like(vp) if vp is not None else None
+            lo, hi = digits[level]
+            segs = []  # distinct segments (several boundaries may share one)
+            for item in todo:
+                if not segs or segs[-1][0] != (item[3], tuple(item[4])):
+                    segs.append(((item[3], tuple(item[4])), item[4], item[5]))
+            local = []
+            for _, starts, counts in segs:
+                a, c = starts[me], counts[me]
+                if c:
+                    sub = self.ops.partition_into(kp[a:a + c], vp[a:a + c] if vp is not None else None, lo, hi,
+                                                  scratch_k[a:a + c], scratch_v[a:a + c] if vp is not None else None)
+                    kp[a:a + c].copy_(scratch_k[a:a + c])
+                    if vp is not None:
+                        vp[a:a + c].copy_(scratch_v[a:a + c])
+                    local.append([sub[b + 1] - sub[b] for b in range(len(sub) - 1)])
+                else:
+                    local.append([0] * (1 << (hi - lo)))
+            seg_hists = self._gather(local)  # [seg][rank][sub-bucket]
+            nxt = []
+            for item in todo:
+                k = next(i for i, sg in enumerate(segs) if sg[0] == (item[3], tuple(item[4])))
+                self._place(item[0], item[1], level, item[3], item[4], seg_hists[k], split, nxt)
+            todo = nxt
+        # 3c. boundaries still inside a segment after the last digit: equal keys, split by
+        # global index (rank-major, each rank's run in local index order)
+        for j, t, _, g0, starts, counts in todo:
+            run = g0
+            for r in range(world):
+                split[j][r] = starts[r] + min(counts[r], max(0, t - run))
+                run += counts[r]
+        send = [[split[j + 1][r] - split[j][r] for j in range(world)] for r in range(world)]
+        recv = [send[src][me] for src in range(world)]
+        # 4. exchange (every source's segment in source-rank order)
         rk = torch.empty(sum(recv), dtype=keys.dtype, device=keys.device)
-        dist.all_to_all_single(_bits(rk), _bits(kp), output_split_sizes=recv,
-                               input_split_sizes=send[self.rank], group=self.group)
+        _all_to_all(_bits(rk), _bits(kp), recv, send[me], self.group)
         rv = None
         if vals is not None:
             rv = torch.empty(sum(recv), dtype=vals.dtype, device=vals.device)
-            dist.all_to_all_single(_bits(rv), _bits(vp), output_split_sizes=recv,
-                                   input_split_sizes=send[self.rank], group=self.group)
+            _all_to_all(_bits(rv), _bits(vp), recv, send[me], self.group)
         # 5. local sort of the received records (source-rank order = global input order)
         ko, vo = self.ops.sort(rk, rv, self.begin, self.end)
-        offset = sum(c for b, c in enumerate(glob) if owner[b] < self.rank)
-        self.last = {"send": send[self.rank], "recv": recv, "owner": owner, "offset": offset,
+        offset = me * N // world
+        self.last = {"send": send[me], "recv": recv, "offset": offset, "refine_levels": levels,
                      "imbalance": max(sum(send[s][j] for s in range(world)) for j in range(world)) /
-                     max(1, sum(glob) / world)}
+                     max(1, N / world)}
         return ko, vo, offset
 
+    def _gather(self, rows):
+        """all_gather of this rank's histogram rows ([k][r] ints) -> [k][rank][r]."""
+        k, r = len(rows), len(rows[0])
+        mine = torch.tensor(rows, dtype=torch.int64).reshape(-1)
+        if self.keys.is_cuda:
+            mine = mine.to(self.keys.device)
+        allv = torch.empty(self.world * k * r, dtype=torch.int64, device=mine.device)
+        _all_gather(allv, mine, self.group)
+        a = allv.view(self.world, k, r).cpu().tolist()
+        return [[a[q][i] for q in range(self.world)] for i in range(k)]
+
+    def _place(self, j, t, level, g0, starts, hists, split, todo):
+        """Global position t falls in the segment whose sub-buckets have per-rank sizes
+        hists[rank][b] (global base g0, local starts[rank]): record its local split
+        position on every rank if t is a sub-bucket edge, else queue the sub-bucket."""
+        world = self.world
+        base = g0
+        local = list(starts)
+        for b in range(len(hists[0])):
+            tot = sum(h[b] for h in hists)
+            if t < base + tot:
+                if t == base:
+                    break
+                todo.append((j, t, level + 1, base, list(local), [h[b] for h in hists]))
+                return
+            base += tot
+            for r in range(world):
+                local[r] += hists[r][b]
+        split[j] = local
     def _offset_identity(self):
         n = torch.tensor([self.keys.numel()], dtype=torch.int64, device=self.keys.device)
         allv = torch.empty(self.world, dtype=torch.int64, device=n.device)
-        dist.all_gather_into_tensor(allv, n, group=self.group)
+        _all_gather(allv, n, self.group)
         return int(allv[: self.rank].sum())
 
 

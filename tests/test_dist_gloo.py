@@ -32,6 +32,13 @@ class OracleOps:
         ko, vo, offs = oracle.partition_pass(keys, vals, lo, hi)
         return _to_torch(ko, keys), (_to_torch(vo, vals) if vals is not None else None), offs
 
+    def partition_into(self, keys, vals, lo, hi, keys_out, vals_out):
+        ko, vo, offs = oracle.partition_pass(keys, vals, lo, hi)
+        keys_out.copy_(_to_torch(ko, keys))
+        if vals is not None:
+            vals_out.copy_(_to_torch(vo, vals))
+        return [int(x) for x in offs]
+
     def sort(self, keys, vals, b, e):
         ko, vo = oracle.sort(keys, vals, b, e)
         return _to_torch(ko, keys), (_to_torch(vo, vals) if vals is not None else None)
@@ -63,8 +70,11 @@ def _worker(rank, world, port, n_per, kbits, dist_name, q):
 
 
 @pytest.mark.parametrize("world,kbits,dist_name", [(2, 32, "uniform"), (2, 64, "and3"), (3, 32, "and4"),
-                                                   (2, 32, "const")])
+                                                   (2, 32, "const"), (4, 32, "and4"), (3, 64, "const"),
+                                                   (4, 64, "uniform")])
 def test_distributed_sort_matches_global_oracle(world, kbits, dist_name):
+    """The rank outputs concatenate to the global stable sort, and every rank holds
+    exactly its N/G share whatever the skew (exact splitting)."""
     n_per = 3000
     ctx = mp.get_context("spawn")
     q = ctx.Queue()
@@ -81,23 +91,29 @@ def test_distributed_sort_matches_global_oracle(world, kbits, dist_name):
     gv = np.arange(world * n_per, dtype=np.uint64)
     ek, ev = oracle.sort(gk, gv, 0, kbits)
     off = 0
+    N = world * n_per
     for rank, (o, ko, vo, last) in enumerate(parts):
         assert o == off, (rank, o, off)
+        assert len(ko) == (rank + 1) * N // world - rank * N // world, (rank, len(ko))
+        assert last["imbalance"] <= 1.0 + world / N
         assert ko == ek[off:off + len(ko)].tolist()
         assert vo == ev[off:off + len(vo)].tolist()
         off += len(ko)
     assert off == world * n_per
 
 
-def test_assignment_is_contiguous_and_balanced():
-    hist = [10] * 256
-    owner = hdist.assign_buckets(hist, 4)
-    assert owner == sorted(owner) and owner[0] == 0 and owner[-1] == 3
-    assert [owner.count(j) for j in range(4)] == [64, 64, 64, 64]
-    # a single heavy bucket cannot be split at first-digit granularity
-    hist = [0] * 100 + [1000] + [0] * 155
-    owner = hdist.assign_buckets(hist, 8)
-    assert owner == sorted(owner) and owner[100] == 0
-    assert hdist.split_counts([hist], owner, 8)[0] == [1000] + [0] * 7
-    send = hdist.split_counts([[1] * 256, [2] * 256], hdist.assign_buckets([3] * 256, 2), 2)
-    assert send == [[128, 128], [256, 256]]
+def test_split_positions_by_global_index():
+    """_place / the final tie split on hand-made histograms (no processes)."""
+    class S(hdist.DistributedSorter):
+        def __init__(self, world):
+            self.world, self.rank = world, 0
+    s = S(3)
+    # 2 ranks x 3 buckets: sizes [[2,0,4],[1,3,0]] -> global [3,3,4], N = 10
+    hists = [[2, 0, 4], [1, 3, 0]]
+    s.world = 2
+    split = [[0, 0] for _ in range(3)]
+    todo = []
+    s._place(1, 3, 0, 0, [0, 0], hists, split, todo)  # t = 3: edge of bucket 1
+    assert split[1] == [2, 1] and not todo
+    s._place(1, 5, 0, 0, [0, 0], hists, split, todo)  # t = 5: inside bucket 1 (3..6)
+    assert todo == [(1, 5, 1, 3, [2, 1], [0, 3])]
