@@ -79,16 +79,30 @@ constexpr uint32_t DEFAULT_MT_DIV = 4;
 #define HRS_SC_MINB 3
 #endif
 
+// wider records (8-byte keys or values) scatter shape
+#ifndef HRS_SC64_THREADS
+#define HRS_SC64_THREADS 256
+#endif
+#ifndef HRS_SC64_KPT
+#define HRS_SC64_KPT 16
+#endif
+#ifndef HRS_SC64_MINB
+#define HRS_SC64_MINB 2
+#endif
+#ifndef HRS_SC64_NBUF
+#define HRS_SC64_NBUF 1
+#endif
+
 // ------------------------------------------------------------------ compile-time configurations
 
 // scatter: THREADS x KPT records per tile (= the largest KPB); MINB resident CTAs per SM
 template <int KB, int VB>
 struct ScatterCfg {
     static constexpr bool SMALL = (KB == 4 && VB <= 4);
-    static constexpr int THREADS = SMALL ? 256 : 512;
-    static constexpr int KPT = SMALL ? HRS_SC_KPT : 8;  // 256 x 13: two staging buffers + the slot index for three CTAs per SM
-    static constexpr int MINB = SMALL ? HRS_SC_MINB : 1;
-    static constexpr int NBUF = SMALL ? HRS_SC_NBUF : 2;
+    static constexpr int THREADS = SMALL ? 256 : HRS_SC64_THREADS;
+    static constexpr int KPT = SMALL ? HRS_SC_KPT : HRS_SC64_KPT;  // 256 x 13: two staging buffers + the slot index for three CTAs per SM
+    static constexpr int MINB = SMALL ? HRS_SC_MINB : HRS_SC64_MINB;
+    static constexpr int NBUF = SMALL ? HRS_SC_NBUF : HRS_SC64_NBUF;
 };
 #ifndef HRS_HIST_THREADS
 #define HRS_HIST_THREADS 256
@@ -289,8 +303,9 @@ struct Plan {
     uint32_t range_cap = 0;  // CTAs of the hist/scatter grid the temp layout allows
     size_t off_auxk = 0, off_auxv = 0, off_buckets[2] = {0, 0}, off_tot[2] = {0, 0}, off_subrel = 0,
            off_seg_last = 0, off_seg_meta = 0, off_carry = 0, off_tiles = 0, off_tile_pref = 0,
-           off_local[HRS_NUM_CLASSES] = {0}, off_local_fb = 0, off_local_fb2 = 0, total = 0;
-    uint32_t local_fb_cap = 0, local_fb2_cap = 0;
+           off_local[HRS_NUM_CLASSES] = {0}, off_local_wide[HRS_NUM_CLASSES] = {0}, off_local_fb2 = 0, total = 0;
+    uint32_t local_wide_cap[HRS_NUM_CLASSES] = {0}, local_fb2_cap = 0;
+    int wide_top = 0;
 };
 
 size_t align_up(size_t x, size_t a) { return (x + a - 1) / a * a; }
@@ -392,10 +407,18 @@ hrs_status make_plan(Plan &pl, uint64_t n, int kb, int vb, int begin, int end, c
         fb += pl.local_cap[c];
     }
     // entries of more than 19 sort bits whose top bits tie in long runs go to the wide
-    // local sort: at most every entry
-    pl.local_fb_cap = static_cast<uint32_t>(std::min<uint64_t>(fb, 0xFFFFFFFFull));
-    pl.off_local_fb = off;
-    off = align_up(off + sizeof(LocalEntry) * static_cast<size_t>(pl.local_fb_cap), 256);
+    // local sort, to the list of the wide configuration of their size class (every entry
+    // of the single-configuration ablation to its one class)
+    (void)fb;
+    pl.wide_top = max_class(kb, vb);
+    uint64_t wcap[HRS_NUM_CLASSES] = {0};
+    for (int c = 0; c < HRS_NUM_CLASSES; ++c)
+        wcap[pl.single_class >= 0 ? pl.single_class : wide_cfg(c, pl.wide_top)] += pl.local_cap[c];
+    for (int c = 0; c < HRS_NUM_CLASSES; ++c) {
+        pl.local_wide_cap[c] = static_cast<uint32_t>(std::min<uint64_t>(wcap[c], 0xFFFFFFFFull));
+        pl.off_local_wide[c] = off;
+        off = align_up(off + sizeof(LocalEntry) * static_cast<size_t>(pl.local_wide_cap[c]), 256);
+    }
     // entries the counting local sort (classes CNT_LO..CNT_HI) hands to the narrow one
     uint64_t fb2 = 0;
     for (int c = CNT_LO; c <= CNT_HI; ++c) fb2 += pl.local_cap[c];
@@ -617,14 +640,21 @@ struct Runner {
             LocalParams lp;
             local_params(lp, pl, temp, kin, kout, vin, vout);
             Ctl *ctl = at<Ctl>(temp, 0);
-            lp.fb_list = at<LocalEntry>(temp, pl.off_local_fb);
-            lp.fb_count = &ctl->nlocal_fb;
-            lp.fb_cap = pl.local_fb_cap;
+            lp.fb_list = nullptr;
+            lp.fb_count = nullptr;
+            lp.fb_cap = 0;
+            for (int c = 0; c < HRS_NUM_CLASSES; ++c) {
+                lp.wide_list[c] = at<LocalEntry>(temp, pl.off_local_wide[c]);
+                lp.wide_cap[c] = pl.local_wide_cap[c];
+            }
+            lp.wide_count = ctl->nlocal_wide;
+            lp.wide_single = pl.single_class;
+            lp.wide_top = pl.wide_top;
             uint32_t cap = pl.local_cap[C];
-            if (which == LIST_FB) {  // the wide variant sorts what the narrow ones handed over
-                lp.list = lp.fb_list;
-                lp.count = &ctl->nlocal_fb;
-                cap = pl.local_fb_cap;
+            if (which == LIST_FB) {  // the wide variant of configuration C sorts what was handed to it
+                lp.list = lp.wide_list[C];
+                lp.count = &ctl->nlocal_wide[C];
+                cap = pl.local_wide_cap[C];
             } else if (which == LIST_FB2) {  // what the counting variant handed over
                 lp.list = at<LocalEntry>(temp, pl.off_local_fb2);
                 lp.count = &ctl->nlocal_fb2;
@@ -638,7 +668,7 @@ struct Runner {
             hrs_status s = grid_for(fn, LC::THREADS, LST::bytes, dev, sms, &grid);
             if (s) return s;
             grid = static_cast<int>(std::min<uint64_t>(grid, std::max<uint32_t>(cap, 1)));
-            LaunchScope ls(st, 3, which == LIST_FB ? 8 : which == LIST_FB2 ? 9 : C);
+            LaunchScope ls(st, 3, which == LIST_FB ? 10 + C : which == LIST_FB2 ? 9 : C);
             launch_pdl(fn, dim3(grid), dim3(LC::THREADS), LST::bytes, st, lp);
             return last_launch();
         }
@@ -662,14 +692,35 @@ struct Runner {
         return local_variant<C, 0>(pl, temp, st, dev, sms, kin, kout, vin, vout);
     }
 
-    // one wide launch (largest configuration) for whatever the narrow ones handed over;
-    // only needed when more than 19 bits can remain to sort
+    // the wide launches for whatever the narrow ones handed over, one per wide
+    // configuration (wide_cfg: 1024, 2048, largest); only needed when more than 19 bits
+    // can remain to sort
     static hrs_status local_wide(const Plan &pl, void *temp, cudaStream_t st, int dev, int sms, const void *kin,
                                  void *kout, const void *vin, void *vout) {
         if (pl.end - pl.begin <= 19) return HRS_SUCCESS;  // every entry fits a narrow composite
-        if (max_class_t<K, V>() == 7)
-            return local_variant<7, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout, LIST_FB);
-        return local_variant<6, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout, LIST_FB);
+        hrs_status s;
+        if (pl.single_class >= 0) {
+            switch (pl.single_class) {
+                case 0: return local_variant<0, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout, LIST_FB);
+                case 1: return local_variant<1, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout, LIST_FB);
+                case 2: return local_variant<2, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout, LIST_FB);
+                case 3: return local_variant<3, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout, LIST_FB);
+                case 4: return local_variant<4, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout, LIST_FB);
+                case 5: return local_variant<5, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout, LIST_FB);
+                case 6: return local_variant<6, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout, LIST_FB);
+                case 7: return local_variant<7, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout, LIST_FB);
+            }
+            return HRS_ERROR_INVALID_VALUE;
+        }
+        const int cmax = size_class_of(pl.lt);
+        if ((s = local_variant<3, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout, LIST_FB))) return s;
+        if (cmax >= 4 && (s = local_variant<4, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout, LIST_FB))) return s;
+        if (cmax >= 5) {
+            if (max_class_t<K, V>() == 7)
+                return local_variant<7, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout, LIST_FB);
+            return local_variant<6, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout, LIST_FB);
+        }
+        return HRS_SUCCESS;
     }
 
     // the narrow k_local over the entries the counting variant handed over (sizes up to

@@ -99,7 +99,7 @@ struct Ctl {
     unsigned long long alloc[HRS_MAX_PASSES + 2];
     uint32_t nlocal[HRS_NUM_CLASSES];       // entries in local list c
     uint32_t claim[HRS_MAX_PASSES + 2];     // k_scatter tile claims of pass p
-    uint32_t nlocal_fb;                     // entries the narrow local sort handed to the wide one
+    uint32_t nlocal_wide[HRS_NUM_CLASSES];  // entries the narrow local sort handed to the wide one, per configuration
     uint32_t nlocal_fb2;                    // entries the counting local sort handed to the narrow one
     uint32_t overflow;
     uint32_t pad_;
@@ -146,6 +146,10 @@ __host__ __device__ __forceinline__ int size_class_of(uint32_t size) {
 }
 
 __host__ __device__ constexpr size_t align16(size_t x) { return (x + 15) & ~size_t(15); }
+
+// The configuration (size class) of the wide local sort that takes a hand-off of size
+// class c: 1024 records (class 3) for small ones, 2048 (class 4), else the largest.
+__host__ __device__ __forceinline__ int wide_cfg(int c, int top) { return c <= 3 ? 3 : (c == 4 ? 4 : top); }
 
 // Exclusive scan of n <= 288 u32 values in shared memory, in place, by warp 0.
 __device__ __forceinline__ void warp0_exclusive_scan(uint32_t *a, int n) {
@@ -1363,9 +1367,16 @@ struct LocalParams {
     void *vals_out;
     const LocalEntry *list;
     const uint32_t *count;  // entries in the list
-    LocalEntry *fb_list;    // narrow variant: entries handed to the wide variant
+    LocalEntry *fb_list;    // k_local_cnt: entries handed to the narrow k_local
     uint32_t *fb_count;
     uint32_t fb_cap;
+    // narrow k_local: entries handed to the wide variant, one list per wide configuration
+    // (class wide_cfg(size class)); wide_single >= 0: the single-configuration ablation
+    LocalEntry *wide_list[HRS_NUM_CLASSES];
+    uint32_t *wide_count;
+    uint32_t wide_cap[HRS_NUM_CLASSES];
+    int wide_single;
+    int wide_top;  // largest wide configuration
     int begin_bit;
 };
 
@@ -1462,10 +1473,15 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
                                                          : prm.src_vals[SRC_OUT]);
     };
     // the recon variant hands entries of more than 19 sort bits to the wide variant
+    // hand an entry to the wide variant's list of its size
+    auto to_wide = [&](const LocalEntry &en) {
+        const int w = prm.wide_single >= 0 ? prm.wide_single : wide_cfg(size_class_of(en.count), prm.wide_top);
+        const uint32_t slot = atomicAdd(&prm.wide_count[w], 1u);
+        if (slot < prm.wide_cap[w]) prm.wide_list[w][slot] = en;
+    };
     auto mine = [&](const LocalEntry &en) {
         if (!LW::RECON || static_cast<int>(en.hi_bit) - prm.begin_bit <= 32 - IB) return true;
-        const uint32_t slot = atomicAdd(prm.fb_count, 1u);
-        if (slot < prm.fb_cap) prm.fb_list[slot] = en;
+        to_wide(en);
         return false;
     };
     __shared__ uint32_t s_fallback;
@@ -1635,8 +1651,25 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
                     }
                 }
             };
-            passes(true);
-            if (moved) {
+            // more sort bits than the composite holds: the tie runs on the top bits are
+            // sorted by insertion afterwards, and a run longer than RUN_MAX sends the
+            // bucket to the wide variant.  AND-skewed keys make the all-zero top field
+            // such a run: count it first and hand the bucket over before any pass.
+            bool early = false;
+            if (!LW::RECON && sb > tb) {
+                uint32_t z = 0;
+#pragma unroll
+                for (int c = 0; c < KPT; ++c)
+                    z += ((!BAL || c < kpt) && wbase + c * 32 + lane < count && (cv[c] >> IB) == 0) ? 1u : 0u;
+                z = __reduce_add_sync(0xffffffffu, z);
+                if (tid == 0) s_fallback = 0;
+                __syncthreads();
+                if (lane == 0 && z) atomicAdd(&s_fallback, z);
+                __syncthreads();
+                early = s_fallback > RUN_MAX;
+            }
+            if (!early) passes(true);
+            if (!early && moved) {
                 // the composites are distinct (index field), so the passes were all stable
                 // iff they end strictly increasing; otherwise put every composite back at
                 // its index and redo the passes with the rank that is stable by construction
@@ -1664,8 +1697,8 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
                 }
             }
             const K *const ksp = ks + sk.pad;
-            bool fallback = false;
-            if (!LW::RECON && sb > tb) {
+            bool fallback = early;
+            if (!early && !LW::RECON && sb > tb) {
                 // ---- runs that tie on the top bits: insertion sort by (low bits, index);
                 // inside a run the records are in index order (the passes are stable), so
                 // shifting only past strictly greater low bits keeps the sort stable
@@ -1675,14 +1708,23 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
                     for (int c = 0; c < KPT; ++c)
                         if ((!BAL || c < kpt) && active) comp[wbase + c * 32 + lane] = cv[c];
                 }
+                // a run longer than RUN_MAX exists iff some slot e has the same top bits as
+                // slot e + RUN_MAX (the slots are sorted by them): then the bucket goes to
+                // the wide variant without any insertion sort
+                bool longrun = false;
+                for (uint32_t e = tid; e + RUN_MAX < count; e += THREADS)
+                    longrun |= (comp[e] >> IB) == (comp[e + RUN_MAX] >> IB);
                 if (tid == 0) s_fallback = 0;
-                __syncthreads();
+                if (__syncthreads_or(longrun)) {
+                    if (tid == 0) s_fallback = 1;
+                    __syncthreads();
+                }
                 const int lb = sb - tb;
                 const K lmask = lb >= static_cast<int>(8 * sizeof(K)) ? ~K(0) : ((K(1) << lb) - 1);
                 auto low = [&](CT x) -> K {
                     return (ksp[static_cast<uint32_t>(x) & ((1u << IB) - 1u)] >> begin_bit) & lmask;
                 };
-                for (uint32_t e = tid; e + 1 < count; e += THREADS) {
+                for (uint32_t e = tid; e + 1 < count && !s_fallback; e += THREADS) {
                     const CT t = comp[e] >> IB;
                     if ((comp[e + 1] >> IB) != t) continue;
                     if (e > 0 && (comp[e - 1] >> IB) == t) continue;  // not the start of the run
@@ -1716,15 +1758,12 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
             }
             if (fallback) {
                 if (tid == 0) {
-                    const uint32_t slot = atomicAdd(prm.fb_count, 1u);
-                    if (slot < prm.fb_cap) {
-                        LocalEntry en;
-                        en.offs = offs;
-                        en.count = count;
-                        en.hi_bit = static_cast<uint16_t>(hi_bit);
-                        en.src = static_cast<uint16_t>(src);
-                        prm.fb_list[slot] = en;
-                    }
+                    LocalEntry en;
+                    en.offs = offs;
+                    en.count = count;
+                    en.hi_bit = static_cast<uint16_t>(hi_bit);
+                    en.src = static_cast<uint16_t>(src);
+                    to_wide(en);
                 }
             } else if (moved || src != SRC_OUT) {
                 K *const kd = kout + offs;
@@ -1744,9 +1783,12 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
                 }
             }
         } else {
-            // ---- pair path (64-bit keys with more than 51 bits to sort): (key, index)
-            // pairs, the key staging buffer doubles as the sort buffer
+            // ---- pair path (64-bit keys, wide variant): (key, index) pairs, the key
+            // staging buffer doubles as the sort buffer.  The passes use the fast rank;
+            // the result is the stable sort iff (sort bits, index) strictly increase along
+            // the slots, else the passes are redone from the source with the exact rank.
             K *skeys = ks;
+            auto pair_passes = [&](bool fast) {
             for (int lo = begin_bit; lo < hi_bit; lo += 8) {
                 const int width = min(8, hi_bit - lo);
                 const uint32_t mask = (1u << width) - 1u;
@@ -1756,7 +1798,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
 #pragma unroll
                 for (int c = 0; c < KPT; ++c)
                     dg[c] = (wbase + c * 32 + lane) < count ? digit_of(key[c], lo, mask) : INVALID_DIGIT;
-                ranker.rank(dg, kpt, active, ltm, false);
+                ranker.rank(dg, kpt, active, ltm, fast);
                 if (active) {
 #pragma unroll
                     for (int c = 0; c < KPT; ++c) {
@@ -1776,6 +1818,31 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
                             idx[c] = sidx[e];
                         }
                     }
+                }
+            }
+            };
+            pair_passes(true);
+            if (moved) {
+                const K smask = sb >= static_cast<int>(8 * sizeof(K)) ? ~K(0) : ((K(1) << sb) - 1);
+                bool bad = false;
+                if (active) {
+#pragma unroll
+                    for (int c = 0; c < KPT; ++c) {
+                        const uint32_t e = wbase + c * 32 + lane;
+                        if ((!BAL || c < kpt) && e > 0 && e < count) {
+                            const K pa = (skeys[e - 1] >> begin_bit) & smask, pb = (key[c] >> begin_bit) & smask;
+                            bad |= pa > pb || (pa == pb && sidx[e - 1] >= idx[c]);
+                        }
+                    }
+                }
+                if (__syncthreads_or(bad)) {
+#pragma unroll
+                    for (int c = 0; c < KPT; ++c) {
+                        const uint32_t e = wbase + c * 32 + lane;
+                        key[c] = e < count ? ksrc[e] : K(0);  // the source is untouched until the write-out
+                        idx[c] = e;
+                    }
+                    pair_passes(false);
                 }
             }
             if (moved || src != SRC_OUT) {
