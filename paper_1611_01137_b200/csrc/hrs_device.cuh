@@ -48,6 +48,9 @@
 #ifndef HRS_WAIT1
 #define HRS_WAIT1 0  // (measured slower when 1) k_hist / k_scatter: one warp waits on the TMA mbarrier, a CTA barrier releases the others
 #endif
+#ifndef HRS_WIDE64
+#define HRS_WIDE64 1  // measured: c4 AND-2/3/4 -4 to -9 %, uniform unchanged
+#endif
 #ifndef HRS_RANK2
 #define HRS_RANK2 1  // Ranker::rank2 for blocks of >= 256 threads
 #endif
@@ -1479,8 +1482,11 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
         const uint32_t slot = atomicAdd(&prm.wide_count[w], 1u);
         if (slot < prm.wide_cap[w]) prm.wide_list[w][slot] = en;
     };
+    // RECON takes at most 19 sort bits (the composite); with HRS_WIDE64 the narrow
+    // variant for 64-bit keys passes entries of more sort bits straight to the wide one
+    constexpr bool DIRECT = LW::RECON || (HRS_WIDE64 && WIDE == 0 && sizeof(K) == 8);
     auto mine = [&](const LocalEntry &en) {
-        if (!LW::RECON || static_cast<int>(en.hi_bit) - prm.begin_bit <= 32 - IB) return true;
+        if (!DIRECT || static_cast<int>(en.hi_bit) - prm.begin_bit <= 32 - IB) return true;
         to_wide(en);
         return false;
     };
