@@ -241,3 +241,15 @@ def test_errors_on_gpu():
         hrs.check(hrs.lib.hrs_sort_ex(ctypes.c_void_p(t.data_ptr()), ctypes.byref(sz),
                                       ctypes.c_void_p(raw.data_ptr() + 1), ctypes.c_void_p(raw.data_ptr() + 404),
                                       None, None, 10, 4, 0, 0, 32, None, None), "misaligned")
+
+
+@pytest.mark.parametrize("kbits,vbits", [(32, 32), (32, 64), (32, 0), (64, 32)])
+@pytest.mark.parametrize("dist_name", ["uniform", "and2"])
+def test_counting_local_sort_paths(kbits, vbits, dist_name):
+    """2^20 records: one counting pass leaves ~4096-record buckets, so the counting local
+    sort (k_local_cnt) runs -- with key reconstruction ([0, 32) of u32 keys), without it
+    (begin > 0: tie fix-up on gathered low key bits; end < 32: carried upper bits), and
+    with AND-2 keys whose 4-bit counters overflow (hand-off to k_local)."""
+    k, v = _inputs((1 << 20) + 3, kbits, vbits, dist_name, seed=31)
+    for b, e in ((0, kbits), (2, kbits), (0, kbits - 1), (5, kbits - 2)):
+        _run_and_check(k, v, b, e)
