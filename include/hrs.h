@@ -38,9 +38,15 @@
  *              No C++ exception crosses this ABI.
  *   Devices:   the library contains sm_100a code only; on any other device the
  *              calls fail with HRS_ERROR_NO_DEVICE.  There is no CPU fallback.
- *   Threads:   stateless apart from the thread-local last error and per-device
- *              launch-configuration caches; concurrent calls on different streams
- *              with different temp buffers are safe.
+ *   Graphs:    sorts of at most 2^22 records are launch-bound: from the second call
+ *              with identical arguments (every pointer included) the library replays
+ *              a CUDA graph of its launch sequence, captured on a private stream, with
+ *              one cudaGraphLaunch into `stream` (not while `stream` is itself being
+ *              captured; environment HRS_GRAPHS=0 disables it).
+ *   Threads:   stateless apart from the thread-local last error, per-device
+ *              launch-configuration caches and the graph cache (mutex-protected);
+ *              concurrent calls on different streams with different temp buffers
+ *              are safe.
  *   Limits:    n <= HRS_MAX_ITEMS.
  */
 #ifndef HRS_H_

@@ -9,6 +9,7 @@
 
 #include <algorithm>
 #include <cstdint>
+#include <cstdlib>
 #include <cstring>
 #include <mutex>
 #include <type_traits>
@@ -869,6 +870,107 @@ hrs_status block_dispatch(int kb, int vb, const Plan &pl, void *temp, const void
 
 bool aligned(const void *p, size_t a) { return (reinterpret_cast<uintptr_t>(p) % a) == 0; }
 
+// ------------------------------------------------------------------ graph cache (small sorts)
+//
+// A sort enqueues a fixed sequence of ~25 launches whatever its size; below ~2^22
+// records the host's launch submissions take longer than the GPU work.  The second
+// call with identical arguments (sizes, bits, tuning, every pointer, device) captures
+// the sequence on a private stream into a CUDA graph (programmatic-dependent-launch
+// edges included), and that and every later such call replays it with one
+// cudaGraphLaunch into the caller's stream.  (The first call runs directly, which
+// also fills the per-kernel grid cache outside any capture.)  HRS_GRAPHS=0 disables it;
+// per-launch profiling bypasses it.
+#ifndef HRS_GRAPH_MAX_N
+#define HRS_GRAPH_MAX_N (1ull << 22)
+#endif
+struct GraphKey {
+    uint64_t v[16];
+    bool operator==(const GraphKey &o) const { return std::memcmp(v, o.v, sizeof(v)) == 0; }
+};
+struct GraphKeyHash {
+    size_t operator()(const GraphKey &k) const {
+        uint64_t h = 0x9E3779B97F4A7C15ull;
+        for (uint64_t x : k.v) h = (h ^ x) * 0xBF58476D1CE4E5B9ull;
+        return static_cast<size_t>(h ^ (h >> 31));
+    }
+};
+struct GraphEntry {
+    cudaGraphExec_t exec = nullptr;  // null: seen once, not captured yet
+    uint64_t launches = 0;
+    uint64_t stamp = 0;
+};
+std::mutex g_gmu;
+std::unordered_map<GraphKey, GraphEntry, GraphKeyHash> g_graphs;
+std::unordered_map<int, cudaStream_t> g_capture_stream;
+uint64_t g_gstamp = 0;
+constexpr size_t GRAPH_CACHE_MAX = 64;
+
+bool graphs_enabled() {
+    static const bool on = [] {
+        const char *e = std::getenv("HRS_GRAPHS");
+        return !(e && e[0] == '0');
+    }();
+    return on;
+}
+
+// Runs `run(stream)` through the graph cache; returns false when the cache does not
+// apply (then the caller launches directly).
+template <typename F>
+bool via_graph(const GraphKey &key, cudaStream_t stream, int dev, hrs_status *out, F &&run) {
+    std::lock_guard<std::mutex> lk(g_gmu);
+    auto it = g_graphs.find(key);
+    if (it == g_graphs.end()) {
+        if (g_graphs.size() >= GRAPH_CACHE_MAX) {  // evict the least recently used
+            auto lru = g_graphs.begin();
+            for (auto j = g_graphs.begin(); j != g_graphs.end(); ++j)
+                if (j->second.stamp < lru->second.stamp) lru = j;
+            if (lru->second.exec) cudaGraphExecDestroy(lru->second.exec);
+            g_graphs.erase(lru);
+        }
+        GraphEntry e;
+        e.stamp = ++g_gstamp;
+        g_graphs.emplace(key, e);
+        return false;  // first call: direct
+    }
+    GraphEntry &e = it->second;
+    e.stamp = ++g_gstamp;
+    if (!e.exec) {
+        cudaStream_t &cs = g_capture_stream[dev];
+        cudaError_t err = cudaSuccess;
+        if (!cs && (err = cudaStreamCreateWithFlags(&cs, cudaStreamNonBlocking)) != cudaSuccess) {
+            cs = nullptr;
+            return false;
+        }
+        if (cudaStreamBeginCapture(cs, cudaStreamCaptureModeThreadLocal) != cudaSuccess) return false;
+        const uint64_t l0 = g_launches;
+        const hrs_status s = run(cs);
+        cudaGraph_t g = nullptr;
+        err = cudaStreamEndCapture(cs, &g);
+        if (s != HRS_SUCCESS || err != cudaSuccess || !g) {
+            if (g) cudaGraphDestroy(g);
+            cudaGetLastError();
+            return false;  // run directly instead
+        }
+        err = cudaGraphInstantiate(&e.exec, g, 0);
+        cudaGraphDestroy(g);
+        if (err != cudaSuccess) {
+            e.exec = nullptr;
+            cudaGetLastError();
+            return false;
+        }
+        e.launches = g_launches - l0;
+        g_launches = l0;  // counted when the graph runs
+    }
+    const cudaError_t err = cudaGraphLaunch(e.exec, stream);
+    if (err != cudaSuccess) {
+        *out = cuda_fail(err);
+        return true;
+    }
+    g_launches += e.launches;
+    *out = HRS_SUCCESS;
+    return true;
+}
+
 }  // namespace
 
 // ====================================================================== C ABI
@@ -908,8 +1010,35 @@ hrs_status hrs_sort_ex(void *d_temp, size_t *temp_bytes, const void *keys_in, vo
     }
     int dev = 0, sms = 0;
     if ((s = check_device(&dev, &sms))) return s;
-    return sort_dispatch(key_bytes, value_bytes, pl, d_temp, keys_in, keys_out, vals_in, vals_out,
-                         reinterpret_cast<cudaStream_t>(stream), dev, sms);
+    cudaStream_t st = reinterpret_cast<cudaStream_t>(stream);
+    auto run = [&](cudaStream_t on) {
+        return sort_dispatch(key_bytes, value_bytes, pl, d_temp, keys_in, keys_out, vals_in, vals_out, on, dev, sms);
+    };
+    cudaStreamCaptureStatus cap = cudaStreamCaptureStatusNone;
+    if (n > 0 && n <= HRS_GRAPH_MAX_N && !g_prof && graphs_enabled() &&
+        cudaStreamIsCapturing(st, &cap) == cudaSuccess && cap == cudaStreamCaptureStatusNone) {
+        GraphKey key;
+        std::memset(&key, 0, sizeof(key));
+        const hrs_tuning t = tuning ? *tuning : hrs_tuning{};
+        uint64_t *v = key.v;
+        v[0] = static_cast<uint64_t>(dev);
+        v[1] = n;
+        v[2] = static_cast<uint64_t>(key_bytes) | (static_cast<uint64_t>(value_bytes) << 8) |
+               (static_cast<uint64_t>(begin_bit) << 16) | (static_cast<uint64_t>(end_bit) << 24);
+        v[3] = t.local_threshold;
+        v[4] = t.merge_threshold;
+        v[5] = t.keys_per_tile;
+        v[6] = t.local_classes;
+        v[7] = reinterpret_cast<uintptr_t>(keys_in);
+        v[8] = reinterpret_cast<uintptr_t>(keys_out);
+        v[9] = reinterpret_cast<uintptr_t>(vals_in);
+        v[10] = reinterpret_cast<uintptr_t>(vals_out);
+        v[11] = reinterpret_cast<uintptr_t>(d_temp);
+        v[12] = *temp_bytes;
+        hrs_status gs = HRS_SUCCESS;
+        if (via_graph(key, st, dev, &gs, run)) return gs;
+    }
+    return run(st);
 }
 
 hrs_status hrs_sort_keys_u32(void *t, size_t *tb, const uint32_t *ki, uint32_t *ko, uint64_t n, int b, int e,

@@ -253,3 +253,28 @@ def test_counting_local_sort_paths(kbits, vbits, dist_name):
     k, v = _inputs((1 << 20) + 3, kbits, vbits, dist_name, seed=31)
     for b, e in ((0, kbits), (2, kbits), (0, kbits - 1), (5, kbits - 2)):
         _run_and_check(k, v, b, e)
+
+
+def test_graph_replay_follows_new_data():
+    """Small sorts replay a captured CUDA graph from the second identical call on: the
+    replays must sort whatever the buffers hold now (new data every call), for several
+    sizes and with HRS_GRAPHS' cache keyed on every argument."""
+    import paper_1611_01137_b200 as hrs
+    for n, kbits, vbits in ((70001, 32, 32), (1 << 20, 32, 0), (300000, 64, 64)):
+        kd = torch.empty(n, dtype=torch.uint32 if kbits == 32 else torch.uint64, device=DEV)
+        vd = torch.empty(n, dtype=torch.uint32 if vbits == 32 else torch.uint64, device=DEV) if vbits else None
+        ko, vo = torch.empty_like(kd), (torch.empty_like(vd) if vbits else None)
+        temp = torch.empty(hrs.temp_bytes(n, kbits // 8, vbits // 8), dtype=torch.uint8, device=DEV)
+        l0 = hrs.launch_count()
+        for i, dist in enumerate(("uniform", "and3", "uniform", "and2")):
+            k, v = _inputs(n, kbits, vbits, dist, seed=100 + i)
+            kd.copy_(k.to(DEV))
+            if vbits:
+                vd.copy_(v.to(DEV))
+            hrs.sort(kd, vd, keys_out=ko, values_out=vo, temp=temp)
+            torch.cuda.synchronize()
+            ek, ev = oracle.sort(k, v, 0, kbits)
+            assert np.array_equal(_np(ko), ek), (n, i)
+            if vbits:
+                assert np.array_equal(_np(vo), ev), (n, i)
+        assert hrs.launch_count() - l0 >= 4 * 10  # replays still count their kernels
