@@ -117,3 +117,29 @@ def test_large_random_values_slice_parity():
     ek, ev = oracle.sort(k, v, 0, 32)
     assert np.array_equal(oracle._u64(ko.cpu()), ek)
     assert np.array_equal(oracle._u64(vo.cpu()), ev)
+
+
+def test_more_than_2_31_records():
+    """n = 2^31 + 12345 u32/u32 (48 GB with outputs and temp): 64-bit bucket and tile
+    offsets, record indices past 2^31.  O(n) certificate, chunked to bound memory."""
+    import paper_1611_01137_b200 as hrs
+    n = (1 << 31) + 12345
+    kd = gen.keys(n, 32, "uniform", device=DEV)
+    vd = gen.values(n, 32, "index", device=DEV)
+    temp = torch.empty(hrs.temp_bytes(n, 4, 4), dtype=torch.uint8, device=DEV)
+    ko, vo = hrs.sort(kd, vd, temp=temp)
+    torch.cuda.synchronize()
+    st = hrs.get_stats(temp)
+    del temp
+    assert st["counting_passes"] == 3 and st["overflow"] == 0
+    ki = kd.view(torch.int32)
+    C = 1 << 27
+    for a in range(0, n, C):
+        b = min(n, a + C + 1)  # one element of overlap with the next chunk
+        idx = vo[a:b].view(torch.int32).to(torch.int64) & 0xFFFFFFFF
+        assert int(idx.max()) < n
+        assert torch.equal(ki[idx], ko[a:b].view(torch.int32)), "keys_out != keys_in[vals_out]"
+        sk = ko[a:b].view(torch.int32).to(torch.int64) & 0xFFFFFFFF
+        ok = (sk[:-1] < sk[1:]) | ((sk[:-1] == sk[1:]) & (idx[:-1] < idx[1:]))
+        assert bool(ok.all()), f"order/stability violated near {a}"
+        del idx, sk, ok
