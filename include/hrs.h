@@ -144,6 +144,24 @@ uint32_t hrs_max_keys_per_tile(int key_bytes, int value_bytes);
 /* Default tuning for the key/value widths (written to *out). */
 hrs_status hrs_default_tuning(int key_bytes, int value_bytes, hrs_tuning *out);
 
+/* ---- signed and floating-point keys (the paper's order-preserving
+ * bijections) ----
+ * Stable sort of n keys of `kind` by their whole value (no bit range), values moved along:
+ *   HRS_KEY_UINT:  unsigned (as hrs_sort_ex over [0, 8 * key_bytes));
+ *   HRS_KEY_INT:   two's-complement signed;
+ *   HRS_KEY_FLOAT: IEEE-754 binary32 (key_bytes 4) / binary64 (8) in the total order
+ *                  -NaN < -inf < ... < -0.0 < +0.0 < ... < +inf < +NaN (NaNs of one sign
+ *                  ordered by their bit patterns: larger payload further out).
+ * Layout, ownership, async behaviour and errors as hrs_sort_ex.  Implementation: a kernel
+ * maps the keys through the bijection into a region of d_temp (ints: flip the sign bit;
+ * floats: flip every bit of a negative key, the sign bit of a positive one), the unsigned
+ * sort runs on that copy, and the inverse map runs in place on keys_out.  Temp therefore
+ * holds the unsigned sort's temp plus n * key_bytes (two-phase size query as usual). */
+typedef enum { HRS_KEY_UINT = 0, HRS_KEY_INT = 1, HRS_KEY_FLOAT = 2 } hrs_key_kind;
+hrs_status hrs_sort_typed(void *d_temp, size_t *temp_bytes, const void *keys_in, void *keys_out,
+                          const void *vals_in, void *vals_out, uint64_t n, int key_bytes, int value_bytes,
+                          hrs_key_kind kind, hrs_stream_t stream);
+
 /* ---- building blocks (kernel-level tests, the distributed driver) ---- */
 
 /* Histogram of digit bits [lo_bit, hi_bit) (1 <= hi_bit - lo_bit <= 8) over all n keys:

@@ -117,3 +117,31 @@ def sort(keys, vals=None, begin_bit: int = 0, end_bit: int | None = None, key_bi
 
 
 from .plan import classify_bucket, simulate_msd, size_class  # noqa: E402,F401
+
+
+def sort_typed(keys, vals, kind: str):
+    """Stable sort of signed ('int') or IEEE-754 ('float') keys by value, the order
+    include/hrs.h documents for hrs_sort_typed (the paper's P:907-918 bijections define
+    the GPU side; this is the plain definition, independent of them):
+      int:   two's-complement numeric order;
+      float: -NaN (larger bit pattern first) < -inf < ... < -0.0 < +0.0 < ... < +inf <
+             +NaN (smaller bit pattern first); equal keys keep input order.
+    keys: numpy int32/int64/float32/float64 array; returns (keys_out, vals_out)."""
+    k = np.asarray(keys)
+    v = None if vals is None else np.asarray(vals)
+    idx = np.arange(k.size)
+    if kind == "int":
+        order = np.argsort(k, kind="stable")
+    elif kind == "float":
+        ub = np.uint32 if k.dtype == np.float32 else np.uint64
+        bits = k.view(ub).astype(np.uint64)
+        sign = (bits >> np.uint64(8 * k.itemsize - 1)).astype(np.int64)
+        nan = np.isnan(k)
+        neg_nan, pos_nan, num = idx[nan & (sign == 1)], idx[nan & (sign == 0)], idx[~nan]
+        order = np.concatenate([
+            neg_nan[np.lexsort((neg_nan, ~bits[neg_nan]))],       # further from zero first
+            num[np.lexsort((num, 1 - sign[num], k[num]))],       # value, then -0.0 before +0.0
+            pos_nan[np.lexsort((pos_nan, bits[pos_nan]))]]).astype(np.int64)
+    else:
+        raise ValueError(kind)
+    return k[order], (None if v is None else v[order])

@@ -19,6 +19,8 @@ __all__ = ["sort", "temp_bytes", "get_stats", "digit_histogram", "partition_pass
            "default_tuning", "max_local_threshold", "max_keys_per_tile", "lib"]
 
 _KEY_DTYPES = {torch.uint32: 4, torch.uint64: 8}
+# signed / floating-point keys: (key bytes, hrs_key_kind) -- hrs_sort_typed
+_TYPED_KEYS = {torch.int32: (4, 1), torch.int64: (8, 1), torch.float32: (4, 2), torch.float64: (8, 2)}
 
 
 def _nbytes(t: torch.Tensor | None, what: str) -> int:
@@ -80,6 +82,9 @@ def sort(keys: torch.Tensor, values: torch.Tensor | None = None, begin_bit: int 
     Enqueued on `stream` (default: torch's current stream); nothing synchronises.
     """
     _check_tensor(keys, "keys")
+    if keys.dtype in _TYPED_KEYS:
+        return sort_typed(keys, values, keys_out=keys_out, values_out=values_out, temp=temp, stream=stream,
+                          begin_bit=begin_bit, end_bit=end_bit, tuning=tuning)
     kb = _nbytes(keys, "keys")
     vb = 0
     if values is not None:
@@ -104,6 +109,45 @@ def sort(keys: torch.Tensor, values: torch.Tensor | None = None, begin_bit: int 
         check(lib.hrs_sort_ex(_ptr(temp), ctypes.byref(sz), _ptr(keys), _ptr(keys_out), _ptr(values),
                               _ptr(values_out), n, kb, vb, begin_bit, end_bit, _tuning(tuning), _stream(stream)),
               "hrs_sort_ex")
+    return keys_out, (values_out if values is not None else None)
+
+
+def typed_temp_bytes(n: int, key_bytes: int, value_bytes: int, kind: int) -> int:
+    sz = ctypes.c_size_t(0)
+    check(lib.hrs_sort_typed(None, ctypes.byref(sz), None, None, None, None, n, key_bytes, value_bytes, kind, None),
+          "hrs_sort_typed")
+    return sz.value
+
+
+def sort_typed(keys: torch.Tensor, values: torch.Tensor | None = None, *, keys_out=None, values_out=None, temp=None,
+               stream=None, begin_bit: int = 0, end_bit: int | None = None, tuning=None):
+    """Stable sort of int32/int64 (two's complement) or float32/float64 (IEEE-754 total
+    order, -0.0 < +0.0, NaNs at the ends by sign) keys by their whole value, with
+    uint32/uint64 values moved along."""
+    _check_tensor(keys, "keys")
+    if keys.dtype not in _TYPED_KEYS:
+        raise TypeError(f"keys must be int32/int64/float32/float64 here, got {keys.dtype}")
+    kb, kind = _TYPED_KEYS[keys.dtype]
+    if begin_bit != 0 or (end_bit is not None and end_bit != 8 * kb) or tuning is not None:
+        raise ValueError("signed/float keys sort by the whole key (no bit range, no tuning)")
+    vb = 0
+    if values is not None:
+        _check_tensor(values, "values")
+        vb = _nbytes(values, "values")
+        if values.numel() != keys.numel():
+            raise ValueError("keys and values differ in length")
+    n = keys.numel()
+    if keys_out is None:
+        keys_out = torch.empty_like(keys)
+    if values is not None and values_out is None:
+        values_out = torch.empty_like(values)
+    tb = typed_temp_bytes(n, kb, vb, kind)
+    if temp is None or temp.numel() < tb:
+        temp = alloc_temp(tb, keys.device)
+    sz = ctypes.c_size_t(temp.numel())
+    with torch.cuda.device(keys.device):
+        check(lib.hrs_sort_typed(_ptr(temp), ctypes.byref(sz), _ptr(keys), _ptr(keys_out), _ptr(values),
+                                 _ptr(values_out), n, kb, vb, kind, _stream(stream)), "hrs_sort_typed")
     return keys_out, (values_out if values is not None else None)
 
 
@@ -139,6 +183,9 @@ def partition_pass(keys: torch.Tensor, values: torch.Tensor | None, lo_bit: int,
                    temp: torch.Tensor | None = None, stream=None):
     """One stable counting pass on digit bits [lo_bit, hi_bit): (keys_out, values_out, offsets[r+1])."""
     _check_tensor(keys, "keys")
+    if keys.dtype in _TYPED_KEYS:
+        return sort_typed(keys, values, keys_out=keys_out, values_out=values_out, temp=temp, stream=stream,
+                          begin_bit=begin_bit, end_bit=end_bit, tuning=tuning)
     kb = _nbytes(keys, "keys")
     vb = 0
     if values is not None:

@@ -1041,6 +1041,58 @@ hrs_status hrs_sort_ex(void *d_temp, size_t *temp_bytes, const void *keys_in, vo
     return run(st);
 }
 
+hrs_status hrs_sort_typed(void *d_temp, size_t *temp_bytes, const void *keys_in, void *keys_out, const void *vals_in,
+                          void *vals_out, uint64_t n, int key_bytes, int value_bytes, hrs_key_kind kind,
+                          hrs_stream_t stream) {
+    if (!temp_bytes) return HRS_ERROR_INVALID_VALUE;
+    if (kind != HRS_KEY_UINT && kind != HRS_KEY_INT && kind != HRS_KEY_FLOAT) return HRS_ERROR_INVALID_VALUE;
+    if (key_bytes != 4 && key_bytes != 8) return HRS_ERROR_INVALID_VALUE;
+    const int kbits = 8 * key_bytes;
+    if (kind == HRS_KEY_UINT)
+        return hrs_sort_ex(d_temp, temp_bytes, keys_in, keys_out, vals_in, vals_out, n, key_bytes, value_bytes, 0,
+                           kbits, nullptr, stream);
+    // temp = [mapped keys: n * key_bytes, 256-aligned | the unsigned sort's temp]
+    size_t inner = 0;
+    hrs_status s = hrs_sort_ex(nullptr, &inner, nullptr, nullptr, nullptr, nullptr, n, key_bytes, value_bytes, 0,
+                               kbits, nullptr, stream);
+    if (s) return s;
+    const size_t mapped = align_up(static_cast<size_t>(n) * key_bytes, 256);
+    if (!d_temp) {
+        *temp_bytes = mapped + inner;
+        return HRS_SUCCESS;
+    }
+    if (*temp_bytes < mapped + inner) return HRS_ERROR_TEMP_TOO_SMALL;
+    if (!aligned(d_temp, 256)) return HRS_ERROR_INVALID_VALUE;
+    if (n == 0) return HRS_SUCCESS;
+    if (!keys_in || !keys_out) return HRS_ERROR_INVALID_VALUE;
+    if (!aligned(keys_in, key_bytes) || !aligned(keys_out, key_bytes)) return HRS_ERROR_INVALID_VALUE;
+    if (overlap(keys_in, n * key_bytes, d_temp, *temp_bytes) || overlap(keys_out, n * key_bytes, d_temp, *temp_bytes) ||
+        (value_bytes && (overlap(vals_in, n * value_bytes, d_temp, mapped) || overlap(vals_out, n * value_bytes, d_temp, mapped))))
+        return HRS_ERROR_ALIASING;
+    int dev = 0, sms = 0;
+    if ((s = check_device(&dev, &sms))) return s;
+    cudaStream_t st = reinterpret_cast<cudaStream_t>(stream);
+    void *mk = d_temp;
+    void *sort_temp = static_cast<unsigned char *>(d_temp) + mapped;
+    const int grid = static_cast<int>(std::min<uint64_t>((n + 255) / 256, static_cast<uint64_t>(sms) * 8));
+    auto map = [&](const void *in, void *out, int inv) -> hrs_status {
+        LaunchScope ls(st, 4, inv);
+        if (key_bytes == 4)
+            launch_pdl(k_key_map<uint32_t>, dim3(grid), dim3(256), 0, st, static_cast<const uint32_t *>(in),
+                       static_cast<uint32_t *>(out), n, static_cast<int>(kind), inv);
+        else
+            launch_pdl(k_key_map<uint64_t>, dim3(grid), dim3(256), 0, st, static_cast<const uint64_t *>(in),
+                       static_cast<uint64_t *>(out), n, static_cast<int>(kind), inv);
+        return last_launch();
+    };
+    if ((s = map(keys_in, mk, 0))) return s;
+    size_t tb = *temp_bytes - mapped;
+    if ((s = hrs_sort_ex(sort_temp, &tb, mk, keys_out, vals_in, vals_out, n, key_bytes, value_bytes, 0, kbits, nullptr,
+                         stream)))
+        return s;
+    return map(keys_out, keys_out, 1);
+}
+
 hrs_status hrs_sort_keys_u32(void *t, size_t *tb, const uint32_t *ki, uint32_t *ko, uint64_t n, int b, int e,
                              hrs_stream_t s) {
     return hrs_sort_ex(t, tb, ki, ko, nullptr, nullptr, n, 4, 0, b, e, nullptr, s);

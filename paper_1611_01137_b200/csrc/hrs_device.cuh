@@ -624,6 +624,25 @@ __global__ void k_init(InitParams prm) {
     }
 }
 
+// Order-preserving bijections of signed / IEEE-754 keys onto unsigned ones:
+// kind 1 (two's complement): flip the sign bit; kind 2 (float): a negative key (sign bit
+// set) has every bit flipped, a positive one only its sign bit.  k_key_map applies the map
+// (inv = 0) from `in` to `out`, or its inverse (inv = 1), which may run in place.
+template <typename K>
+__global__ void k_key_map(const K *in, K *out, uint64_t n, int kind, int inv) {
+    pdl_wait();
+    constexpr K SIGN = K(1) << (8 * sizeof(K) - 1);
+    const uint64_t stride = static_cast<uint64_t>(gridDim.x) * blockDim.x;
+    for (uint64_t i = static_cast<uint64_t>(blockIdx.x) * blockDim.x + threadIdx.x; i < n; i += stride) {
+        const K x = in[i];
+        K y;
+        if (kind == 1) y = x ^ SIGN;
+        else if (!inv) y = (x & SIGN) ? ~x : (x ^ SIGN);
+        else y = (x & SIGN) ? (x ^ SIGN) : ~x;
+        out[i] = y;
+    }
+}
+
 template <typename T>
 __global__ void k_copy(const T *__restrict__ in, T *__restrict__ out, uint64_t n) {
     const uint64_t stride = static_cast<uint64_t>(gridDim.x) * blockDim.x;

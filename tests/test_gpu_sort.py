@@ -278,3 +278,27 @@ def test_graph_replay_follows_new_data():
             if vbits:
                 assert np.array_equal(_np(vo), ev), (n, i)
         assert hrs.launch_count() - l0 >= 4 * 10  # replays still count their kernels
+
+
+@pytest.mark.parametrize("dtype,vbits", [(torch.int32, 32), (torch.int64, 64), (torch.float32, 32),
+                                         (torch.float64, 0), (torch.float32, 64)])
+@pytest.mark.parametrize("n", [1, 1000, 70001, (1 << 20) + 9])
+def test_typed_keys(dtype, vbits, n):
+    """Signed and IEEE-754 keys (hrs_sort_typed) against the oracle's
+    plain definition of their order: random bit patterns (so NaNs with every payload,
+    ±inf, ±0, denormals and int min/max occur) plus AND-3 skew, bit-exact keys and values."""
+    import paper_1611_01137_b200 as hrs
+    kb = 32 if dtype in (torch.int32, torch.float32) else 64
+    kind = "int" if dtype in (torch.int32, torch.int64) else "float"
+    for dist in ("uniform", "and3"):
+        bits = gen.keys(n, kb, dist, seed=41)
+        k = bits.view(dtype)
+        v = gen.values(n, vbits, "index") if vbits else None
+        ko, vo = hrs.sort(k.to(DEV), v.to(DEV) if vbits else None)
+        torch.cuda.synchronize()
+        kn = k.numpy() if dtype != torch.int32 else k.numpy()
+        ek, ev = oracle.sort_typed(kn, None if v is None else oracle._u64(v), kind)
+        ub = np.uint32 if kb == 32 else np.uint64
+        assert np.array_equal(ko.cpu().numpy().view(ub), ek.view(ub)), (dtype, n, dist)
+        if vbits:
+            assert np.array_equal(oracle._u64(vo.cpu()), ev), (dtype, n, dist)

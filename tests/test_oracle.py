@@ -232,3 +232,41 @@ def test_uniform_structure_prediction():
     r = plan.simulate_msd(k, None, 0, 32, 6144, 3000, 4096)
     assert r.counting_passes == 1 and r.local_buckets == 256 and r.merged_groups == 0
     assert plan.bytes_min(r, 4, 0) == 20 * n
+
+
+def test_sort_typed_against_comparison_sort():
+    """oracle.sort_typed (numpy) against a pure-Python stable comparison sort written from
+    the documented order, on small inputs with the special values (±0, ±inf, NaN payloads,
+    denormals, int min/max)."""
+    import functools
+    import struct
+    rng = np.random.default_rng(5)
+    ints = np.concatenate([rng.integers(-2**31, 2**31, 300), [-2**31, 2**31 - 1, 0, -1, 1, 0, -2**31]]).astype(np.int32)
+    ek, ev = oracle.sort_typed(ints, np.arange(ints.size), "int")
+    pairs = sorted(zip(ints.tolist(), range(ints.size)))  # (value, index) = stable numeric order
+    assert ek.tolist() == [p[0] for p in pairs] and ev.tolist() == [p[1] for p in pairs]
+
+    specials = [0.0, -0.0, np.inf, -np.inf, 1e-40, -1e-40, 1.5, -1.5, 0.0, -0.0]
+    nans = [struct.unpack("<f", struct.pack("<I", b))[0] for b in (0x7FC00000, 0x7F800001, 0xFFC00000, 0xFF800001)]
+    fl = np.concatenate([rng.standard_normal(200), specials, nans, specials]).astype(np.float32)
+    bits = fl.view(np.uint32).tolist()
+
+    def rank(i):  # documented total order as a tuple
+        b = bits[i]
+        neg, isnan = b >> 31, (b & 0x7F800000) == 0x7F800000 and (b & 0x7FFFFF) != 0
+        if isnan:
+            return (0, -b, i) if neg else (3, b, i)
+        return (1 if neg else 2, float(fl[i]), i)
+
+    def cmp(i, j):
+        a, c = rank(i), rank(j)
+        if a[0] != c[0]:
+            return -1 if a[0] < c[0] else 1
+        if a[1] != c[1]:
+            return -1 if a[1] < c[1] else 1
+        return -1 if i < j else (1 if i > j else 0)
+
+    want = sorted(range(fl.size), key=functools.cmp_to_key(cmp))
+    gk, gv = oracle.sort_typed(fl, np.arange(fl.size), "float")
+    assert gv.tolist() == want
+    assert gk.view(np.uint32).tolist() == [bits[i] for i in want]
