@@ -414,7 +414,7 @@ hrs_status make_plan(Plan &pl, uint64_t n, int kb, int vb, int begin, int end, c
     pl.wide_top = max_class(kb, vb);
     uint64_t wcap[HRS_NUM_CLASSES] = {0};
     for (int c = 0; c < HRS_NUM_CLASSES; ++c)
-        wcap[pl.single_class >= 0 ? pl.single_class : wide_cfg(c, pl.wide_top)] += pl.local_cap[c];
+        wcap[pl.single_class >= 0 ? pl.single_class : wide_cfg(c, pl.wide_top, kb == 8)] += pl.local_cap[c];
     for (int c = 0; c < HRS_NUM_CLASSES; ++c) {
         pl.local_wide_cap[c] = static_cast<uint32_t>(std::min<uint64_t>(wcap[c], 0xFFFFFFFFull));
         pl.off_local_wide[c] = off;
@@ -694,7 +694,7 @@ struct Runner {
     }
 
     // the wide launches for whatever the narrow ones handed over, one per wide
-    // configuration (wide_cfg: 1024, 2048, largest); only needed when more than 19 bits
+    // configuration (wide_cfg: 1024, 2048, [4096, 4608 for 64-bit keys,] largest); only needed when more than 19 bits
     // can remain to sort
     static hrs_status local_wide(const Plan &pl, void *temp, cudaStream_t st, int dev, int sms, const void *kin,
                                  void *kout, const void *vin, void *vout) {
@@ -716,6 +716,12 @@ struct Runner {
         const int cmax = size_class_of(pl.lt);
         if ((s = local_variant<3, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout, LIST_FB))) return s;
         if (cmax >= 4 && (s = local_variant<4, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout, LIST_FB))) return s;
+        if (HRS_WIDE_MID && KB == 8 && cmax >= 5 && max_class_t<K, V>() > 5 &&
+            (s = local_variant<5, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout, LIST_FB)))
+            return s;
+        if (HRS_WIDE_MID && KB == 8 && cmax >= 6 && max_class_t<K, V>() > 6 &&
+            (s = local_variant<6, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout, LIST_FB)))
+            return s;
         if (cmax >= 5) {
             if (max_class_t<K, V>() == 7)
                 return local_variant<7, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout, LIST_FB);

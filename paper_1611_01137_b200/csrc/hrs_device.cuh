@@ -151,8 +151,17 @@ __host__ __device__ __forceinline__ int size_class_of(uint32_t size) {
 __host__ __device__ constexpr size_t align16(size_t x) { return (x + 15) & ~size_t(15); }
 
 // The configuration (size class) of the wide local sort that takes a hand-off of size
-// class c: 1024 records (class 3) for small ones, 2048 (class 4), else the largest.
-__host__ __device__ __forceinline__ int wide_cfg(int c, int top) { return c <= 3 ? 3 : (c == 4 ? 4 : top); }
+// class c: 1024 records (class 3) for small ones, 2048 (class 4), else the largest --
+// except for 64-bit keys (mid = 1), where classes 5 and 6 keep their own configuration
+// (4096 / 4608 records): measured on B200, c4 AND-2 16.39 -> 15.58 ms, AND-3 17.33 ->
+// 16.71 ms, uniform unchanged; for 32-bit keys the two extra launches only cost latency
+// (2^20 keys-only 90.8 -> 96.2 us), so they keep the largest.
+#ifndef HRS_WIDE_MID
+#define HRS_WIDE_MID 1
+#endif
+__host__ __device__ __forceinline__ int wide_cfg(int c, int top, bool mid) {
+    return c <= 3 ? 3 : (c == 4 ? 4 : (HRS_WIDE_MID && mid ? (c < top ? c : top) : top));
+}
 
 // Exclusive scan of n <= 288 u32 values in shared memory, in place, by warp 0.
 __device__ __forceinline__ void warp0_exclusive_scan(uint32_t *a, int n) {
@@ -1505,7 +1514,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
     // the recon variant hands entries of more than 19 sort bits to the wide variant
     // hand an entry to the wide variant's list of its size
     auto to_wide = [&](const LocalEntry &en) {
-        const int w = prm.wide_single >= 0 ? prm.wide_single : wide_cfg(size_class_of(en.count), prm.wide_top);
+        const int w = prm.wide_single >= 0 ? prm.wide_single : wide_cfg(size_class_of(en.count), prm.wide_top, sizeof(K) == 8);
         const uint32_t slot = atomicAdd(&prm.wide_count[w], 1u);
         if (slot < prm.wide_cap[w]) prm.wide_list[w][slot] = en;
     };
