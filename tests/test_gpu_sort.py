@@ -302,3 +302,14 @@ def test_typed_keys(dtype, vbits, n):
         assert np.array_equal(ko.cpu().numpy().view(ub), ek.view(ub)), (dtype, n, dist)
         if vbits:
             assert np.array_equal(oracle._u64(vo.cpu()), ev), (dtype, n, dist)
+
+
+@pytest.mark.parametrize("kbits,vbits", [(64, 0), (64, 32), (64, 64)])
+@pytest.mark.parametrize("n", [786431, (1 << 20) + 5, 1572869])
+def test_wide_configurations_64bit(kbits, vbits, n):
+    """One counting pass leaves 256 buckets of ~n/256 records with 56 sort bits, which
+    the 64-bit local sort hands to the wide variant: mean 3072 / 4096 / 6144 records put
+    them in the wide lists of size class 5 (<= 4096), 6 (<= 4608) and the largest."""
+    for dist in ("uniform", "and2"):
+        k, v = _inputs(n, kbits, vbits, dist, seed=n % 1000 + kbits + vbits)
+        _run_and_check(k, v, 0, kbits)
