@@ -328,7 +328,7 @@ def run_e2e(torch, hrs, keys, vals, temp, args, n, kb, vb):
     for i in range(2):
         step(i)
     torch.cuda.synchronize()
-    k = max(4, min(args.steps, 8))
+    k = max(4, args.steps)  # the same K as the device-timed steps (at least 4)
     t0, t1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
     t0.record(s_in)
     s_out.wait_event(t0)
