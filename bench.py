@@ -162,7 +162,8 @@ def run_hrs(args):
     n = 1 << logn
     kb, vb = kbits // 8, vbits // 8
     pg = None
-    if world > 1:
+    use_dist = world > 1 or args.force_dist
+    if use_dist:
         import torch.distributed as dist
         dist.init_process_group("nccl", device_id=dev)
         pg = dist.group.WORLD
@@ -172,7 +173,7 @@ def run_hrs(args):
     vals = gen.values(n, vbits, "index", start=rank * n, device=dev) if vbits else None
     stream = torch.cuda.current_stream()
 
-    if world > 1:
+    if use_dist:
         from paper_1611_01137_b200 import dist as hdist
         sorter = hdist.DistributedSorter(keys, vals, group=pg)
         step = sorter.step
@@ -226,7 +227,11 @@ def run_hrs(args):
            "gpu_launches": launches, "clocks": clocks,
            "step_ms": {"median": statistics.median(step_ms), "min": min(step_ms), "max": max(step_ms)}}
 
-    if world == 1:
+    if use_dist:
+        out["exchange"] = run_exchange(torch, sorter, pg, dev, kb, vb)
+        if not args.no_e2e:
+            out["e2e"] = run_e2e_dist(torch, sorter, pg, args, n, dev)
+    else:
         st = hrs.get_stats(temp)
         bmin = st["bytes_min"]
         out["sort_roofline"] = {
@@ -276,6 +281,82 @@ def run_hrs(args):
     if pg is not None:
         torch.distributed.destroy_process_group()
     return 0
+
+
+def _max_over_ranks(torch, x, pg, dev):
+    if pg is None:
+        return x
+    t = torch.tensor([x], dtype=torch.float64, device=dev)
+    torch.distributed.all_reduce(t, op=torch.distributed.ReduceOp.MAX, group=pg)
+    return float(t.item())
+
+
+def run_exchange(torch, sorter, pg, dev, kb, vb, reps=3):
+    """The NCCL all-to-all of the distributed sort (step 4) against NVLink: bytes this
+    rank sends to other ranks / the exchange's CUDA-event time, max time over ranks."""
+    sorter.time_exchange = True
+    ms = []
+    for _ in range(reps):
+        sorter.step()
+        torch.cuda.synchronize()
+        e0, e1 = sorter.exchange_events
+        ms.append(e0.elapsed_time(e1))
+    sorter.time_exchange = False
+    me = sorter.rank
+    sent = sum(c for j, c in enumerate(sorter.last["send"]) if j != me) * (kb + vb)
+    recv = sum(c for j, c in enumerate(sorter.last["recv"]) if j != me) * (kb + vb)
+    t = _max_over_ranks(torch, statistics.median(ms), pg, dev)
+    peak = 900.0  # NVLink 5 per direction per GPU (GB/s), nominal
+    ach = sent / (t * 1e-3) / 1e9 if t > 0 else 0.0
+    return {"bound": "nvlink", "ms": t, "bytes_sent_to_peers": sent, "bytes_recv_from_peers": recv,
+            "achieved": ach, "peak": peak, "unit": "GB/s", "frac": ach / peak, "peak_source": "nominal",
+            "imbalance": sorter.last.get("imbalance"), "refine_levels": sorter.last.get("refine_levels"),
+            "note": "rank 0's peer bytes over the max-over-ranks all-to-all time (keys + values)"}
+
+
+def run_e2e_dist(torch, sorter, pg, args, n, dev):
+    """End to end at N GPUs: every step copies this rank's shard H2D from pinned memory
+    into the sorter's input tensors, runs the distributed sort (hrs.dist), and copies
+    this rank's sorted slice D2H; CUDA events on the current stream, max over ranks."""
+    hk = torch.empty(sorter.keys.shape, dtype=sorter.keys.dtype, pin_memory=True)
+    hk.copy_(sorter.keys)
+    hv = None
+    if sorter.vals is not None:
+        hv = torch.empty(sorter.vals.shape, dtype=sorter.vals.dtype, pin_memory=True)
+        hv.copy_(sorter.vals)
+    hko = torch.empty(2 * n, dtype=sorter.keys.dtype, pin_memory=True)
+    hvo = torch.empty(2 * n, dtype=sorter.vals.dtype, pin_memory=True) if hv is not None else None
+    k = max(4, args.steps)
+    stream = torch.cuda.current_stream()
+
+    def step():
+        sorter.keys.copy_(hk, non_blocking=True)
+        if hv is not None:
+            sorter.vals.copy_(hv, non_blocking=True)
+        ko, vo, _ = sorter.step()
+        hko[:ko.numel()].copy_(ko, non_blocking=True)
+        if vo is not None:
+            hvo[:vo.numel()].copy_(vo, non_blocking=True)
+        return ko.numel()
+
+    step()
+    torch.cuda.synchronize()
+    if pg is not None:
+        torch.distributed.barrier(group=pg)
+    t0, t1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+    t0.record(stream)
+    got = 0
+    for _ in range(k):
+        got = step()
+    t1.record(stream)
+    torch.cuda.synchronize()
+    t = _max_over_ranks(torch, t0.elapsed_time(t1) / k, pg, dev)
+    world = sorter.world
+    nb_in = n * (sorter.keys.element_size() + (sorter.vals.element_size() if hv is not None else 0))
+    nb_out = got * (sorter.keys.element_size() + (sorter.vals.element_size() if hv is not None else 0))
+    return {"value": n * world / (t * 1e-3), "unit": "records/s", "ms_per_step": t, "h2d_bytes_per_step": nb_in,
+            "d2h_bytes_per_step": nb_out, "steps": k,
+            "path": "pinned host -> H2D -> hrs.dist (partition, NCCL all-to-all, C-ABI local sort) -> D2H, per rank"}
 
 
 def run_e2e(torch, hrs, keys, vals, temp, args, n, kb, vb):
@@ -367,6 +448,8 @@ def main(argv=None):
     ap.add_argument("--config", default="c2", choices=sorted(CONFIGS))
     ap.add_argument("--dist", default="uniform", choices=["uniform", "and2", "and3", "and4", "const"])
     ap.add_argument("--no-e2e", action="store_true")
+    ap.add_argument("--force-dist", action="store_true",
+                    help="run the distributed path (NCCL) even at world size 1 (tests the N>1 code path on one GPU)")
     ap.add_argument("--no-cpu", action="store_true")
     ap.add_argument("--cpu-log2", type=int, default=26)
     ap.add_argument("--ref-log2", type=int, default=24)

@@ -99,6 +99,10 @@ class DistributedSorter:
         self.world = dist.get_world_size(group)
         self.rank = dist.get_rank(group)
         self.last = {}
+        # time_exchange: CUDA events around step 4 (the all-to-all) on the current stream,
+        # so bench.py can report the exchange against NVLink bandwidth
+        self.time_exchange = False
+        self.exchange_events = None
 
     def digits(self):
         """The (lo, hi) bit ranges of the 8-bit digits, most significant first."""
@@ -172,11 +176,17 @@ class DistributedSorter:
         recv = [send[src][me] for src in range(world)]
         # 4. exchange (every source's segment in source-rank order)
         rk = torch.empty(sum(recv), dtype=keys.dtype, device=keys.device)
+        rv = torch.empty(sum(recv), dtype=vals.dtype, device=vals.device) if vals is not None else None
+        ev = None
+        if self.time_exchange and keys.is_cuda:
+            ev = (torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True))
+            ev[0].record()
         _all_to_all(_bits(rk), _bits(kp), recv, send[me], self.group)
-        rv = None
         if vals is not None:
-            rv = torch.empty(sum(recv), dtype=vals.dtype, device=vals.device)
             _all_to_all(_bits(rv), _bits(vp), recv, send[me], self.group)
+        if ev is not None:
+            ev[1].record()
+        self.exchange_events = ev
         # 5. local sort of the received records (source-rank order = global input order)
         ko, vo = self.ops.sort(rk, rv, self.begin, self.end)
         offset = me * N // world
