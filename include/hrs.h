@@ -83,13 +83,24 @@ typedef enum {
  *   merge_threshold  ∂   neighbouring sub-buckets merge while their total < ∂ (1 .. ∂ˆ; 1 = no merging)
  *   keys_per_tile    KPB records per tile ("key block") (1 .. hrs_max_keys_per_tile)
  *   local_classes    0 = size classes [1,128], (128,256], ...; 1 = a single
- *                    local-sort configuration for every bucket (the ablation of Figs 11-14) */
+ *                    local-sort configuration for every bucket (the ablation of Figs 11-14)
+ *   flags            HRS_FLAG_* test switches (0 in production).  HRS_FLAG_FORCE_REDO makes
+ *                    every stability check of the fast rank fail, so the scatter and the
+ *                    local sorts always take their stable-by-construction redo path (the
+ *                    fast rank takes the lane order of returning shared-memory atomics as
+ *                    the in-warp order, which PTX does not guarantee; the checks catch a
+ *                    device that reorders, and this flag is how tests exercise the redo
+ *                    code).  The environment variable HRS_FORCE_REDO=1, read once when the
+ *                    library loads, ORs it into every call.  Results are identical either
+ *                    way; only the time changes. */
 typedef struct {
     uint32_t local_threshold;
     uint32_t merge_threshold;
     uint32_t keys_per_tile;
     uint32_t local_classes;
+    uint32_t flags;
 } hrs_tuning;
+#define HRS_FLAG_FORCE_REDO 1u
 
 #define HRS_MAX_PASSES 8
 #define HRS_NUM_CLASSES 8
@@ -108,6 +119,8 @@ typedef struct {
     uint64_t merged_groups;                    /* local entries made of >= 2 merged sub-buckets */
     uint64_t local_in_class[HRS_NUM_CLASSES];  /* local entries per size class */
     uint64_t bytes_min;                        /* sum_p R_p (K + 2(K+V)) + R_L 2(K+V) */
+    uint64_t redo_blocks;                      /* tiles / buckets redone with the stable-by-construction rank
+                                                  (0 unless a stability check failed or HRS_FLAG_FORCE_REDO) */
 } hrs_stats;
 
 /* ---- full sorts; arguments: temp, size, keys in/out, [values in/out], n, bit range, stream ---- */
@@ -143,6 +156,13 @@ uint32_t hrs_max_local_threshold(int key_bytes, int value_bytes);
 uint32_t hrs_max_keys_per_tile(int key_bytes, int value_bytes);
 /* Default tuning for the key/value widths (written to *out). */
 hrs_status hrs_default_tuning(int key_bytes, int value_bytes, hrs_tuning *out);
+/* Capacity (largest size) of local-sort size class c, 0 <= c < HRS_NUM_CLASSES (0 for c out
+ * of range): a bucket of s records goes to the smallest class whose capacity is >= s
+ * (hrs_stats.local_in_class counts entries per class).  P:562-566 gives the classes
+ * [1,128], (128,256], (256,512], ... as an example; this build uses powers of two up to
+ * 4096, then 4608 and 8192 (reading #20: uniform 2^28 inputs leave buckets of
+ * 4096 +- 200 records after two passes). */
+uint32_t hrs_class_capacity(int c);
 
 /* ---- signed and floating-point keys (the paper's order-preserving
  * bijections) ----

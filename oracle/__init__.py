@@ -33,14 +33,101 @@ import numpy as np
 _HERE = os.path.dirname(os.path.abspath(__file__))
 _SRC = os.path.join(_HERE, "oracle.c")
 _LIB = os.path.join(_HERE, "liboracle.so")
+_CPU_SRC = os.path.join(_HERE, "cpu_baseline.cc")
+_CPU_LIB = os.path.join(_HERE, "libcpu_baseline.so")
 _lib = None
+_cpu = None
 
 
 def build(force: bool = False) -> str:
-    """Compile oracle.c with gcc (plain C, -O2, single thread)."""
+    """Compile oracle.c with gcc (plain C, -O2, single thread) and cpu_baseline.cc with g++
+    (the multi-threaded LSD baseline and the std::stable_sort cross-check)."""
     if force or not os.path.exists(_LIB) or os.path.getmtime(_LIB) < os.path.getmtime(_SRC):
         subprocess.check_call(["gcc", "-O2", "-std=c99", "-shared", "-fPIC", "-o", _LIB, _SRC])
+    if force or not os.path.exists(_CPU_LIB) or os.path.getmtime(_CPU_LIB) < os.path.getmtime(_CPU_SRC):
+        subprocess.check_call(["g++", "-O3", "-std=c++17", "-pthread", "-shared", "-fPIC", "-o", _CPU_LIB,
+                               _CPU_SRC])
     return _LIB
+
+
+def _load_cpu():
+    global _cpu
+    if _cpu is None:
+        build()
+        lib = ctypes.CDLL(_CPU_LIB)
+        P, U, I = ctypes.c_void_p, ctypes.c_uint64, ctypes.c_int
+        lib.cpu_lsd_sort.argtypes = [P, P, U, I, I, I, I, P, P, I]
+        lib.cpu_stable_sort.argtypes = [P, P, U, I, I, I, I, P, P]
+        lib.cpu_lsd_sort.restype = I
+        lib.cpu_stable_sort.restype = I
+        _cpu = lib
+    return _cpu
+
+
+def host_cores() -> int:
+    """Cores this process may run on (sched_getaffinity), the baseline's thread count."""
+    try:
+        return len(os.sched_getaffinity(0))
+    except AttributeError:  # pragma: no cover
+        return os.cpu_count() or 1
+
+
+def host_model() -> str:
+    """CPU model name (lscpu / /proc/cpuinfo), for the cpu_baseline record."""
+    try:
+        for line in open("/proc/cpuinfo", encoding="utf-8"):
+            if line.startswith("model name"):
+                return line.split(":", 1)[1].strip()
+    except OSError:  # pragma: no cover
+        pass
+    return "unknown"
+
+
+def _native(a):
+    """A numpy uint32/uint64 view of a numpy array or torch CPU tensor (no widening)."""
+    if hasattr(a, "numpy"):
+        a = a.cpu()
+        import torch
+        if a.dtype == torch.uint32:
+            return a.view(torch.int32).numpy().view(np.uint32)
+        if a.dtype == torch.uint64:
+            return a.view(torch.int64).numpy().view(np.uint64)
+        a = a.numpy()
+    a = np.ascontiguousarray(a)
+    if a.dtype not in (np.uint32, np.uint64):
+        raise TypeError(a.dtype)
+    return a
+
+
+def cpu_lsd_sort(keys, vals=None, begin_bit: int = 0, end_bit: int | None = None, threads: int | None = None):
+    """Multi-threaded stable LSD radix sort (the timed CPU baseline) on the
+    native widths; byte-identical to sort() for any thread count."""
+    k = _native(keys)
+    v = _native(vals) if vals is not None else None
+    if end_bit is None:
+        end_bit = 8 * k.itemsize
+    ko = np.empty_like(k)
+    vo = np.empty_like(v) if v is not None else None
+    rc = _load_cpu().cpu_lsd_sort(_ptr(k), _ptr(v), k.size, k.itemsize, 0 if v is None else v.itemsize, begin_bit,
+                                  end_bit, _ptr(ko), _ptr(vo), threads or host_cores())
+    if rc:
+        raise ValueError(f"cpu_lsd_sort rc={rc}")
+    return ko, vo
+
+
+def cpu_stable_sort(keys, vals=None, begin_bit: int = 0, end_bit: int | None = None):
+    """std::stable_sort of the (key, value) records by key bits [begin, end), one thread."""
+    k = _native(keys)
+    v = _native(vals) if vals is not None else None
+    if end_bit is None:
+        end_bit = 8 * k.itemsize
+    ko = np.empty_like(k)
+    vo = np.empty_like(v) if v is not None else None
+    rc = _load_cpu().cpu_stable_sort(_ptr(k), _ptr(v), k.size, k.itemsize, 0 if v is None else v.itemsize,
+                                     begin_bit, end_bit, _ptr(ko), _ptr(vo))
+    if rc:
+        raise ValueError(f"cpu_stable_sort rc={rc}")
+    return ko, vo
 
 
 def _load():

@@ -42,16 +42,25 @@ def digit_plan(begin_bit: int, end_bit: int):
     return out
 
 
+NUM_CLASSES = 8
+
+
 def class_capacity(c: int) -> int:
-    """Upper size of local-sort class c.  P:562-566 gives [1,128], (128,256], (256,512],
-    ... as an example; reading #20: powers of two up to 4096, then 4608, 8192."""
-    return (128 << c) if c < 6 else (4608 if c == 6 else 8192)
+    """Upper size of local-sort class c as P:562-566 gives it: [1,128], (128,256],
+    (256,512], ... -- powers of two, 128 * 2^c."""
+    return 128 << c
 
 
-def size_class(size: int) -> int:
-    """Smallest class whose capacity holds `size` records (capped at class 7)."""
+PAPER_CLASSES = tuple(class_capacity(c) for c in range(NUM_CLASSES))
+
+
+def size_class(size: int, capacities=PAPER_CLASSES) -> int:
+    """Smallest class whose capacity holds `size` records (capped at the last class).
+    `capacities` is the class table (default: the paper's powers of two); a build whose
+    tuning uses other boundaries (reading #20) passes its own table, which the
+    classes then only rename -- the sort, pass and bucket structure do not depend on it."""
     c = 0
-    while class_capacity(c) < size and c < 7:
+    while capacities[c] < size and c < len(capacities) - 1:
         c += 1
     return c
 
@@ -121,8 +130,9 @@ def _sk(keys: np.ndarray, lo: int, hi: int) -> np.ndarray:
 
 def simulate_msd(keys, vals=None, begin_bit: int = 0, end_bit: int = 32,
                  local_threshold: int = 4096, merge_threshold: int = 3000,
-                 keys_per_tile: int = 4096) -> MsdResult:
-    """Run the MSD hybrid sort on uint64 arrays; returns sorted data plus its structure."""
+                 keys_per_tile: int = 4096, class_capacities=PAPER_CLASSES) -> MsdResult:
+    """Run the MSD hybrid sort on uint64 arrays; returns sorted data plus its structure.
+    Local entries are labelled with their size class under `class_capacities`."""
     k = np.array(keys, dtype=np.uint64, copy=True)
     v = None if vals is None else np.array(vals, dtype=np.uint64, copy=True)
     n = k.size
@@ -136,7 +146,7 @@ def simulate_msd(keys, vals=None, begin_bit: int = 0, end_bit: int = 32,
         k[seg] = k[seg][order]
         if v is not None:
             v[seg] = v[seg][order]
-        res.local_entries.append((off, cnt, hi_bit, size_class(cnt), p))
+        res.local_entries.append((off, cnt, hi_bit, size_class(cnt, class_capacities), p))
 
     if n <= local_threshold:
         local_sort(0, n, end_bit, 0)

@@ -16,7 +16,7 @@ import torch
 from ._lib import HRS_MAX_ITEMS, HrsError, Stats, Tuning, check, lib  # noqa: F401
 
 __all__ = ["sort", "temp_bytes", "get_stats", "digit_histogram", "partition_pass", "HrsError", "Tuning",
-           "default_tuning", "max_local_threshold", "max_keys_per_tile", "lib"]
+           "default_tuning", "max_local_threshold", "max_keys_per_tile", "class_capacities", "lib"]
 
 _KEY_DTYPES = {torch.uint32: 4, torch.uint64: 8}
 # signed / floating-point keys: (key bytes, hrs_key_kind) -- hrs_sort_typed
@@ -48,6 +48,31 @@ def _stream(stream) -> ctypes.c_void_p:
     if stream is None:
         stream = torch.cuda.current_stream()
     return ctypes.c_void_p(stream.cuda_stream if hasattr(stream, "cuda_stream") else int(stream))
+
+
+def _on_stream(stream, *tensors) -> None:
+    """Tensors the binding allocated (on torch's current stream) but the library uses on
+    `stream`: tell the caching allocator, so a block freed on return is not handed to a
+    new allocation while the sort is still running on `stream`."""
+    if stream is None or not isinstance(stream, torch.cuda.Stream):
+        return
+    if stream == torch.cuda.current_stream(stream.device):
+        return
+    for t in tensors:
+        if t is not None:
+            t.record_stream(stream)
+
+
+def _out(t: torch.Tensor | None, like: torch.Tensor, what: str) -> torch.Tensor:
+    """An output buffer: allocated like `like`, or the caller's, checked for length, dtype
+    and device (the library writes n elements through the raw pointer)."""
+    if t is None:
+        return torch.empty_like(like)
+    _check_tensor(t, what)
+    if t.dtype != like.dtype or t.numel() != like.numel() or t.device != like.device:
+        raise ValueError(f"{what} must be a {like.dtype} tensor of {like.numel()} elements on {like.device}, "
+                         f"got {t.dtype} x {t.numel()} on {t.device}")
+    return t
 
 
 def _tuning(tuning) -> ctypes.POINTER(Tuning) | None:
@@ -97,13 +122,13 @@ def sort(keys: torch.Tensor, values: torch.Tensor | None = None, begin_bit: int 
     n = keys.numel()
     if end_bit is None:
         end_bit = 8 * kb
-    if keys_out is None:
-        keys_out = torch.empty_like(keys)
-    if values is not None and values_out is None:
-        values_out = torch.empty_like(values)
+    keys_out = _out(keys_out, keys, "keys_out")
+    if values is not None:
+        values_out = _out(values_out, values, "values_out")
     tb = temp_bytes(n, kb, vb, begin_bit, end_bit, tuning)
     if temp is None or temp.numel() < tb:
         temp = alloc_temp(tb, keys.device)
+    _on_stream(stream, temp, keys_out, values_out)
     sz = ctypes.c_size_t(temp.numel())
     with torch.cuda.device(keys.device):
         check(lib.hrs_sort_ex(_ptr(temp), ctypes.byref(sz), _ptr(keys), _ptr(keys_out), _ptr(values),
@@ -137,13 +162,13 @@ def sort_typed(keys: torch.Tensor, values: torch.Tensor | None = None, *, keys_o
         if values.numel() != keys.numel():
             raise ValueError("keys and values differ in length")
     n = keys.numel()
-    if keys_out is None:
-        keys_out = torch.empty_like(keys)
-    if values is not None and values_out is None:
-        values_out = torch.empty_like(values)
+    keys_out = _out(keys_out, keys, "keys_out")
+    if values is not None:
+        values_out = _out(values_out, values, "values_out")
     tb = typed_temp_bytes(n, kb, vb, kind)
     if temp is None or temp.numel() < tb:
         temp = alloc_temp(tb, keys.device)
+    _on_stream(stream, temp, keys_out, values_out)
     sz = ctypes.c_size_t(temp.numel())
     with torch.cuda.device(keys.device):
         check(lib.hrs_sort_typed(_ptr(temp), ctypes.byref(sz), _ptr(keys), _ptr(keys_out), _ptr(values),
@@ -171,6 +196,7 @@ def digit_histogram(keys: torch.Tensor, lo_bit: int, hi_bit: int, *, temp: torch
     if temp is None or temp.numel() < sz.value:
         temp = alloc_temp(sz.value, keys.device)
     hist = torch.empty(1 << (hi_bit - lo_bit), dtype=torch.uint64, device=keys.device)
+    _on_stream(stream, temp, hist)
     sz = ctypes.c_size_t(temp.numel())
     with torch.cuda.device(keys.device):
         check(lib.hrs_digit_histogram(_ptr(temp), ctypes.byref(sz), _ptr(keys), n, kb, lo_bit, hi_bit, _ptr(hist),
@@ -184,24 +210,27 @@ def partition_pass(keys: torch.Tensor, values: torch.Tensor | None, lo_bit: int,
     """One stable counting pass on digit bits [lo_bit, hi_bit): (keys_out, values_out, offsets[r+1])."""
     _check_tensor(keys, "keys")
     if keys.dtype in _TYPED_KEYS:
-        return sort_typed(keys, values, keys_out=keys_out, values_out=values_out, temp=temp, stream=stream,
-                          begin_bit=begin_bit, end_bit=end_bit, tuning=tuning)
+        raise TypeError("partition_pass takes unsigned keys (torch.uint32 / torch.uint64): a digit of a "
+                        "signed or floating-point key is a digit of its order-preserving image (P:907-918); "
+                        "map the keys first or use sort()")
     kb = _nbytes(keys, "keys")
     vb = 0
     if values is not None:
         _check_tensor(values, "values")
         vb = _nbytes(values, "values")
+        if values.numel() != keys.numel() or values.device != keys.device:
+            raise ValueError("keys and values differ in length or device")
     n = keys.numel()
     sz = ctypes.c_size_t(0)
     check(lib.hrs_partition_pass(None, ctypes.byref(sz), None, None, None, None, n, kb, vb, lo_bit, hi_bit, None,
                                  None), "hrs_partition_pass(size query)")
     if temp is None or temp.numel() < sz.value:
         temp = alloc_temp(sz.value, keys.device)
-    if keys_out is None:
-        keys_out = torch.empty_like(keys)
-    if values is not None and values_out is None:
-        values_out = torch.empty_like(values)
+    keys_out = _out(keys_out, keys, "keys_out")
+    if values is not None:
+        values_out = _out(values_out, values, "values_out")
     offs = torch.empty((1 << (hi_bit - lo_bit)) + 1, dtype=torch.uint64, device=keys.device)
+    _on_stream(stream, temp, keys_out, values_out, offs)
     sz = ctypes.c_size_t(temp.numel())
     with torch.cuda.device(keys.device):
         check(lib.hrs_partition_pass(_ptr(temp), ctypes.byref(sz), _ptr(keys), _ptr(keys_out), _ptr(values),
@@ -222,6 +251,12 @@ def max_local_threshold(key_bytes: int, value_bytes: int) -> int:
 
 def max_keys_per_tile(key_bytes: int, value_bytes: int) -> int:
     return lib.hrs_max_keys_per_tile(key_bytes, value_bytes)
+
+
+def class_capacities() -> list:
+    """Capacity of every local-sort size class of this build (hrs_class_capacity)."""
+    from ._lib import HRS_NUM_CLASSES
+    return [lib.hrs_class_capacity(c) for c in range(HRS_NUM_CLASSES)]
 
 
 def profile_enable(on: bool = True) -> None:

@@ -41,7 +41,11 @@ class Tuning(ctypes.Structure):
         ("merge_threshold", ctypes.c_uint32),
         ("keys_per_tile", ctypes.c_uint32),
         ("local_classes", ctypes.c_uint32),
+        ("flags", ctypes.c_uint32),
     ]
+
+
+HRS_FLAG_FORCE_REDO = 1
 
 
 class Stats(ctypes.Structure):
@@ -59,6 +63,7 @@ class Stats(ctypes.Structure):
         ("merged_groups", ctypes.c_uint64),
         ("local_in_class", ctypes.c_uint64 * HRS_NUM_CLASSES),
         ("bytes_min", ctypes.c_uint64),
+        ("redo_blocks", ctypes.c_uint64),
     ]
 
     def to_dict(self) -> dict:
@@ -77,6 +82,7 @@ class Stats(ctypes.Structure):
             "merged_groups": self.merged_groups,
             "local_in_class": list(self.local_in_class),
             "bytes_min": self.bytes_min,
+            "redo_blocks": self.redo_blocks,
         }
 
 
@@ -105,6 +111,7 @@ SIGNATURES = {
     "hrs_max_local_threshold": (ctypes.c_uint32, [_I, _I]),
     "hrs_max_keys_per_tile": (ctypes.c_uint32, [_I, _I]),
     "hrs_default_tuning": (_ST, [_I, _I, ctypes.POINTER(Tuning)]),
+    "hrs_class_capacity": (ctypes.c_uint32, [_I]),
     "hrs_digit_histogram": (_ST, [_P, _SZP, _P, _U64, _I, _I, _I, _P, _P]),
     "hrs_partition_pass": (_ST, [_P, _SZP, _P, _P, _P, _P, _U64, _I, _I, _I, _I, _P, _P]),
     "hrs_profile_enable": (None, [_I]),

@@ -307,7 +307,17 @@ struct Plan {
            off_local[HRS_NUM_CLASSES] = {0}, off_local_wide[HRS_NUM_CLASSES] = {0}, off_local_fb2 = 0, total = 0;
     uint32_t local_wide_cap[HRS_NUM_CLASSES] = {0}, local_fb2_cap = 0;
     int wide_top = 0;
+    int force_redo = 0;  // HRS_FLAG_FORCE_REDO (tuning flags or the HRS_FORCE_REDO environment variable)
 };
+
+// HRS_FORCE_REDO=1 in the environment ORs HRS_FLAG_FORCE_REDO into every call (include/hrs.h)
+uint32_t env_flags() {
+    static const uint32_t f = [] {
+        const char *e = std::getenv("HRS_FORCE_REDO");
+        return (e && e[0] == '1') ? HRS_FLAG_FORCE_REDO : 0u;
+    }();
+    return f;
+}
 
 size_t align_up(size_t x, size_t a) { return (x + a - 1) / a * a; }
 
@@ -322,13 +332,17 @@ hrs_status make_plan(Plan &pl, uint64_t n, int kb, int vb, int begin, int end, c
     t.merge_threshold = 8192 / DEFAULT_MT_DIV;
     t.keys_per_tile = max_kpb(kb, vb);
     t.local_classes = 0;
+    t.flags = 0;
     if (tu) {
         if (tu->local_threshold) t.local_threshold = tu->local_threshold;
         if (tu->merge_threshold) t.merge_threshold = tu->merge_threshold;
         else if (tu->local_threshold) t.merge_threshold = std::max<uint32_t>(1, t.local_threshold / DEFAULT_MT_DIV);
         if (tu->keys_per_tile) t.keys_per_tile = tu->keys_per_tile;
         t.local_classes = tu->local_classes;
+        t.flags = tu->flags;
     }
+    if (t.flags & ~HRS_FLAG_FORCE_REDO) return HRS_ERROR_INVALID_VALUE;
+    pl.force_redo = ((t.flags | env_flags()) & HRS_FLAG_FORCE_REDO) ? 1 : 0;
     if (t.local_threshold < 1 || t.local_threshold > max_lt(kb, vb)) return HRS_ERROR_INVALID_VALUE;
     if (t.merge_threshold < 1 || t.merge_threshold > t.local_threshold) return HRS_ERROR_INVALID_VALUE;
     if (t.keys_per_tile < 1 || t.keys_per_tile > max_kpb(kb, vb)) return HRS_ERROR_INVALID_VALUE;
@@ -566,6 +580,7 @@ struct Runner {
         sp.tiles = at<TileDesc>(temp, pl.off_tiles);
         sp.tile_pref = at<uint32_t>(temp, pl.off_tile_pref);
         sp.ctl = at<Ctl>(temp, 0);
+        sp.force_redo = pl.force_redo;
         auto fn = k_scatter<K, V, SC::THREADS, SC::KPT, SC::MINB, SC::NBUF>;
         const size_t smem = ScatterSmem<K, V, SC::THREADS, SC::KPT, SC::NBUF>::bytes;
         int grid = 0;
@@ -592,6 +607,8 @@ struct Runner {
         lp.keys_out = kout;
         lp.vals_out = vout;
         lp.begin_bit = pl.begin;
+        lp.force_redo = pl.force_redo;
+        lp.redo = &at<Ctl>(temp, 0)->redo;
     }
 
     // the counting local sort of class C; hands what it does not take to LIST_FB2
@@ -1041,6 +1058,7 @@ hrs_status hrs_sort_ex(void *d_temp, size_t *temp_bytes, const void *keys_in, vo
         v[10] = reinterpret_cast<uintptr_t>(vals_out);
         v[11] = reinterpret_cast<uintptr_t>(d_temp);
         v[12] = *temp_bytes;
+        v[13] = t.flags | env_flags();
         hrs_status gs = HRS_SUCCESS;
         if (via_graph(key, st, dev, &gs, run)) return gs;
     }
@@ -1155,6 +1173,7 @@ hrs_status hrs_get_stats(const void *d_temp, hrs_stats *out, hrs_stream_t stream
     }
     out->local_recs = c.local_recs;
     out->merged_groups = c.merged_groups;
+    out->redo_blocks = c.redo;
     out->bytes_min = bytes + c.local_recs * 2 * R;
     return HRS_SUCCESS;
 }
@@ -1172,8 +1191,11 @@ hrs_status hrs_default_tuning(int key_bytes, int value_bytes, hrs_tuning *out) {
     out->merge_threshold = pl.mt;
     out->keys_per_tile = pl.kpb;
     out->local_classes = 0;
+    out->flags = 0;
     return HRS_SUCCESS;
 }
+
+uint32_t hrs_class_capacity(int c) { return (c >= 0 && c < HRS_NUM_CLASSES) ? class_capacity(c) : 0u; }
 
 static hrs_status block_common(void *d_temp, size_t *temp_bytes, const void *keys_in, void *keys_out,
                                const void *vals_in, void *vals_out, uint64_t n, int kb, int vb, int lo, int hi,

@@ -109,6 +109,7 @@ struct Ctl {
     unsigned long long recs_in_pass[HRS_MAX_PASSES + 2];
     unsigned long long local_recs;
     unsigned long long merged_groups;
+    unsigned long long redo;  // blocks that redid a tile / bucket with the stable-by-construction rank
 };
 
 // ------------------------------------------------------------------ small helpers
@@ -979,7 +980,7 @@ __device__ void classify_bucket(const ClassifyParams &prm, const Bucket &bk, uin
         glead[d] = 0;
         gmulti[d] = 0;
         const bool cnt = !prm.last && v > prm.lt;
-        ct[d] = cnt ? (v + prm.kpb - 1) / prm.kpb : 0u;
+        ct[d] = cnt ? v / prm.kpb + (v % prm.kpb != 0u) : 0u;  // (no u32 wrap near 2^32)
         cb[d] = cnt ? 1u : 0u;
     }
     if (tid < 32) misc[tid] = 0;
@@ -1090,7 +1091,7 @@ __device__ void classify_bucket(const ClassifyParams &prm, const Bucket &bk, uin
             nb.offs = boffs + start[tid];
             nb.count = s;
             nb.first_tile = bt + ct[tid];
-            nb.ntiles = (s + prm.kpb - 1) / prm.kpb;
+            nb.ntiles = s / prm.kpb + (s % prm.kpb != 0u);
             nb.pad = 0;
             prm.next_buckets[id] = nb;
         }
@@ -1173,6 +1174,7 @@ struct ScatterParams {
     const TileDesc *tiles;
     const uint32_t *tile_pref;
     Ctl *ctl;
+    int force_redo;  // HRS_FLAG_FORCE_REDO: every stability check fails (tests of the redo path)
 };
 
 struct StageInfo {
@@ -1363,9 +1365,10 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
             }
             __syncthreads();
             const bool bad = write_out(true);
-            if (__syncthreads_or(bad)) {
+            if (__syncthreads_or(bad || prm.force_redo)) {
                 // the atomics did not serve the lanes in order: redo the tile with the
                 // rank that is stable by construction (same digit starts, so gs holds)
+                if (tid == 0) atomicAdd(&prm.ctl->redo, 1ull);
 #pragma unroll
                 for (int c = 0; c < KPT; ++c) {
                     const uint32_t e = wbase + c * 32 + lane;
@@ -1417,6 +1420,8 @@ struct LocalParams {
     int wide_single;
     int wide_top;  // largest wide configuration
     int begin_bit;
+    int force_redo;  // HRS_FLAG_FORCE_REDO: every stability check of the fast rank fails
+    unsigned long long *redo;  // Ctl::redo
 };
 
 // Shared memory of one local-sort CTA: NSTAGE staging buffers {keys, values}; after
@@ -1723,7 +1728,8 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
                         if ((!BAL || c < kpt) && e > 0 && e < count) bad |= comp[e - 1] >= cv[c];
                     }
                 }
-                if (__syncthreads_or(bad)) {
+                if (__syncthreads_or(bad || prm.force_redo)) {
+                    if (tid == 0) atomicAdd(prm.redo, 1ull);
                     if (active) {
 #pragma unroll
                         for (int c = 0; c < KPT; ++c)
@@ -1877,7 +1883,8 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
                         }
                     }
                 }
-                if (__syncthreads_or(bad)) {
+                if (__syncthreads_or(bad || prm.force_redo)) {
+                    if (tid == 0) atomicAdd(prm.redo, 1ull);
 #pragma unroll
                     for (int c = 0; c < KPT; ++c) {
                         const uint32_t e = wbase + c * 32 + lane;

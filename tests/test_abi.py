@@ -101,3 +101,19 @@ def test_python_wrapper_rejects_cpu_tensors():
     import paper_1611_01137_b200 as hrs
     with pytest.raises(ValueError, match="CUDA"):
         hrs.sort(torch.zeros(4, dtype=torch.uint32))
+
+
+def test_class_capacities_and_flags():
+    """The size-class table the library exports is increasing, starts at the paper's
+    [1,128] class and ends at the largest local-sort threshold; unknown tuning
+    flags are rejected."""
+    import paper_1611_01137_b200 as hrs
+    from paper_1611_01137_b200 import _lib
+    caps = hrs.class_capacities()
+    assert caps[0] == 128 and all(a < b for a, b in zip(caps, caps[1:]))
+    assert max(hrs.max_local_threshold(kb, vb) for kb, vb in ((4, 0), (4, 4), (8, 8))) <= caps[-1]
+    assert _lib.lib.hrs_class_capacity(-1) == 0 and _lib.lib.hrs_class_capacity(8) == 0
+    ok = _lib.Tuning(flags=_lib.HRS_FLAG_FORCE_REDO)
+    assert _sz(_lib.lib.hrs_sort_ex, None, None, None, None, 10, 4, 0, 0, 32, ctypes.byref(ok), None)[0] == 0
+    bad = _lib.Tuning(flags=2)
+    assert _sz(_lib.lib.hrs_sort_ex, None, None, None, None, 10, 4, 0, 0, 32, ctypes.byref(bad), None)[0] == 1

@@ -66,7 +66,7 @@ def _top_digit_runs(keys_out, kbits):
     return torch.bincount(top, minlength=256).cpu().numpy().astype(np.uint64), top
 
 
-@pytest.mark.parametrize("dist", ["uniform", "and2", "and3", "and4"])
+@pytest.mark.parametrize("dist", ["uniform", "and2", "and3", "and4", "const"])
 def test_c2_c3_pairs_u32(dist):
     n = 1 << 28
     k = gen.keys(n, 32, dist, device=DEV)
@@ -84,7 +84,7 @@ def test_c2_c3_pairs_u32(dist):
         assert st["local_recs"] == n and st["bytes_min"] == 56 * n
 
 
-@pytest.mark.parametrize("dist", ["uniform", "and3"])
+@pytest.mark.parametrize("dist", ["uniform", "and2", "and3", "and4", "const"])
 def test_c4_pairs_u64(dist):
     n = 1 << 28
     k = gen.keys(n, 64, dist, device=DEV)

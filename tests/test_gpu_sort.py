@@ -129,8 +129,11 @@ def test_threshold_overrides_and_structure(tuning, dist, kbits, vbits):
     st = hrs.get_stats(temp)
     ek, ev = oracle.sort(k, v, 0, kbits)
     assert np.array_equal(_np(ko), ek) and np.array_equal(_np(vo), ev)
+    # the library's own size-class table (hrs_class_capacity) labels the oracle's entries:
+    # the class boundaries are a tuning of this build (reading #20), not part of the method
     sim = plan.simulate_msd(oracle._u64(k), None, 0, kbits, tuning["local_threshold"],
-                            tuning["merge_threshold"], tuning["keys_per_tile"])
+                            tuning["merge_threshold"], tuning["keys_per_tile"],
+                            class_capacities=tuple(hrs.class_capacities()))
     assert st["overflow"] == 0
     assert st["counting_passes"] == sim.counting_passes
     assert st["recs_in_pass"] == sim.recs_in_pass
@@ -313,3 +316,61 @@ def test_wide_configurations_64bit(kbits, vbits, n):
     for dist in ("uniform", "and2"):
         k, v = _inputs(n, kbits, vbits, dist, seed=n % 1000 + kbits + vbits)
         _run_and_check(k, v, 0, kbits)
+
+
+# ------------------------------------------------------------- the named §8(b) entry points
+
+@pytest.mark.parametrize("name,kbits,vbits", [("hrs_sort_keys_u32", 32, 0), ("hrs_sort_keys_u64", 64, 0),
+                                              ("hrs_sort_pairs_u32_u32", 32, 32),
+                                              ("hrs_sort_pairs_u32_u64", 32, 64),
+                                              ("hrs_sort_pairs_u64_u32", 64, 32),
+                                              ("hrs_sort_pairs_u64_u64", 64, 64)])
+def test_named_entry_points(name, kbits, vbits):
+    """Each typed C entry point of include/hrs.h called directly through ctypes (two-phase
+    temp protocol, raw device pointers, the current stream), against the oracle."""
+    import ctypes
+    import paper_1611_01137_b200 as hrs
+    fn = getattr(hrs.lib, name)
+    for n, dist, (b, e) in ((100003, "and2", (0, kbits)), (4097, "uniform", (3, kbits - 2)), (0, "uniform", (0, kbits)),
+                            (1 << 20, "uniform", (0, kbits))):
+        k, v = _inputs(n, kbits, vbits, dist, seed=n + 5)
+        kd = k.to(DEV)
+        ko = torch.empty_like(kd)
+        vd = v.to(DEV) if v is not None else None
+        vo = torch.empty_like(vd) if v is not None else None
+        P = ctypes.c_void_p
+        ptr = lambda t: P(t.data_ptr()) if t is not None and t.numel() else P(0)  # noqa: E731
+        data = [ptr(kd), ptr(ko)] + ([ptr(vd), ptr(vo)] if vbits else [])
+        sz = ctypes.c_size_t(0)
+        hrs.check(fn(None, ctypes.byref(sz), *data, n, b, e, None), name + "(size)")
+        temp = torch.empty(max(sz.value, 256), dtype=torch.uint8, device=DEV)
+        sz = ctypes.c_size_t(temp.numel())
+        stream = P(torch.cuda.current_stream().cuda_stream)
+        hrs.check(fn(P(temp.data_ptr()), ctypes.byref(sz), *data, n, b, e, stream), name)
+        torch.cuda.synchronize()
+        ek, ev = oracle.sort(k, v, b, e)
+        assert np.array_equal(_np(ko), ek), (name, n)
+        if vbits:
+            assert np.array_equal(_np(vo), ev), (name, n)
+
+
+def test_binding_checks_outputs_and_streams():
+    """The binding rejects short / mistyped output buffers (the library writes n elements
+    through raw pointers) and typed keys in partition_pass; a sort on a side stream with
+    binding-allocated temp gives the oracle's result."""
+    import paper_1611_01137_b200 as hrs
+    k = gen.keys(5000, 32, "uniform", seed=1).to(DEV)
+    with pytest.raises(ValueError):
+        hrs.sort(k, None, keys_out=torch.empty(4999, dtype=torch.uint32, device=DEV))
+    with pytest.raises(ValueError):
+        hrs.sort(k, k.clone(), values_out=torch.empty(5000, dtype=torch.uint64, device=DEV))
+    with pytest.raises(TypeError):
+        hrs.partition_pass(k.view(torch.int32), None, 24, 32)
+    s = torch.cuda.Stream()
+    kk, vv = _inputs(1 << 20, 32, 32, "and2", seed=3)
+    kd, vd = kk.to(DEV), vv.to(DEV)
+    s.wait_stream(torch.cuda.current_stream())
+    ko, vo = hrs.sort(kd, vd, stream=s)
+    s.synchronize()
+    ek, ev = oracle.sort(kk, vv, 0, 32)
+    assert np.array_equal(_np(ko), ek) and np.array_equal(_np(vo), ev)

@@ -200,10 +200,12 @@ def test_merge_rule_worked_vector():
 
 
 def test_size_classes():
-    # [1,128] -> 0, (128,256] -> 1, (256,512] -> 2, ..., (2048,4096] -> 5,
-    # then (4096,4608] -> 6 and (4608,8192] -> 7 (reading #20)
-    assert [plan.size_class(s) for s in (1, 128, 129, 256, 257, 512, 513, 4096, 4097, 4608, 4609, 8192)] == \
-        [0, 0, 1, 1, 2, 2, 3, 5, 6, 6, 7, 7]
+    # [1,128] -> 0, (128,256] -> 1, (256,512] -> 2, and so on by powers of two
+    assert [plan.size_class(s) for s in (1, 128, 129, 256, 257, 512, 513, 4096, 4097, 8192, 8193, 16384, 10**6)] == \
+        [0, 0, 1, 1, 2, 2, 3, 5, 6, 6, 7, 7, 7]
+    # another class table only relabels: boundaries are where the table says
+    tab = (128, 256, 512, 1024, 2048, 4096, 4608, 8192)
+    assert [plan.size_class(s, tab) for s in (4096, 4097, 4608, 4609, 8192)] == [5, 6, 6, 7, 7]
 
 
 @pytest.mark.parametrize("dist", ["uniform", "and2", "and3", "and4", "const"])
@@ -270,3 +272,42 @@ def test_sort_typed_against_comparison_sort():
     gk, gv = oracle.sort_typed(fl, np.arange(fl.size), "float")
     assert gv.tolist() == want
     assert gk.view(np.uint32).tolist() == [bits[i] for i in want]
+
+
+# ---------------------------------------------------------------- std::stable_sort and the CPU baseline
+
+@pytest.mark.parametrize("kbits,vbits", [(32, 0), (32, 32), (32, 64), (64, 0), (64, 32), (64, 64)])
+@pytest.mark.parametrize("dist", ["uniform", "and3", "const"])
+def test_oracle_equals_std_stable_sort_and_parallel_lsd(kbits, vbits, dist):
+    """The library routine BJ north_star names: std::stable_sort of the (key, value)
+    records by sk gives the oracle's bytes (a plausible oracle mistake -- a wrong digit
+    order, an unstable scatter, a dropped narrow digit -- would differ).  The
+    multi-threaded LSD (the timed CPU baseline) is byte-identical to the
+    one-thread oracle for every thread count, including more threads than records."""
+    n = 20011
+    k = gen.keys(n, kbits, dist, seed=29)
+    v = gen.values(n, vbits, "random", seed=29) if vbits else None
+    kn = oracle._native(k)
+    vn = oracle._native(v) if v is not None else None
+    for b, e in ((0, kbits), (3, kbits - 5), (kbits - 1, kbits), (7, 7)):
+        ek, ev = oracle.sort(kn, vn, b, e)
+        sk, sv = oracle.cpu_stable_sort(kn, vn, b, e)
+        assert np.array_equal(sk.astype(np.uint64), ek), (b, e)
+        if v is not None:
+            assert np.array_equal(sv.astype(np.uint64), ev), (b, e)
+        for t in (1, 3, 8, 64):
+            pk, pv = oracle.cpu_lsd_sort(kn, vn, b, e, threads=t)
+            assert pk.dtype == kn.dtype
+            assert np.array_equal(pk.astype(np.uint64), ek), (b, e, t)
+            if v is not None:
+                assert np.array_equal(pv.astype(np.uint64), ev), (b, e, t)
+    # tiny inputs with more threads than records
+    for n2 in (0, 1, 5):
+        kk = kn[:n2].copy()
+        pk, _ = oracle.cpu_lsd_sort(kk, None, 0, kbits, threads=16)
+        assert np.array_equal(pk.astype(np.uint64), oracle.sort(kk, None, 0, kbits)[0])
+
+
+def test_host_description():
+    assert oracle.host_cores() >= 1
+    assert isinstance(oracle.host_model(), str)
