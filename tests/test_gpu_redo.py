@@ -99,7 +99,10 @@ def test_forced_redo_env_typed_and_fullsize():
     code = r"""
 import numpy as np, torch, gen, oracle
 import paper_1611_01137_b200 as hrs
-from tests.test_gpu_fullsize import certificate
+import importlib.util
+_spec = importlib.util.spec_from_file_location("fullsize", "tests/test_gpu_fullsize.py")
+_m = importlib.util.module_from_spec(_spec); _spec.loader.exec_module(_m)
+certificate = _m.certificate
 DEV = "cuda:0"
 for dtype, kind in ((torch.int32, "int"), (torch.float64, "float")):
     kb = 32 if dtype == torch.int32 else 64
