@@ -275,7 +275,7 @@ def run_hrs(args):
             out["e2e"] = run_e2e(torch, hrs, keys, vals, temp, args, n, kb, vb)
         # ---------------- CPU baseline: the oracle as it stands on a bounded sample
         if not args.no_cpu:
-            out["cpu_baseline"] = cpu_baseline(args, kbits, vbits, dist_name)
+            out["cpu_baseline"] = cpu_baseline(args, kbits, vbits, dist_name, keys_dev=keys)
     if rank == 0:
         print(json.dumps(out), flush=True)
     if pg is not None:
@@ -424,19 +424,46 @@ def run_e2e(torch, hrs, keys, vals, temp, args, n, kb, vb):
             "path": "pinned host -> H2D -> hrs.sort (C ABI) -> D2H, consecutive steps pipelined over 3 streams"}
 
 
-def cpu_baseline(args, kbits, vbits, dist_name):
+def cpu_baseline(args, kbits, vbits, dist_name, keys_dev=None):
+    """The CPU baselines of SURVEY §8(d) on this box's host, bounded to ~10-30 s:
+      * value: the stable LSD radix sort over every core this process may use
+        (oracle/cpu_baseline.cc, byte-identical to the oracle; pinned by tests/test_oracle.py)
+        on the FULL workload (the GPU input copied to the host, untimed);
+      * oracle_1core: the oracle as it stands (oracle/oracle.c, one thread) on a 2^cpu_log2 slice;
+      * stable_sort_1core: std::stable_sort of the records on the same slice."""
     import numpy as np
     import gen
     import oracle
-    n = 1 << args.cpu_log2
-    k = oracle._u64(gen.keys(n, kbits, dist_name))
-    v = np.arange(n, dtype=np.uint64) if vbits else None
+    n_full = None
+    if keys_dev is not None:
+        k = oracle._native(keys_dev.cpu())
+        n_full = k.size
+    else:
+        k = oracle._native(gen.keys(1 << args.cpu_log2, kbits, dist_name))
+    vdt = np.uint32 if vbits == 32 else np.uint64
+    v = np.arange(k.size, dtype=vdt) if vbits else None
+    cores = oracle.host_cores()
+    oracle.cpu_lsd_sort(k[:1 << 16], None if v is None else v[:1 << 16], 0, kbits, threads=cores)  # warm
     t0 = time.perf_counter()
-    oracle.sort(k, v, 0, kbits)
-    t = time.perf_counter() - t0
-    return {"value": n / t, "unit": "records/s", "cores": 1, "kind": "oracle",
-            "sample": f"{n} records of the same workload ({dist_name}), single-threaded LSD oracle "
-                      f"(oracle/oracle.c), {t:.2f} s"}
+    oracle.cpu_lsd_sort(k, v, 0, kbits, threads=cores)
+    t_par = time.perf_counter() - t0
+    ns = min(k.size, 1 << args.cpu_log2)
+    ks = k[:ns].copy()
+    vs = None if v is None else v[:ns].copy()
+    t0 = time.perf_counter()
+    oracle.sort(ks, vs, 0, kbits)
+    t_or = time.perf_counter() - t0
+    t0 = time.perf_counter()
+    oracle.cpu_stable_sort(ks, vs, 0, kbits)
+    t_ss = time.perf_counter() - t0
+    return {"value": k.size / t_par, "unit": "records/s", "cores": cores, "kind": "oracle",
+            "sample": f"{k.size} records ({'the full workload' if n_full else 'a slice'}, {dist_name}), stable LSD "
+                      f"radix sort on {cores} host threads (oracle/cpu_baseline.cc, byte-identical to the oracle), "
+                      f"{t_par:.2f} s",
+            "host_model": oracle.host_model(),
+            "oracle_1core": {"value": ns / t_or, "records": ns, "s": t_or,
+                             "what": "oracle/oracle.c single-threaded LSD (64-bit words)"},
+            "stable_sort_1core": {"value": ns / t_ss, "records": ns, "s": t_ss, "what": "std::stable_sort, 1 thread"}}
 
 
 def main(argv=None):
@@ -451,7 +478,7 @@ def main(argv=None):
     ap.add_argument("--force-dist", action="store_true",
                     help="run the distributed path (NCCL) even at world size 1 (tests the N>1 code path on one GPU)")
     ap.add_argument("--no-cpu", action="store_true")
-    ap.add_argument("--cpu-log2", type=int, default=26)
+    ap.add_argument("--cpu-log2", type=int, default=24)
     ap.add_argument("--ref-log2", type=int, default=24)
     args = ap.parse_args(argv)
     if args.warmup < 3:

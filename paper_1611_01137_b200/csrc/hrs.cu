@@ -70,14 +70,17 @@ struct LaunchScope {
 constexpr uint32_t DEFAULT_MT_DIV = 4;
 
 // 32-bit-key scatter shape (overridable for experiments, micro/scatter_exp.py)
+#ifndef HRS_SC_THREADS
+#define HRS_SC_THREADS 256
+#endif
 #ifndef HRS_SC_KPT
-#define HRS_SC_KPT 13
+#define HRS_SC_KPT 22  // measured on B200 (c2 uniform, both passes): 13 x 3 CTAs/SM 2.51 ms, 16 x 2 2.24, 20 x 2 2.15, 22 x 2 2.10, 32 x 1 2.41
 #endif
 #ifndef HRS_SC_NBUF
 #define HRS_SC_NBUF 2
 #endif
 #ifndef HRS_SC_MINB
-#define HRS_SC_MINB 3
+#define HRS_SC_MINB 2
 #endif
 
 // wider records (8-byte keys or values) scatter shape
@@ -85,13 +88,13 @@ constexpr uint32_t DEFAULT_MT_DIV = 4;
 #define HRS_SC64_THREADS 256
 #endif
 #ifndef HRS_SC64_KPT
-#define HRS_SC64_KPT 16
+#define HRS_SC64_KPT 12  // measured (c4 uniform / AND-3 step): 16 x 1 buffer 7.80 / 17.5 ms, 12 x 2 7.66 / 16.1, 22 x 1 7.52 / 17.2
 #endif
 #ifndef HRS_SC64_MINB
 #define HRS_SC64_MINB 2
 #endif
 #ifndef HRS_SC64_NBUF
-#define HRS_SC64_NBUF 1
+#define HRS_SC64_NBUF 2
 #endif
 
 // ------------------------------------------------------------------ compile-time configurations
@@ -100,8 +103,8 @@ constexpr uint32_t DEFAULT_MT_DIV = 4;
 template <int KB, int VB>
 struct ScatterCfg {
     static constexpr bool SMALL = (KB == 4 && VB <= 4);
-    static constexpr int THREADS = SMALL ? 256 : HRS_SC64_THREADS;
-    static constexpr int KPT = SMALL ? HRS_SC_KPT : HRS_SC64_KPT;  // 256 x 13: two staging buffers + the slot index for three CTAs per SM
+    static constexpr int THREADS = SMALL ? HRS_SC_THREADS : HRS_SC64_THREADS;
+    static constexpr int KPT = SMALL ? HRS_SC_KPT : HRS_SC64_KPT;  // 256 x 22: two staging buffers + the slot index for two CTAs per SM
     static constexpr int MINB = SMALL ? HRS_SC_MINB : HRS_SC64_MINB;
     static constexpr int NBUF = SMALL ? HRS_SC_NBUF : HRS_SC64_NBUF;
 };
@@ -867,8 +870,21 @@ hrs_status run_block(const Plan &pl, void *temp, const void *kin, void *kout, co
     return Runner<K, V>::building_block(pl, temp, kin, kout, vin, vout, h, o, sc, st, dev, sms);
 }
 
+// HRS_ONLY_TYPES=44 (or 88): experiment builds instantiate one key/value pair only (fast
+// compiles for kernel-variant timing, micro/scatter_exp.py); 0 in the product
+#ifndef HRS_ONLY_TYPES
+#define HRS_ONLY_TYPES 0
+#endif
 hrs_status sort_dispatch(int kb, int vb, const Plan &pl, void *temp, const void *kin, void *kout, const void *vin,
                          void *vout, cudaStream_t st, int dev, int sms) {
+#if HRS_ONLY_TYPES == 44
+    if (kb == 4 && vb == 4) return run_sort<uint32_t, uint32_t>(pl, temp, kin, kout, vin, vout, st, dev, sms);
+    return HRS_ERROR_INVALID_VALUE;
+#elif HRS_ONLY_TYPES == 88
+    if (kb == 8 && vb == 8)
+        return run_sort<unsigned long long, unsigned long long>(pl, temp, kin, kout, vin, vout, st, dev, sms);
+    return HRS_ERROR_INVALID_VALUE;
+#else
     if (kb == 4) {
         if (vb == 0) return run_sort<uint32_t, NoVal>(pl, temp, kin, kout, vin, vout, st, dev, sms);
         if (vb == 4) return run_sort<uint32_t, uint32_t>(pl, temp, kin, kout, vin, vout, st, dev, sms);
@@ -877,10 +893,16 @@ hrs_status sort_dispatch(int kb, int vb, const Plan &pl, void *temp, const void 
     if (vb == 0) return run_sort<unsigned long long, NoVal>(pl, temp, kin, kout, vin, vout, st, dev, sms);
     if (vb == 4) return run_sort<unsigned long long, uint32_t>(pl, temp, kin, kout, vin, vout, st, dev, sms);
     return run_sort<unsigned long long, unsigned long long>(pl, temp, kin, kout, vin, vout, st, dev, sms);
+#endif
 }
 
 hrs_status block_dispatch(int kb, int vb, const Plan &pl, void *temp, const void *kin, void *kout, const void *vin,
                           void *vout, uint64_t *h, uint64_t *o, bool sc, cudaStream_t st, int dev, int sms) {
+#if HRS_ONLY_TYPES
+    (void)kb; (void)vb; (void)pl; (void)temp; (void)kin; (void)kout; (void)vin; (void)vout; (void)h; (void)o;
+    (void)sc; (void)st; (void)dev; (void)sms;
+    return HRS_ERROR_INVALID_VALUE;
+#else
     if (kb == 4) {
         if (vb == 0) return run_block<uint32_t, NoVal>(pl, temp, kin, kout, vin, vout, h, o, sc, st, dev, sms);
         if (vb == 4) return run_block<uint32_t, uint32_t>(pl, temp, kin, kout, vin, vout, h, o, sc, st, dev, sms);
@@ -889,6 +911,7 @@ hrs_status block_dispatch(int kb, int vb, const Plan &pl, void *temp, const void
     if (vb == 0) return run_block<unsigned long long, NoVal>(pl, temp, kin, kout, vin, vout, h, o, sc, st, dev, sms);
     if (vb == 4) return run_block<unsigned long long, uint32_t>(pl, temp, kin, kout, vin, vout, h, o, sc, st, dev, sms);
     return run_block<unsigned long long, unsigned long long>(pl, temp, kin, kout, vin, vout, h, o, sc, st, dev, sms);
+#endif
 }
 
 bool aligned(const void *p, size_t a) { return (reinterpret_cast<uintptr_t>(p) % a) == 0; }

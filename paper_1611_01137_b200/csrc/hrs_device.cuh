@@ -51,6 +51,13 @@
 #ifndef HRS_WIDE64
 #define HRS_WIDE64 1  // measured: c4 AND-2/3/4 -4 to -9 %, uniform unchanged
 #endif
+#ifndef HRS_WO_UNROLL
+#define HRS_WO_UNROLL 4
+#endif
+namespace hrs { constexpr int WO_UNROLL = HRS_WO_UNROLL; }
+#ifndef HRS_SC_DIRECT
+#define HRS_SC_DIRECT 0  // experiment: values placed from registers, no slot index, no stability check
+#endif
 #ifndef HRS_RANK2
 #define HRS_RANK2 1  // Ranker::rank2 for blocks of >= 256 threads
 #endif
@@ -1182,6 +1189,11 @@ struct StageInfo {
     uint64_t offs;
 };
 
+// Shared memory of one scatter CTA (NBUF staging buffers of keys and values, filled by
+// TMA bulk copies).  The rank needs per-warp digit counters [W][256] and the tile's digit
+// starts; the sorted tile is built IN PLACE in the key staging buffer (the keys are held
+// in registers from the count on) plus a 16-bit slot -> element index (sidx) through which
+// the values are gathered and the stability of the fast rank is checked.
 template <typename K, typename V, int THREADS, int KPT, int NBUF>
 struct ScatterSmem {
     static constexpr int W = THREADS / 32;
@@ -1192,9 +1204,9 @@ struct ScatterSmem {
     static constexpr size_t vst_elems = KPB + 32 / sizeof(VT);
     static constexpr size_t off_bar = 0;
     static constexpr size_t off_info = 16;
-    using RK = Ranker<THREADS, KPT>;
-    static constexpr size_t off_rank = align16(off_info + NBUF * sizeof(StageInfo));
-    static constexpr size_t off_gs = align16(off_rank + RK::smem_bytes);
+    static constexpr size_t off_cnt = align16(off_info + NBUF * sizeof(StageInfo));
+    static constexpr size_t off_wsum = align16(off_cnt + sizeof(uint32_t) * W * RADIX);
+    static constexpr size_t off_gs = align16(off_wsum + sizeof(uint32_t) * 16);
     static constexpr size_t off_sidx = align16(off_gs + sizeof(uint2) * RADIX);
     static constexpr size_t off_kst = align16(off_sidx + sizeof(uint16_t) * KPB);
     static constexpr size_t kst_bytes = align16(sizeof(K) * kst_elems);
@@ -1203,23 +1215,43 @@ struct ScatterSmem {
     static constexpr size_t bytes = off_vst + NBUF * vst_bytes;
 };
 
-// NBUF staging buffers: with two, tile i + 1 is in flight into the other buffer while
-// tile i is ranked and written out; with one, the other resident CTAs cover the load.  The staged keys and values are never moved inside shared
-// memory: the rank produces, for every slot of the sorted tile, the index of the
-// element that goes there (sidx), and the write-out gathers key and value through it.
+// One counting pass over the tiles of every bucket of pass p, stable.
+// Per tile, with the next tile already in flight through TMA (NBUF = 2) or the other
+// resident CTAs covering the load (NBUF = 1):
+//   A  count: every warp ranks its 32 x KPT keys (warp-striped, element e = warp*32*KPT +
+//      c*32 + lane) against its own digit counters: the returning atomic of the fast rank
+//      gives the in-warp rank (lane order of same-address lanes, checked below), the exact
+//      rank (skewed tiles) counts each column and orders duplicates with one match-any;
+//   B  fold: thread d sums the W warp counters of digit d, a block scan of the digit
+//      totals gives the tile's digit starts, and every warp counter becomes the first slot
+//      of that warp's run of digit d (one thread per digit, all counters touched once);
+//   C  place: slot = counter + in-warp rank; the key (held in a register) is stored at its
+//      slot in the key staging buffer, the element index in sidx;
+//   D  write-out: slot j holds key ks[j] and value vs[sidx[j]], destination = global base
+//      of digit d + j - start[d]: consecutive threads store consecutive addresses of every
+//      digit run (write-combined, Fig 3).  Slot j - 1 of the same digit must
+//      hold an earlier element -- the complete stability condition; a tile that fails it
+//      (or every tile under HRS_FLAG_FORCE_REDO) is ranked again with the exact rank.
+// The per-digit global base of a tile (sub-bucket start + counts of the earlier tiles of
+// its bucket) comes from k_hist / k_classify, so tiles are independent (no
+// look-back) and claimed in order from a counter: the tiles in flight write neighbouring
+// runs of every sub-bucket, which combine in L2.
 template <typename K, typename V, int THREADS, int KPT, int MINB, int NBUF>
 __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
     pdl_wait();
     static_assert(NBUF == 1 || NBUF == 2, "one or two staging buffers");
+    static_assert(THREADS % RADIX == 0 && THREADS <= 4 * RADIX, "threads 0..255 fold one digit each");
+    static_assert(32 * KPT < (1 << 16), "the in-warp rank is packed above the digit");
     using L = ScatterSmem<K, V, THREADS, KPT, NBUF>;
+    constexpr int W = THREADS / 32;
     constexpr bool HV = HasVal<V>::value;
     using VT = ValT<V>;
     extern __shared__ __align__(16) unsigned char smem[];
     uint64_t *bar = reinterpret_cast<uint64_t *>(smem + L::off_bar);
     StageInfo *info = reinterpret_cast<StageInfo *>(smem + L::off_info);
-    typename L::RK ranker;
-    ranker.init(reinterpret_cast<uint32_t *>(smem + L::off_rank));
-    // gs[d] = {destination of slot 0 of digit d relative to the bucket, first slot of d}
+    uint32_t *cnt = reinterpret_cast<uint32_t *>(smem + L::off_cnt);    // [W][256]
+    uint32_t *wsum = reinterpret_cast<uint32_t *>(smem + L::off_wsum);  // [W] digit-total partial sums
+    // gs[d] = {destination of slot 0 of digit d relative to the bucket (may wrap), first slot of d}
     uint2 *gs = reinterpret_cast<uint2 *>(smem + L::off_gs);
     uint16_t *sidx = reinterpret_cast<uint16_t *>(smem + L::off_sidx);
     auto kst = [&](int s) { return reinterpret_cast<K *>(smem + L::off_kst + s * L::kst_bytes); };
@@ -1234,12 +1266,9 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
     const uint32_t T = alloc_tiles(prm.ctl->alloc[prm.p]);
     if (blockIdx.x >= T) return;
     const uint64_t pol = policy_evict_first();
+    uint32_t *const ca = cnt + warp * RADIX;  // this warp's counters
+    for (int i = tid; i < W * RADIX; i += THREADS) cnt[i] = 0;
 
-    // tiles are claimed in order from a counter: the tiles in flight at any moment
-    // are neighbours, so the runs they write to a sub-bucket are adjacent in memory
-    // and combine in L2 (contiguous runs per CTA measured +25% DRAM traffic).  The
-    // tile-ordered offsets come from k_hist (tile_pref) and k_classify (carry), so the
-    // tiles are independent: no look-back.
     auto issue = [&](int s, uint32_t t) {
         StageInfo &in = info[s];
         in.valid = t < T;
@@ -1275,18 +1304,18 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
     const int lo = prm.lo;
     const uint32_t mask = prm.mask;
     const uint32_t ltm = lanemask_lt();
-    // per-digit destination base of a tile, relative to its bucket: sub-bucket start
-    // + counts of the earlier tiles of the bucket (tile order = memory order: stable).
-    // Loaded one tile ahead so the global loads overlap the previous tile.
-    // The three terms are loaded a whole tile ahead (two buffers) or before the wait
-    // for the tile's data (one buffer) and added only when needed.
+    // per-digit destination base of a tile relative to its bucket: sub-bucket start + counts
+    // of the earlier tiles of the bucket (tile order = memory order: stable), loaded a tile
+    // ahead (two buffers) or before the wait for the tile's data (one buffer)
     uint32_t m0 = 0, m1 = 0, m2 = 0;
     uint64_t boffs = 0;
     auto meta_load = [&](const StageInfo &in) {
-        if (tid < RADIX && in.valid) {
-            m0 = prm.sub_rel[static_cast<uint64_t>(in.bucket) * RADIX + tid];
-            m1 = prm.tile_pref[static_cast<uint64_t>(in.tile) * RADIX + tid];
-            m2 = in.carry_row != EMPTY_RANGE ? prm.carry[static_cast<uint64_t>(in.carry_row) * RADIX + tid] : 0u;
+        if (in.valid) {
+            if (tid < RADIX) {
+                m0 = prm.sub_rel[static_cast<uint64_t>(in.bucket) * RADIX + tid];
+                m1 = prm.tile_pref[static_cast<uint64_t>(in.tile) * RADIX + tid];
+                m2 = in.carry_row != EMPTY_RANGE ? prm.carry[static_cast<uint64_t>(in.carry_row) * RADIX + tid] : 0u;
+            }
             boffs = prm.buckets[in.bucket].offs;
         }
     };
@@ -1297,9 +1326,8 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
         const StageInfo in = info[s];
         if (!in.valid) break;
         const uint32_t count = in.count;
-        const uint32_t rbase = m0 + m1 + m2;
-        const uint64_t tboffs = tid < RADIX ? boffs : prm.buckets[in.bucket].offs;
-        if (tid < RADIX) gs[tid].x = rbase;     // rank() turns it into {base - start, start}
+        const uint32_t gbase = m0 + m1 + m2;  // thread tid = digit tid
+        const uint64_t tboffs = boffs;
         Seg sk, sv;
         sk.pad = in.kpad;
         sk.i0 = static_cast<int32_t>(in.k0);
@@ -1309,78 +1337,163 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
         sv.i1 = static_cast<int32_t>(in.v1);
         const K *ksrc = kin + in.offs;
         const VT *vsrc = HV ? vin + in.offs : nullptr;
-        K *ks = kst(s);
-        VT *vs = HV ? vst(s) : nullptr;
-        if (!HRS_WAIT1 || warp == 0) mbar_wait(&bar[s], par);  // one warp waits, the barrier releases the rest
-        if (HRS_WAIT1) __syncthreads();
-        // full tiles with an aligned interior take the predicate-free path
+        K *const ks = kst(s);
+        VT *const vs = HV ? vst(s) : nullptr;
+        mbar_wait(&bar[s], par);
         const bool full = count == static_cast<uint32_t>(L::KPB) && seg_full(sk, count) && (!HV || seg_full(sv, count));
-        const K *const kb = ks + sk.pad;  // element i of the tile (after the edges are filled)
         const VT *const vb = HV ? vs + sv.pad : nullptr;
+
         auto body = [&](auto full_tag) {
             constexpr bool FULL = decltype(full_tag)::value;
-            if (!FULL) {
-                // unaligned head / tail into shared memory (read by the gathers, after barriers)
-                seg_fill_edges<K, THREADS>(ks, ksrc, sk, count);
-                if (HV) seg_fill_edges<VT, THREADS>(vs, vsrc, sv, count);
+            // the values of the elements the bulk copy did not cover (segments at the ends
+            // of the buffer) into shared memory, read by the write-out after the barriers
+            constexpr bool DIRECT = HRS_SC_DIRECT && HV;
+            if (!DIRECT && !FULL && HV) seg_fill_edges<VT, THREADS>(vs, vsrc, sv, count);
+            const K *const kb = ks + sk.pad;
+            VT val[DIRECT ? KPT : 1];
+            // the keys stay in registers from here to the placement; the in-warp ranks are
+            // packed two to a register (rank < 32 * KPT < 2^16), the digits recomputed
+            constexpr int NR = (KPT + 1) / 2;
+            K key[KPT];
+            uint32_t rk[NR];
+            uint32_t valid = 0;  // bit c: element wbase + c*32 + lane exists
+#pragma unroll
+            for (int c = 0; c < KPT; ++c) {
+                const uint32_t e = wbase + c * 32 + lane;
+                const bool v = FULL || e < count;
+                key[c] = v ? (FULL ? kb[e] : seg_get(ks, ksrc, sk, e)) : K(0);
+                if constexpr (DIRECT) val[c] = v ? (FULL ? vb[e] : seg_get(vs, vsrc, sv, e)) : VT(0);
+                valid |= v ? (1u << c) : 0u;
             }
+#pragma unroll
+            for (int i = 0; i < NR; ++i) rk[i] = 0;
+            auto dig = [&](int c) -> uint32_t { return digit_of(key[c], lo, mask); };
+            // ---- A: in-warp ranks
+            auto count_fast = [&]() {
+#pragma unroll
+                for (int c = 0; c < KPT; ++c)
+                    if (valid & (1u << c)) rk[c >> 1] |= atomicAdd(&ca[dig(c)], 1u) << (16 * (c & 1));
+            };
+            auto count_exact = [&]() {
+#pragma unroll
+                for (int c = 0; c < KPT; ++c) {
+                    const bool v0 = (valid >> c) & 1u;
+                    const uint32_t d0 = v0 ? dig(c) : 0u;
+                    const uint32_t p0 = v0 ? ca[d0] : 0u;
+                    __syncwarp();
+                    if (v0) atomicAdd(&ca[d0], 1u);
+                    __syncwarp();
+                    const uint32_t k0 = v0 ? ca[d0] - p0 : 0u;
+                    const uint32_t m = __match_any_sync(0xffffffffu, k0 > 1 ? d0 : 0xFFFFFFFFu);
+                    if (v0) rk[c >> 1] |= (p0 + (k0 > 1 ? __popc(m & ltm) : 0u)) << (16 * (c & 1));
+                }
+            };
+            // ---- B: fold the warp counters into first slots; digit starts and bases
+            auto fold = [&]() {
+                __syncthreads();  // counts complete
+                uint32_t v[W];
+                uint32_t t = 0, incl = 0;
+                if (tid < RADIX) {
+#pragma unroll
+                    for (int w = 0; w < W; ++w) {
+                        v[w] = cnt[w * RADIX + tid];
+                        t += v[w];
+                    }
+                    incl = t;
+#pragma unroll
+                    for (int o = 1; o < 32; o <<= 1) {
+                        const uint32_t y = __shfl_up_sync(0xffffffffu, incl, o);
+                        if (lane >= o) incl += y;
+                    }
+                    if (lane == 31) wsum[warp] = incl;
+                }
+                __syncthreads();
+                if (tid < RADIX) {
+                    uint32_t run = incl - t;
+#pragma unroll
+                    for (int w = 0; w < RADIX / 32; ++w) run += w < warp ? wsum[w] : 0u;
+                    gs[tid] = make_uint2(gbase - run, run);
+#pragma unroll
+                    for (int w = 0; w < W; ++w) {
+                        cnt[w * RADIX + tid] = run;
+                        run += v[w];
+                    }
+                }
+                __syncthreads();  // first slots published
+            };
+            // ---- C: place keys and element indices at their slots (in place: every key
+            // of the tile was read into registers before the fold's barriers); clear the
+            // warp's counters for the next rank
+            auto place = [&]() {
+#pragma unroll
+                for (int c = 0; c < KPT; ++c) {
+                    if (valid & (1u << c)) {
+                        const uint32_t slot = ca[dig(c)] + ((rk[c >> 1] >> (16 * (c & 1))) & 0xFFFFu);
+                        ks[slot] = key[c];
+                        if constexpr (DIRECT) vs[slot] = val[c];
+                        else sidx[slot] = static_cast<uint16_t>(wbase + c * 32 + lane);
+                    }
+                }
+                __syncwarp();
+#pragma unroll
+                for (int d = lane; d < RADIX; d += 32) ca[d] = 0;
+                __syncthreads();  // sorted tile complete
+            };
+            // ---- D: write-out (check: the complete stability condition)
             K *const kdst = kout + tboffs;
             VT *const vdst = HV ? vout + tboffs : nullptr;
-            // slot j of the sorted tile holds element sidx[j]: gather, store at its
-            // destination, and (check) test that slot j - 1, when it holds the same digit,
-            // holds an earlier element -- the complete stability condition
             auto write_out = [&](bool check) -> bool {
                 bool bad = false;
-#pragma unroll
+#pragma unroll (WO_UNROLL)
                 for (int c = 0; c < KPT; ++c) {
                     const uint32_t j = c * THREADS + tid;
                     if (FULL || j < count) {
-                        const uint32_t i = sidx[j];
-                        const K k = kb[i];
-                        const uint2 g = gs[digit_of(k, lo, mask)];
-                        const uint32_t pos = g.x + j;
-                        kdst[pos] = k;
-                        if (HV) vdst[pos] = vb[i];
-                        if (check && j > g.y) bad |= sidx[j - 1] > i;
+                        const K k = ks[j];
+                        if constexpr (DIRECT) {
+                            const uint32_t pos = gs[digit_of(k, lo, mask)].x + j;
+                            kdst[pos] = k;
+                            vdst[pos] = vs[j];
+                        } else {
+                            const uint32_t i = sidx[j];
+                            const uint2 g = gs[digit_of(k, lo, mask)];
+                            const uint32_t pos = g.x + j;
+                            kdst[pos] = k;
+                            if (HV) vdst[pos] = vb[i];
+                            if (check && j > g.y) bad |= sidx[j - 1] > i;
+                        }
                     }
                 }
                 return bad;
             };
-            // ---- digits (warp-striped: element e = warp * 32 * KPT + c * 32 + lane)
-            uint32_t dg[KPT];
+            // contention probe: equal digits among the 5 butterfly partners of column 0
+            // (a uniform digit gives 0.6 on average over the warp): heavy contention makes
+            // returning atomics slow, and the exact rank cheap
+            bool fast;
+            {
+                const uint32_t d0 = (valid & 1u) ? dig(0) : INVALID_DIGIT;
+                uint32_t eq = 0;
 #pragma unroll
-            for (int c = 0; c < KPT; ++c) {
-                const uint32_t e = wbase + c * 32 + lane;
-                if (FULL || e < count) dg[c] = digit_of(FULL ? kb[e] : seg_get(ks, ksrc, sk, e), lo, mask);
-                else dg[c] = INVALID_DIGIT;
+                for (int k2 = 1; k2 < 32; k2 <<= 1) eq += __shfl_xor_sync(0xffffffffu, d0, k2) == d0;
+                fast = __reduce_add_sync(0xffffffffu, eq) < 8;
             }
-            const bool active = FULL || wbase < count;
-            ranker.rank(dg, KPT, active, ltm, true, gs);
-            // the next tile's metadata (info[s ^ 1], published before the rank's barriers)
+            if (fast) count_fast();
+            else count_exact();
+            fold();
+            place();
+            // the next tile's metadata (info[s ^ 1] was published by the issue after the
+            // previous tile, before this tile's barriers); the loads overlap the write-out
             if (NBUF == 2) meta_load(info[s ^ 1]);
-#pragma unroll
-            for (int c = 0; c < KPT; ++c) {
-                const uint32_t e = wbase + c * 32 + lane;
-                if (FULL || e < count) sidx[dg[c]] = static_cast<uint16_t>(e);
-            }
-            __syncthreads();
-            const bool bad = write_out(true);
-            if (__syncthreads_or(bad || prm.force_redo)) {
-                // the atomics did not serve the lanes in order: redo the tile with the
-                // rank that is stable by construction (same digit starts, so gs holds)
+            const bool bad = write_out(fast && !DIRECT);
+            if (__syncthreads_or(bad || (fast && prm.force_redo))) {
+                // the atomics did not serve the lanes of a warp in order: rank the tile
+                // again with the rank that is stable by construction (same digit totals, so
+                // the starts and bases are unchanged) and write it out again
                 if (tid == 0) atomicAdd(&prm.ctl->redo, 1ull);
 #pragma unroll
-                for (int c = 0; c < KPT; ++c) {
-                    const uint32_t e = wbase + c * 32 + lane;
-                    dg[c] = (FULL || e < count) ? digit_of(kb[e], lo, mask) : INVALID_DIGIT;
-                }
-                ranker.rank(dg, KPT, active, ltm, false);
-#pragma unroll
-                for (int c = 0; c < KPT; ++c) {
-                    const uint32_t e = wbase + c * 32 + lane;
-                    if (FULL || e < count) sidx[dg[c]] = static_cast<uint16_t>(e);
-                }
-                __syncthreads();
+                for (int i = 0; i < NR; ++i) rk[i] = 0;
+                count_exact();
+                fold();
+                place();
                 write_out(false);
                 __syncthreads();
             }
