@@ -61,7 +61,8 @@ def test_forced_redo_default_tuning(kbits, vbits, dist):
     v = gen.values(n, vbits, "random", seed=13) if vbits else None
     st = _forced_sort(k, v, 0, kbits)
     assert st["overflow"] == 0
-    if st["counting_passes"]:
+    if dist in ("uniform", "and2"):
+        # (constant / AND-4 digits make every warp take the exact rank, which needs no check)
         assert st["redo_blocks"] > 0, "the forced redo branch did not run"
 
 
