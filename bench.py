@@ -36,7 +36,11 @@ CONFIGS = {
     "c2": (28, 32, 32, "2^28 uint32 key + uint32 value pairs"),
     "c3": (28, 32, 32, "2^28 uint32 key + uint32 value pairs, AND-skewed"),
     "c4": (28, 64, 64, "2^28 uint64 key + uint64 value pairs"),
+    # BASELINE.json configs[4]: 64 GiB of u64/u64 records in total, split over the N GPUs
+    # (strong scaling); needs N >= 2 (input + output + aux of 64 GiB exceed one GPU's HBM)
+    "c5": (32, 64, 64, "2^32 uint64 key + uint64 value pairs (64 GiB) in total"),
 }
+STRONG = {"c5"}
 METRIC = "sorted records/sec and % of B200 HBM roofline (1/2/4/8 GPU)"
 
 
@@ -159,7 +163,14 @@ def run_hrs(args):
     dist_name = args.dist
     if args.config == "c3" and dist_name == "uniform":
         dist_name = "and3"
-    n = 1 << logn
+    strong = args.config in STRONG
+    n = (1 << logn) // world if strong else 1 << logn  # records per GPU
+    if strong and world < 2 and not args.force_dist:
+        if rank == 0:
+            print(json.dumps({"metric": METRIC, "config": {"workload": f"{args.config}:{desc}"}, "n_gpus": world,
+                              "unavailable": "64 GiB of input plus its output and aux exceed one GPU's HBM; "
+                                             "c5 runs at N >= 2 (or one rank's shard with --force-dist)"}))
+        return 0
     kb, vb = kbits // 8, vbits // 8
     pg = None
     use_dist = world > 1 or args.force_dist
@@ -218,7 +229,8 @@ def run_hrs(args):
 
     peak, peak_kind = _peaks()
     out = {"metric": METRIC, "value": value, "unit": "records/s", "n_gpus": world, "steps": args.steps,
-           "warmup": args.warmup, "ms_per_step": t_ms, "higher_is_better": True, "scaling": "weak",
+           "warmup": args.warmup, "ms_per_step": t_ms, "higher_is_better": True,
+           "scaling": "strong" if strong else "weak",
            "vs_baseline": None, "dtype": "u32" if kbits == 32 else "u64", "data": "synthetic",
            "config": {"workload": f"{args.config}:{desc}, {dist_name}", "n_per_gpu": n, "key_bits": kbits,
                       "value_bits": vbits, "bits": [0, kbits], "values": "input index",
@@ -466,6 +478,28 @@ def cpu_baseline(args, kbits, vbits, dist_name, keys_dev=None):
             "stable_sort_1core": {"value": ns / t_ss, "records": ns, "s": t_ss, "what": "std::stable_sort, 1 thread"}}
 
 
+def _self_launch(args, argv) -> int | None:
+    """`bench.py --gpus N` without torchrun's environment: start N ranks of this script
+    with torch.distributed.run (one process per GPU, 127.0.0.1 rendezvous) and return its
+    exit code; under torchrun, check that --gpus agrees with WORLD_SIZE."""
+    ws = os.environ.get("WORLD_SIZE")
+    if ws is not None:
+        if int(ws) != args.gpus:
+            sys.stderr.write(f"bench.py: --gpus {args.gpus} but WORLD_SIZE={ws}\n")
+            raise SystemExit(2)
+        return None
+    if args.gpus <= 1:
+        return None
+    import socket
+    with socket.socket() as sk:
+        sk.bind(("127.0.0.1", 0))
+        port = sk.getsockname()[1]
+    cmd = [sys.executable, "-m", "torch.distributed.run", "--nnodes=1", f"--nproc-per-node={args.gpus}",
+           "--master-addr", "127.0.0.1", "--master-port", str(port), os.path.abspath(__file__),
+           *(argv if argv is not None else sys.argv[1:])]
+    return subprocess.call(cmd)
+
+
 def main(argv=None):
     ap = argparse.ArgumentParser()
     ap.add_argument("--gpus", type=int, default=1)
@@ -483,6 +517,9 @@ def main(argv=None):
     args = ap.parse_args(argv)
     if args.warmup < 3:
         args.warmup = 3
+    rc = _self_launch(args, argv)
+    if rc is not None:
+        return rc
     if args.impl == "reference":
         return run_reference(args)
     return run_hrs(args)

@@ -83,6 +83,17 @@ class CudaOps:
     def sort(self, keys, vals, begin_bit, end_bit):
         return self.hrs.sort(keys, vals, begin_bit, end_bit)
 
+    def sort_into(self, keys, vals, begin_bit, end_bit, keys_out, vals_out, temp_holder):
+        """Sort into caller buffers with a temp kept across calls (temp_holder: a one-element
+        list holding the temp tensor or None): no allocation on the step's critical path."""
+        kb, vb = keys.element_size(), (vals.element_size() if vals is not None else 0)
+        need = self.hrs.temp_bytes(keys.numel(), kb, vb, begin_bit, end_bit)
+        if temp_holder[0] is None or temp_holder[0].numel() < need:
+            temp_holder[0] = None
+            temp_holder[0] = self.hrs.alloc_temp(need, keys.device)
+        return self.hrs.sort(keys, vals, begin_bit, end_bit, keys_out=keys_out, values_out=vals_out,
+                             temp=temp_holder[0])
+
 
 class DistributedSorter:
     """Sorts the global array formed by concatenating every rank's (keys, vals) shard
@@ -103,6 +114,27 @@ class DistributedSorter:
         # so bench.py can report the exchange against NVLink bandwidth
         self.time_exchange = False
         self.exchange_events = None
+        # buffers kept across steps (memory at C5 scale): the partition output
+        # (= send buffer, later the local sort's output), the receive buffer (= refinement
+        # scratch before the exchange) and the local sort's temp
+        self._kp = self._vp = None
+        self._rk = self._rv = None
+        self._temp = [None]
+
+    def _send_buffers(self, n):
+        if self._kp is None or self._kp.numel() != n:
+            self._kp = self._vp = None
+            self._kp = torch.empty_like(self.keys)
+            self._vp = torch.empty_like(self.vals) if self.vals is not None else None
+        return self._kp, self._vp
+
+    def _recv_buffers(self, cap):
+        if self._rk is None or self._rk.numel() < cap:
+            self._rk = self._rv = None
+            self._rk = torch.empty(cap, dtype=self.keys.dtype, device=self.keys.device)
+            self._rv = (torch.empty(cap, dtype=self.vals.dtype, device=self.vals.device)
+                        if self.vals is not None else None)
+        return self._rk, self._rv
 
     def digits(self):
         """The (lo, hi) bit ranges of the 8-bit digits, most significant first."""
@@ -120,12 +152,13 @@ class DistributedSorter:
             return keys.clone(), (vals.clone() if vals is not None else None), self._offset_identity()
         digits = self.digits()
         # 1-3a. first-digit partition of the whole shard; its histogram, gathered
-        kp = torch.empty_like(keys)
-        vp = torch.empty_like(vals) if vals is not None else None
+        kp, vp = self._send_buffers(keys.numel())
         lo, hi = digits[0]
         offs = self.ops.partition_into(keys, vals, lo, hi, kp, vp)
         hists = self._gather([[offs[b + 1] - offs[b] for b in range(len(offs) - 1)]])[0]  # [rank][bucket]
         N = sum(sum(h) for h in hists)
+        cap = max((j + 1) * N // world - j * N // world for j in range(world))  # largest receive
+        rk_all, rv_all = self._recv_buffers(cap)
         # split[j][r]: local position on rank r of global sorted position t_j = j N / G
         split = [[0] * world for _ in range(world + 1)]
         split[world] = [sum(h) for h in hists]
@@ -140,8 +173,14 @@ class DistributedSorter:
                 break
             levels = level
             if scratch_k is None:
-                scratch_k = torch.empty_like(kp)
-                scratch_v = torch.empty_like(vp) if vp is not None else None
+                # the receive buffer is not in use before the exchange: it is the scratch of
+                # the refinement passes (a refined sub-range larger than it gets its own)
+                big = max(it[5][me] for it in todo)
+                if big <= rk_all.numel():
+                    scratch_k, scratch_v = rk_all, rv_all
+                else:
+                    scratch_k = torch.empty(big, dtype=kp.dtype, device=kp.device)
+                    scratch_v = torch.empty(big, dtype=vp.dtype, device=vp.device) if vp is not None else None
             lo, hi = digits[level]
             segs = []  # distinct segments (several boundaries may share one)
             for item in todo:
@@ -152,10 +191,10 @@ class DistributedSorter:
                 a, c = starts[me], counts[me]
                 if c:
                     sub = self.ops.partition_into(kp[a:a + c], vp[a:a + c] if vp is not None else None, lo, hi,
-                                                  scratch_k[a:a + c], scratch_v[a:a + c] if vp is not None else None)
-                    kp[a:a + c].copy_(scratch_k[a:a + c])
+                                                  scratch_k[:c], scratch_v[:c] if vp is not None else None)
+                    kp[a:a + c].copy_(scratch_k[:c])
                     if vp is not None:
-                        vp[a:a + c].copy_(scratch_v[a:a + c])
+                        vp[a:a + c].copy_(scratch_v[:c])
                     local.append([sub[b + 1] - sub[b] for b in range(len(sub) - 1)])
                 else:
                     local.append([0] * (1 << (hi - lo)))
@@ -175,8 +214,9 @@ class DistributedSorter:
         send = [[split[j + 1][r] - split[j][r] for j in range(world)] for r in range(world)]
         recv = [send[src][me] for src in range(world)]
         # 4. exchange (every source's segment in source-rank order)
-        rk = torch.empty(sum(recv), dtype=keys.dtype, device=keys.device)
-        rv = torch.empty(sum(recv), dtype=vals.dtype, device=vals.device) if vals is not None else None
+        m = sum(recv)
+        rk = rk_all[:m]
+        rv = rv_all[:m] if vals is not None else None
         ev = None
         if self.time_exchange and keys.is_cuda:
             ev = (torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True))
@@ -187,8 +227,13 @@ class DistributedSorter:
         if ev is not None:
             ev[1].record()
         self.exchange_events = ev
-        # 5. local sort of the received records (source-rank order = global input order)
-        ko, vo = self.ops.sort(rk, rv, self.begin, self.end)
+        # 5. local sort of the received records (source-rank order = global input order),
+        # into the send buffers (dead after the exchange) when they are large enough
+        if hasattr(self.ops, "sort_into") and m <= kp.numel():
+            ko, vo = self.ops.sort_into(rk, rv, self.begin, self.end, kp[:m], vp[:m] if vp is not None else None,
+                                        self._temp)
+        else:
+            ko, vo = self.ops.sort(rk, rv, self.begin, self.end)
         offset = me * N // world
         self.last = {"send": send[me], "recv": recv, "offset": offset, "refine_levels": levels,
                      "imbalance": max(sum(send[s][j] for s in range(world)) for j in range(world)) /

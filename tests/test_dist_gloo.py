@@ -43,6 +43,15 @@ class OracleOps:
         ko, vo = oracle.sort(keys, vals, b, e)
         return _to_torch(ko, keys), (_to_torch(vo, vals) if vals is not None else None)
 
+    def sort_into(self, keys, vals, b, e, keys_out, vals_out, temp_holder):
+        """Into the driver's reused buffers (the send buffer), as the CUDA path does."""
+        ko, vo = self.sort(keys, vals, b, e)
+        keys_out.copy_(ko)
+        if vals is not None:
+            vals_out.copy_(vo)
+        temp_holder[0] = "used"
+        return keys_out, vals_out
+
 
 def _free_port():
     s = socket.socket()
@@ -61,6 +70,12 @@ def _worker(rank, world, port, n_per, kbits, dist_name, q):
         v = gen.values(n_per, 64, "index", start=rank * n_per)
         sorter = hdist.DistributedSorter(k, v, ops=OracleOps())
         ko, vo, off = sorter.step()
+        ko = ko.clone()
+        # a second step reuses every buffer (send / receive / temp) and must give the same
+        ko2, vo2, off2 = sorter.step()
+        assert off2 == off and torch.equal(ko2.view(torch.int64 if kbits == 64 else torch.int32),
+                                           ko.view(torch.int64 if kbits == 64 else torch.int32))
+        assert sorter._temp[0] == "used" and ko2.data_ptr() == sorter._kp.data_ptr()
         parts = [None] * world
         dist.all_gather_object(parts, (off, oracle._u64(ko).tolist(), oracle._u64(vo).tolist(), sorter.last))
         if rank == 0:
