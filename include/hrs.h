@@ -147,6 +147,24 @@ hrs_status hrs_sort_ex(void *d_temp, size_t *temp_bytes, const void *keys_in, vo
                        const void *vals_in, void *vals_out, uint64_t n, int key_bytes, int value_bytes,
                        int begin_bit, int end_bit, const hrs_tuning *tuning, hrs_stream_t stream);
 
+/* The same stable sort for an input that is ALREADY GROUPED by its first (most
+ * significant) digit: the digit of bits [max(begin_bit, end_bit - 8), end_bit), the first
+ * digit of the plan, with the records of digit value 0 first, then 1, ... --
+ * e.g. what a partition pass on that digit (hrs_partition_pass) or the bucket-major
+ * exchange of the distributed sort produces.  d_first_digit_hist (device, 2^width uint64)
+ * holds the number of records of every digit value; it must sum to n.  The library takes
+ * the first counting pass as done (its histogram, exclusive prefix and sub-bucket
+ * classification, run from d_first_digit_hist; nothing is moved) and
+ * continues at the second digit, so the sort reads and writes every record once less.
+ * Output, temp size, layout, ownership, async behaviour and errors as hrs_sort_ex
+ * (HRS_ERROR_INVALID_VALUE if d_first_digit_hist is NULL for a non-trivial sort).  The
+ * grouping is a precondition, not checked: an input that is not grouped, or a histogram
+ * that does not describe it, gives an unspecified permutation of the input. */
+hrs_status hrs_sort_grouped(void *d_temp, size_t *temp_bytes, const void *keys_in, void *keys_out,
+                            const void *vals_in, void *vals_out, uint64_t n, int key_bytes, int value_bytes,
+                            int begin_bit, int end_bit, const uint64_t *d_first_digit_hist, const hrs_tuning *tuning,
+                            hrs_stream_t stream);
+
 /* Copies the stats block of the last sort that used d_temp to *out.  Synchronises
  * `stream`; call it outside any timed region. */
 hrs_status hrs_get_stats(const void *d_temp, hrs_stats *out, hrs_stream_t stream);

@@ -15,7 +15,7 @@ import torch
 
 from ._lib import HRS_MAX_ITEMS, HrsError, Stats, Tuning, check, lib  # noqa: F401
 
-__all__ = ["sort", "temp_bytes", "get_stats", "digit_histogram", "partition_pass", "HrsError", "Tuning",
+__all__ = ["sort", "sort_grouped", "temp_bytes", "get_stats", "digit_histogram", "partition_pass", "HrsError", "Tuning",
            "default_tuning", "max_local_threshold", "max_keys_per_tile", "class_capacities", "lib"]
 
 _KEY_DTYPES = {torch.uint32: 4, torch.uint64: 8}
@@ -100,7 +100,7 @@ def alloc_temp(nbytes: int, device) -> torch.Tensor:
 
 def sort(keys: torch.Tensor, values: torch.Tensor | None = None, begin_bit: int = 0, end_bit: int | None = None,
          *, tuning=None, keys_out: torch.Tensor | None = None, values_out: torch.Tensor | None = None,
-         temp: torch.Tensor | None = None, stream=None):
+         temp: torch.Tensor | None = None, stream=None, first_digit_hist: torch.Tensor | None = None):
     """Stable sort of `keys` (and `values`) by key bits [begin_bit, end_bit).
 
     Returns (keys_out, values_out); values_out is None for keys-only sorts.
@@ -108,6 +108,8 @@ def sort(keys: torch.Tensor, values: torch.Tensor | None = None, begin_bit: int 
     """
     _check_tensor(keys, "keys")
     if keys.dtype in _TYPED_KEYS:
+        if first_digit_hist is not None:
+            raise TypeError("grouped sorts take unsigned keys")
         return sort_typed(keys, values, keys_out=keys_out, values_out=values_out, temp=temp, stream=stream,
                           begin_bit=begin_bit, end_bit=end_bit, tuning=tuning)
     kb = _nbytes(keys, "keys")
@@ -131,10 +133,36 @@ def sort(keys: torch.Tensor, values: torch.Tensor | None = None, begin_bit: int 
     _on_stream(stream, temp, keys_out, values_out)
     sz = ctypes.c_size_t(temp.numel())
     with torch.cuda.device(keys.device):
-        check(lib.hrs_sort_ex(_ptr(temp), ctypes.byref(sz), _ptr(keys), _ptr(keys_out), _ptr(values),
-                              _ptr(values_out), n, kb, vb, begin_bit, end_bit, _tuning(tuning), _stream(stream)),
-              "hrs_sort_ex")
+        if first_digit_hist is None:
+            check(lib.hrs_sort_ex(_ptr(temp), ctypes.byref(sz), _ptr(keys), _ptr(keys_out), _ptr(values),
+                                  _ptr(values_out), n, kb, vb, begin_bit, end_bit, _tuning(tuning),
+                                  _stream(stream)), "hrs_sort_ex")
+        else:
+            check(lib.hrs_sort_grouped(_ptr(temp), ctypes.byref(sz), _ptr(keys), _ptr(keys_out), _ptr(values),
+                                       _ptr(values_out), n, kb, vb, begin_bit, end_bit, _ptr(first_digit_hist),
+                                       _tuning(tuning), _stream(stream)), "hrs_sort_grouped")
     return keys_out, (values_out if values is not None else None)
+
+
+def sort_grouped(keys: torch.Tensor, values: torch.Tensor | None, first_digit_hist, begin_bit: int = 0,
+                 end_bit: int | None = None, **kw):
+    """hrs_sort_grouped: the stable sort of an input already grouped by its first digit
+    (bits [max(begin, end - 8), end)) in ascending order, with that digit's counts
+    `first_digit_hist` (a sequence or a tensor of 2^width counts); skips the first pass."""
+    if keys.dtype in _TYPED_KEYS:
+        raise TypeError("sort_grouped takes unsigned keys")
+    if end_bit is None:
+        end_bit = 8 * _nbytes(keys, "keys")
+    width = min(8, end_bit - begin_bit)
+    h = first_digit_hist
+    if not isinstance(h, torch.Tensor) or h.dtype != torch.uint64 or not h.is_cuda:
+        h = torch.as_tensor([int(x) for x in (h.tolist() if isinstance(h, torch.Tensor) else h)],
+                            dtype=torch.int64).view(torch.uint64).to(keys.device)
+    if end_bit > begin_bit and h.numel() != (1 << width):
+        raise ValueError(f"first_digit_hist needs {1 << width} counts")
+    stream = kw.get("stream")
+    _on_stream(stream, h)
+    return sort(keys, values, begin_bit, end_bit, first_digit_hist=h, **kw)
 
 
 def typed_temp_bytes(n: int, key_bytes: int, value_bytes: int, kind: int) -> int:

@@ -468,8 +468,11 @@ struct Runner {
     static constexpr int HIST_CAP = ScatterCfg<KB, VB>::THREADS * ScatterCfg<KB, VB>::KPT;
     using SC = ScatterCfg<KB, (VB == 0 ? 4 : VB)>;
 
-    static hrs_status init(const Plan &pl, void *temp, cudaStream_t st, int sms, int root_class, int counting) {
+    static hrs_status init(const Plan &pl, void *temp, cudaStream_t st, int sms, int root_class, int counting,
+                           const uint64_t *grouped_hist = nullptr) {
         InitParams ip;
+        ip.grouped_hist = grouped_hist;
+        ip.grouped_radix = 1u << (pl.hi[0] - pl.lo[0]);
         ip.ctl = at<Ctl>(temp, 0);
         ip.buckets = at<Bucket>(temp, pl.off_buckets[1]);
         ip.tot = at<uint32_t>(temp, pl.off_tot[1]);
@@ -774,17 +777,22 @@ struct Runner {
         return HRS_ERROR_INVALID_VALUE;
     }
 
+    // grouped: the input is already grouped by its first digit (hrs_sort_grouped) with the
+    // device histogram `grouped`; pass 1's partition is skipped (X_1 = the input)
     static hrs_status sort(const Plan &pl, void *temp, const void *kin, void *kout, const void *vin, void *vout,
-                           cudaStream_t st, int dev, int sms) {
+                           cudaStream_t st, int dev, int sms, const uint64_t *grouped = nullptr) {
         hrs_status s;
         const int root_class =
             pl.counting ? -1
                         : (pl.single_class >= 0 ? pl.single_class
                                                 : size_class_of((uint32_t)std::max<uint64_t>(pl.n, 1)));
-        if ((s = init(pl, temp, st, sms, pl.n > 0 && pl.begin < pl.end ? root_class : -1, pl.counting ? 1 : 0)))
+        // a grouped input on a single digit is already the stable sort: one copy
+        const bool copy_only = grouped && pl.counting && pl.D == 1;
+        if ((s = init(pl, temp, st, sms, pl.n > 0 && pl.begin < pl.end ? root_class : -1, pl.counting ? 1 : 0,
+                      pl.counting && !copy_only ? grouped : nullptr)))
             return s;
         if (pl.n == 0) return HRS_SUCCESS;
-        if (pl.begin == pl.end) {
+        if (pl.begin == pl.end || copy_only) {
             using VC = typename std::conditional<VB == 8, uint64_t, uint32_t>::type;
             const int grid = static_cast<int>(std::min<uint64_t>((pl.n + 255) / 256, static_cast<uint64_t>(sms) * 8));
             {
@@ -809,6 +817,12 @@ struct Runner {
                 const bool to_out = ((pl.D - p) % 2) == 0;
                 void *yk = to_out ? kout : auxk;
                 void *yv = to_out ? vout : auxv;
+                if (p == 1 && grouped) {
+                    // the partition on digit 1 is given: classify its histogram (no per-CTA
+                    // ranges), the sub-buckets stay in the input (X_1 = in)
+                    if ((s = classify(pl, temp, st, dev, sms, 1, SRC_IN, nullptr, nullptr, false, 0))) return s;
+                    continue;
+                }
                 if ((s = hist(pl, temp, st, dev, sms, p, xk, G))) return s;
                 if ((s = classify(pl, temp, st, dev, sms, p, to_out ? SRC_OUT : SRC_AUX, nullptr, nullptr,
                                   p == pl.D, G)))
@@ -860,8 +874,8 @@ struct Runner {
 
 template <typename K, typename V>
 hrs_status run_sort(const Plan &pl, void *temp, const void *kin, void *kout, const void *vin, void *vout,
-                    cudaStream_t st, int dev, int sms) {
-    return Runner<K, V>::sort(pl, temp, kin, kout, vin, vout, st, dev, sms);
+                    cudaStream_t st, int dev, int sms, const uint64_t *grouped) {
+    return Runner<K, V>::sort(pl, temp, kin, kout, vin, vout, st, dev, sms, grouped);
 }
 
 template <typename K, typename V>
@@ -876,23 +890,23 @@ hrs_status run_block(const Plan &pl, void *temp, const void *kin, void *kout, co
 #define HRS_ONLY_TYPES 0
 #endif
 hrs_status sort_dispatch(int kb, int vb, const Plan &pl, void *temp, const void *kin, void *kout, const void *vin,
-                         void *vout, cudaStream_t st, int dev, int sms) {
+                         void *vout, cudaStream_t st, int dev, int sms, const uint64_t *grouped = nullptr) {
 #if HRS_ONLY_TYPES == 44
-    if (kb == 4 && vb == 4) return run_sort<uint32_t, uint32_t>(pl, temp, kin, kout, vin, vout, st, dev, sms);
+    if (kb == 4 && vb == 4) return run_sort<uint32_t, uint32_t>(pl, temp, kin, kout, vin, vout, st, dev, sms, grouped);
     return HRS_ERROR_INVALID_VALUE;
 #elif HRS_ONLY_TYPES == 88
     if (kb == 8 && vb == 8)
-        return run_sort<unsigned long long, unsigned long long>(pl, temp, kin, kout, vin, vout, st, dev, sms);
+        return run_sort<unsigned long long, unsigned long long>(pl, temp, kin, kout, vin, vout, st, dev, sms, grouped);
     return HRS_ERROR_INVALID_VALUE;
 #else
     if (kb == 4) {
-        if (vb == 0) return run_sort<uint32_t, NoVal>(pl, temp, kin, kout, vin, vout, st, dev, sms);
-        if (vb == 4) return run_sort<uint32_t, uint32_t>(pl, temp, kin, kout, vin, vout, st, dev, sms);
-        return run_sort<uint32_t, unsigned long long>(pl, temp, kin, kout, vin, vout, st, dev, sms);
+        if (vb == 0) return run_sort<uint32_t, NoVal>(pl, temp, kin, kout, vin, vout, st, dev, sms, grouped);
+        if (vb == 4) return run_sort<uint32_t, uint32_t>(pl, temp, kin, kout, vin, vout, st, dev, sms, grouped);
+        return run_sort<uint32_t, unsigned long long>(pl, temp, kin, kout, vin, vout, st, dev, sms, grouped);
     }
-    if (vb == 0) return run_sort<unsigned long long, NoVal>(pl, temp, kin, kout, vin, vout, st, dev, sms);
-    if (vb == 4) return run_sort<unsigned long long, uint32_t>(pl, temp, kin, kout, vin, vout, st, dev, sms);
-    return run_sort<unsigned long long, unsigned long long>(pl, temp, kin, kout, vin, vout, st, dev, sms);
+    if (vb == 0) return run_sort<unsigned long long, NoVal>(pl, temp, kin, kout, vin, vout, st, dev, sms, grouped);
+    if (vb == 4) return run_sort<unsigned long long, uint32_t>(pl, temp, kin, kout, vin, vout, st, dev, sms, grouped);
+    return run_sort<unsigned long long, unsigned long long>(pl, temp, kin, kout, vin, vout, st, dev, sms, grouped);
 #endif
 }
 
@@ -1023,9 +1037,31 @@ bool via_graph(const GraphKey &key, cudaStream_t stream, int dev, hrs_status *ou
 
 extern "C" {
 
+static hrs_status sort_common(void *d_temp, size_t *temp_bytes, const void *keys_in, void *keys_out,
+                              const void *vals_in, void *vals_out, uint64_t n, int key_bytes, int value_bytes,
+                              int begin_bit, int end_bit, const hrs_tuning *tuning, const uint64_t *grouped,
+                              hrs_stream_t stream);
+
 hrs_status hrs_sort_ex(void *d_temp, size_t *temp_bytes, const void *keys_in, void *keys_out, const void *vals_in,
                        void *vals_out, uint64_t n, int key_bytes, int value_bytes, int begin_bit, int end_bit,
                        const hrs_tuning *tuning, hrs_stream_t stream) {
+    return sort_common(d_temp, temp_bytes, keys_in, keys_out, vals_in, vals_out, n, key_bytes, value_bytes,
+                       begin_bit, end_bit, tuning, nullptr, stream);
+}
+
+hrs_status hrs_sort_grouped(void *d_temp, size_t *temp_bytes, const void *keys_in, void *keys_out,
+                            const void *vals_in, void *vals_out, uint64_t n, int key_bytes, int value_bytes,
+                            int begin_bit, int end_bit, const uint64_t *d_first_digit_hist, const hrs_tuning *tuning,
+                            hrs_stream_t stream) {
+    if (d_temp && n > 0 && begin_bit < end_bit && !d_first_digit_hist) return HRS_ERROR_INVALID_VALUE;
+    return sort_common(d_temp, temp_bytes, keys_in, keys_out, vals_in, vals_out, n, key_bytes, value_bytes,
+                       begin_bit, end_bit, tuning, d_first_digit_hist, stream);
+}
+
+static hrs_status sort_common(void *d_temp, size_t *temp_bytes, const void *keys_in, void *keys_out,
+                              const void *vals_in, void *vals_out, uint64_t n, int key_bytes, int value_bytes,
+                              int begin_bit, int end_bit, const hrs_tuning *tuning, const uint64_t *grouped,
+                              hrs_stream_t stream) {
     if (!temp_bytes) return HRS_ERROR_INVALID_VALUE;
     if (key_bytes != 4 && key_bytes != 8) return HRS_ERROR_INVALID_VALUE;
     if (value_bytes != 0 && value_bytes != 4 && value_bytes != 8) return HRS_ERROR_INVALID_VALUE;
@@ -1058,7 +1094,8 @@ hrs_status hrs_sort_ex(void *d_temp, size_t *temp_bytes, const void *keys_in, vo
     if ((s = check_device(&dev, &sms))) return s;
     cudaStream_t st = reinterpret_cast<cudaStream_t>(stream);
     auto run = [&](cudaStream_t on) {
-        return sort_dispatch(key_bytes, value_bytes, pl, d_temp, keys_in, keys_out, vals_in, vals_out, on, dev, sms);
+        return sort_dispatch(key_bytes, value_bytes, pl, d_temp, keys_in, keys_out, vals_in, vals_out, on, dev, sms,
+                             grouped);
     };
     cudaStreamCaptureStatus cap = cudaStreamCaptureStatusNone;
     if (n > 0 && n <= HRS_GRAPH_MAX_N && !g_prof && graphs_enabled() &&
@@ -1082,6 +1119,7 @@ hrs_status hrs_sort_ex(void *d_temp, size_t *temp_bytes, const void *keys_in, vo
         v[11] = reinterpret_cast<uintptr_t>(d_temp);
         v[12] = *temp_bytes;
         v[13] = t.flags | env_flags();
+        v[14] = reinterpret_cast<uintptr_t>(grouped);
         hrs_status gs = HRS_SUCCESS;
         if (via_graph(key, st, dev, &gs, run)) return gs;
     }

@@ -599,6 +599,10 @@ struct InitParams {
     int counting;  // 1: the root bucket is counting-sorted
     int end_bit;
     uint32_t key_bytes, value_bytes;
+    // hrs_sort_grouped: the input is already grouped by the first digit with these counts
+    // (2^width u64): pass 1's partition is given, its histogram is this, it moves nothing
+    const uint64_t *grouped_hist;
+    uint32_t grouped_radix;
 };
 
 __global__ void k_init(InitParams prm) {
@@ -609,7 +613,10 @@ __global__ void k_init(InitParams prm) {
         uint32_t *w = reinterpret_cast<uint32_t *>(prm.ctl);
         for (int i = threadIdx.x; i < static_cast<int>(sizeof(Ctl) / 4); i += blockDim.x) w[i] = 0;
         if (prm.counting)
-            for (int i = threadIdx.x; i < RADIX; i += blockDim.x) prm.tot[i] = 0;
+            for (int i = threadIdx.x; i < RADIX; i += blockDim.x)
+                prm.tot[i] = (prm.grouped_hist && static_cast<uint32_t>(i) < prm.grouped_radix)
+                                 ? static_cast<uint32_t>(prm.grouped_hist[i])
+                                 : 0u;
         __syncthreads();
         if (threadIdx.x == 0) {
             Ctl *c = prm.ctl;
@@ -618,8 +625,9 @@ __global__ void k_init(InitParams prm) {
             c->key_bytes = prm.key_bytes;
             c->value_bytes = prm.value_bytes;
             if (prm.counting) {
-                c->alloc[1] = (static_cast<unsigned long long>(T1) << 32) | 1ull;
-                c->recs_in_pass[1] = n;
+                // (grouped input: pass 1 has its bucket but no tiles and moves no record)
+                c->alloc[1] = (static_cast<unsigned long long>(prm.grouped_hist ? 0u : T1) << 32) | 1ull;
+                c->recs_in_pass[1] = prm.grouped_hist ? 0ull : n;
                 Bucket b;
                 b.offs = 0;
                 b.count = static_cast<uint32_t>(n);

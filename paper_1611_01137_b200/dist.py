@@ -83,14 +83,23 @@ class CudaOps:
     def sort(self, keys, vals, begin_bit, end_bit):
         return self.hrs.sort(keys, vals, begin_bit, end_bit)
 
-    def sort_into(self, keys, vals, begin_bit, end_bit, keys_out, vals_out, temp_holder):
-        """Sort into caller buffers with a temp kept across calls (temp_holder: a one-element
-        list holding the temp tensor or None): no allocation on the step's critical path."""
+    def sort_grouped_into(self, keys, vals, first_hist, begin_bit, end_bit, keys_out, vals_out, temp_holder):
+        """hrs_sort_grouped into caller buffers (the input is grouped by its first digit)."""
+        self._temp_for(keys, vals, begin_bit, end_bit, temp_holder)
+        return self.hrs.sort_grouped(keys, vals, first_hist, begin_bit, end_bit, keys_out=keys_out,
+                                     values_out=vals_out, temp=temp_holder[0])
+
+    def _temp_for(self, keys, vals, begin_bit, end_bit, temp_holder):
         kb, vb = keys.element_size(), (vals.element_size() if vals is not None else 0)
         need = self.hrs.temp_bytes(keys.numel(), kb, vb, begin_bit, end_bit)
         if temp_holder[0] is None or temp_holder[0].numel() < need:
             temp_holder[0] = None
             temp_holder[0] = self.hrs.alloc_temp(need, keys.device)
+
+    def sort_into(self, keys, vals, begin_bit, end_bit, keys_out, vals_out, temp_holder):
+        """Sort into caller buffers with a temp kept across calls (temp_holder: a one-element
+        list holding the temp tensor or None): no allocation on the step's critical path."""
+        self._temp_for(keys, vals, begin_bit, end_bit, temp_holder)
         return self.hrs.sort(keys, vals, begin_bit, end_bit, keys_out=keys_out, values_out=vals_out,
                              temp=temp_holder[0])
 
@@ -101,12 +110,17 @@ class DistributedSorter:
     global offset."""
 
     def __init__(self, keys: torch.Tensor, vals: torch.Tensor | None = None, group=None, begin_bit: int = 0,
-                 end_bit: int | None = None, ops=None):
+                 end_bit: int | None = None, ops=None, exchange: str = "grouped"):
         self.keys, self.vals, self.group = keys, vals, group
         self.kbits = 8 * keys.element_size()
         self.begin = begin_bit
         self.end = self.kbits if end_bit is None else end_bit
         self.ops = ops if ops is not None else CudaOps()
+        if exchange not in ("grouped", "a2a"):
+            raise ValueError(exchange)
+        # "grouped": bucket-major point-to-point exchange, the receiver skips the first pass;
+        # "a2a": one all_to_all_single per array, the receiver sorts from the first digit
+        self.exchange = exchange
         self.world = dist.get_world_size(group)
         self.rank = dist.get_rank(group)
         self.last = {}
@@ -213,7 +227,6 @@ class DistributedSorter:
                 run += counts[r]
         send = [[split[j + 1][r] - split[j][r] for j in range(world)] for r in range(world)]
         recv = [send[src][me] for src in range(world)]
-        # 4. exchange (every source's segment in source-rank order)
         m = sum(recv)
         rk = rk_all[:m]
         rv = rv_all[:m] if vals is not None else None
@@ -221,17 +234,33 @@ class DistributedSorter:
         if self.time_exchange and keys.is_cuda:
             ev = (torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True))
             ev[0].record()
-        _all_to_all(_bits(rk), _bits(kp), recv, send[me], self.group)
-        if vals is not None:
-            _all_to_all(_bits(rv), _bits(vp), recv, send[me], self.group)
+        grouped = self.exchange == "grouped" and len(digits) >= 1
+        if grouped:
+            # 4. bucket-major exchange: every (source, first-digit bucket) piece lands at its
+            # place in the receiver's buffer -- bucket b's pieces from sources 0..G-1 in rank
+            # order -- so the received records are grouped by the first digit and, within a
+            # bucket, in global input order (reading #17)
+            sends, recvs, rhist = self._grouped_plan(hists, split)
+            self._p2p(rk, kp, sends, recvs)
+            if vals is not None:
+                self._p2p(rv, vp, sends, recvs)
+        else:
+            # 4. all-to-all (every source's segment in source-rank order)
+            _all_to_all(_bits(rk), _bits(kp), recv, send[me], self.group)
+            if vals is not None:
+                _all_to_all(_bits(rv), _bits(vp), recv, send[me], self.group)
         if ev is not None:
             ev[1].record()
         self.exchange_events = ev
-        # 5. local sort of the received records (source-rank order = global input order),
-        # into the send buffers (dead after the exchange) when they are large enough
-        if hasattr(self.ops, "sort_into") and m <= kp.numel():
-            ko, vo = self.ops.sort_into(rk, rv, self.begin, self.end, kp[:m], vp[:m] if vp is not None else None,
-                                        self._temp)
+        # 5. local sort of the received records, into the send buffers (dead after the
+        # exchange) when they are large enough; a grouped receive buffer starts at the
+        # second digit (hrs_sort_grouped: the first pass is already done by the exchange)
+        outk = kp[:m] if m <= kp.numel() else None
+        outv = (vp[:m] if vp is not None else None) if outk is not None else None
+        if grouped and hasattr(self.ops, "sort_grouped_into") and outk is not None:
+            ko, vo = self.ops.sort_grouped_into(rk, rv, rhist, self.begin, self.end, outk, outv, self._temp)
+        elif hasattr(self.ops, "sort_into") and outk is not None:
+            ko, vo = self.ops.sort_into(rk, rv, self.begin, self.end, outk, outv, self._temp)
         else:
             ko, vo = self.ops.sort(rk, rv, self.begin, self.end)
         offset = me * N // world
@@ -239,6 +268,70 @@ class DistributedSorter:
                      "imbalance": max(sum(send[s][j] for s in range(world)) for j in range(world)) /
                      max(1, N / world)}
         return ko, vo, offset
+
+    def _grouped_plan(self, hists, split):
+        """Pieces of the bucket-major exchange.  Rank r's partition output holds bucket b at
+        [O_r(b), O_r(b+1)) (O_r = prefix of hists[r]); it sends [split[j][r], split[j+1][r])
+        to rank j.  Receiver j stores, for every bucket b in ascending order, the pieces of
+        sources 0..G-1 in rank order.  Returns this rank's sends [(peer, src_off, len,
+        dst_off)], receives [(peer, dst_off, len)] (both in bucket order per peer, so the
+        messages of a pair match in issue order) and the received first-digit histogram."""
+        world, me = self.world, self.rank
+        R = len(hists[0])
+        O = []
+        for r in range(world):
+            o, run = [0] * (R + 1), 0
+            for b in range(R):
+                o[b] = run
+                run += hists[r][b]
+            o[R] = run
+            O.append(o)
+
+        def pieces(j):  # [(b, r, src_off, len)] of receiver j, bucket-major
+            out = []
+            for b in range(R):
+                for r in range(world):
+                    a = max(split[j][r], O[r][b])
+                    z = min(split[j + 1][r], O[r][b + 1])
+                    if z > a:
+                        out.append((b, r, a, z - a))
+            return out
+
+        sends, recvs = [], []
+        rhist = [0] * R
+        for j in range(world):
+            dst = 0
+            for b, r, a, ln in pieces(j):
+                if r == me:
+                    sends.append((j, a, ln, dst))
+                if j == me:
+                    recvs.append((r, dst, ln))
+                    rhist[b] += ln
+                dst += ln
+        return sends, recvs, rhist
+
+    def _p2p(self, rbuf, sbuf, sends, recvs):
+        """The pieces as one batch of point-to-point messages (NCCL groups them; NVLink),
+        this rank's own pieces as device copies."""
+        me = self.rank
+        staged = _host_staged(self.group, sbuf)
+        sb = sbuf.cpu() if staged else sbuf
+        rb = torch.empty_like(rbuf, device="cpu") if staged else rbuf
+        sbv, rbv = _bits(sb), _bits(rb)
+        ops = []
+        for peer, a, ln, d in sends:
+            if peer == me:
+                rbv[d:d + ln].copy_(sbv[a:a + ln])
+            else:
+                ops.append(dist.P2POp(dist.isend, sbv[a:a + ln], peer, self.group))
+        for peer, d, ln in recvs:
+            if peer != me:
+                ops.append(dist.P2POp(dist.irecv, rbv[d:d + ln], peer, self.group))
+        if ops:
+            for req in dist.batch_isend_irecv(ops):
+                req.wait()
+        if staged:
+            rbuf.copy_(rb)
 
     def _gather(self, rows):
         """all_gather of this rank's histogram rows ([k][r] ints) -> [k][rank][r]."""
@@ -276,6 +369,6 @@ class DistributedSorter:
         return int(allv[: self.rank].sum())
 
 
-def sort(keys, vals=None, group=None, begin_bit: int = 0, end_bit: int | None = None):
+def sort(keys, vals=None, group=None, begin_bit: int = 0, end_bit: int | None = None, exchange: str = "grouped"):
     """hrs.dist.sort(keys, values, group) -> (keys_out, values_out, global_rank_offset)."""
-    return DistributedSorter(keys, vals, group, begin_bit, end_bit).step()
+    return DistributedSorter(keys, vals, group, begin_bit, end_bit, exchange=exchange).step()

@@ -43,6 +43,16 @@ class OracleOps:
         ko, vo = oracle.sort(keys, vals, b, e)
         return _to_torch(ko, keys), (_to_torch(vo, vals) if vals is not None else None)
 
+    def sort_grouped_into(self, keys, vals, first_hist, b, e, keys_out, vals_out, temp_holder):
+        """The bucket-major exchange must deliver the records grouped by their first digit
+        with exactly this histogram (hrs_sort_grouped's precondition): checked, then sorted."""
+        lo = max(b, e - 8)
+        dig = (oracle._u64(keys) >> np.uint64(lo)) & np.uint64((1 << (e - lo)) - 1)
+        assert bool(np.all(dig[1:] >= dig[:-1])), "receive buffer not grouped by the first digit"
+        assert np.bincount(dig.astype(np.int64), minlength=len(first_hist)).tolist() == list(first_hist)
+        self.grouped_calls = getattr(self, "grouped_calls", 0) + 1
+        return self.sort_into(keys, vals, b, e, keys_out, vals_out, temp_holder)
+
     def sort_into(self, keys, vals, b, e, keys_out, vals_out, temp_holder):
         """Into the driver's reused buffers (the send buffer), as the CUDA path does."""
         ko, vo = self.sort(keys, vals, b, e)
@@ -61,14 +71,15 @@ def _free_port():
     return p
 
 
-def _worker(rank, world, port, n_per, kbits, dist_name, q):
+def _worker(rank, world, port, n_per, kbits, dist_name, q, exchange="grouped"):
     os.environ["MASTER_ADDR"] = "127.0.0.1"
     os.environ["MASTER_PORT"] = str(port)
     dist.init_process_group("gloo", rank=rank, world_size=world)
     try:
         k = gen.keys(n_per, kbits, dist_name, start=rank * n_per)
         v = gen.values(n_per, 64, "index", start=rank * n_per)
-        sorter = hdist.DistributedSorter(k, v, ops=OracleOps())
+        ops = OracleOps()
+        sorter = hdist.DistributedSorter(k, v, ops=ops, exchange=exchange)
         ko, vo, off = sorter.step()
         ko = ko.clone()
         # a second step reuses every buffer (send / receive / temp) and must give the same
@@ -76,6 +87,7 @@ def _worker(rank, world, port, n_per, kbits, dist_name, q):
         assert off2 == off and torch.equal(ko2.view(torch.int64 if kbits == 64 else torch.int32),
                                            ko.view(torch.int64 if kbits == 64 else torch.int32))
         assert sorter._temp[0] == "used" and ko2.data_ptr() == sorter._kp.data_ptr()
+        assert getattr(ops, "grouped_calls", 0) == (2 if exchange == "grouped" else 0)
         parts = [None] * world
         dist.all_gather_object(parts, (off, oracle._u64(ko).tolist(), oracle._u64(vo).tolist(), sorter.last))
         if rank == 0:
@@ -84,17 +96,20 @@ def _worker(rank, world, port, n_per, kbits, dist_name, q):
         dist.destroy_process_group()
 
 
-@pytest.mark.parametrize("world,kbits,dist_name", [(2, 32, "uniform"), (2, 64, "and3"), (3, 32, "and4"),
-                                                   (2, 32, "const"), (4, 32, "and4"), (3, 64, "const"),
-                                                   (4, 64, "uniform")])
-def test_distributed_sort_matches_global_oracle(world, kbits, dist_name):
+@pytest.mark.parametrize("world,kbits,dist_name,exchange", [(2, 32, "uniform", "grouped"), (2, 64, "and3", "grouped"),
+                                                            (3, 32, "and4", "grouped"), (2, 32, "const", "grouped"),
+                                                            (4, 32, "and4", "grouped"), (3, 64, "const", "grouped"),
+                                                            (4, 64, "uniform", "grouped"), (3, 32, "and3", "a2a"),
+                                                            (2, 64, "uniform", "a2a")])
+def test_distributed_sort_matches_global_oracle(world, kbits, dist_name, exchange):
     """The rank outputs concatenate to the global stable sort, and every rank holds
     exactly its N/G share whatever the skew (exact splitting)."""
     n_per = 3000
     ctx = mp.get_context("spawn")
     q = ctx.Queue()
     port = _free_port()
-    procs = [ctx.Process(target=_worker, args=(r, world, port, n_per, kbits, dist_name, q)) for r in range(world)]
+    procs = [ctx.Process(target=_worker, args=(r, world, port, n_per, kbits, dist_name, q, exchange))
+             for r in range(world)]
     for p in procs:
         p.start()
     parts = q.get(timeout=240)

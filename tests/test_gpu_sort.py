@@ -374,3 +374,54 @@ def test_binding_checks_outputs_and_streams():
     s.synchronize()
     ek, ev = oracle.sort(kk, vv, 0, 32)
     assert np.array_equal(_np(ko), ek) and np.array_equal(_np(vo), ev)
+
+
+# ------------------------------------------------------------- grouped input (first pass given)
+
+@pytest.mark.parametrize("kbits,vbits", TYPES)
+@pytest.mark.parametrize("dist", ["uniform", "and3", "const"])
+def test_sort_grouped(kbits, vbits, dist):
+    """hrs_sort_grouped: an input stably partitioned on its first digit (the oracle's pass,
+    P:503-509) with that digit's histogram; the library starts at the second digit.  A
+    stable partition followed by the stable sort of the rest is the stable sort of the
+    original input, so the result must equal the oracle's sort of the ungrouped data;
+    bit ranges with a narrow first digit and tiny thresholds (deep recursion) included."""
+    import paper_1611_01137_b200 as hrs
+    for n, (b, e), tun in ((300001, (0, kbits), None), (70001, (3, kbits - 4), None),
+                           (20011, (0, kbits), dict(local_threshold=64, merge_threshold=40, keys_per_tile=32)),
+                           (5000, (0, 5), None), (100003, (kbits - 8, kbits), None), (9000, (0, 12), None)):
+        k, v = _inputs(n, kbits, vbits, dist, seed=n)
+        lo, hi = max(b, e - 8), e
+        gk, gv, offs = oracle.partition_pass(k, v, lo, hi)
+        hist = np.diff(offs.astype(np.int64))
+        tk = torch.from_numpy(gk.astype(np.uint64).view(np.int64)).to(DEV)
+        tk = tk.view(torch.uint64) if kbits == 64 else tk.to(torch.int32).view(torch.uint32)
+        tv = None
+        if v is not None:
+            tv = torch.from_numpy(gv.astype(np.uint64).view(np.int64)).to(DEV)
+            tv = tv.view(torch.uint64) if vbits == 64 else tv.to(torch.int32).view(torch.uint32)
+        ko, vo = hrs.sort_grouped(tk, tv, hist.tolist(), b, e, tuning=tun)
+        torch.cuda.synchronize()
+        ek, ev = oracle.sort(k, v, b, e)
+        assert np.array_equal(_np(ko), ek), (n, b, e, tun)
+        if v is not None:
+            assert np.array_equal(_np(vo), ev), (n, b, e, tun)
+
+
+def test_sort_grouped_stats_skip_first_pass():
+    """The first pass moves nothing: bytes_min drops by R(K + 2(K+V)) for that pass."""
+    import paper_1611_01137_b200 as hrs
+    n = 1 << 22
+    k = gen.keys(n, 32, "uniform", seed=7)
+    v = gen.values(n, 32, "index")
+    gk, gv, offs = oracle.partition_pass(k, v, 24, 32)
+    tk = torch.from_numpy(gk.astype(np.int64)).to(torch.int32).view(torch.uint32).to(DEV)
+    tv = torch.from_numpy(gv.astype(np.int64)).to(torch.int32).view(torch.uint32).to(DEV)
+    temp = torch.empty(hrs.temp_bytes(n, 4, 4), dtype=torch.uint8, device=DEV)
+    ko, vo = hrs.sort_grouped(tk, tv, np.diff(offs.astype(np.int64)).tolist(), temp=temp)
+    st = hrs.get_stats(temp)
+    full = plan.simulate_msd(oracle._u64(k), None, 0, 32, 8192, 2048, hrs.max_keys_per_tile(4, 4))
+    assert st["recs_in_pass"][0] == 0 and st["recs_in_pass"][1:] == full.recs_in_pass[1:]
+    assert st["bytes_min"] == plan.bytes_min(full, 4, 4) - n * (4 + 2 * 8)
+    ek, ev = oracle.sort(k, v, 0, 32)
+    assert np.array_equal(_np(ko), ek) and np.array_equal(_np(vo), ev)
