@@ -176,6 +176,13 @@ def run_hrs(args):
     use_dist = world > 1 or args.force_dist
     if use_dist:
         import torch.distributed as dist
+        if "RANK" not in os.environ:  # --force-dist without torchrun: a world of one
+            import socket
+            with socket.socket() as sk:
+                sk.bind(("127.0.0.1", 0))
+                os.environ.setdefault("MASTER_PORT", str(sk.getsockname()[1]))
+            os.environ.update(RANK="0", WORLD_SIZE="1", LOCAL_RANK="0")
+            os.environ.setdefault("MASTER_ADDR", "127.0.0.1")
         dist.init_process_group("nccl", device_id=dev)
         pg = dist.group.WORLD
 

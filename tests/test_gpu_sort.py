@@ -108,7 +108,7 @@ TUNINGS = [
     dict(local_threshold=300, merge_threshold=100, keys_per_tile=128),
     dict(local_threshold=3, merge_threshold=2, keys_per_tile=4),
     dict(local_threshold=200, merge_threshold=1, keys_per_tile=1),
-    dict(local_threshold=4096, merge_threshold=4096, keys_per_tile=3328),
+    dict(local_threshold=4096, merge_threshold=4096, keys_per_tile=3072),
 ]
 
 
