@@ -1309,6 +1309,27 @@ hrs_status hrs_partition_pass(void *d_temp, size_t *temp_bytes, const void *keys
                         hi_bit, nullptr, d_offsets, true, stream);
 }
 
+hrs_status hrs_copy_pieces(void *dst, const void *src, int elem_bytes, const uint64_t *d_pieces, uint64_t npieces,
+                           hrs_stream_t stream) {
+    if (elem_bytes != 4 && elem_bytes != 8) return HRS_ERROR_INVALID_VALUE;
+    if (npieces == 0) return HRS_SUCCESS;
+    if (!dst || !src || !d_pieces) return HRS_ERROR_INVALID_VALUE;
+    if (!aligned(dst, elem_bytes) || !aligned(src, elem_bytes) || !aligned(d_pieces, 8)) return HRS_ERROR_INVALID_VALUE;
+    int dev = 0, sms = 0;
+    hrs_status s = check_device(&dev, &sms);
+    if (s) return s;
+    cudaStream_t st = reinterpret_cast<cudaStream_t>(stream);
+    LaunchScope ls(st, 4, 0);
+    if (elem_bytes == 4)
+        launch_pdl(k_copy_pieces<uint32_t>, dim3(sms * 4), dim3(256), 0, st, static_cast<const uint32_t *>(src),
+                   static_cast<uint32_t *>(dst), d_pieces, npieces);
+    else
+        launch_pdl(k_copy_pieces<unsigned long long>, dim3(sms * 4), dim3(256), 0, st,
+                   static_cast<const unsigned long long *>(src), static_cast<unsigned long long *>(dst), d_pieces,
+                   npieces);
+    return last_launch();
+}
+
 const char *hrs_status_string(hrs_status s) {
     switch (s) {
         case HRS_SUCCESS: return "success";

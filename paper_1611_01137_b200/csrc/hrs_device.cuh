@@ -675,6 +675,25 @@ __global__ void k_copy(const T *__restrict__ in, T *__restrict__ out, uint64_t n
         out[i] = in[i];
 }
 
+// Copies of many pieces in one launch (the distributed sort's own pieces of the
+// bucket-major exchange): tab holds npieces x {src_off, dst_off, count} in elements; the
+// CTAs of the grid walk the pieces, each piece cut into chunks of CHUNK elements.
+template <typename T>
+__global__ void __launch_bounds__(256) k_copy_pieces(const T *__restrict__ src, T *__restrict__ dst,
+                                                     const uint64_t *__restrict__ tab, uint64_t npieces) {
+    pdl_wait();
+    constexpr uint64_t CHUNK = 1u << 16;
+    for (uint64_t pc = 0; pc < npieces; ++pc) {
+        const uint64_t so = tab[3 * pc], d = tab[3 * pc + 1], cnt = tab[3 * pc + 2];
+        const uint64_t nch = (cnt + CHUNK - 1) / CHUNK;
+        // chunk c of piece pc goes to CTA (pc + c) % grid: pieces are spread over the grid
+        for (uint64_t c = (blockIdx.x + gridDim.x - pc % gridDim.x) % gridDim.x; c < nch; c += gridDim.x) {
+            const uint64_t a = c * CHUNK, z = min(cnt, a + CHUNK);
+            for (uint64_t i = a + threadIdx.x; i < z; i += blockDim.x) dst[d + i] = src[so + i];
+        }
+    }
+}
+
 __global__ void k_fill_u64(uint64_t *p, uint64_t n, uint64_t v) {
     for (uint64_t i = static_cast<uint64_t>(blockIdx.x) * blockDim.x + threadIdx.x; i < n;
          i += static_cast<uint64_t>(gridDim.x) * blockDim.x)

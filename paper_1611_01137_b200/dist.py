@@ -83,6 +83,9 @@ class CudaOps:
     def sort(self, keys, vals, begin_bit, end_bit):
         return self.hrs.sort(keys, vals, begin_bit, end_bit)
 
+    def copy_pieces(self, dst, src, pieces):
+        self.hrs.copy_pieces(dst, src, pieces)
+
     def sort_grouped_into(self, keys, vals, first_hist, begin_bit, end_bit, keys_out, vals_out, temp_holder):
         """hrs_sort_grouped into caller buffers (the input is grouped by its first digit)."""
         self._temp_for(keys, vals, begin_bit, end_bit, temp_holder)
@@ -318,12 +321,21 @@ class DistributedSorter:
         sb = sbuf.cpu() if staged else sbuf
         rb = torch.empty_like(rbuf, device="cpu") if staged else rbuf
         sbv, rbv = _bits(sb), _bits(rb)
-        ops = []
+        ops, own = [], []
         for peer, a, ln, d in sends:
             if peer == me:
-                rbv[d:d + ln].copy_(sbv[a:a + ln])
+                if own and own[-1][0] + own[-1][2] == a and own[-1][1] + own[-1][2] == d:
+                    own[-1] = (own[-1][0], own[-1][1], own[-1][2] + ln)  # contiguous on both sides
+                else:
+                    own.append((a, d, ln))
             else:
                 ops.append(dist.P2POp(dist.isend, sbv[a:a + ln], peer, self.group))
+        if own:
+            if hasattr(self.ops, "copy_pieces") and not staged:
+                self.ops.copy_pieces(rbv, sbv, own)  # one launch for all own pieces
+            else:
+                for a, d, ln in own:
+                    rbv[d:d + ln].copy_(sbv[a:a + ln])
         for peer, d, ln in recvs:
             if peer != me:
                 ops.append(dist.P2POp(dist.irecv, rbv[d:d + ln], peer, self.group))

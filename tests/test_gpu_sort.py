@@ -425,3 +425,23 @@ def test_sort_grouped_stats_skip_first_pass():
     assert st["bytes_min"] == plan.bytes_min(full, 4, 4) - n * (4 + 2 * 8)
     ek, ev = oracle.sort(k, v, 0, 32)
     assert np.array_equal(_np(ko), ek) and np.array_equal(_np(vo), ev)
+
+
+def test_copy_pieces():
+    """hrs_copy_pieces (the distributed sort's own pieces): random pieces against numpy."""
+    import paper_1611_01137_b200 as hrs
+    rng = np.random.default_rng(5)
+    for dt in (torch.int32, torch.int64):
+        src = torch.arange(300000, dtype=dt, device=DEV)
+        dst = torch.full((300000,), -1, dtype=dt, device=DEV)
+        cuts = np.sort(rng.choice(np.arange(1, 300000), 40, replace=False))
+        lens = np.diff(np.concatenate([[0], cuts, [300000]]))
+        perm = rng.permutation(len(lens))
+        soffs = np.concatenate([[0], np.cumsum(lens)[:-1]])
+        pieces, d = [], 0
+        for i in perm:
+            pieces.append((int(soffs[i]), d, int(lens[i])))
+            d += int(lens[i])
+        hrs.copy_pieces(dst, src, pieces + [(0, 0, 0)])
+        exp = np.concatenate([np.arange(soffs[i], soffs[i] + lens[i]) for i in perm])
+        assert np.array_equal(dst.cpu().numpy(), exp)
