@@ -214,11 +214,13 @@ hrs_status hrs_partition_pass(void *d_temp, size_t *temp_bytes, const void *keys
                               const void *vals_in, void *vals_out, uint64_t n, int key_bytes, int value_bytes,
                               int lo_bit, int hi_bit, uint64_t *d_offsets, hrs_stream_t stream);
 
-/* Copies npieces pieces of elem_bytes-wide elements (4 or 8) from src to dst in one launch:
- * d_pieces (device) holds npieces x {src_offset, dst_offset, count} uint64, in elements.
- * The pieces must not overlap in dst, and src and dst must not overlap.  The distributed
- * sort's placement of a rank's own pieces in the bucket-major exchange (SURVEY §8(e)
- * step 6: the pieces of every first-digit bucket from every source, in source order). */
+/* Copies npieces pieces of elem_bytes-wide elements (4 or 8) from src to dst (device):
+ * `pieces` is a HOST array of npieces x {src_offset, dst_offset, count} uint64, in
+ * elements, read during the call (it travels in kernel parameters, 256 pieces per
+ * launch; no device memory is needed for it).  The pieces must not overlap in dst, and
+ * src and dst must not overlap.  The distributed sort's placement of a rank's own pieces
+ * in the bucket-major exchange (the pieces of every first-digit
+ * bucket from every source, in source order). */
 hrs_status hrs_copy_pieces(void *dst, const void *src, int elem_bytes, const uint64_t *d_pieces, uint64_t npieces,
                            hrs_stream_t stream);
 

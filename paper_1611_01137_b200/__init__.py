@@ -268,21 +268,21 @@ def partition_pass(keys: torch.Tensor, values: torch.Tensor | None, lo_bit: int,
 
 
 def copy_pieces(dst: torch.Tensor, src: torch.Tensor, pieces, stream=None) -> None:
-    """hrs_copy_pieces: dst[d:d+c] = src[s:s+c] for every (s, d, c) in `pieces` (one launch)."""
+    """hrs_copy_pieces: dst[d:d+c] = src[s:s+c] for every (s, d, c) in `pieces` (host list)."""
     _check_tensor(dst, "dst")
     _check_tensor(src, "src")
     if dst.dtype != src.dtype or dst.element_size() not in (4, 8):
         raise TypeError("copy_pieces takes two tensors of one 4- or 8-byte dtype")
-    flat = [int(x) for pc in pieces for x in pc]
-    if not flat:
+    pcs = [(int(a), int(d), int(c)) for a, d, c in pieces if int(c) > 0]
+    if not pcs:
         return
-    for so, d, c in pieces:
+    for so, d, c in pcs:
         if so < 0 or d < 0 or so + c > src.numel() or d + c > dst.numel():
             raise ValueError("piece out of range")
-    tab = torch.tensor(flat, dtype=torch.int64).view(torch.uint64).to(dst.device, non_blocking=False)
-    _on_stream(stream, tab)
+    tab = (ctypes.c_uint64 * (3 * len(pcs)))(*[x for pc in pcs for x in pc])
     with torch.cuda.device(dst.device):
-        check(lib.hrs_copy_pieces(_ptr(dst), _ptr(src), dst.element_size(), _ptr(tab), len(pieces), _stream(stream)),
+        check(lib.hrs_copy_pieces(_ptr(dst), _ptr(src), dst.element_size(), ctypes.cast(tab, ctypes.c_void_p),
+                                  len(pcs), _stream(stream)),
               "hrs_copy_pieces")
 
 

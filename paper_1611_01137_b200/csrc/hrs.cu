@@ -1309,25 +1309,30 @@ hrs_status hrs_partition_pass(void *d_temp, size_t *temp_bytes, const void *keys
                         hi_bit, nullptr, d_offsets, true, stream);
 }
 
-hrs_status hrs_copy_pieces(void *dst, const void *src, int elem_bytes, const uint64_t *d_pieces, uint64_t npieces,
+hrs_status hrs_copy_pieces(void *dst, const void *src, int elem_bytes, const uint64_t *pieces, uint64_t npieces,
                            hrs_stream_t stream) {
     if (elem_bytes != 4 && elem_bytes != 8) return HRS_ERROR_INVALID_VALUE;
     if (npieces == 0) return HRS_SUCCESS;
-    if (!dst || !src || !d_pieces) return HRS_ERROR_INVALID_VALUE;
-    if (!aligned(dst, elem_bytes) || !aligned(src, elem_bytes) || !aligned(d_pieces, 8)) return HRS_ERROR_INVALID_VALUE;
+    if (!dst || !src || !pieces) return HRS_ERROR_INVALID_VALUE;
+    if (!aligned(dst, elem_bytes) || !aligned(src, elem_bytes)) return HRS_ERROR_INVALID_VALUE;
     int dev = 0, sms = 0;
     hrs_status s = check_device(&dev, &sms);
     if (s) return s;
     cudaStream_t st = reinterpret_cast<cudaStream_t>(stream);
-    LaunchScope ls(st, 4, 0);
-    if (elem_bytes == 4)
-        launch_pdl(k_copy_pieces<uint32_t>, dim3(sms * 4), dim3(256), 0, st, static_cast<const uint32_t *>(src),
-                   static_cast<uint32_t *>(dst), d_pieces, npieces);
-    else
-        launch_pdl(k_copy_pieces<unsigned long long>, dim3(sms * 4), dim3(256), 0, st,
-                   static_cast<const unsigned long long *>(src), static_cast<unsigned long long *>(dst), d_pieces,
-                   npieces);
-    return last_launch();
+    for (uint64_t p0 = 0; p0 < npieces; p0 += COPY_PIECES_MAX) {  // the table goes in the kernel parameters
+        CopyPieces cp;
+        cp.npieces = static_cast<uint32_t>(std::min<uint64_t>(COPY_PIECES_MAX, npieces - p0));
+        std::memcpy(cp.tab, pieces + 3 * p0, sizeof(uint64_t) * 3 * cp.npieces);
+        LaunchScope ls(st, 4, 0);
+        if (elem_bytes == 4)
+            launch_pdl(k_copy_pieces<uint32_t>, dim3(sms * 4), dim3(256), 0, st, static_cast<const uint32_t *>(src),
+                       static_cast<uint32_t *>(dst), cp);
+        else
+            launch_pdl(k_copy_pieces<unsigned long long>, dim3(sms * 4), dim3(256), 0, st,
+                       static_cast<const unsigned long long *>(src), static_cast<unsigned long long *>(dst), cp);
+        if ((s = last_launch())) return s;
+    }
+    return HRS_SUCCESS;
 }
 
 const char *hrs_status_string(hrs_status s) {

@@ -676,20 +676,41 @@ __global__ void k_copy(const T *__restrict__ in, T *__restrict__ out, uint64_t n
 }
 
 // Copies of many pieces in one launch (the distributed sort's own pieces of the
-// bucket-major exchange): tab holds npieces x {src_off, dst_off, count} in elements; the
-// CTAs of the grid walk the pieces, each piece cut into chunks of CHUNK elements.
+// bucket-major exchange): the piece table travels in the kernel parameters (no host to
+// device copy), {src_off, dst_off, count} in elements; the CTAs of the grid walk the
+// pieces, each piece cut into chunks of CHUNK elements, 16-byte vectors where src and dst
+// are equally aligned.
+constexpr int COPY_PIECES_MAX = 256;
+struct CopyPieces {
+    uint64_t tab[3 * COPY_PIECES_MAX];
+    uint32_t npieces;
+};
 template <typename T>
 __global__ void __launch_bounds__(256) k_copy_pieces(const T *__restrict__ src, T *__restrict__ dst,
-                                                     const uint64_t *__restrict__ tab, uint64_t npieces) {
+                                                     const __grid_constant__ CopyPieces prm) {
     pdl_wait();
     constexpr uint64_t CHUNK = 1u << 16;
-    for (uint64_t pc = 0; pc < npieces; ++pc) {
-        const uint64_t so = tab[3 * pc], d = tab[3 * pc + 1], cnt = tab[3 * pc + 2];
+    constexpr uint64_t VE = 16 / sizeof(T);
+    for (uint32_t pc = 0; pc < prm.npieces; ++pc) {
+        const uint64_t so = prm.tab[3 * pc], d = prm.tab[3 * pc + 1], cnt = prm.tab[3 * pc + 2];
         const uint64_t nch = (cnt + CHUNK - 1) / CHUNK;
         // chunk c of piece pc goes to CTA (pc + c) % grid: pieces are spread over the grid
         for (uint64_t c = (blockIdx.x + gridDim.x - pc % gridDim.x) % gridDim.x; c < nch; c += gridDim.x) {
             const uint64_t a = c * CHUNK, z = min(cnt, a + CHUNK);
-            for (uint64_t i = a + threadIdx.x; i < z; i += blockDim.x) dst[d + i] = src[so + i];
+            const T *sp = src + so;
+            T *dp = dst + d;
+            if (((so ^ d) % VE) == 0) {
+                // scalar head to 16-byte alignment, vectors, scalar tail
+                const uint64_t h = min(z, a + (VE - (so + a) % VE) % VE);
+                for (uint64_t i = a + threadIdx.x; i < h; i += blockDim.x) dp[i] = sp[i];
+                const uint64_t nv = (z - h) / VE;
+                const uint4 *sv = reinterpret_cast<const uint4 *>(sp + h);
+                uint4 *dv = reinterpret_cast<uint4 *>(dp + h);
+                for (uint64_t v = threadIdx.x; v < nv; v += blockDim.x) dv[v] = sv[v];
+                for (uint64_t i = h + nv * VE + threadIdx.x; i < z; i += blockDim.x) dp[i] = sp[i];
+            } else {
+                for (uint64_t i = a + threadIdx.x; i < z; i += blockDim.x) dp[i] = sp[i];
+            }
         }
     }
 }

@@ -233,17 +233,18 @@ class DistributedSorter:
         m = sum(recv)
         rk = rk_all[:m]
         rv = rv_all[:m] if vals is not None else None
+        grouped = self.exchange == "grouped" and len(digits) >= 1
+        if grouped:
+            sends, recvs, rhist = self._grouped_plan(hists, split)
         ev = None
         if self.time_exchange and keys.is_cuda:
             ev = (torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True))
             ev[0].record()
-        grouped = self.exchange == "grouped" and len(digits) >= 1
         if grouped:
             # 4. bucket-major exchange: every (source, first-digit bucket) piece lands at its
             # place in the receiver's buffer -- bucket b's pieces from sources 0..G-1 in rank
             # order -- so the received records are grouped by the first digit and, within a
             # bucket, in global input order (reading #17)
-            sends, recvs, rhist = self._grouped_plan(hists, split)
             self._p2p(rk, kp, sends, recvs)
             if vals is not None:
                 self._p2p(rv, vp, sends, recvs)
@@ -279,38 +280,22 @@ class DistributedSorter:
         sources 0..G-1 in rank order.  Returns this rank's sends [(peer, src_off, len,
         dst_off)], receives [(peer, dst_off, len)] (both in bucket order per peer, so the
         messages of a pair match in issue order) and the received first-digit histogram."""
+        import numpy as np
         world, me = self.world, self.rank
-        R = len(hists[0])
-        O = []
-        for r in range(world):
-            o, run = [0] * (R + 1), 0
-            for b in range(R):
-                o[b] = run
-                run += hists[r][b]
-            o[R] = run
-            O.append(o)
-
-        def pieces(j):  # [(b, r, src_off, len)] of receiver j, bucket-major
-            out = []
-            for b in range(R):
-                for r in range(world):
-                    a = max(split[j][r], O[r][b])
-                    z = min(split[j + 1][r], O[r][b + 1])
-                    if z > a:
-                        out.append((b, r, a, z - a))
-            return out
-
-        sends, recvs = [], []
-        rhist = [0] * R
-        for j in range(world):
-            dst = 0
-            for b, r, a, ln in pieces(j):
-                if r == me:
-                    sends.append((j, a, ln, dst))
-                if j == me:
-                    recvs.append((r, dst, ln))
-                    rhist[b] += ln
-                dst += ln
+        H = np.asarray(hists, dtype=np.int64)                 # [rank][bucket]
+        R = H.shape[1]
+        O = np.zeros((world, R + 1), dtype=np.int64)
+        O[:, 1:] = np.cumsum(H, axis=1)                       # bucket starts per rank
+        S = np.asarray(split, dtype=np.int64)                 # [j][rank] split positions
+        # piece (j, b, r) = [max(S[j][r], O[r][b]), min(S[j+1][r], O[r][b+1]))
+        a = np.maximum(S[:-1, None, :], O.T[None, :-1, :])    # [j][b][r]
+        z = np.minimum(S[1:, None, :], O.T[None, 1:, :])
+        ln = np.maximum(z - a, 0)
+        dst = np.cumsum(ln.reshape(world, -1), axis=1).reshape(ln.shape) - ln  # receiver offsets, (b, r)-major
+        sends = [(int(j), int(a[j, b, me]), int(ln[j, b, me]), int(dst[j, b, me]))
+                 for j, b in zip(*np.nonzero(ln[:, :, me]))]
+        recvs = [(int(r), int(dst[me, b, r]), int(ln[me, b, r])) for b, r in zip(*np.nonzero(ln[me]))]
+        rhist = ln[me].sum(axis=1).tolist()
         return sends, recvs, rhist
 
     def _p2p(self, rbuf, sbuf, sends, recvs):
