@@ -118,9 +118,11 @@ typedef struct {
     uint64_t local_recs;                       /* records finished by a local sort */
     uint64_t merged_groups;                    /* local entries made of >= 2 merged sub-buckets */
     uint64_t local_in_class[HRS_NUM_CLASSES];  /* local entries per size class */
-    uint64_t bytes_min;                        /* sum_p R_p (K + 2(K+V)) + R_L 2(K+V) */
+    uint64_t bytes_min;                        /* sum_p [R_p K + (R_p - S_p) 2(K+V)] + R_L 2(K+V) */
     uint64_t redo_blocks;                      /* tiles / buckets redone with the stable-by-construction rank
                                                   (0 unless a stability check failed or HRS_FLAG_FORCE_REDO) */
+    uint64_t skipped_recs_in_pass[HRS_MAX_PASSES]; /* S_p: records of buckets whose digit p is constant and that
+                                                  never moved: their scatter is skipped (reading #22) */
 } hrs_stats;
 
 /* ---- full sorts; arguments: temp, size, keys in/out, [values in/out], n, bit range, stream ---- */

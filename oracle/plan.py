@@ -110,6 +110,7 @@ class MsdResult:
     buckets_in_pass: list = field(default_factory=list)
     local_entries: list = field(default_factory=list)  # (offset, count, hi_bit, class, pass)
     merged_groups: int = 0
+    skipped_in_pass: list = field(default_factory=list)  # S_p: records whose pass-p scatter is skipped
 
     @property
     def local_buckets(self):
@@ -153,17 +154,22 @@ def simulate_msd(keys, vals=None, begin_bit: int = 0, end_bit: int = 32,
         return res
 
     plan = digit_plan(begin_bit, end_bit)
-    buckets = [(0, n)]
+    # (offset, count, moved): `moved` -- some earlier pass scattered the bucket's records out
+    # of the input buffer.  Reading #22: a bucket that never moved and whose
+    # digit is the same for all its records is not scattered (a scatter would only copy it),
+    # except in the last pass (whose output is the final result).
+    buckets = [(0, n, False)]
     for p, (lo, hi) in enumerate(plan, start=1):
         if not buckets:
             break
         res.counting_passes = p
-        res.recs_in_pass.append(sum(c for _, c in buckets))
-        res.tiles_in_pass.append(sum(-(-c // keys_per_tile) for _, c in buckets))
+        res.recs_in_pass.append(sum(c for _, c, _ in buckets))
+        res.tiles_in_pass.append(sum(-(-c // keys_per_tile) for _, c, _ in buckets))
         res.buckets_in_pass.append(len(buckets))
+        res.skipped_in_pass.append(0)
         last = p == len(plan)
         nxt = []
-        for off, cnt in buckets:
+        for off, cnt, moved in buckets:
             seg = slice(off, off + cnt)
             dig = _sk(k[seg], lo, hi)
             order = np.argsort(dig, kind="stable")  # the stable partition of this bucket
@@ -172,10 +178,13 @@ def simulate_msd(keys, vals=None, begin_bit: int = 0, end_bit: int = 32,
                 v[seg] = v[seg][order]
             tot = np.bincount(dig.astype(np.int64), minlength=1 << (hi - lo))
             starts = np.concatenate([[0], np.cumsum(tot)[:-1]]) + off
+            skip = not last and not moved and int(np.count_nonzero(tot)) == 1
+            if skip:
+                res.skipped_in_pass[-1] += cnt
             for kind, ds, size in classify_bucket(tot, last, local_threshold, merge_threshold):
                 start = int(starts[ds[0]])
                 if kind == "count":
-                    nxt.append((start, size))
+                    nxt.append((start, size, not skip))
                 elif kind == "local":
                     if len(ds) >= 2:
                         res.merged_groups += 1
@@ -185,6 +194,8 @@ def simulate_msd(keys, vals=None, begin_bit: int = 0, end_bit: int = 32,
 
 
 def bytes_min(res: MsdResult, key_bytes: int, value_bytes: int) -> int:
-    """sum_p R_p (K + 2(K+V)) + R_L * 2(K+V)."""
+    """sum_p [R_p K + (R_p - S_p) 2(K+V)] + R_L * 2(K+V) -- every record of a
+    pass is histogrammed, the records of skipped buckets (S_p, reading #22) are not moved."""
     rec = key_bytes + value_bytes
-    return sum(r * (key_bytes + 2 * rec) for r in res.recs_in_pass) + res.local_recs * 2 * rec
+    return sum(r * key_bytes + (r - sk) * 2 * rec for r, sk in zip(res.recs_in_pass, res.skipped_in_pass)) + \
+        res.local_recs * 2 * rec

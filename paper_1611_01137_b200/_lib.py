@@ -64,6 +64,7 @@ class Stats(ctypes.Structure):
         ("local_in_class", ctypes.c_uint64 * HRS_NUM_CLASSES),
         ("bytes_min", ctypes.c_uint64),
         ("redo_blocks", ctypes.c_uint64),
+        ("skipped_recs_in_pass", ctypes.c_uint64 * HRS_MAX_PASSES),
     ]
 
     def to_dict(self) -> dict:
@@ -83,6 +84,7 @@ class Stats(ctypes.Structure):
             "local_in_class": list(self.local_in_class),
             "bytes_min": self.bytes_min,
             "redo_blocks": self.redo_blocks,
+            "skipped_recs_in_pass": list(self.skipped_recs_in_pass)[:p],
         }
 
 

@@ -501,11 +501,28 @@ struct Runner {
         return HRS_SUCCESS;
     }
 
-    static hrs_status hist(const Plan &pl, void *temp, cudaStream_t st, int dev, int sms, int p, const void *xin,
+    // the three buffers a bucket can live in (Bucket::src): the input, the aux buffer in
+    // temp and the output
+    struct Bufs {
+        const void *k[3];
+        const void *v[3];
+    };
+    static Bufs bufs(const Plan &pl, void *temp, const void *kin, void *kout, const void *vin, void *vout) {
+        Bufs b;
+        b.k[SRC_IN] = kin;
+        b.k[SRC_AUX] = at<void>(temp, pl.off_auxk);
+        b.k[SRC_OUT] = kout;
+        b.v[SRC_IN] = vin;
+        b.v[SRC_AUX] = VB ? at<void>(temp, pl.off_auxv) : nullptr;
+        b.v[SRC_OUT] = vout;
+        return b;
+    }
+
+    static hrs_status hist(const Plan &pl, void *temp, cudaStream_t st, int dev, int sms, int p, const Bufs &bf,
                            uint32_t G) {
         HistParams hp;
         hp.n = pl.n;
-        hp.keys = xin;
+        for (int i = 0; i < 3; ++i) hp.src_keys[i] = bf.k[i];
         hp.p = p;
         hp.lo = pl.lo[p - 1];
         hp.mask = (1u << (pl.hi[p - 1] - pl.lo[p - 1])) - 1u;
@@ -569,13 +586,15 @@ struct Runner {
         return last_launch();
     }
 
-    static hrs_status scatter(const Plan &pl, void *temp, cudaStream_t st, int dev, int sms, int p, const void *kin,
-                              void *kout, const void *vin, void *vout, uint32_t G) {
+    static hrs_status scatter(const Plan &pl, void *temp, cudaStream_t st, int dev, int sms, int p, const Bufs &bf,
+                              void *kout, void *vout, uint32_t G) {
         ScatterParams sp;
         sp.n = pl.n;
-        sp.keys_in = kin;
+        for (int i = 0; i < 3; ++i) {
+            sp.src_keys[i] = bf.k[i];
+            sp.src_vals[i] = bf.v[i];
+        }
         sp.keys_out = kout;
-        sp.vals_in = vin;
         sp.vals_out = vout;
         sp.p = p;
         sp.lo = pl.lo[p - 1];
@@ -812,7 +831,7 @@ struct Runner {
         if (pl.counting) {
             uint32_t G = 0;
             if ((s = range_grid(pl, dev, sms, &G))) return s;
-            const void *xk = kin, *xv = vin;
+            const Bufs bf = bufs(pl, temp, kin, kout, vin, vout);
             for (int p = 1; p <= pl.D; ++p) {
                 const bool to_out = ((pl.D - p) % 2) == 0;
                 void *yk = to_out ? kout : auxk;
@@ -823,13 +842,11 @@ struct Runner {
                     if ((s = classify(pl, temp, st, dev, sms, 1, SRC_IN, nullptr, nullptr, false, 0))) return s;
                     continue;
                 }
-                if ((s = hist(pl, temp, st, dev, sms, p, xk, G))) return s;
+                if ((s = hist(pl, temp, st, dev, sms, p, bf, G))) return s;
                 if ((s = classify(pl, temp, st, dev, sms, p, to_out ? SRC_OUT : SRC_AUX, nullptr, nullptr,
                                   p == pl.D, G)))
                     return s;
-                if ((s = scatter(pl, temp, st, dev, sms, p, xk, yk, xv, yv, G))) return s;
-                xk = yk;
-                xv = yv;
+                if ((s = scatter(pl, temp, st, dev, sms, p, bf, yk, yv, G))) return s;
             }
             const int cmax = pl.single_class >= 0 ? pl.single_class : size_class_of(pl.lt);
             bool cnt = false;
@@ -865,9 +882,10 @@ struct Runner {
         }
         uint32_t G = 0;
         if ((s = range_grid(pl, dev, sms, &G))) return s;
-        if ((s = hist(pl, temp, st, dev, sms, 1, kin, G))) return s;
+        const Bufs bf = bufs(pl, temp, kin, kout, vin, vout);
+        if ((s = hist(pl, temp, st, dev, sms, 1, bf, G))) return s;
         if ((s = classify(pl, temp, st, dev, sms, 1, SRC_OUT, out_hist, out_offsets, true, G))) return s;
-        if (do_scatter && (s = scatter(pl, temp, st, dev, sms, 1, kin, kout, vin, vout, G))) return s;
+        if (do_scatter && (s = scatter(pl, temp, st, dev, sms, 1, bf, kout, vout, G))) return s;
         return HRS_SUCCESS;
     }
 };
@@ -1226,7 +1244,9 @@ hrs_status hrs_get_stats(const void *d_temp, hrs_stats *out, hrs_stream_t stream
         out->recs_in_pass[p - 1] = c.recs_in_pass[p];
         out->tiles_in_pass[p - 1] = tiles;
         out->buckets_in_pass[p - 1] = bks;
-        bytes += c.recs_in_pass[p] * (K + 2 * R);
+        out->skipped_recs_in_pass[p - 1] = c.skipped_in_pass[p];
+        // the histogram reads every record of the pass, the scatter moves the unskipped ones
+        bytes += c.recs_in_pass[p] * K + (c.recs_in_pass[p] - c.skipped_in_pass[p]) * 2 * R;
     }
     for (int k = 0; k < HRS_NUM_CLASSES; ++k) {
         out->local_in_class[k] = c.nlocal[k];

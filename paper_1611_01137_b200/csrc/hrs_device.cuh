@@ -79,7 +79,9 @@ struct Bucket {
     uint32_t count;
     uint32_t first_tile;
     uint32_t ntiles;
-    uint32_t pad;
+    uint16_t src;   // SrcCode of the buffer holding the bucket's records at the start of the pass
+    uint16_t skip;  // set by k_classify: the digit is constant over the bucket and it never
+                    // moved (src == SRC_IN): k_scatter leaves its records where they are
 };
 // One tile as k_hist saw it, for k_scatter: records [offs, offs + count) of bucket
 // `bucket`; carry_row = the hist CTA whose carry applies (tile in the first bucket
@@ -117,6 +119,7 @@ struct Ctl {
     unsigned long long local_recs;
     unsigned long long merged_groups;
     unsigned long long redo;  // blocks that redid a tile / bucket with the stable-by-construction rank
+    unsigned long long skipped_in_pass[HRS_MAX_PASSES + 2];  // records of skipped buckets (no scatter)
 };
 
 // ------------------------------------------------------------------ small helpers
@@ -633,7 +636,8 @@ __global__ void k_init(InitParams prm) {
                 b.count = static_cast<uint32_t>(n);
                 b.first_tile = 0;
                 b.ntiles = T1;
-                b.pad = 0;
+                b.src = SRC_IN;
+                b.skip = 0;
                 prm.buckets[0] = b;
             } else if (n > 0 && prm.root_local) {
                 LocalEntry e;
@@ -724,8 +728,8 @@ __global__ void k_fill_u64(uint64_t *p, uint64_t n, uint64_t v) {
 // ------------------------------------------------------------------ histogram
 
 struct HistParams {
-    const void *keys;  // X_{p-1}
-    uint64_t n;        // elements of the buffer
+    const void *src_keys[3];  // indexed by SrcCode: each bucket's keys are in its src buffer
+    uint64_t n;               // elements of the buffers
     int p;
     int lo;
     uint32_t mask;
@@ -765,7 +769,7 @@ __global__ void __launch_bounds__(THREADS) k_hist(HistParams prm) {
     auto stage = [&](int s) {
         return reinterpret_cast<K *>(smem + L::off_stage + s * align16(sizeof(K) * L::stage_elems));
     };
-    const K *__restrict__ keys = static_cast<const K *>(prm.keys);
+    __shared__ const K *src_of[NSTAGE];  // key buffer of the tile in stage s
     const int tid = threadIdx.x, warp = tid >> 5;
     const unsigned long long al = prm.ctl->alloc[prm.p];
     const uint32_t T = alloc_tiles(al), NB = alloc_buckets(al);
@@ -786,6 +790,8 @@ __global__ void __launch_bounds__(THREADS) k_hist(HistParams prm) {
         if (!cur.valid()) return;
         const uint64_t o = cur.offs();
         const uint32_t cnt = cur.count();
+        const K *keys = static_cast<const K *>(prm.src_keys[cur.bk.src]);
+        src_of[s] = keys;
         Seg sg;
         const uint32_t bytes = seg_plan(keys + o, cnt, keys, keys + prm.n, sg);
         in[1] = cnt;
@@ -823,7 +829,7 @@ __global__ void __launch_bounds__(THREADS) k_hist(HistParams prm) {
         sg.i0 = static_cast<int32_t>(in[4]);
         sg.i1 = static_cast<int32_t>(in[5]);
         const uint64_t toffs = offs_of[s];
-        const K *src = keys + toffs;
+        const K *src = src_of[s] + toffs;
         // one block histogram per tile, double-buffered: the counts of tile i are read
         // and cleared while tile i + 1 is counted into the other buffer
         uint32_t *my = wh + (it & 1u) * RADIX;
@@ -909,7 +915,7 @@ struct ClassifyParams {
     int last;  // 1: digit p is the least-significant one (no further classification)
     int lo;    // digit bits [lo, lo + width)
     int width;
-    const Bucket *buckets;
+    Bucket *buckets;  // (k_classify sets Bucket::skip)
     const uint32_t *tot;  // this pass
     uint32_t *tot_next;   // next pass (rows of created buckets are cleared)
     Bucket *next_buckets;
@@ -1056,6 +1062,16 @@ __device__ void classify_bucket(const ClassifyParams &prm, const Bucket &bk, uin
     }
     if (prm.last) return;
 
+    // ---- a bucket that never moved (still in the input) whose digit p is the same for all
+    // of its records keeps its records where they are: the scatter of pass p would only copy
+    // it (reading #22); its child and local entries point at the input
+    const bool skip = __syncthreads_or(tid < RADIX && tot[tid] == bk.count) && bk.src == SRC_IN;
+    const uint16_t child_src = skip ? static_cast<uint16_t>(SRC_IN) : prm.src_code;
+    if (skip && tid == 0) {
+        prm.buckets[bucket_id].skip = 1;
+        atomicAdd(&prm.ctl->skipped_in_pass[prm.p], static_cast<unsigned long long>(bk.count));
+    }
+
     // ---- counting children: next-pass buckets (R2) and their tile ranges (R4); one
     // 64-bit atomic allocates both so bucket order stays tile order
     const uint32_t TT = ct[RADIX];
@@ -1132,7 +1148,7 @@ __device__ void classify_bucket(const ClassifyParams &prm, const Bucket &bk, uin
             e.offs = boffs + start[tid];
             e.count = glead[tid];
             e.hi_bit = static_cast<uint16_t>(gmulti[tid] ? hi_p : prm.lo);
-            e.src = prm.src_code;
+            e.src = child_src;
             prm.local[my_cls][slot] = e;
         }
     }
@@ -1147,7 +1163,8 @@ __device__ void classify_bucket(const ClassifyParams &prm, const Bucket &bk, uin
             nb.count = s;
             nb.first_tile = bt + ct[tid];
             nb.ntiles = s / prm.kpb + (s % prm.kpb != 0u);
-            nb.pad = 0;
+            nb.src = child_src;
+            nb.skip = 0;
             prm.next_buckets[id] = nb;
         }
     }
@@ -1216,9 +1233,9 @@ __global__ void __launch_bounds__(THREADS) k_classify(ClassifyParams prm) {
 
 struct ScatterParams {
     uint64_t n;  // elements of the buffers
-    const void *keys_in;
-    void *keys_out;
-    const void *vals_in;
+    const void *src_keys[3];  // indexed by SrcCode (Bucket::src): where each bucket's records are
+    void *keys_out;           // X_p
+    const void *src_vals[3];
     void *vals_out;
     int p;
     int lo;
@@ -1233,7 +1250,7 @@ struct ScatterParams {
 };
 
 struct StageInfo {
-    uint32_t valid, count, bucket, carry_row, kpad, k0, k1, vpad, v0, v1, tile, pad_;
+    uint32_t valid, count, bucket, carry_row, kpad, k0, k1, vpad, v0, v1, tile, src;
     uint64_t offs;
 };
 
@@ -1305,10 +1322,10 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
     auto kst = [&](int s) { return reinterpret_cast<K *>(smem + L::off_kst + s * L::kst_bytes); };
     auto vst = [&](int s) { return reinterpret_cast<VT *>(smem + L::off_vst + s * L::vst_bytes); };
 
-    const K *__restrict__ kin = static_cast<const K *>(prm.keys_in);
     K *__restrict__ kout = static_cast<K *>(prm.keys_out);
-    const VT *__restrict__ vin = static_cast<const VT *>(prm.vals_in);
     VT *__restrict__ vout = static_cast<VT *>(prm.vals_out);
+    auto kin_of = [&](uint32_t src) { return static_cast<const K *>(prm.src_keys[src]); };
+    auto vin_of = [&](uint32_t src) { return static_cast<const VT *>(prm.src_vals[src]); };
     const int tid = threadIdx.x, lane = tid & 31, warp = tid >> 5;
     const uint32_t wbase = static_cast<uint32_t>(warp) * 32 * KPT;
     const uint32_t T = alloc_tiles(prm.ctl->alloc[prm.p]);
@@ -1319,9 +1336,20 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
 
     auto issue = [&](int s, uint32_t t) {
         StageInfo &in = info[s];
+        TileDesc td;
+        uint32_t src = SRC_IN;
+        while (t < T) {  // (the tiles of skipped buckets are claimed and passed over)
+            td = prm.tiles[t];
+            const Bucket bk = prm.buckets[td.bucket];
+            src = bk.src;
+            if (!bk.skip) break;
+            t = atomicAdd(&prm.ctl->claim[prm.p], 1u);
+        }
         in.valid = t < T;
         if (t >= T) return;
-        const TileDesc td = prm.tiles[t];
+        const K *kin = kin_of(src);
+        const VT *vin = HV ? vin_of(src) : nullptr;
+        in.src = src;
         in.count = td.count;
         in.bucket = td.bucket;
         in.carry_row = td.carry_row;
@@ -1383,8 +1411,8 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
         sv.pad = in.vpad;
         sv.i0 = static_cast<int32_t>(in.v0);
         sv.i1 = static_cast<int32_t>(in.v1);
-        const K *ksrc = kin + in.offs;
-        const VT *vsrc = HV ? vin + in.offs : nullptr;
+        const K *ksrc = kin_of(in.src) + in.offs;
+        const VT *vsrc = HV ? vin_of(in.src) + in.offs : nullptr;
         K *const ks = kst(s);
         VT *const vs = HV ? vst(s) : nullptr;
         mbar_wait(&bar[s], par);

@@ -142,6 +142,7 @@ def test_threshold_overrides_and_structure(tuning, dist, kbits, vbits):
     assert st["local_buckets"] == sim.local_buckets
     assert st["local_recs"] == sim.local_recs
     assert st["merged_groups"] == sim.merged_groups
+    assert st["skipped_recs_in_pass"] == sim.skipped_in_pass
     per_class = [0] * 8
     for e in sim.local_entries:
         per_class[e[3]] += 1
@@ -445,3 +446,38 @@ def test_copy_pieces():
         hrs.copy_pieces(dst, src, pieces + [(0, 0, 0)])
         exp = np.concatenate([np.arange(soffs[i], soffs[i] + lens[i]) for i in perm])
         assert np.array_equal(dst.cpu().numpy(), exp)
+
+
+@pytest.mark.parametrize("kbits,vbits", TYPES)
+def test_leading_constant_digits_skip(kbits, vbits):
+    """Reading #22: buckets still in the input whose digit is constant are not scattered.
+    Constant keys, 64-bit keys below 2^32 (four leading constant digits), keys with a
+    constant top byte, and a constant second digit after a real pass (no skip): output
+    against the oracle, structure (skipped records per pass) against the MSD simulation."""
+    import paper_1611_01137_b200 as hrs
+    n = 200003
+    base = gen.keys(n, kbits, "uniform", seed=8)
+    bo = oracle._u64(base)
+    cases = [np.full(n, 0x5A5A5A5A5A5A5A5A if kbits == 64 else 0x5A5A5A5A, dtype=np.uint64),
+             bo & np.uint64(0x00FFFFFF if kbits == 32 else 0xFFFFFFFF),
+             (bo & np.uint64((1 << (kbits - 8)) - 1)) | np.uint64(0xC3 << (kbits - 8)),
+             (bo & ~np.uint64(0xFF << (kbits - 16))) | np.uint64(0x5 << (kbits - 16))]
+    tun = dict(local_threshold=2048, merge_threshold=512, keys_per_tile=1024)
+    for kk in cases:
+        k = torch.from_numpy(kk.view(np.int64).copy())
+        k = k.view(torch.uint64) if kbits == 64 else k.to(torch.int32).view(torch.uint32)
+        v = gen.values(n, vbits, "random", seed=9) if vbits else None
+        for t in (None, tun):
+            kd, vd = k.to(DEV), (v.to(DEV) if v is not None else None)
+            temp = torch.empty(hrs.temp_bytes(n, kbits // 8, vbits // 8, 0, kbits, t), dtype=torch.uint8, device=DEV)
+            ko, vo = hrs.sort(kd, vd, tuning=t, temp=temp)
+            st = hrs.get_stats(temp)
+            ek, ev = oracle.sort(k, v, 0, kbits)
+            assert np.array_equal(_np(ko), ek)
+            if v is not None:
+                assert np.array_equal(_np(vo), ev)
+            dt = t or hrs.default_tuning(kbits // 8, vbits // 8)
+            sim = plan.simulate_msd(kk, None, 0, kbits, dt["local_threshold"], dt["merge_threshold"],
+                                    dt["keys_per_tile"])
+            assert st["skipped_recs_in_pass"] == sim.skipped_in_pass
+            assert st["bytes_min"] == plan.bytes_min(sim, kbits // 8, vbits // 8)

@@ -311,3 +311,28 @@ def test_oracle_equals_std_stable_sort_and_parallel_lsd(kbits, vbits, dist):
 def test_host_description():
     assert oracle.host_cores() >= 1
     assert isinstance(oracle.host_model(), str)
+
+
+def test_leading_constant_digit_skip_rule():
+    """Reading #22: a bucket still in the input whose digit is the same for all its records
+    is not scattered (except in the last pass).  Closed forms: constant u32/u32 keys skip
+    passes 1-3 and move once (4 x 4 B histogram reads + 16 B = 32 B/record); keys below
+    2^24 skip pass 1 only; uniform keys never skip; a second constant digit after a real
+    pass does not skip (the bucket moved)."""
+    n = 50000
+    lt, mt, kpb = 4096, 1024, 3072
+    r = plan.simulate_msd(np.full(n, 0xA5A5A5A5, dtype=np.uint64), None, 0, 32, lt, mt, kpb)
+    assert r.counting_passes == 4 and r.skipped_in_pass == [n, n, n, 0]
+    assert plan.bytes_min(r, 4, 4) == 32 * n
+    k = oracle._u64(gen.keys(n, 32, "uniform", seed=3)) & np.uint64(0x00FFFFFF)
+    r = plan.simulate_msd(k, None, 0, 32, lt, mt, kpb)
+    assert r.skipped_in_pass[0] == n and r.skipped_in_pass[1] == 0
+    r = plan.simulate_msd(oracle._u64(gen.keys(n, 32, "uniform", seed=3)), None, 0, 32, lt, mt, kpb)
+    assert r.counting_passes == 1 and r.skipped_in_pass == [0]
+    assert plan.bytes_min(r, 4, 4) == 20 * n + 16 * n  # one pass (4 + 16 B) and the local sorts (16 B)
+    # top digit varies, the second is constant: pass 2 moves (the buckets moved in pass 1)
+    k = (oracle._u64(gen.keys(n, 32, "uniform", seed=4)) & np.uint64(0xFF00FFFF)) | np.uint64(0x00370000)
+    r = plan.simulate_msd(k, None, 0, 32, 64, 16, 32)
+    assert r.counting_passes >= 2 and r.skipped_in_pass[:2] == [0, 0]
+    ks, _ = oracle.sort(k, None, 0, 32)
+    assert np.array_equal(r.keys, ks)
