@@ -1338,11 +1338,12 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
         StageInfo &in = info[s];
         TileDesc td;
         uint32_t src = SRC_IN;
-        while (t < T) {  // (the tiles of skipped buckets are claimed and passed over)
+        while (t < T) {  // (the tiles of a skipped bucket are passed over: the claim jumps past them)
             td = prm.tiles[t];
             const Bucket bk = prm.buckets[td.bucket];
             src = bk.src;
             if (!bk.skip) break;
+            atomicMax(&prm.ctl->claim[prm.p], bk.first_tile + bk.ntiles);
             t = atomicAdd(&prm.ctl->claim[prm.p], 1u);
         }
         in.valid = t < T;
