@@ -202,6 +202,22 @@ hrs_status hrs_sort_typed(void *d_temp, size_t *temp_bytes, const void *keys_in,
                           const void *vals_in, void *vals_out, uint64_t n, int key_bytes, int value_bytes,
                           hrs_key_kind kind, hrs_stream_t stream);
 
+/* ---- records stored interleaved (array of structs) ----
+ * Record i is key_bytes + value_bytes bytes at records_in + i * (key_bytes + value_bytes),
+ * its key at byte offset key_offset (0: key first, value_bytes: value first), both parts
+ * little-endian; records are 4-byte aligned.  The records are decomposed into a key array
+ * and a value array (one pass at memory bandwidth; the key of a signed / float kind goes
+ * through the order-preserving bijection of hrs_sort_typed on the way), sorted
+ * as pairs (hrs_sort_ex; stable), and recomposed into records_out (the inverse bijection
+ * fused into that pass).  kind HRS_KEY_UINT sorts by key bits [begin_bit, end_bit); the
+ * other kinds by the whole key (begin_bit = 0, end_bit = 8 * key_bytes, else
+ * HRS_ERROR_INVALID_BITS).  Temp = 2 n (key_bytes + value_bytes) + the pair sort's temp
+ * (two-phase size query); records_in, records_out and temp must not overlap.  Otherwise
+ * as hrs_sort_ex. */
+hrs_status hrs_sort_records(void *d_temp, size_t *temp_bytes, const void *records_in, void *records_out, uint64_t n,
+                            int key_bytes, int value_bytes, int key_offset, int begin_bit, int end_bit,
+                            hrs_key_kind kind, hrs_stream_t stream);
+
 /* ---- building blocks (kernel-level tests, the distributed driver) ---- */
 
 /* Histogram of digit bits [lo_bit, hi_bit) (1 <= hi_bit - lo_bit <= 8) over all n keys:

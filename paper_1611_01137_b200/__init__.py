@@ -15,7 +15,7 @@ import torch
 
 from ._lib import HRS_MAX_ITEMS, HrsError, Stats, Tuning, check, lib  # noqa: F401
 
-__all__ = ["sort", "sort_grouped", "temp_bytes", "get_stats", "digit_histogram", "partition_pass", "HrsError", "Tuning",
+__all__ = ["sort", "sort_grouped", "sort_records", "temp_bytes", "get_stats", "digit_histogram", "partition_pass", "HrsError", "Tuning",
            "default_tuning", "max_local_threshold", "max_keys_per_tile", "class_capacities", "lib"]
 
 _KEY_DTYPES = {torch.uint32: 4, torch.uint64: 8}
@@ -202,6 +202,44 @@ def sort_typed(keys: torch.Tensor, values: torch.Tensor | None = None, *, keys_o
         check(lib.hrs_sort_typed(_ptr(temp), ctypes.byref(sz), _ptr(keys), _ptr(keys_out), _ptr(values),
                                  _ptr(values_out), n, kb, vb, kind, _stream(stream)), "hrs_sort_typed")
     return keys_out, (values_out if values is not None else None)
+
+
+_KINDS = {"uint": 0, "int": 1, "float": 2}
+
+
+def sort_records(records: torch.Tensor, key_bytes: int, value_bytes: int, *, key_first: bool = True,
+                 kind: str = "uint", begin_bit: int = 0, end_bit: int | None = None, records_out=None, temp=None,
+                 stream=None) -> torch.Tensor:
+    """hrs_sort_records: stable sort of interleaved records (array of structs).
+    `records` is a contiguous CUDA tensor whose bytes are n records of key_bytes +
+    value_bytes each (e.g. a uint8 tensor of shape (n, R) or an int32 tensor of (n, R/4));
+    the key is the first (key_first) or the last field.  Returns records_out (same shape)."""
+    if not records.is_cuda or not records.is_contiguous():
+        raise ValueError("records must be a contiguous CUDA tensor")
+    rbytes = key_bytes + value_bytes
+    total = records.numel() * records.element_size()
+    if total % rbytes:
+        raise ValueError(f"{total} bytes is not a whole number of {rbytes}-byte records")
+    n = total // rbytes
+    if end_bit is None:
+        end_bit = 8 * key_bytes
+    if records_out is None:
+        records_out = torch.empty_like(records)
+    elif records_out.numel() * records_out.element_size() != total or not records_out.is_cuda:
+        raise ValueError("records_out must have the size of records")
+    sz = ctypes.c_size_t(0)
+    ko = 0 if key_first else value_bytes
+    check(lib.hrs_sort_records(None, ctypes.byref(sz), None, None, n, key_bytes, value_bytes, ko, begin_bit,
+                               end_bit, _KINDS[kind], None), "hrs_sort_records(size)")
+    if temp is None or temp.numel() < sz.value:
+        temp = alloc_temp(sz.value, records.device)
+    _on_stream(stream, temp, records_out)
+    sz = ctypes.c_size_t(temp.numel())
+    with torch.cuda.device(records.device):
+        check(lib.hrs_sort_records(_ptr(temp), ctypes.byref(sz), _ptr(records), _ptr(records_out), n, key_bytes,
+                                   value_bytes, ko, begin_bit, end_bit, _KINDS[kind], _stream(stream)),
+              "hrs_sort_records")
+    return records_out
 
 
 def get_stats(temp: torch.Tensor, stream=None) -> dict:

@@ -109,6 +109,7 @@ SIGNATURES = {
     "hrs_sort_pairs_u64_u64": (_ST, [_P, _SZP, _P, _P, _P, _P, _U64, _I, _I, _P]),
     "hrs_sort_ex": (_ST, [_P, _SZP, _P, _P, _P, _P, _U64, _I, _I, _I, _I, ctypes.POINTER(Tuning), _P]),
     "hrs_sort_typed": (_ST, [_P, _SZP, _P, _P, _P, _P, _U64, _I, _I, _I, _P]),
+    "hrs_sort_records": (_ST, [_P, _SZP, _P, _P, _U64, _I, _I, _I, _I, _I, _I, _P]),
     "hrs_sort_grouped": (_ST, [_P, _SZP, _P, _P, _P, _P, _U64, _I, _I, _I, _I, _P, ctypes.POINTER(Tuning), _P]),
     "hrs_get_stats": (_ST, [_P, ctypes.POINTER(Stats), _P]),
     "hrs_max_local_threshold": (ctypes.c_uint32, [_I, _I]),

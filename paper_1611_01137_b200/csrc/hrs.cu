@@ -1196,6 +1196,86 @@ hrs_status hrs_sort_typed(void *d_temp, size_t *temp_bytes, const void *keys_in,
     return map(keys_out, keys_out, 1);
 }
 
+}  // extern "C"
+
+namespace {
+template <typename K, typename V, int RW, bool KF>
+void launch_records(const void *ri, void *ro, void *keys, void *vals, uint64_t n, int kind, int recompose, int grid,
+                    cudaStream_t st) {
+    LaunchScope ls(st, 4, recompose);
+    launch_pdl(k_records<K, V, RW, KF>, dim3(grid), dim3(256), 0, st, static_cast<const uint32_t *>(ri),
+               static_cast<uint32_t *>(ro), static_cast<K *>(keys), static_cast<ValT<V> *>(vals), n, kind, recompose);
+}
+template <typename K, typename V>
+void records_kv(bool kf, const void *ri, void *ro, void *keys, void *vals, uint64_t n, int kind, int rc, int grid,
+                cudaStream_t st) {
+    constexpr int RW = static_cast<int>(sizeof(K) + (HasVal<V>::value ? sizeof(ValT<V>) : 0)) / 4;
+    if (kf) launch_records<K, V, RW, true>(ri, ro, keys, vals, n, kind, rc, grid, st);
+    else launch_records<K, V, RW, false>(ri, ro, keys, vals, n, kind, rc, grid, st);
+}
+void records_pass(int kb, int vb, bool kf, const void *ri, void *ro, void *keys, void *vals, uint64_t n, int kind,
+                  int rc, int grid, cudaStream_t st) {
+    if (kb == 4) {
+        if (vb == 0) records_kv<uint32_t, NoVal>(kf, ri, ro, keys, vals, n, kind, rc, grid, st);
+        else if (vb == 4) records_kv<uint32_t, uint32_t>(kf, ri, ro, keys, vals, n, kind, rc, grid, st);
+        else records_kv<uint32_t, unsigned long long>(kf, ri, ro, keys, vals, n, kind, rc, grid, st);
+    } else {
+        if (vb == 0) records_kv<unsigned long long, NoVal>(kf, ri, ro, keys, vals, n, kind, rc, grid, st);
+        else if (vb == 4) records_kv<unsigned long long, uint32_t>(kf, ri, ro, keys, vals, n, kind, rc, grid, st);
+        else records_kv<unsigned long long, unsigned long long>(kf, ri, ro, keys, vals, n, kind, rc, grid, st);
+    }
+}
+}  // namespace
+
+extern "C" {
+
+hrs_status hrs_sort_records(void *d_temp, size_t *temp_bytes, const void *records_in, void *records_out, uint64_t n,
+                            int key_bytes, int value_bytes, int key_offset, int begin_bit, int end_bit,
+                            hrs_key_kind kind, hrs_stream_t stream) {
+    if (!temp_bytes) return HRS_ERROR_INVALID_VALUE;
+    if (key_bytes != 4 && key_bytes != 8) return HRS_ERROR_INVALID_VALUE;
+    if (value_bytes != 0 && value_bytes != 4 && value_bytes != 8) return HRS_ERROR_INVALID_VALUE;
+    if (key_offset != 0 && key_offset != value_bytes) return HRS_ERROR_INVALID_VALUE;
+    if (kind != HRS_KEY_UINT && kind != HRS_KEY_INT && kind != HRS_KEY_FLOAT) return HRS_ERROR_INVALID_VALUE;
+    if (begin_bit < 0 || end_bit > 8 * key_bytes || begin_bit > end_bit) return HRS_ERROR_INVALID_BITS;
+    if (kind != HRS_KEY_UINT && (begin_bit != 0 || end_bit != 8 * key_bytes)) return HRS_ERROR_INVALID_BITS;
+    if (n > HRS_MAX_ITEMS) return HRS_ERROR_TOO_LARGE;
+    // temp = [keys n*K | values n*V | sorted keys n*K | sorted values n*V | the pair sort's temp]
+    size_t inner = 0;
+    hrs_status s = hrs_sort_ex(nullptr, &inner, nullptr, nullptr, nullptr, nullptr, n, key_bytes, value_bytes,
+                               begin_bit, end_bit, nullptr, stream);
+    if (s) return s;
+    const size_t nk = align_up(static_cast<size_t>(n) * key_bytes, 256), nv = align_up(static_cast<size_t>(n) * value_bytes, 256);
+    const size_t need = 2 * (nk + nv) + inner;
+    if (!d_temp) {
+        *temp_bytes = need;
+        return HRS_SUCCESS;
+    }
+    if (*temp_bytes < need) return HRS_ERROR_TEMP_TOO_SMALL;
+    if (!aligned(d_temp, 256)) return HRS_ERROR_INVALID_VALUE;
+    if (n == 0) return HRS_SUCCESS;
+    if (!records_in || !records_out || !aligned(records_in, 4) || !aligned(records_out, 4)) return HRS_ERROR_INVALID_VALUE;
+    const size_t rb = static_cast<size_t>(n) * (key_bytes + value_bytes);
+    if (overlap(records_in, rb, records_out, rb) || overlap(records_in, rb, d_temp, *temp_bytes) ||
+        overlap(records_out, rb, d_temp, *temp_bytes))
+        return HRS_ERROR_ALIASING;
+    int dev = 0, sms = 0;
+    if ((s = check_device(&dev, &sms))) return s;
+    cudaStream_t st = reinterpret_cast<cudaStream_t>(stream);
+    unsigned char *t = static_cast<unsigned char *>(d_temp);
+    void *k0 = t, *v0 = t + nk, *k1 = t + nk + nv, *v1 = t + 2 * nk + nv, *inner_t = t + 2 * (nk + nv);
+    const int grid = static_cast<int>(std::min<uint64_t>((n + 255) / 256, static_cast<uint64_t>(sms) * 8));
+    const bool kf = key_offset == 0;
+    records_pass(key_bytes, value_bytes, kf, records_in, nullptr, k0, value_bytes ? v0 : nullptr, n, kind, 0, grid, st);
+    if ((s = last_launch())) return s;
+    size_t tb = inner;
+    if ((s = hrs_sort_ex(inner_t, &tb, k0, k1, value_bytes ? v0 : nullptr, value_bytes ? v1 : nullptr, n, key_bytes,
+                         value_bytes, begin_bit, end_bit, nullptr, stream)))
+        return s;
+    records_pass(key_bytes, value_bytes, kf, nullptr, records_out, k1, value_bytes ? v1 : nullptr, n, kind, 1, grid, st);
+    return last_launch();
+}
+
 hrs_status hrs_sort_keys_u32(void *t, size_t *tb, const uint32_t *ki, uint32_t *ko, uint64_t n, int b, int e,
                              hrs_stream_t s) {
     return hrs_sort_ex(t, tb, ki, ko, nullptr, nullptr, n, 4, 0, b, e, nullptr, s);

@@ -672,6 +672,62 @@ __global__ void k_key_map(const K *in, K *out, uint64_t n, int kind, int inv) {
     }
 }
 
+// Array-of-structs records: decomposition into a key array and a value array,
+// and the recomposition after the sort, one pass each at memory bandwidth.  A record is
+// RW 4-byte words (key_bytes + value_bytes, the key at word KO); the key goes through the
+// order-preserving bijection of its kind on the way in and back on the way out
+// (P:907-918), fused into these passes.  Value words travel as opaque u32 / u64.
+template <typename K>
+__device__ __forceinline__ K key_map(K x, int kind, bool inv) {
+    constexpr K SIGN = K(1) << (8 * sizeof(K) - 1);
+    if (kind == 1) return x ^ SIGN;
+    if (kind == 2) return !inv ? ((x & SIGN) ? ~x : (x ^ SIGN)) : ((x & SIGN) ? (x ^ SIGN) : ~x);
+    return x;
+}
+template <typename K, typename V, int RW, bool KEYFIRST>
+__global__ void k_records(const uint32_t *__restrict__ rec_in, uint32_t *__restrict__ rec_out, K *keys,
+                          ValT<V> *vals, uint64_t n, int kind, int recompose) {
+    pdl_wait();
+    constexpr int KW = sizeof(K) / 4;
+    constexpr int VW = HasVal<V>::value ? static_cast<int>(sizeof(ValT<V>)) / 4 : 0;
+    constexpr int ko = KEYFIRST ? 0 : VW;  // word offset of the key
+    static_assert(KW + VW == RW, "record = key + value words");
+    const uint64_t stride = static_cast<uint64_t>(gridDim.x) * blockDim.x;
+    for (uint64_t i = static_cast<uint64_t>(blockIdx.x) * blockDim.x + threadIdx.x; i < n; i += stride) {
+        if (!recompose) {
+            uint32_t w[RW];
+#pragma unroll
+            for (int j = 0; j < RW; ++j) w[j] = rec_in[i * RW + j];
+            K k = 0;
+#pragma unroll
+            for (int j = 0; j < KW; ++j) k |= static_cast<K>(w[ko + j]) << (32 * j);
+            keys[i] = key_map(k, kind, false);
+            if constexpr (VW > 0) {
+                ValT<V> v = 0;
+                int q = 0;
+#pragma unroll
+                for (int j = 0; j < RW; ++j)
+                    if (j < ko || j >= ko + KW) v |= static_cast<ValT<V>>(w[j]) << (32 * q++);
+                vals[i] = v;
+            }
+        } else {
+            const K k = key_map(keys[i], kind, true);
+            uint32_t w[RW];
+#pragma unroll
+            for (int j = 0; j < KW; ++j) w[ko + j] = static_cast<uint32_t>(k >> (32 * j));
+            if constexpr (VW > 0) {
+                const ValT<V> v = vals[i];
+                int q = 0;
+#pragma unroll
+                for (int j = 0; j < RW; ++j)
+                    if (j < ko || j >= ko + KW) w[j] = static_cast<uint32_t>(v >> (32 * q++));
+            }
+#pragma unroll
+            for (int j = 0; j < RW; ++j) rec_out[i * RW + j] = w[j];
+        }
+    }
+}
+
 template <typename T>
 __global__ void k_copy(const T *__restrict__ in, T *__restrict__ out, uint64_t n) {
     const uint64_t stride = static_cast<uint64_t>(gridDim.x) * blockDim.x;

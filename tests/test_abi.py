@@ -117,3 +117,14 @@ def test_class_capacities_and_flags():
     assert _sz(_lib.lib.hrs_sort_ex, None, None, None, None, 10, 4, 0, 0, 32, ctypes.byref(ok), None)[0] == 0
     bad = _lib.Tuning(flags=2)
     assert _sz(_lib.lib.hrs_sort_ex, None, None, None, None, 10, 4, 0, 0, 32, ctypes.byref(bad), None)[0] == 1
+
+
+def test_records_argument_checks():
+    from paper_1611_01137_b200 import _lib
+    lib = _lib.lib
+    sz = ctypes.c_size_t(0)
+    assert lib.hrs_sort_records(None, ctypes.byref(sz), None, None, 1000, 4, 4, 0, 0, 32, 0, None) == 0
+    assert sz.value > 1000 * 8 * 3   # two decomposed copies + the pair sort (with its aux)
+    assert lib.hrs_sort_records(None, ctypes.byref(sz), None, None, 10, 4, 4, 2, 0, 32, 0, None) == 1  # key offset
+    assert lib.hrs_sort_records(None, ctypes.byref(sz), None, None, 10, 4, 4, 0, 1, 32, 1, None) == 2  # typed range
+    assert lib.hrs_sort_records(None, ctypes.byref(sz), None, None, 10, 4, 3, 0, 0, 32, 0, None) == 1  # value bytes

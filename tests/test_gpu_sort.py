@@ -481,3 +481,33 @@ def test_leading_constant_digits_skip(kbits, vbits):
                                     dt["keys_per_tile"])
             assert st["skipped_recs_in_pass"] == sim.skipped_in_pass
             assert st["bytes_min"] == plan.bytes_min(sim, kbits // 8, vbits // 8)
+
+
+# ------------------------------------------------------------- array-of-structs records
+
+@pytest.mark.parametrize("kb,vb", [(4, 4), (4, 8), (8, 4), (8, 8), (4, 0), (8, 0)])
+@pytest.mark.parametrize("key_first", [True, False])
+def test_sort_records(kb, vb, key_first):
+    """hrs_sort_records: interleaved records decomposed, sorted, recomposed.  Unsigned keys
+    over a bit range and signed / float keys by value; the oracle sorts the (key, record
+    index) pairs stably and the expected output is the records in that order."""
+    import paper_1611_01137_b200 as hrs
+    n = 100003
+    rng = np.random.default_rng(kb * 10 + vb + key_first)
+    raw = rng.integers(0, 256, size=(n, kb + vb), dtype=np.uint8)
+    raw[: n // 3, :] = raw[n // 2: n // 2 + n // 3, :]  # duplicate records: ties
+    koff = 0 if key_first else vb
+    kdt = {4: np.uint32, 8: np.uint64}[kb]
+    keys = np.ascontiguousarray(raw[:, koff:koff + kb]).view(kdt).reshape(-1)
+    rd = torch.from_numpy(raw.copy()).to(DEV)
+    for kind, (b, e) in (("uint", (0, 8 * kb)), ("uint", (3, 8 * kb - 5)), ("int", (0, 8 * kb)), ("float", (0, 8 * kb))):
+        out = hrs.sort_records(rd, kb, vb, key_first=key_first, kind=kind, begin_bit=b, end_bit=e)
+        torch.cuda.synchronize()
+        idx = np.arange(n, dtype=np.uint64)
+        if kind == "uint":
+            _, order = oracle.sort(keys, idx, b, e)
+        else:
+            tdt = {("int", 4): np.int32, ("int", 8): np.int64, ("float", 4): np.float32, ("float", 8): np.float64}
+            _, order = oracle.sort_typed(keys.view(tdt[(kind, kb)]), idx, kind)
+        exp = raw[order.astype(np.int64)]
+        assert np.array_equal(out.cpu().numpy(), exp), (kind, b, e)
