@@ -192,11 +192,12 @@ uint32_t hrs_class_capacity(int c);
  *   HRS_KEY_FLOAT: IEEE-754 binary32 (key_bytes 4) / binary64 (8) in the total order
  *                  -NaN < -inf < ... < -0.0 < +0.0 < ... < +inf < +NaN (NaNs of one sign
  *                  ordered by their bit patterns: larger payload further out).
- * Layout, ownership, async behaviour and errors as hrs_sort_ex.  Implementation: a kernel
- * maps the keys through the bijection into a region of d_temp (ints: flip the sign bit;
- * floats: flip every bit of a negative key, the sign bit of a positive one), the unsigned
- * sort runs on that copy, and the inverse map runs in place on keys_out.  Temp therefore
- * holds the unsigned sort's temp plus n * key_bytes (two-phase size query as usual). */
+ * Layout, ownership, async behaviour and errors as hrs_sort_ex; temp as hrs_sort_ex for
+ * unsigned keys of the same width.  The bijection (ints: flip the sign bit; floats: flip
+ * every bit of a negative key, the sign bit of a positive one) is fused into the sort as
+ * P:914-918 describes: a key read from the input is mapped where it is read (the first
+ * histogram and scatter, the local sorts of buckets that never moved), and mapped back
+ * where it is written for the last time (the last counting pass, the local sorts). */
 typedef enum { HRS_KEY_UINT = 0, HRS_KEY_INT = 1, HRS_KEY_FLOAT = 2 } hrs_key_kind;
 hrs_status hrs_sort_typed(void *d_temp, size_t *temp_bytes, const void *keys_in, void *keys_out,
                           const void *vals_in, void *vals_out, uint64_t n, int key_bytes, int value_bytes,

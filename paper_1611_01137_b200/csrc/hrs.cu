@@ -311,6 +311,7 @@ struct Plan {
     uint32_t local_wide_cap[HRS_NUM_CLASSES] = {0}, local_fb2_cap = 0;
     int wide_top = 0;
     int force_redo = 0;  // HRS_FLAG_FORCE_REDO (tuning flags or the HRS_FORCE_REDO environment variable)
+    int kind = 0;        // hrs_key_kind of the keys (signed / float: the bijection fused into the kernels)
 };
 
 // HRS_FORCE_REDO=1 in the environment ORs HRS_FLAG_FORCE_REDO into every call (include/hrs.h)
@@ -523,6 +524,7 @@ struct Runner {
         HistParams hp;
         hp.n = pl.n;
         for (int i = 0; i < 3; ++i) hp.src_keys[i] = bf.k[i];
+        hp.kind = pl.kind;
         hp.p = p;
         hp.lo = pl.lo[p - 1];
         hp.mask = (1u << (pl.hi[p - 1] - pl.lo[p - 1])) - 1u;
@@ -606,6 +608,8 @@ struct Runner {
         sp.tile_pref = at<uint32_t>(temp, pl.off_tile_pref);
         sp.ctl = at<Ctl>(temp, 0);
         sp.force_redo = pl.force_redo;
+        sp.kind = pl.kind;
+        sp.final_pass = p == pl.D ? 1 : 0;
         auto fn = k_scatter<K, V, SC::THREADS, SC::KPT, SC::MINB, SC::NBUF>;
         const size_t smem = ScatterSmem<K, V, SC::THREADS, SC::KPT, SC::NBUF>::bytes;
         int grid = 0;
@@ -634,6 +638,7 @@ struct Runner {
         lp.begin_bit = pl.begin;
         lp.force_redo = pl.force_redo;
         lp.redo = &at<Ctl>(temp, 0)->redo;
+        lp.kind = pl.kind;
     }
 
     // the counting local sort of class C; hands what it does not take to LIST_FB2
@@ -1058,7 +1063,7 @@ extern "C" {
 static hrs_status sort_common(void *d_temp, size_t *temp_bytes, const void *keys_in, void *keys_out,
                               const void *vals_in, void *vals_out, uint64_t n, int key_bytes, int value_bytes,
                               int begin_bit, int end_bit, const hrs_tuning *tuning, const uint64_t *grouped,
-                              hrs_stream_t stream);
+                              hrs_stream_t stream, int kind = 0);
 
 hrs_status hrs_sort_ex(void *d_temp, size_t *temp_bytes, const void *keys_in, void *keys_out, const void *vals_in,
                        void *vals_out, uint64_t n, int key_bytes, int value_bytes, int begin_bit, int end_bit,
@@ -1079,7 +1084,7 @@ hrs_status hrs_sort_grouped(void *d_temp, size_t *temp_bytes, const void *keys_i
 static hrs_status sort_common(void *d_temp, size_t *temp_bytes, const void *keys_in, void *keys_out,
                               const void *vals_in, void *vals_out, uint64_t n, int key_bytes, int value_bytes,
                               int begin_bit, int end_bit, const hrs_tuning *tuning, const uint64_t *grouped,
-                              hrs_stream_t stream) {
+                              hrs_stream_t stream, int kind) {
     if (!temp_bytes) return HRS_ERROR_INVALID_VALUE;
     if (key_bytes != 4 && key_bytes != 8) return HRS_ERROR_INVALID_VALUE;
     if (value_bytes != 0 && value_bytes != 4 && value_bytes != 8) return HRS_ERROR_INVALID_VALUE;
@@ -1088,6 +1093,7 @@ static hrs_status sort_common(void *d_temp, size_t *temp_bytes, const void *keys
     Plan pl;
     hrs_status s = make_plan(pl, n, key_bytes, value_bytes, begin_bit, end_bit, tuning, MODE_SORT);
     if (s) return s;
+    pl.kind = kind;
     if (!d_temp) {
         *temp_bytes = pl.total;
         return HRS_SUCCESS;
@@ -1138,6 +1144,7 @@ static hrs_status sort_common(void *d_temp, size_t *temp_bytes, const void *keys
         v[12] = *temp_bytes;
         v[13] = t.flags | env_flags();
         v[14] = reinterpret_cast<uintptr_t>(grouped);
+        v[15] = static_cast<uint64_t>(kind);
         hrs_status gs = HRS_SUCCESS;
         if (via_graph(key, st, dev, &gs, run)) return gs;
     }
@@ -1150,50 +1157,11 @@ hrs_status hrs_sort_typed(void *d_temp, size_t *temp_bytes, const void *keys_in,
     if (!temp_bytes) return HRS_ERROR_INVALID_VALUE;
     if (kind != HRS_KEY_UINT && kind != HRS_KEY_INT && kind != HRS_KEY_FLOAT) return HRS_ERROR_INVALID_VALUE;
     if (key_bytes != 4 && key_bytes != 8) return HRS_ERROR_INVALID_VALUE;
-    const int kbits = 8 * key_bytes;
-    if (kind == HRS_KEY_UINT)
-        return hrs_sort_ex(d_temp, temp_bytes, keys_in, keys_out, vals_in, vals_out, n, key_bytes, value_bytes, 0,
-                           kbits, nullptr, stream);
-    // temp = [mapped keys: n * key_bytes, 256-aligned | the unsigned sort's temp]
-    size_t inner = 0;
-    hrs_status s = hrs_sort_ex(nullptr, &inner, nullptr, nullptr, nullptr, nullptr, n, key_bytes, value_bytes, 0,
-                               kbits, nullptr, stream);
-    if (s) return s;
-    const size_t mapped = align_up(static_cast<size_t>(n) * key_bytes, 256);
-    if (!d_temp) {
-        *temp_bytes = mapped + inner;
-        return HRS_SUCCESS;
-    }
-    if (*temp_bytes < mapped + inner) return HRS_ERROR_TEMP_TOO_SMALL;
-    if (!aligned(d_temp, 256)) return HRS_ERROR_INVALID_VALUE;
-    if (n == 0) return HRS_SUCCESS;
-    if (!keys_in || !keys_out) return HRS_ERROR_INVALID_VALUE;
-    if (!aligned(keys_in, key_bytes) || !aligned(keys_out, key_bytes)) return HRS_ERROR_INVALID_VALUE;
-    if (overlap(keys_in, n * key_bytes, d_temp, *temp_bytes) || overlap(keys_out, n * key_bytes, d_temp, *temp_bytes) ||
-        (value_bytes && (overlap(vals_in, n * value_bytes, d_temp, mapped) || overlap(vals_out, n * value_bytes, d_temp, mapped))))
-        return HRS_ERROR_ALIASING;
-    int dev = 0, sms = 0;
-    if ((s = check_device(&dev, &sms))) return s;
-    cudaStream_t st = reinterpret_cast<cudaStream_t>(stream);
-    void *mk = d_temp;
-    void *sort_temp = static_cast<unsigned char *>(d_temp) + mapped;
-    const int grid = static_cast<int>(std::min<uint64_t>((n + 255) / 256, static_cast<uint64_t>(sms) * 8));
-    auto map = [&](const void *in, void *out, int inv) -> hrs_status {
-        LaunchScope ls(st, 4, inv);
-        if (key_bytes == 4)
-            launch_pdl(k_key_map<uint32_t>, dim3(grid), dim3(256), 0, st, static_cast<const uint32_t *>(in),
-                       static_cast<uint32_t *>(out), n, static_cast<int>(kind), inv);
-        else
-            launch_pdl(k_key_map<uint64_t>, dim3(grid), dim3(256), 0, st, static_cast<const uint64_t *>(in),
-                       static_cast<uint64_t *>(out), n, static_cast<int>(kind), inv);
-        return last_launch();
-    };
-    if ((s = map(keys_in, mk, 0))) return s;
-    size_t tb = *temp_bytes - mapped;
-    if ((s = hrs_sort_ex(sort_temp, &tb, mk, keys_out, vals_in, vals_out, n, key_bytes, value_bytes, 0, kbits, nullptr,
-                         stream)))
-        return s;
-    return map(keys_out, keys_out, 1);
+    // the bijection is fused into the kernels: a key read from the input is
+    // mapped on the way in (histogram, first scatter, local sorts of unmoved buckets) and
+    // mapped back where it is written for the last time (last scatter pass, local sorts)
+    return sort_common(d_temp, temp_bytes, keys_in, keys_out, vals_in, vals_out, n, key_bytes, value_bytes, 0,
+                       8 * key_bytes, nullptr, nullptr, stream, static_cast<int>(kind));
 }
 
 }  // extern "C"

@@ -797,6 +797,7 @@ struct HistParams {
     TileDesc *tiles;           // [tile]: descriptor for k_scatter
     uint32_t *tile_pref;       // [tile][256]: digit counts of the earlier tiles of its bucket segment
     Ctl *ctl;
+    int kind;  // hrs_key_kind: keys still in the input go through the bijection
 };
 
 template <typename K, int THREADS, int NSTAGE, int CAP>
@@ -886,6 +887,7 @@ __global__ void __launch_bounds__(THREADS) k_hist(HistParams prm) {
         sg.i1 = static_cast<int32_t>(in[5]);
         const uint64_t toffs = offs_of[s];
         const K *src = src_of[s] + toffs;
+        const bool mapin = prm.kind != 0 && src_of[s] == static_cast<const K *>(prm.src_keys[SRC_IN]);
         // one block histogram per tile, double-buffered: the counts of tile i are read
         // and cleared while tile i + 1 is counted into the other buffer
         uint32_t *my = wh + (it & 1u) * RADIX;
@@ -918,7 +920,7 @@ __global__ void __launch_bounds__(THREADS) k_hist(HistParams prm) {
                 const uint4 w = vb[v];
                 const K *kk = reinterpret_cast<const K *>(&w);
 #pragma unroll
-                for (int j = 0; j < VK; ++j) atomicAdd(&my[digit_of(kk[j], prm.lo, prm.mask)], 1u);
+                for (int j = 0; j < VK; ++j) atomicAdd(&my[digit_of(mapin ? key_map(kk[j], prm.kind, false) : kk[j], prm.lo, prm.mask)], 1u);
             }
             // edge vectors: v = 0 when it starts before element 0, v = vhi when partial
             const int32_t ve = tid == 0 ? (vlo ? 0 : -1) : (tid == 1 && vhi < nq && vhi >= vlo ? vhi : -1);
@@ -929,7 +931,7 @@ __global__ void __launch_bounds__(THREADS) k_hist(HistParams prm) {
 #pragma unroll
                 for (int j = 0; j < VK; ++j)
                     if (i + j >= 0 && i + j < static_cast<int32_t>(count))
-                        atomicAdd(&my[digit_of(kk[j], prm.lo, prm.mask)], 1u);
+                        atomicAdd(&my[digit_of(mapin ? key_map(kk[j], prm.kind, false) : kk[j], prm.lo, prm.mask)], 1u);
             }
         }
         // elements the copy did not cover (segments at the ends of the buffer) from global
@@ -938,7 +940,7 @@ __global__ void __launch_bounds__(THREADS) k_hist(HistParams prm) {
             const uint32_t tl = sg.i1 > sg.i0 ? static_cast<uint32_t>(min(sg.i1, static_cast<int32_t>(count))) : count;
             for (uint32_t j = tid; j < h + (count - tl); j += THREADS) {
                 const uint32_t i = j < h ? j : tl + (j - h);
-                atomicAdd(&my[digit_of(src[i], prm.lo, prm.mask)], 1u);
+                atomicAdd(&my[digit_of(mapin ? key_map(src[i], prm.kind, false) : src[i], prm.lo, prm.mask)], 1u);
             }
         }
         __syncthreads();
@@ -1303,6 +1305,8 @@ struct ScatterParams {
     const uint32_t *tile_pref;
     Ctl *ctl;
     int force_redo;  // HRS_FLAG_FORCE_REDO: every stability check fails (tests of the redo path)
+    int kind;        // hrs_key_kind: the bijection on the way out of the input, its inverse
+    int final_pass;  //   on the way into the final output (the last pass)
 };
 
 struct StageInfo {
@@ -1474,6 +1478,8 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
         VT *const vs = HV ? vst(s) : nullptr;
         mbar_wait(&bar[s], par);
         const bool full = count == static_cast<uint32_t>(L::KPB) && seg_full(sk, count) && (!HV || seg_full(sv, count));
+        const bool mapin = prm.kind != 0 && in.src == SRC_IN;          // records still in the input
+        const bool unmap = prm.kind != 0 && prm.final_pass != 0;       // their final place
         const VT *const vb = HV ? vs + sv.pad : nullptr;
 
         auto body = [&](auto full_tag) {
@@ -1495,6 +1501,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
                 const uint32_t e = wbase + c * 32 + lane;
                 const bool v = FULL || e < count;
                 key[c] = v ? (FULL ? kb[e] : seg_get(ks, ksrc, sk, e)) : K(0);
+                if (mapin) key[c] = key_map(key[c], prm.kind, false);
                 if constexpr (DIRECT) val[c] = v ? (FULL ? vb[e] : seg_get(vs, vsrc, sv, e)) : VT(0);
                 valid |= v ? (1u << c) : 0u;
             }
@@ -1584,13 +1591,13 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
                         const K k = ks[j];
                         if constexpr (DIRECT) {
                             const uint32_t pos = gs[digit_of(k, lo, mask)].x + j;
-                            kdst[pos] = k;
+                            kdst[pos] = unmap ? key_map(k, prm.kind, true) : k;
                             vdst[pos] = vs[j];
                         } else {
                             const uint32_t i = sidx[j];
                             const uint2 g = gs[digit_of(k, lo, mask)];
                             const uint32_t pos = g.x + j;
-                            kdst[pos] = k;
+                            kdst[pos] = unmap ? key_map(k, prm.kind, true) : k;
                             if (HV) vdst[pos] = vb[i];
                             if (check && j > g.y) bad |= sidx[j - 1] > i;
                         }
@@ -1668,6 +1675,7 @@ struct LocalParams {
     int begin_bit;
     int force_redo;  // HRS_FLAG_FORCE_REDO: every stability check of the fast rank fails
     unsigned long long *redo;  // Ctl::redo
+    int kind;        // hrs_key_kind: keys read from the input are mapped, every write is final (unmapped)
 };
 
 // Shared memory of one local-sort CTA: NSTAGE staging buffers {keys, values}; after
@@ -1840,6 +1848,13 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
         const uint32_t count = in[1];
         const int hi_bit = static_cast<int>(in[2]);
         const uint32_t src = in[3];
+        // signed / float keys (hrs_sort_typed): keys read from the input are mapped to their
+        // order-preserving image, every key this kernel writes is final and mapped back
+        const bool mapin = prm.kind != 0 && src == SRC_IN;
+        auto kin_map = [&](K x) -> K { return mapin ? key_map(x, prm.kind, false) : x; };
+        auto kout_map = [&](K x) -> K { return prm.kind != 0 ? key_map(x, prm.kind, true) : x; };
+        // a staged key copied to the output: the original if it came from the input
+        auto kout_raw = [&](K x) -> K { return (prm.kind != 0 && !mapin) ? key_map(x, prm.kind, true) : x; };
         const uint64_t offs = static_cast<uint64_t>(in[4]) | (static_cast<uint64_t>(in[5]) << 32);
         Seg sk, sv;
         sk.pad = in[6];
@@ -1870,7 +1885,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
         for (int c = 0; c < KPT; ++c) {
             const uint32_t e = wbase + c * 32 + lane;
             idx[c] = e;
-            key[c] = (!BAL || c < kpt) ? (e < count ? seg_get(ks, ksrc, sk, e) : ks[sk.pad + e]) : K(0);  // past count: stale, never written out
+            key[c] = kin_map((!BAL || c < kpt) ? (e < count ? seg_get(ks, ksrc, sk, e) : ks[sk.pad + e]) : K(0));  // past count: stale, never written out
             const bool v = (!BAL || c < kpt) && e < count;
             a &= v ? key[c] : ~K(0);
             o |= v ? key[c] : K(0);
@@ -2016,7 +2031,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
                 const int lb = sb - tb;
                 const K lmask = lb >= static_cast<int>(8 * sizeof(K)) ? ~K(0) : ((K(1) << lb) - 1);
                 auto low = [&](CT x) -> K {
-                    return (ksp[static_cast<uint32_t>(x) & ((1u << IB) - 1u)] >> begin_bit) & lmask;
+                    return (kin_map(ksp[static_cast<uint32_t>(x) & ((1u << IB) - 1u)]) >> begin_bit) & lmask;
                 };
                 for (uint32_t e = tid; e + 1 < count && !s_fallback; e += THREADS) {
                     const CT t = comp[e] >> IB;
@@ -2059,7 +2074,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
                     en.src = static_cast<uint16_t>(src);
                     to_wide(en);
                 }
-            } else if (moved || src != SRC_OUT) {
+            } else if (moved || src != SRC_OUT || prm.kind != 0) {
                 K *const kd = kout + offs;
                 VT *const vd = HV ? vout + offs : nullptr;
                 const VT *const vsp = HV ? vs + sv.pad : nullptr;
@@ -2071,7 +2086,8 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
                     const uint32_t e = wbase + c * 32 + lane;
                     if ((!BAL || c < kpt) && e < count) {
                         const uint32_t ix = static_cast<uint32_t>(cv[c]) & ((1u << IB) - 1u);
-                        kd[e] = LW::RECON ? (khigh | static_cast<K>(static_cast<uint32_t>(cv[c]) >> IB)) : ksp[ix];
+                        kd[e] = LW::RECON ? kout_map(khigh | static_cast<K>(static_cast<uint32_t>(cv[c]) >> IB))
+                                          : kout_raw(ksp[ix]);
                         if (HV) vd[e] = vsp[ix];
                     }
                 }
@@ -2134,13 +2150,13 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
 #pragma unroll
                     for (int c = 0; c < KPT; ++c) {
                         const uint32_t e = wbase + c * 32 + lane;
-                        key[c] = e < count ? ksrc[e] : K(0);  // the source is untouched until the write-out
+                        key[c] = e < count ? kin_map(ksrc[e]) : K(0);  // the source is untouched until the write-out
                         idx[c] = e;
                     }
                     pair_passes(false);
                 }
             }
-            if (moved || src != SRC_OUT) {
+            if (moved || src != SRC_OUT || prm.kind != 0) {
                 K *const kd = kout + offs;
                 VT *const vd = HV ? vout + offs : nullptr;
                 const VT *const vsp = HV ? vs + sv.pad : nullptr;
@@ -2148,7 +2164,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
                 for (int c = 0; c < KPT; ++c) {
                     const uint32_t e = wbase + c * 32 + lane;
                     if ((!BAL || c < kpt) && e < count) {
-                        kd[e] = key[c];
+                        kd[e] = kout_map(key[c]);
                         if (HV) vd[e] = vsp[idx[c]];
                     }
                 }
@@ -2332,6 +2348,13 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
         const uint32_t count = in[1];
         const int hi_bit = static_cast<int>(in[2]);
         const uint32_t src = in[3];
+        // signed / float keys (hrs_sort_typed): keys read from the input are mapped to their
+        // order-preserving image, every key this kernel writes is final and mapped back
+        const bool mapin = prm.kind != 0 && src == SRC_IN;
+        auto kin_map = [&](K x) -> K { return mapin ? key_map(x, prm.kind, false) : x; };
+        auto kout_map = [&](K x) -> K { return prm.kind != 0 ? key_map(x, prm.kind, true) : x; };
+        // a staged key copied to the output: the original if it came from the input
+        auto kout_raw = [&](K x) -> K { return (prm.kind != 0 && !mapin) ? key_map(x, prm.kind, true) : x; };
         const uint64_t offs = static_cast<uint64_t>(in[4]) | (static_cast<uint64_t>(in[5]) << 32);
         Seg sk, sv;
         sk.pad = in[6];
@@ -2357,7 +2380,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
 #pragma unroll
         for (int c = 0; c < KPT; ++c) {
             const uint32_t e = c * THREADS + tid;
-            key[c] = ksp[e < count ? e : 0u];  // past the end: a copy of key 0 (neutral for and/or)
+            key[c] = kin_map(ksp[e < count ? e : 0u]);  // past the end: a copy of key 0 (neutral for and/or)
             a &= key[c];
             o |= key[c];
         }
@@ -2389,12 +2412,12 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
         const VT *const vsp = HV ? vs + sv.pad : nullptr;
         if (nosort) {
             // every record has the same sort bits: the stable order is the input order
-            if (src != SRC_OUT) {
+            if (src != SRC_OUT || prm.kind != 0) {
 #pragma unroll
                 for (int c = 0; c < KPT; ++c) {
                     const uint32_t e = c * THREADS + tid;
                     if (e < count) {
-                        kd[e] = key[c];
+                        kd[e] = kout_map(key[c]);
                         if (HV) vd[e] = vsp[e];
                     }
                 }
@@ -2487,7 +2510,8 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
                 auto less = [&](uint32_t x, uint32_t y) -> bool {
                     if ((x >> IB) != (y >> IB)) return x < y;
                     if (low) {
-                        const K lx = (ksp[x & IMASK] >> begin_bit) & lmask, ly = (ksp[y & IMASK] >> begin_bit) & lmask;
+                        const K lx = (kin_map(ksp[x & IMASK]) >> begin_bit) & lmask,
+                                ly = (kin_map(ksp[y & IMASK]) >> begin_bit) & lmask;
                         if (lx != ly) return lx < ly;
                     }
                     return x < y;
@@ -2527,7 +2551,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
                     const uint32_t e = c * THREADS + tid;
                     if (e < count) {
                         const uint32_t x = comp[e], ix = x & IMASK;
-                        kd[e] = RECON ? (khigh | static_cast<K>(x >> IB)) : ksp[ix];
+                        kd[e] = RECON ? kout_map(khigh | static_cast<K>(x >> IB)) : kout_raw(ksp[ix]);
                         if (HV) vd[e] = vsp[ix];
                     }
                 }

@@ -294,7 +294,7 @@ def test_typed_keys(dtype, vbits, n):
     import paper_1611_01137_b200 as hrs
     kb = 32 if dtype in (torch.int32, torch.float32) else 64
     kind = "int" if dtype in (torch.int32, torch.int64) else "float"
-    for dist in ("uniform", "and3"):
+    for dist in ("uniform", "and3", "const"):
         bits = gen.keys(n, kb, dist, seed=41)
         k = bits.view(dtype)
         v = gen.values(n, vbits, "index") if vbits else None
