@@ -608,7 +608,7 @@ struct InitParams {
     uint32_t grouped_radix;
 };
 
-__global__ void k_init(InitParams prm) {
+static __global__ void k_init(InitParams prm) {
     pdl_wait();
     const uint64_t n = prm.n;
     const uint32_t T1 = prm.counting ? static_cast<uint32_t>((n + prm.kpb - 1) / prm.kpb) : 0u;
@@ -650,25 +650,6 @@ __global__ void k_init(InitParams prm) {
                 c->local_recs = n;
             }
         }
-    }
-}
-
-// Order-preserving bijections of signed / IEEE-754 keys onto unsigned ones:
-// kind 1 (two's complement): flip the sign bit; kind 2 (float): a negative key (sign bit
-// set) has every bit flipped, a positive one only its sign bit.  k_key_map applies the map
-// (inv = 0) from `in` to `out`, or its inverse (inv = 1), which may run in place.
-template <typename K>
-__global__ void k_key_map(const K *in, K *out, uint64_t n, int kind, int inv) {
-    pdl_wait();
-    constexpr K SIGN = K(1) << (8 * sizeof(K) - 1);
-    const uint64_t stride = static_cast<uint64_t>(gridDim.x) * blockDim.x;
-    for (uint64_t i = static_cast<uint64_t>(blockIdx.x) * blockDim.x + threadIdx.x; i < n; i += stride) {
-        const K x = in[i];
-        K y;
-        if (kind == 1) y = x ^ SIGN;
-        else if (!inv) y = (x & SIGN) ? ~x : (x ^ SIGN);
-        else y = (x & SIGN) ? (x ^ SIGN) : ~x;
-        out[i] = y;
     }
 }
 
@@ -775,7 +756,7 @@ __global__ void __launch_bounds__(256) k_copy_pieces(const T *__restrict__ src, 
     }
 }
 
-__global__ void k_fill_u64(uint64_t *p, uint64_t n, uint64_t v) {
+static __global__ void k_fill_u64(uint64_t *p, uint64_t n, uint64_t v) {
     for (uint64_t i = static_cast<uint64_t>(blockIdx.x) * blockDim.x + threadIdx.x; i < n;
          i += static_cast<uint64_t>(gridDim.x) * blockDim.x)
         p[i] = v;
@@ -811,7 +792,7 @@ struct HistSmem {
     static constexpr size_t bytes = off_stage + NSTAGE * align16(sizeof(K) * stage_elems);
 };
 
-template <typename K, int THREADS, int NSTAGE, int CAP>
+template <typename K, int THREADS, int NSTAGE, int CAP, bool TY>
 __global__ void __launch_bounds__(THREADS) k_hist(HistParams prm) {
     pdl_wait();
     using L = HistSmem<K, THREADS, NSTAGE, CAP>;
@@ -887,7 +868,7 @@ __global__ void __launch_bounds__(THREADS) k_hist(HistParams prm) {
         sg.i1 = static_cast<int32_t>(in[5]);
         const uint64_t toffs = offs_of[s];
         const K *src = src_of[s] + toffs;
-        const bool mapin = prm.kind != 0 && src_of[s] == static_cast<const K *>(prm.src_keys[SRC_IN]);
+        const bool mapin = TY && prm.kind != 0 && src_of[s] == static_cast<const K *>(prm.src_keys[SRC_IN]);
         // one block histogram per tile, double-buffered: the counts of tile i are read
         // and cleared while tile i + 1 is counted into the other buffer
         uint32_t *my = wh + (it & 1u) * RADIX;
@@ -1361,7 +1342,7 @@ struct ScatterSmem {
 // its bucket) comes from k_hist / k_classify, so tiles are independent (no
 // look-back) and claimed in order from a counter: the tiles in flight write neighbouring
 // runs of every sub-bucket, which combine in L2.
-template <typename K, typename V, int THREADS, int KPT, int MINB, int NBUF>
+template <typename K, typename V, int THREADS, int KPT, int MINB, int NBUF, bool TY>
 __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
     pdl_wait();
     static_assert(NBUF == 1 || NBUF == 2, "one or two staging buffers");
@@ -1478,8 +1459,8 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
         VT *const vs = HV ? vst(s) : nullptr;
         mbar_wait(&bar[s], par);
         const bool full = count == static_cast<uint32_t>(L::KPB) && seg_full(sk, count) && (!HV || seg_full(sv, count));
-        const bool mapin = prm.kind != 0 && in.src == SRC_IN;          // records still in the input
-        const bool unmap = prm.kind != 0 && prm.final_pass != 0;       // their final place
+        const bool mapin = TY && prm.kind != 0 && in.src == SRC_IN;     // records still in the input
+        const bool unmap = TY && prm.kind != 0 && prm.final_pass != 0;  // their final place
         const VT *const vb = HV ? vs + sv.pad : nullptr;
 
         auto body = [&](auto full_tag) {
@@ -1489,7 +1470,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
             constexpr bool DIRECT = HRS_SC_DIRECT && HV;
             if (!DIRECT && !FULL && HV) seg_fill_edges<VT, THREADS>(vs, vsrc, sv, count);
             const K *const kb = ks + sk.pad;
-            VT val[DIRECT ? KPT : 1];
+            [[maybe_unused]] VT val[DIRECT ? KPT : 1];
             // the keys stay in registers from here to the placement; the in-warp ranks are
             // packed two to a register (rank < 32 * KPT < 2^16), the digits recomputed
             constexpr int NR = (KPT + 1) / 2;
@@ -1731,7 +1712,7 @@ __device__ __forceinline__ unsigned long long warp_or(unsigned long long x) {
     return (static_cast<unsigned long long>(hi) << 32) | lo;
 }
 
-template <typename K, typename V, int THREADS, int KPT, int NSTAGE, int MINB, int WIDE>
+template <typename K, typename V, int THREADS, int KPT, int NSTAGE, int MINB, int WIDE, bool TY>
 __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
     pdl_wait();
     using L = LocalSmem<K, V, THREADS, KPT, NSTAGE, WIDE>;
@@ -1850,11 +1831,12 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
         const uint32_t src = in[3];
         // signed / float keys (hrs_sort_typed): keys read from the input are mapped to their
         // order-preserving image, every key this kernel writes is final and mapped back
-        const bool mapin = prm.kind != 0 && src == SRC_IN;
+        const bool typed = TY && prm.kind != 0;
+        const bool mapin = typed && src == SRC_IN;
         auto kin_map = [&](K x) -> K { return mapin ? key_map(x, prm.kind, false) : x; };
-        auto kout_map = [&](K x) -> K { return prm.kind != 0 ? key_map(x, prm.kind, true) : x; };
+        auto kout_map = [&](K x) -> K { return typed ? key_map(x, prm.kind, true) : x; };
         // a staged key copied to the output: the original if it came from the input
-        auto kout_raw = [&](K x) -> K { return (prm.kind != 0 && !mapin) ? key_map(x, prm.kind, true) : x; };
+        auto kout_raw = [&](K x) -> K { return (typed && !mapin) ? key_map(x, prm.kind, true) : x; };
         const uint64_t offs = static_cast<uint64_t>(in[4]) | (static_cast<uint64_t>(in[5]) << 32);
         Seg sk, sv;
         sk.pad = in[6];
@@ -2074,7 +2056,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
                     en.src = static_cast<uint16_t>(src);
                     to_wide(en);
                 }
-            } else if (moved || src != SRC_OUT || prm.kind != 0) {
+            } else if (moved || src != SRC_OUT || typed) {
                 K *const kd = kout + offs;
                 VT *const vd = HV ? vout + offs : nullptr;
                 const VT *const vsp = HV ? vs + sv.pad : nullptr;
@@ -2156,7 +2138,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
                     pair_passes(false);
                 }
             }
-            if (moved || src != SRC_OUT || prm.kind != 0) {
+            if (moved || src != SRC_OUT || typed) {
                 K *const kd = kout + offs;
                 VT *const vd = HV ? vout + offs : nullptr;
                 const VT *const vsp = HV ? vs + sv.pad : nullptr;
@@ -2241,7 +2223,7 @@ struct LocalCntSmem {
     static constexpr size_t bytes = off_vst + NSTAGE * vst_bytes;
 };
 
-template <typename K, typename V, int THREADS, int KPT, int NSTAGE, int MINB, int CB, bool RECON>
+template <typename K, typename V, int THREADS, int KPT, int NSTAGE, int MINB, int CB, bool RECON, bool TY>
 __global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
     pdl_wait();
     using L = LocalCntSmem<K, V, THREADS, KPT, NSTAGE, CB, RECON>;
@@ -2350,11 +2332,12 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
         const uint32_t src = in[3];
         // signed / float keys (hrs_sort_typed): keys read from the input are mapped to their
         // order-preserving image, every key this kernel writes is final and mapped back
-        const bool mapin = prm.kind != 0 && src == SRC_IN;
+        const bool typed = TY && prm.kind != 0;
+        const bool mapin = typed && src == SRC_IN;
         auto kin_map = [&](K x) -> K { return mapin ? key_map(x, prm.kind, false) : x; };
-        auto kout_map = [&](K x) -> K { return prm.kind != 0 ? key_map(x, prm.kind, true) : x; };
+        auto kout_map = [&](K x) -> K { return typed ? key_map(x, prm.kind, true) : x; };
         // a staged key copied to the output: the original if it came from the input
-        auto kout_raw = [&](K x) -> K { return (prm.kind != 0 && !mapin) ? key_map(x, prm.kind, true) : x; };
+        auto kout_raw = [&](K x) -> K { return (typed && !mapin) ? key_map(x, prm.kind, true) : x; };
         const uint64_t offs = static_cast<uint64_t>(in[4]) | (static_cast<uint64_t>(in[5]) << 32);
         Seg sk, sv;
         sk.pad = in[6];
@@ -2412,7 +2395,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
         const VT *const vsp = HV ? vs + sv.pad : nullptr;
         if (nosort) {
             // every record has the same sort bits: the stable order is the input order
-            if (src != SRC_OUT || prm.kind != 0) {
+            if (src != SRC_OUT || typed) {
 #pragma unroll
                 for (int c = 0; c < KPT; ++c) {
                     const uint32_t e = c * THREADS + tid;
