@@ -34,6 +34,7 @@ std::mutex g_mu;
 std::unordered_map<uint64_t, KernelInfo> g_kinfo;
 std::unordered_map<int, int> g_dev_ok;
 std::unordered_map<int, int> g_dev_sms;
+thread_local GraphCtx *g_gx = nullptr;
 }  // namespace hrs_host
 
 namespace {
@@ -89,6 +90,16 @@ std::unordered_map<int, cudaStream_t> g_capture_stream;
 uint64_t g_gstamp = 0;
 constexpr size_t GRAPH_CACHE_MAX = 64;
 
+std::unordered_map<int, GraphCtx> g_gctx;  // conditional-capture streams per device
+
+bool cond_graphs_enabled() {
+    static const bool on = [] {
+        const char *e = std::getenv("HRS_GRAPH_COND");
+        return !(e && e[0] == '0');
+    }();
+    return on;
+}
+
 bool graphs_enabled() {
     static const bool on = [] {
         const char *e = std::getenv("HRS_GRAPHS");
@@ -125,25 +136,41 @@ bool via_graph(const GraphKey &key, cudaStream_t stream, int dev, hrs_status *ou
             cs = nullptr;
             return false;
         }
-        if (cudaStreamBeginCapture(cs, cudaStreamCaptureModeThreadLocal) != cudaSuccess) return false;
+        // first with conditional nodes (empty passes and lists are skipped on the device),
+        // then, if any conditional-graph call fails, as a plain capture
         const uint64_t l0 = g_launches;
-        const hrs_status s = run(cs);
-        cudaGraph_t g = nullptr;
-        err = cudaStreamEndCapture(cs, &g);
-        if (s != HRS_SUCCESS || err != cudaSuccess || !g) {
-            if (g) cudaGraphDestroy(g);
-            cudaGetLastError();
+        bool done = false;
+        for (int attempt = cond_graphs_enabled() ? 0 : 1; attempt < 2 && !done; ++attempt) {
+            if (cudaStreamBeginCapture(cs, cudaStreamCaptureModeThreadLocal) != cudaSuccess) return false;
+            GraphCtx &gc = g_gctx[dev];
+            gc.depth = 0;
+            gc.ok = true;
+            g_gx = attempt == 0 ? &gc : nullptr;
+            g_launches = l0;
+            const hrs_status s = run(cs);
+            g_gx = nullptr;
+            cudaGraph_t g = nullptr;
+            err = cudaStreamEndCapture(cs, &g);
+            if (s != HRS_SUCCESS || err != cudaSuccess || !g || !gc.ok) {
+                if (g) cudaGraphDestroy(g);
+                cudaGetLastError();
+                continue;
+            }
+            err = cudaGraphInstantiate(&e.exec, g, 0);
+            cudaGraphDestroy(g);
+            if (err != cudaSuccess) {
+                e.exec = nullptr;
+                cudaGetLastError();
+                continue;
+            }
+            done = true;
+        }
+        if (!done) {
+            g_launches = l0;
             return false;  // run directly instead
         }
-        err = cudaGraphInstantiate(&e.exec, g, 0);
-        cudaGraphDestroy(g);
-        if (err != cudaSuccess) {
-            e.exec = nullptr;
-            cudaGetLastError();
-            return false;
-        }
-        e.launches = g_launches - l0;
-        g_launches = l0;  // counted when the graph runs
+        e.launches = g_launches - l0;  // (launches captured, including the conditional ones)
+        g_launches = l0;               // counted when the graph runs
     }
     const cudaError_t err = cudaGraphLaunch(e.exec, stream);
     if (err != cudaSuccess) {

@@ -756,6 +756,26 @@ __global__ void __launch_bounds__(256) k_copy_pieces(const T *__restrict__ src, 
     }
 }
 
+// Sets the values of conditional graph nodes from the control block (small sorts replayed as
+// a CUDA graph): what[i] = c < 8: local class list c is non-empty; 8: the counting local
+// sort's hand-off list; 16 + c: the wide list of configuration c.
+constexpr int MAX_CONDS = 16;
+struct CondSet {
+    cudaGraphConditionalHandle h[MAX_CONDS];
+    uint32_t what[MAX_CONDS];
+    int n;
+    const Ctl *ctl;
+};
+static __global__ void k_set_conds(const __grid_constant__ CondSet cs) {
+    pdl_wait();
+    const int i = threadIdx.x;
+    if (i < cs.n) {
+        const uint32_t w = cs.what[i];
+        const uint32_t v = w < 8 ? cs.ctl->nlocal[w] : (w == 8 ? cs.ctl->nlocal_fb2 : cs.ctl->nlocal_wide[w - 16]);
+        cudaGraphSetConditional(cs.h[i], v != 0u ? 1u : 0u);
+    }
+}
+
 static __global__ void k_fill_u64(uint64_t *p, uint64_t n, uint64_t v) {
     for (uint64_t i = static_cast<uint64_t>(blockIdx.x) * blockDim.x + threadIdx.x; i < n;
          i += static_cast<uint64_t>(gridDim.x) * blockDim.x)
@@ -1288,6 +1308,10 @@ struct ScatterParams {
     int force_redo;  // HRS_FLAG_FORCE_REDO: every stability check fails (tests of the redo path)
     int kind;        // hrs_key_kind: the bijection on the way out of the input, its inverse
     int final_pass;  //   on the way into the final output (the last pass)
+    // small sorts replayed as a CUDA graph: the next pass is a conditional node whose value
+    // this scatter sets (the next pass has buckets), so empty passes cost nothing
+    cudaGraphConditionalHandle next_cond;
+    int has_next_cond;
 };
 
 struct StageInfo {
@@ -1370,6 +1394,8 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
     const int tid = threadIdx.x, lane = tid & 31, warp = tid >> 5;
     const uint32_t wbase = static_cast<uint32_t>(warp) * 32 * KPT;
     const uint32_t T = alloc_tiles(prm.ctl->alloc[prm.p]);
+    if (prm.has_next_cond && blockIdx.x == 0 && threadIdx.x == 0)  // (k_classify of this pass has completed)
+        cudaGraphSetConditional(prm.next_cond, alloc_buckets(prm.ctl->alloc[prm.p + 1]) != 0u ? 1u : 0u);
     if (blockIdx.x >= T) return;
     const uint64_t pol = policy_evict_first();
     uint32_t *const ca = cnt + warp * RADIX;  // this warp's counters

@@ -286,6 +286,67 @@ inline hrs_status last_launch() {
     return HRS_SUCCESS;
 }
 
+// ------------------------------------------------------------------ conditional graph capture (small sorts)
+//
+// While a small sort's launch sequence is captured into a CUDA graph (hrs.cu, via_graph),
+// g_gx points at this context: every pass after the first becomes a conditional IF node
+// (nested: pass p + 1 inside pass p) whose value the previous pass's scatter sets, and the
+// local-sort launches IF nodes whose values one small kernel sets from the list counts.
+// A replay then runs only the launches that have work (constant launches per
+// pass -- but a pass with no bucket needs none).  Any API failure abandons the capture (the
+// caller falls back to a plain capture).
+struct GraphCtx {
+    std::vector<cudaStream_t> pool;  // capture streams of the nested bodies
+    size_t depth = 0;
+    bool ok = true;
+    bool graph_of(cudaStream_t st, cudaGraph_t *g, const cudaGraphNode_t **deps, size_t *nd) {
+        cudaStreamCaptureStatus cs = cudaStreamCaptureStatusNone;
+        if (cudaStreamGetCaptureInfo(st, &cs, nullptr, g, deps, nd) != cudaSuccess ||
+            cs != cudaStreamCaptureStatusActive)
+            return ok = false;
+        return true;
+    }
+    bool handle(cudaStream_t st, cudaGraphConditionalHandle *h) {
+        cudaGraph_t g;
+        const cudaGraphNode_t *deps;
+        size_t nd;
+        if (!graph_of(st, &g, &deps, &nd)) return false;
+        if (cudaGraphConditionalHandleCreate(h, g, 0, cudaGraphCondAssignDefault) != cudaSuccess) return ok = false;
+        return true;
+    }
+    // IF(h) after the work captured so far on st; returns the stream capturing its body
+    cudaStream_t if_begin(cudaStream_t st, cudaGraphConditionalHandle h) {
+        cudaGraph_t g;
+        const cudaGraphNode_t *deps;
+        size_t nd;
+        if (!graph_of(st, &g, &deps, &nd)) return nullptr;
+        cudaGraphNodeParams np = {cudaGraphNodeTypeConditional};
+        np.conditional.handle = h;
+        np.conditional.type = cudaGraphCondTypeIf;
+        np.conditional.size = 1;
+        cudaGraphNode_t node;
+        if (cudaGraphAddNode(&node, g, deps, nd, &np) != cudaSuccess) return ok = false, nullptr;
+        if (cudaStreamUpdateCaptureDependencies(st, &node, 1, cudaStreamSetCaptureDependencies) != cudaSuccess)
+            return ok = false, nullptr;
+        if (depth == pool.size()) {
+            cudaStream_t ns = nullptr;
+            if (cudaStreamCreateWithFlags(&ns, cudaStreamNonBlocking) != cudaSuccess) return ok = false, nullptr;
+            pool.push_back(ns);
+        }
+        cudaStream_t bs = pool[depth++];
+        if (cudaStreamBeginCaptureToGraph(bs, np.conditional.phGraph_out[0], nullptr, nullptr, 0,
+                                          cudaStreamCaptureModeThreadLocal) != cudaSuccess)
+            return ok = false, nullptr;
+        return bs;
+    }
+    void if_end(cudaStream_t bs) {
+        cudaGraph_t g = nullptr;
+        if (cudaStreamEndCapture(bs, &g) != cudaSuccess) ok = false;
+        --depth;
+    }
+};
+extern thread_local GraphCtx *g_gx;
+
 // ------------------------------------------------------------------ plan + temp layout
 
 enum Mode { MODE_SORT = 0, MODE_HIST = 1, MODE_PARTITION = 2 };
@@ -586,8 +647,13 @@ struct Runner {
     }
 
     static hrs_status scatter(const Plan &pl, void *temp, cudaStream_t st, int dev, int sms, int p, const Bufs &bf,
-                              void *kout, void *vout, uint32_t G) {
+                              void *kout, void *vout, uint32_t G, const cudaGraphConditionalHandle *next = nullptr) {
         ScatterParams sp;
+        std::memset(&sp, 0, sizeof(sp));
+        if (next) {
+            sp.next_cond = *next;
+            sp.has_next_cond = 1;
+        }
         sp.n = pl.n;
         for (int i = 0; i < 3; ++i) {
             sp.src_keys[i] = bf.k[i];
@@ -737,41 +803,83 @@ struct Runner {
         return local_variant<C, 0>(pl, temp, st, dev, sms, kin, kout, vin, vout);
     }
 
+    // launch(i, stream) for every i: directly, or -- under a conditional graph capture --
+    // each inside IF(the list `what[i]` is non-empty), one k_set_conds in front
+    template <typename F>
+    static hrs_status cond_group(cudaStream_t st, void *temp, const int *what, int n, F &&launch) {
+        GraphCtx *gx = g_gx;
+        if (!gx) {
+            for (int i = 0; i < n; ++i) {
+                const hrs_status s = launch(i, st);
+                if (s) return s;
+            }
+            return HRS_SUCCESS;
+        }
+        for (int i0 = 0; i0 < n; i0 += MAX_CONDS) {
+            const int m = std::min(n - i0, MAX_CONDS);
+            CondSet cs;
+            std::memset(&cs, 0, sizeof(cs));
+            cs.n = m;
+            cs.ctl = at<Ctl>(temp, 0);
+            for (int i = 0; i < m; ++i) {
+                if (!gx->handle(st, &cs.h[i])) return HRS_ERROR_CUDA;
+                cs.what[i] = static_cast<uint32_t>(what[i0 + i]);
+            }
+            {
+                LaunchScope ls(st, 4, 0);
+                launch_pdl(k_set_conds, dim3(1), dim3(32), 0, st, cs);
+            }
+            hrs_status s = last_launch();
+            if (s) return s;
+            for (int i = 0; i < m; ++i) {
+                cudaStream_t bs = gx->if_begin(st, cs.h[i]);
+                if (!bs) return HRS_ERROR_CUDA;
+                s = launch(i0 + i, bs);
+                gx->if_end(bs);
+                if (s) return s;
+                if (!gx->ok) return HRS_ERROR_CUDA;
+            }
+        }
+        return HRS_SUCCESS;
+    }
+
+    static hrs_status wide_one(int c, const Plan &pl, void *temp, cudaStream_t st, int dev, int sms, const void *kin,
+                               void *kout, const void *vin, void *vout) {
+        switch (c) {
+            case 0: return local_variant<0, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout, LIST_FB);
+            case 1: return local_variant<1, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout, LIST_FB);
+            case 2: return local_variant<2, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout, LIST_FB);
+            case 3: return local_variant<3, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout, LIST_FB);
+            case 4: return local_variant<4, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout, LIST_FB);
+            case 5: return local_variant<5, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout, LIST_FB);
+            case 6: return local_variant<6, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout, LIST_FB);
+            case 7: return local_variant<7, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout, LIST_FB);
+        }
+        return HRS_ERROR_INVALID_VALUE;
+    }
+
     // the wide launches for whatever the narrow ones handed over, one per wide
     // configuration (wide_cfg: 1024, 2048, [4096, 4608 for 64-bit keys,] largest); only needed when more than 19 bits
     // can remain to sort
     static hrs_status local_wide(const Plan &pl, void *temp, cudaStream_t st, int dev, int sms, const void *kin,
                                  void *kout, const void *vin, void *vout) {
         if (pl.end - pl.begin <= 19) return HRS_SUCCESS;  // every entry fits a narrow composite
-        hrs_status s;
+        int cfg[8], n = 0;
         if (pl.single_class >= 0) {
-            switch (pl.single_class) {
-                case 0: return local_variant<0, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout, LIST_FB);
-                case 1: return local_variant<1, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout, LIST_FB);
-                case 2: return local_variant<2, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout, LIST_FB);
-                case 3: return local_variant<3, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout, LIST_FB);
-                case 4: return local_variant<4, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout, LIST_FB);
-                case 5: return local_variant<5, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout, LIST_FB);
-                case 6: return local_variant<6, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout, LIST_FB);
-                case 7: return local_variant<7, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout, LIST_FB);
-            }
-            return HRS_ERROR_INVALID_VALUE;
+            cfg[n++] = pl.single_class;
+        } else {
+            const int cmax = size_class_of(pl.lt);
+            cfg[n++] = 3;
+            if (cmax >= 4) cfg[n++] = 4;
+            if (HRS_WIDE_MID && KB == 8 && cmax >= 5 && max_class_t<K, V>() > 5) cfg[n++] = 5;
+            if (HRS_WIDE_MID && KB == 8 && cmax >= 6 && max_class_t<K, V>() > 6) cfg[n++] = 6;
+            if (cmax >= 5) cfg[n++] = max_class_t<K, V>() == 7 ? 7 : 6;
         }
-        const int cmax = size_class_of(pl.lt);
-        if ((s = local_variant<3, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout, LIST_FB))) return s;
-        if (cmax >= 4 && (s = local_variant<4, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout, LIST_FB))) return s;
-        if (HRS_WIDE_MID && KB == 8 && cmax >= 5 && max_class_t<K, V>() > 5 &&
-            (s = local_variant<5, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout, LIST_FB)))
-            return s;
-        if (HRS_WIDE_MID && KB == 8 && cmax >= 6 && max_class_t<K, V>() > 6 &&
-            (s = local_variant<6, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout, LIST_FB)))
-            return s;
-        if (cmax >= 5) {
-            if (max_class_t<K, V>() == 7)
-                return local_variant<7, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout, LIST_FB);
-            return local_variant<6, 1>(pl, temp, st, dev, sms, kin, kout, vin, vout, LIST_FB);
-        }
-        return HRS_SUCCESS;
+        int what[8];
+        for (int i = 0; i < n; ++i) what[i] = 16 + cfg[i];
+        return cond_group(st, temp, what, n, [&](int i, cudaStream_t s2) {
+            return wide_one(cfg[i], pl, temp, s2, dev, sms, kin, kout, vin, vout);
+        });
     }
 
     // the narrow k_local over the entries the counting variant handed over (sizes up to
@@ -834,6 +942,10 @@ struct Runner {
             uint32_t G = 0;
             if ((s = range_grid(pl, dev, sms, &G))) return s;
             const Bufs bf = bufs(pl, temp, kin, kout, vin, vout);
+            GraphCtx *gx = g_gx;
+            cudaStream_t cur = st;  // (inside the nested conditional bodies under graph capture)
+            cudaStream_t opened[HRS_MAX_PASSES + 1];
+            int nopen = 0;
             for (int p = 1; p <= pl.D; ++p) {
                 const bool to_out = ((pl.D - p) % 2) == 0;
                 void *yk = to_out ? kout : auxk;
@@ -841,22 +953,42 @@ struct Runner {
                 if (p == 1 && grouped) {
                     // the partition on digit 1 is given: classify its histogram (no per-CTA
                     // ranges), the sub-buckets stay in the input (X_1 = in)
-                    if ((s = classify(pl, temp, st, dev, sms, 1, SRC_IN, nullptr, nullptr, false, 0))) return s;
+                    if ((s = classify(pl, temp, cur, dev, sms, 1, SRC_IN, nullptr, nullptr, false, 0))) return s;
                     continue;
                 }
-                if ((s = hist(pl, temp, st, dev, sms, p, bf, G))) return s;
-                if ((s = classify(pl, temp, st, dev, sms, p, to_out ? SRC_OUT : SRC_AUX, nullptr, nullptr,
+                if ((s = hist(pl, temp, cur, dev, sms, p, bf, G))) return s;
+                if ((s = classify(pl, temp, cur, dev, sms, p, to_out ? SRC_OUT : SRC_AUX, nullptr, nullptr,
                                   p == pl.D, G)))
                     return s;
-                if ((s = scatter(pl, temp, st, dev, sms, p, bf, yk, yv, G))) return s;
+                cudaGraphConditionalHandle hn;
+                const bool cond = gx && p < pl.D;
+                if (cond && !gx->handle(cur, &hn)) return HRS_ERROR_CUDA;
+                if ((s = scatter(pl, temp, cur, dev, sms, p, bf, yk, yv, G, cond ? &hn : nullptr))) return s;
+                if (cond) {  // pass p + 1 runs iff it has buckets
+                    cur = gx->if_begin(cur, hn);
+                    if (!cur) return HRS_ERROR_CUDA;
+                    opened[nopen++] = cur;
+                }
             }
+            while (nopen > 0) gx->if_end(opened[--nopen]);
+            if (gx && !gx->ok) return HRS_ERROR_CUDA;
             const int cmax = pl.single_class >= 0 ? pl.single_class : size_class_of(pl.lt);
+            const int c0 = pl.single_class >= 0 ? pl.single_class : 0;
+            int what[HRS_NUM_CLASSES];
             bool cnt = false;
-            for (int c = (pl.single_class >= 0 ? pl.single_class : 0); c <= cmax; ++c) {
-                if ((s = local(pl, temp, st, dev, sms, c, kin, kout, vin, vout))) return s;
+            for (int c = c0; c <= cmax; ++c) {
+                what[c - c0] = c;
                 cnt = cnt || (pl.single_class < 0 && cnt_ok(c));
             }
-            if (cnt && (s = local_fb2(pl, temp, st, dev, sms, kin, kout, vin, vout))) return s;
+            if ((s = cond_group(st, temp, what, cmax - c0 + 1, [&](int i, cudaStream_t s2) {
+                     return local(pl, temp, s2, dev, sms, c0 + i, kin, kout, vin, vout);
+                 })))
+                return s;
+            const int w8 = 8;
+            if (cnt && (s = cond_group(st, temp, &w8, 1, [&](int, cudaStream_t s2) {
+                            return local_fb2(pl, temp, s2, dev, sms, kin, kout, vin, vout);
+                        })))
+                return s;
         } else {
             if ((s = local(pl, temp, st, dev, sms, root_class, kin, kout, vin, vout))) return s;
             if (pl.single_class < 0 && cnt_ok(root_class) &&
