@@ -511,3 +511,28 @@ def test_sort_records(kb, vb, key_first):
             _, order = oracle.sort_typed(keys.view(tdt[(kind, kb)]), idx, kind)
         exp = raw[order.astype(np.int64)]
         assert np.array_equal(out.cpu().numpy(), exp), (kind, b, e)
+
+
+def test_conditional_graph_replays():
+    """Small sorts replay a captured CUDA graph whose later passes and local-sort launches are
+    conditional nodes set on the device: replays of inputs with different structure (one
+    pass + local sorts, all passes for constant keys, deep AND-4 recursion with merging and
+    hand-offs, tiny thresholds) through the same cached graph must all match the oracle."""
+    import paper_1611_01137_b200 as hrs
+    for n, kbits, vbits, tun in ((1 << 20, 32, 0, None), (200003, 64, 64, None), (150001, 32, 32,
+                                 dict(local_threshold=300, merge_threshold=100, keys_per_tile=128))):
+        kd = torch.empty(n, dtype=torch.uint32 if kbits == 32 else torch.uint64, device=DEV)
+        vd = torch.empty(n, dtype=torch.uint32 if vbits == 32 else torch.uint64, device=DEV) if vbits else None
+        ko, vo = torch.empty_like(kd), (torch.empty_like(vd) if vbits else None)
+        temp = torch.empty(hrs.temp_bytes(n, kbits // 8, vbits // 8, 0, kbits, tun), dtype=torch.uint8, device=DEV)
+        for i, dist in enumerate(("uniform", "uniform", "const", "and4", "uniform", "and2", "const", "and3")):
+            k, v = _inputs(n, kbits, vbits, dist, seed=200 + i)
+            kd.copy_(k.to(DEV))
+            if vbits:
+                vd.copy_(v.to(DEV))
+            hrs.sort(kd, vd, keys_out=ko, values_out=vo, temp=temp, tuning=tun)
+            torch.cuda.synchronize()
+            ek, ev = oracle.sort(k, v, 0, kbits)
+            assert np.array_equal(_np(ko), ek), (n, dist, i)
+            if vbits:
+                assert np.array_equal(_np(vo), ev), (n, dist, i)
