@@ -2,6 +2,8 @@
 
 All integer work, so the bar is bit-exact keys and values (BJ north_star).  Inputs are
 seeded synthetic workloads from gen/ (uniform and AND-m skew)."""
+import os
+
 import numpy as np
 import pytest
 import torch
@@ -11,6 +13,7 @@ import oracle
 from oracle import plan
 
 pytestmark = pytest.mark.gpu
+ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
 
 DEV = "cuda:0"
 TYPES = [(32, 0), (32, 32), (32, 64), (64, 0), (64, 32), (64, 64)]
@@ -514,6 +517,17 @@ def test_sort_records(kb, vb, key_first):
 
 
 def test_conditional_graph_replays():
+    """(run in a fresh process with HRS_GRAPH_COND=1: conditional capture is opt-in)"""
+    import subprocess
+    import sys
+    code = ("import sys; sys.path.insert(0, 'tests'); import test_gpu_sort as t; "
+            "t._conditional_graph_replays()")
+    env = dict(os.environ, HRS_GRAPH_COND="1", PYTHONPATH=ROOT)
+    r = subprocess.run([sys.executable, "-c", code], cwd=ROOT, env=env, capture_output=True, text=True, timeout=600)
+    assert r.returncode == 0, r.stdout[-2000:] + r.stderr[-4000:]
+
+
+def _conditional_graph_replays():
     """Small sorts replay a captured CUDA graph whose later passes and local-sort launches are
     conditional nodes set on the device: replays of inputs with different structure (one
     pass + local sorts, all passes for constant keys, deep AND-4 recursion with merging and
