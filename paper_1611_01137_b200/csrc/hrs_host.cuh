@@ -132,18 +132,27 @@ template <> struct LocalCfg<7> { static constexpr int THREADS = 512, KPT = 16; }
 // two-stage TMA prefetch when three CTAs still fit per SM, else one stage; the
 // register cap (launch bounds) is set for the occupancy the shared memory allows
 template <typename K, typename V, int C, int WIDE = 0>
+#ifndef HRS_WIDE_NSTAGE
+#define HRS_WIDE_NSTAGE 1  // wide local sort of 8-byte keys: one staging buffer (measured, c4 AND-2 wide class 4: 5.61 -> 5.16 ms)
+#endif
+#ifndef HRS_WIDE_OCC
+#define HRS_WIDE_OCC 6  // ... registers for six CTAs per SM (96, no spill) instead of three (167)
+#endif
 struct LocalStages {
     using LC = LocalCfg<C>;
     static constexpr size_t SM_BUDGET = 228 * 1024;  // shared memory per SM; 1 KB reserved per CTA
+    static constexpr bool W64 = WIDE == 1 && sizeof(K) == 8;
     static constexpr int NSTAGE =
-        3 * (LocalSmem<K, V, LC::THREADS, LC::KPT, 2, WIDE>::bytes + 1024) <= SM_BUDGET ? 2 : 1;
+        (W64 && HRS_WIDE_NSTAGE) ? HRS_WIDE_NSTAGE
+        : (3 * (LocalSmem<K, V, LC::THREADS, LC::KPT, 2, WIDE>::bytes + 1024) <= SM_BUDGET ? 2 : 1);
     static constexpr size_t bytes = LocalSmem<K, V, LC::THREADS, LC::KPT, NSTAGE, WIDE>::bytes;
     static constexpr bool fits = bytes <= SMEM_LIMIT && LocalSmem<K, V, LC::THREADS, LC::KPT, 1, 1>::bytes <= SMEM_LIMIT &&
                                  LocalSmem<K, V, LC::THREADS, LC::KPT, 1, 0>::bytes <= SMEM_LIMIT;
     static constexpr int by_smem = static_cast<int>(SM_BUDGET / (bytes + 1024));
     static constexpr int by_threads = 2048 / LC::THREADS;
     static constexpr int OCC0 = by_smem < by_threads ? by_smem : by_threads;
-    static constexpr int OCC = OCC0 < 1 ? 1 : (OCC0 > 4 ? 4 : OCC0);
+    static constexpr int OCC_CAP = W64 ? HRS_WIDE_OCC : 4;
+    static constexpr int OCC = OCC0 < 1 ? 1 : (OCC0 > OCC_CAP ? OCC_CAP : OCC0);
 };
 
 // counting local sort (k_local_cnt) for the large classes: 2^15 counted values for 8-byte
