@@ -233,6 +233,22 @@ hrs_status hrs_partition_pass(void *d_temp, size_t *temp_bytes, const void *keys
                               const void *vals_in, void *vals_out, uint64_t n, int key_bytes, int value_bytes,
                               int lo_bit, int hi_bit, uint64_t *d_offsets, hrs_stream_t stream);
 
+/* The same stable counting pass, with every digit's run written to its own window: the
+ * records of digit d go, in input order, to key window w = dst_offsets[d] >> 48 at element
+ * offset dst_offsets[d] & (2^48 - 1) (values likewise, to value window w).  dst_offsets,
+ * key_windows and value_windows are HOST arrays (2^(hi-lo) offsets; nwindows <= 64 device
+ * addresses each, naturally aligned), copied into d_temp during the call (the call
+ * synchronises `stream` once for that copy).  A window may be another GPU's memory mapped
+ * into this process (CUDA IPC / symmetric memory over NVLink): this is the fused exchange of
+ * the partition scatter stores every bucket run straight into the
+ * receiving GPU's buffer, with no local partition buffer and no separate all-to-all.  The
+ * runs must not overlap each other or the input; the caller synchronises with the
+ * receivers.  Temp size: two-phase query as usual (larger than hrs_partition_pass's). */
+hrs_status hrs_partition_pass_to(void *d_temp, size_t *temp_bytes, const void *keys_in, const void *vals_in,
+                                 uint64_t n, int key_bytes, int value_bytes, int lo_bit, int hi_bit,
+                                 const uint64_t *dst_offsets, int nwindows, const uint64_t *key_windows,
+                                 const uint64_t *value_windows, hrs_stream_t stream);
+
 /* Copies npieces pieces of elem_bytes-wide elements (4 or 8) from src to dst (device):
  * `pieces` is a HOST array of npieces x {src_offset, dst_offset, count} uint64, in
  * elements, read during the call (it travels in kernel parameters, 256 pieces per

@@ -324,6 +324,41 @@ def copy_pieces(dst: torch.Tensor, src: torch.Tensor, pieces, stream=None) -> No
               "hrs_copy_pieces")
 
 
+def partition_pass_to(keys: torch.Tensor, values: torch.Tensor | None, lo_bit: int, hi_bit: int, dst_offsets,
+                      key_windows, value_windows=None, *, temp: torch.Tensor | None = None, stream=None) -> None:
+    """hrs_partition_pass_to: one stable counting pass on digit bits [lo_bit, hi_bit) whose
+    digit-d records go to key_windows[w][o : o + count_d] (values likewise), with
+    (w, o) = (dst_offsets[d] >> 48, dst_offsets[d] & (2^48 - 1)).  Windows are tensors
+    (or raw device addresses, e.g. another GPU's buffer mapped over NVLink)."""
+    _check_tensor(keys, "keys")
+    kb = _nbytes(keys, "keys")
+    vb = 0
+    if values is not None:
+        _check_tensor(values, "values")
+        vb = _nbytes(values, "values")
+    n = keys.numel()
+    addr = lambda t: int(t) if isinstance(t, int) else t.data_ptr()  # noqa: E731
+    kw = [addr(t) for t in key_windows]
+    vw = [addr(t) for t in value_windows] if values is not None else [0] * len(kw)
+    offs = [int(x) for x in dst_offsets]
+    sz = ctypes.c_size_t(0)
+    check(lib.hrs_partition_pass_to(None, ctypes.byref(sz), None, None, n, kb, vb, lo_bit, hi_bit, None, 0, None,
+                                    None, None), "hrs_partition_pass_to(size query)")
+    if temp is None or temp.numel() < sz.value:
+        temp = alloc_temp(sz.value, keys.device)
+    _on_stream(stream, temp)
+    U = ctypes.c_uint64
+    to = (U * len(offs))(*offs)
+    tk = (U * len(kw))(*kw)
+    tv = (U * len(vw))(*vw)
+    sz = ctypes.c_size_t(temp.numel())
+    with torch.cuda.device(keys.device):
+        check(lib.hrs_partition_pass_to(_ptr(temp), ctypes.byref(sz), _ptr(keys), _ptr(values), n, kb, vb, lo_bit,
+                                        hi_bit, ctypes.cast(to, ctypes.c_void_p), len(kw),
+                                        ctypes.cast(tk, ctypes.c_void_p), ctypes.cast(tv, ctypes.c_void_p),
+                                        _stream(stream)), "hrs_partition_pass_to")
+
+
 def default_tuning(key_bytes: int, value_bytes: int) -> dict:
     t = Tuning()
     check(lib.hrs_default_tuning(key_bytes, value_bytes, ctypes.byref(t)), "hrs_default_tuning")

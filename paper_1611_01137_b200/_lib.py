@@ -119,6 +119,7 @@ SIGNATURES = {
     "hrs_digit_histogram": (_ST, [_P, _SZP, _P, _U64, _I, _I, _I, _P, _P]),
     "hrs_partition_pass": (_ST, [_P, _SZP, _P, _P, _P, _P, _U64, _I, _I, _I, _I, _P, _P]),
     "hrs_copy_pieces": (_ST, [_P, _P, _I, _P, _U64, _P]),
+    "hrs_partition_pass_to": (_ST, [_P, _SZP, _P, _P, _U64, _I, _I, _I, _I, _P, _I, _P, _P, _P]),
     "hrs_profile_enable": (None, [_I]),
     "hrs_profile_collect": (_I, [ctypes.POINTER(ProfileRecord), _I]),
     "hrs_launch_count": (ctypes.c_uint64, []),

@@ -457,9 +457,16 @@ hrs_status hrs_default_tuning(int key_bytes, int value_bytes, hrs_tuning *out) {
 
 uint32_t hrs_class_capacity(int c) { return (c >= 0 && c < HRS_NUM_CLASSES) ? class_capacity(c) : 0u; }
 
+struct DstArgs {
+    const uint64_t *offsets;  // host, 2^(hi-lo)
+    int nwin;
+    const uint64_t *kwin, *vwin;  // host, nwin device addresses
+};
+
 static hrs_status block_common(void *d_temp, size_t *temp_bytes, const void *keys_in, void *keys_out,
                                const void *vals_in, void *vals_out, uint64_t n, int kb, int vb, int lo, int hi,
-                               uint64_t *h, uint64_t *o, bool scatter, hrs_stream_t stream) {
+                               uint64_t *h, uint64_t *o, bool scatter, hrs_stream_t stream,
+                               const DstArgs *dst = nullptr) {
     if (!temp_bytes) return HRS_ERROR_INVALID_VALUE;
     if (kb != 4 && kb != 8) return HRS_ERROR_INVALID_VALUE;
     if (vb != 0 && vb != 4 && vb != 8) return HRS_ERROR_INVALID_VALUE;
@@ -478,9 +485,9 @@ static hrs_status block_common(void *d_temp, size_t *temp_bytes, const void *key
     if (!aligned(d_temp, 256)) return HRS_ERROR_INVALID_VALUE;
     if (!scatter && !h) return HRS_ERROR_INVALID_VALUE;
     if (n > 0) {
-        if (!keys_in || (scatter && !keys_out)) return HRS_ERROR_INVALID_VALUE;
-        if (scatter && vb && (!vals_in || !vals_out)) return HRS_ERROR_INVALID_VALUE;
-        if (!aligned(keys_in, kb) || (scatter && !aligned(keys_out, kb))) return HRS_ERROR_INVALID_VALUE;
+        if (!keys_in || (scatter && !dst && !keys_out)) return HRS_ERROR_INVALID_VALUE;
+        if (scatter && !dst && vb && (!vals_in || !vals_out)) return HRS_ERROR_INVALID_VALUE;
+        if (!aligned(keys_in, kb) || (scatter && !dst && !aligned(keys_out, kb))) return HRS_ERROR_INVALID_VALUE;
         const size_t nk = n * kb, nv = n * vb;
         const void *bufs[5] = {keys_in, scatter ? keys_out : nullptr, vb ? vals_in : nullptr,
                                vb ? vals_out : nullptr, d_temp};
@@ -491,6 +498,30 @@ static hrs_status block_common(void *d_temp, size_t *temp_bytes, const void *key
     }
     int dev = 0, sms = 0;
     if ((s = check_device(&dev, &sms))) return s;
+    if (dst) {
+        // the window tables into temp (pageable host memory: the copy is staged before the call returns)
+        if (!dst->offsets || dst->nwin < 1 || dst->nwin > MAX_WINDOWS || !dst->kwin || (vb && !dst->vwin))
+            return HRS_ERROR_INVALID_VALUE;
+        const int r = 1 << (hi - lo);
+        std::vector<uint64_t> tab(RADIX + 2 * MAX_WINDOWS, 0);
+        for (int d = 0; d < r; ++d) {
+            if ((dst->offsets[d] >> 48) >= static_cast<uint64_t>(dst->nwin)) return HRS_ERROR_INVALID_VALUE;
+            tab[d] = dst->offsets[d];
+        }
+        for (int w = 0; w < dst->nwin; ++w) {
+            if (!dst->kwin[w] || (dst->kwin[w] % kb) || (vb && (!dst->vwin[w] || dst->vwin[w] % vb)))
+                return HRS_ERROR_INVALID_VALUE;
+            tab[RADIX + w] = dst->kwin[w];
+            tab[RADIX + MAX_WINDOWS + w] = vb ? dst->vwin[w] : 0;
+        }
+        cudaStream_t st = reinterpret_cast<cudaStream_t>(stream);
+        cudaError_t e = cudaMemcpyAsync(static_cast<unsigned char *>(d_temp) + pl.off_dst, tab.data(),
+                                        sizeof(uint64_t) * tab.size(), cudaMemcpyHostToDevice, st);
+        if (e != cudaSuccess) return cuda_fail(e);
+        e = cudaStreamSynchronize(st);  // (tab is a local: the copy must be done before it goes)
+        if (e != cudaSuccess) return cuda_fail(e);
+        pl.dst = true;
+    }
     return block_dispatch(kb, vb, pl, d_temp, keys_in, keys_out, vals_in, vals_out, h, o, scatter,
                           reinterpret_cast<cudaStream_t>(stream), dev, sms);
 }
@@ -499,6 +530,15 @@ hrs_status hrs_digit_histogram(void *d_temp, size_t *temp_bytes, const void *key
                                int lo_bit, int hi_bit, uint64_t *d_hist, hrs_stream_t stream) {
     return block_common(d_temp, temp_bytes, keys, nullptr, nullptr, nullptr, n, key_bytes, 0, lo_bit, hi_bit,
                         d_hist, nullptr, false, stream);
+}
+
+hrs_status hrs_partition_pass_to(void *d_temp, size_t *temp_bytes, const void *keys_in, const void *vals_in,
+                                 uint64_t n, int key_bytes, int value_bytes, int lo_bit, int hi_bit,
+                                 const uint64_t *dst_offsets, int nwindows, const uint64_t *key_windows,
+                                 const uint64_t *value_windows, hrs_stream_t stream) {
+    DstArgs da{dst_offsets, nwindows, key_windows, value_windows};
+    return block_common(d_temp, temp_bytes, keys_in, nullptr, vals_in, nullptr, n, key_bytes, value_bytes, lo_bit,
+                        hi_bit, nullptr, nullptr, true, stream, d_temp ? &da : nullptr);
 }
 
 hrs_status hrs_partition_pass(void *d_temp, size_t *temp_bytes, const void *keys_in, void *keys_out,

@@ -1312,7 +1312,15 @@ struct ScatterParams {
     // this scatter sets (the next pass has buckets), so empty passes cost nothing
     cudaGraphConditionalHandle next_cond;
     int has_next_cond;
+    // DST instantiation (hrs_partition_pass_to, the fused exchange of SURVEY §8(f) N2): digit
+    // d's run goes to window w = dst_off[d] >> 48 at element offset dst_off[d] & (2^48 - 1);
+    // window w is the device address of a key (value) array, possibly another GPU's memory
+    // mapped over NVLink
+    const unsigned long long *dst_off;    // [2^width]
+    const unsigned long long *dst_kwin;   // [windows]
+    const unsigned long long *dst_vwin;   // [windows]
 };
+constexpr unsigned long long DST_OFF_MASK = (1ull << 48) - 1;
 
 struct StageInfo {
     uint32_t valid, count, bucket, carry_row, kpad, k0, k1, vpad, v0, v1, tile, src;
@@ -1324,7 +1332,7 @@ struct StageInfo {
 // starts; the sorted tile is built IN PLACE in the key staging buffer (the keys are held
 // in registers from the count on) plus a 16-bit slot -> element index (sidx) through which
 // the values are gathered and the stability of the fast rank is checked.
-template <typename K, typename V, int THREADS, int KPT, int NBUF>
+template <typename K, typename V, int THREADS, int KPT, int NBUF, bool DST = false>
 struct ScatterSmem {
     static constexpr int W = THREADS / 32;
     static constexpr int KPB = THREADS * KPT;
@@ -1337,7 +1345,8 @@ struct ScatterSmem {
     static constexpr size_t off_cnt = align16(off_info + NBUF * sizeof(StageInfo));
     static constexpr size_t off_wsum = align16(off_cnt + sizeof(uint32_t) * W * RADIX);
     static constexpr size_t off_gs = align16(off_wsum + sizeof(uint32_t) * 16);
-    static constexpr size_t off_sidx = align16(off_gs + sizeof(uint2) * RADIX);
+    static constexpr size_t off_start = align16(off_gs + sizeof(uint2) * RADIX);  // DST: digit starts
+    static constexpr size_t off_sidx = align16(off_start + (DST ? sizeof(uint32_t) * RADIX : 0));
     static constexpr size_t off_kst = align16(off_sidx + sizeof(uint16_t) * KPB);
     static constexpr size_t kst_bytes = align16(sizeof(K) * kst_elems);
     static constexpr size_t off_vst = off_kst + NBUF * kst_bytes;
@@ -1366,13 +1375,13 @@ struct ScatterSmem {
 // its bucket) comes from k_hist / k_classify, so tiles are independent (no
 // look-back) and claimed in order from a counter: the tiles in flight write neighbouring
 // runs of every sub-bucket, which combine in L2.
-template <typename K, typename V, int THREADS, int KPT, int MINB, int NBUF, bool TY>
+template <typename K, typename V, int THREADS, int KPT, int MINB, int NBUF, bool TY, bool DST = false>
 __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
     pdl_wait();
     static_assert(NBUF == 1 || NBUF == 2, "one or two staging buffers");
     static_assert(THREADS % RADIX == 0 && THREADS <= 4 * RADIX, "threads 0..255 fold one digit each");
     static_assert(32 * KPT < (1 << 16), "the in-warp rank is packed above the digit");
-    using L = ScatterSmem<K, V, THREADS, KPT, NBUF>;
+    using L = ScatterSmem<K, V, THREADS, KPT, NBUF, DST>;
     constexpr int W = THREADS / 32;
     constexpr bool HV = HasVal<V>::value;
     using VT = ValT<V>;
@@ -1383,6 +1392,8 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
     uint32_t *wsum = reinterpret_cast<uint32_t *>(smem + L::off_wsum);  // [W] digit-total partial sums
     // gs[d] = {destination of slot 0 of digit d relative to the bucket (may wrap), first slot of d}
     uint2 *gs = reinterpret_cast<uint2 *>(smem + L::off_gs);
+    // DST: gs[d] = the 64-bit (window << 48 | element offset of slot 0 of digit d), sstart[d]
+    uint32_t *sstart = reinterpret_cast<uint32_t *>(smem + L::off_start);
     uint16_t *sidx = reinterpret_cast<uint16_t *>(smem + L::off_sidx);
     auto kst = [&](int s) { return reinterpret_cast<K *>(smem + L::off_kst + s * L::kst_bytes); };
     auto vst = [&](int s) { return reinterpret_cast<VT *>(smem + L::off_vst + s * L::vst_bytes); };
@@ -1452,11 +1463,12 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
     // of the earlier tiles of the bucket (tile order = memory order: stable), loaded a tile
     // ahead (two buffers) or before the wait for the tile's data (one buffer)
     uint32_t m0 = 0, m1 = 0, m2 = 0;
-    uint64_t boffs = 0;
+    uint64_t boffs = 0, mdst = 0;
     auto meta_load = [&](const StageInfo &in) {
         if (in.valid) {
             if (tid < RADIX) {
-                m0 = prm.sub_rel[static_cast<uint64_t>(in.bucket) * RADIX + tid];
+                if constexpr (DST) mdst = tid <= static_cast<int>(prm.mask) ? prm.dst_off[tid] : 0ull;
+                else m0 = prm.sub_rel[static_cast<uint64_t>(in.bucket) * RADIX + tid];
                 m1 = prm.tile_pref[static_cast<uint64_t>(in.tile) * RADIX + tid];
                 m2 = in.carry_row != EMPTY_RANGE ? prm.carry[static_cast<uint64_t>(in.carry_row) * RADIX + tid] : 0u;
             }
@@ -1471,6 +1483,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
         if (!in.valid) break;
         const uint32_t count = in.count;
         const uint32_t gbase = m0 + m1 + m2;  // thread tid = digit tid
+        const uint64_t gdst = mdst;
         const uint64_t tboffs = boffs;
         Seg sk, sv;
         sk.pad = in.kpad;
@@ -1559,7 +1572,13 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
                     uint32_t run = incl - t;
 #pragma unroll
                     for (int w = 0; w < RADIX / 32; ++w) run += w < warp ? wsum[w] : 0u;
-                    gs[tid] = make_uint2(gbase - run, run);
+                    if constexpr (DST) {
+                        const uint64_t v = (gdst & ~DST_OFF_MASK) | ((gdst & DST_OFF_MASK) + gbase - run);
+                        gs[tid] = make_uint2(static_cast<uint32_t>(v), static_cast<uint32_t>(v >> 32));
+                        sstart[tid] = run;
+                    } else {
+                        gs[tid] = make_uint2(gbase - run, run);
+                    }
 #pragma unroll
                     for (int w = 0; w < W; ++w) {
                         cnt[w * RADIX + tid] = run;
@@ -1596,7 +1615,17 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
                     const uint32_t j = c * THREADS + tid;
                     if (FULL || j < count) {
                         const K k = ks[j];
-                        if constexpr (DIRECT) {
+                        if constexpr (DST) {
+                            const uint32_t i = sidx[j];
+                            const uint32_t d = digit_of(k, lo, mask);
+                            const uint2 g = gs[d];
+                            const uint64_t v = (static_cast<uint64_t>(g.y) << 32) | g.x;
+                            const uint64_t pos = (v & DST_OFF_MASK) + j;
+                            const uint32_t w = static_cast<uint32_t>(v >> 48);
+                            reinterpret_cast<K *>(prm.dst_kwin[w])[pos] = k;
+                            if (HV) reinterpret_cast<VT *>(prm.dst_vwin[w])[pos] = vb[i];
+                            if (check && j > sstart[d]) bad |= sidx[j - 1] > i;
+                        } else if constexpr (DIRECT) {
                             const uint32_t pos = gs[digit_of(k, lo, mask)].x + j;
                             kdst[pos] = unmap ? key_map(k, prm.kind, true) : k;
                             vdst[pos] = vs[j];

@@ -379,7 +379,10 @@ struct Plan {
     int wide_top = 0;
     int force_redo = 0;  // HRS_FLAG_FORCE_REDO (tuning flags or the HRS_FORCE_REDO environment variable)
     int kind = 0;        // hrs_key_kind of the keys (signed / float: the bijection fused into the kernels)
+    bool dst = false;    // hrs_partition_pass_to: the scatter writes each digit to its own window
+    size_t off_dst = 0;  //   (tables in temp: 256 digit offsets, MAX_WINDOWS key / value windows)
 };
+constexpr int MAX_WINDOWS = 64;
 
 // HRS_FORCE_REDO=1 in the environment ORs HRS_FLAG_FORCE_REDO into every call (include/hrs.h)
 inline uint32_t env_flags() {
@@ -511,6 +514,8 @@ inline hrs_status make_plan(Plan &pl, uint64_t n, int kb, int vb, int begin, int
     pl.local_fb2_cap = static_cast<uint32_t>(std::min<uint64_t>(fb2, 0xFFFFFFFFull));
     pl.off_local_fb2 = off;
     off = align_up(off + sizeof(LocalEntry) * static_cast<size_t>(pl.local_fb2_cap), 256);
+    pl.off_dst = off;
+    if (mode == MODE_PARTITION) off = align_up(off + sizeof(uint64_t) * (RADIX + 2 * MAX_WINDOWS), 256);
     pl.total = off;
     return HRS_SUCCESS;
 }
@@ -682,6 +687,21 @@ struct Runner {
         sp.force_redo = pl.force_redo;
         sp.kind = pl.kind;
         sp.final_pass = p == pl.D ? 1 : 0;
+        if constexpr (!TY) {
+            if (pl.dst) {  // hrs_partition_pass_to: every digit to its own window
+                sp.dst_off = at<unsigned long long>(temp, pl.off_dst);
+                sp.dst_kwin = sp.dst_off + RADIX;
+                sp.dst_vwin = sp.dst_kwin + MAX_WINDOWS;
+                auto fd = k_scatter<K, V, SC::THREADS, SC::KPT, SC::MINB, SC::NBUF, false, true>;
+                const size_t smd = ScatterSmem<K, V, SC::THREADS, SC::KPT, SC::NBUF, true>::bytes;
+                int gd = 0;
+                hrs_status sd = grid_for(fd, SC::THREADS, smd, dev, sms, &gd);
+                if (sd) return sd;
+                LaunchScope ls(st, 2, p);
+                launch_pdl(fd, dim3(gd), dim3(SC::THREADS), smd, st, sp);
+                return last_launch();
+            }
+        }
         auto fn = k_scatter<K, V, SC::THREADS, SC::KPT, SC::MINB, SC::NBUF, TY>;
         const size_t smem = ScatterSmem<K, V, SC::THREADS, SC::KPT, SC::NBUF>::bytes;
         int grid = 0;

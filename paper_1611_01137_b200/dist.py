@@ -86,6 +86,9 @@ class CudaOps:
     def copy_pieces(self, dst, src, pieces):
         self.hrs.copy_pieces(dst, src, pieces)
 
+    def partition_pass_to(self, keys, vals, lo, hi, offsets, key_windows, value_windows):
+        self.hrs.partition_pass_to(keys, vals, lo, hi, offsets, key_windows, value_windows)
+
     def sort_grouped_into(self, keys, vals, first_hist, begin_bit, end_bit, keys_out, vals_out, temp_holder):
         """hrs_sort_grouped into caller buffers (the input is grouped by its first digit)."""
         self._temp_for(keys, vals, begin_bit, end_bit, temp_holder)
@@ -119,11 +122,15 @@ class DistributedSorter:
         self.begin = begin_bit
         self.end = self.kbits if end_bit is None else end_bit
         self.ops = ops if ops is not None else CudaOps()
-        if exchange not in ("grouped", "a2a"):
+        if exchange not in ("grouped", "a2a", "fused"):
             raise ValueError(exchange)
         # "grouped": bucket-major point-to-point exchange, the receiver skips the first pass;
-        # "a2a": one all_to_all_single per array, the receiver sorts from the first digit
+        # "a2a": one all_to_all_single per array, the receiver sorts from the first digit;
+        # "fused": the partition scatter stores every bucket a single rank owns straight into
+        #   that rank's receive buffer (mapped with CUDA IPC: NVLink peer memory on a node),
+        #   only the buckets a rank boundary cuts are staged, refined and sent
         self.exchange = exchange
+        self._windows_cache = None
         self.world = dist.get_world_size(group)
         self.rank = dist.get_rank(group)
         self.last = {}
@@ -168,14 +175,22 @@ class DistributedSorter:
         if self.end == self.begin:  # empty bit range: the stable sort is the identity
             return keys.clone(), (vals.clone() if vals is not None else None), self._offset_identity()
         digits = self.digits()
+        fused = self.exchange == "fused"
         # 1-3a. first-digit partition of the whole shard; its histogram, gathered
         kp, vp = self._send_buffers(keys.numel())
         lo, hi = digits[0]
-        offs = self.ops.partition_into(keys, vals, lo, hi, kp, vp)
-        hists = self._gather([[offs[b + 1] - offs[b] for b in range(len(offs) - 1)]])[0]  # [rank][bucket]
+        if fused:  # histogram first: the fused partition needs every rank's counts
+            h = self.ops.digit_histogram(keys, lo, hi)
+            hists = self._gather([[int(x) for x in h.view(torch.int64).cpu().tolist()]])[0]
+        else:
+            offs = self.ops.partition_into(keys, vals, lo, hi, kp, vp)
+            hists = self._gather([[offs[b + 1] - offs[b] for b in range(len(offs) - 1)]])[0]  # [rank][bucket]
         N = sum(sum(h) for h in hists)
         cap = max((j + 1) * N // world - j * N // world for j in range(world))  # largest receive
         rk_all, rv_all = self._recv_buffers(cap)
+        boundary = None
+        if fused:
+            boundary = self._fused_partition(keys, vals, hists, N, lo, hi, kp, vp, rk_all, rv_all)
         # split[j][r]: local position on rank r of global sorted position t_j = j N / G
         split = [[0] * world for _ in range(world + 1)]
         split[world] = [sum(h) for h in hists]
@@ -233,9 +248,17 @@ class DistributedSorter:
         m = sum(recv)
         rk = rk_all[:m]
         rv = rv_all[:m] if vals is not None else None
-        grouped = self.exchange == "grouped" and len(digits) >= 1
+        grouped = self.exchange in ("grouped", "fused") and len(digits) >= 1
         if grouped:
             sends, recvs, rhist = self._grouped_plan(hists, split)
+            if fused:
+                # the fused scatter already stored every bucket that one rank owns; what is
+                # left are the pieces of the (at most G - 1) buckets a rank boundary cuts,
+                # which were staged locally and refined.  Every rank's stores must be done
+                # before any receiver reads its buffer.
+                sends = [x for x in sends if boundary[x[4]]]
+                recvs = [x for x in recvs if boundary[x[3]]]
+                self._barrier_after_device_work()
         ev = None
         if self.time_exchange and keys.is_cuda:
             ev = (torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True))
@@ -292,9 +315,9 @@ class DistributedSorter:
         z = np.minimum(S[1:, None, :], O.T[None, 1:, :])
         ln = np.maximum(z - a, 0)
         dst = np.cumsum(ln.reshape(world, -1), axis=1).reshape(ln.shape) - ln  # receiver offsets, (b, r)-major
-        sends = [(int(j), int(a[j, b, me]), int(ln[j, b, me]), int(dst[j, b, me]))
+        sends = [(int(j), int(a[j, b, me]), int(ln[j, b, me]), int(dst[j, b, me]), int(b))
                  for j, b in zip(*np.nonzero(ln[:, :, me]))]
-        recvs = [(int(r), int(dst[me, b, r]), int(ln[me, b, r])) for b, r in zip(*np.nonzero(ln[me]))]
+        recvs = [(int(r), int(dst[me, b, r]), int(ln[me, b, r]), int(b)) for b, r in zip(*np.nonzero(ln[me]))]
         rhist = ln[me].sum(axis=1).tolist()
         return sends, recvs, rhist
 
@@ -307,7 +330,7 @@ class DistributedSorter:
         rb = torch.empty_like(rbuf, device="cpu") if staged else rbuf
         sbv, rbv = _bits(sb), _bits(rb)
         ops, own = [], []
-        for peer, a, ln, d in sends:
+        for peer, a, ln, d, *_ in sends:
             if peer == me:
                 if own and own[-1][0] + own[-1][2] == a and own[-1][1] + own[-1][2] == d:
                     own[-1] = (own[-1][0], own[-1][1], own[-1][2] + ln)  # contiguous on both sides
@@ -321,7 +344,7 @@ class DistributedSorter:
             else:
                 for a, d, ln in own:
                     rbv[d:d + ln].copy_(sbv[a:a + ln])
-        for peer, d, ln in recvs:
+        for peer, d, ln, *_ in recvs:
             if peer != me:
                 ops.append(dist.P2POp(dist.irecv, rbv[d:d + ln], peer, self.group))
         if ops:
@@ -329,6 +352,66 @@ class DistributedSorter:
                 req.wait()
         if staged:
             rbuf.copy_(rb)
+
+    def _fused_partition(self, keys, vals, hists, N, lo, hi, kp, vp, rk_all, rv_all):
+        """The fused exchange's partition (hrs_partition_pass_to): bucket b that lies inside
+        rank j's range [t_j, t_{j+1}) goes to j's receive buffer at its bucket-major place
+        (C[b] - t_j + the counts of b on ranks before this one); a bucket that a boundary t_j
+        cuts goes to this rank's staging buffer at its partitioned place.  Returns the
+        boundary flags per bucket."""
+        import numpy as np
+        world, me = self.world, self.rank
+        H = np.asarray(hists, dtype=np.int64)
+        R = H.shape[1]
+        tot = H.sum(axis=0)
+        C = np.concatenate([[0], np.cumsum(tot)])
+        t = np.array([j * N // world for j in range(world + 1)], dtype=np.int64)
+        before = np.concatenate([np.zeros((1, R), dtype=np.int64), np.cumsum(H, axis=0)])[me]  # ranks < me
+        O = np.concatenate([[0], np.cumsum(H[me])])
+        boundary = [False] * R
+        offs = [0] * R
+        for b in range(R):
+            if tot[b] == 0:
+                continue
+            j = int(np.searchsorted(t, C[b], side="right") - 1)  # t_j <= C[b] < t_{j+1}
+            j = min(j, world - 1)
+            if C[b + 1] > t[j + 1]:  # a rank boundary cuts the bucket
+                boundary[b] = True
+                offs[b] = (world << 48) | int(O[b])
+            else:
+                offs[b] = (j << 48) | int(C[b] - t[j] + before[b])
+        kw, vw = self._windows(rk_all, rv_all)
+        self.ops.partition_pass_to(keys, vals, lo, hi, offs, kw + [kp.data_ptr()],
+                                   (vw + [vp.data_ptr()]) if vals is not None else None)
+        return boundary
+
+    def _windows(self, rk_all, rv_all):
+        """Device addresses of every rank's receive buffers in this process: our own, and the
+        peers' opened through CUDA IPC (exchanged once per buffer)."""
+        key = (rk_all.data_ptr(), rv_all.data_ptr() if rv_all is not None else 0)
+        if self._windows_cache is None or self._windows_cache[0] != key:
+            from . import ipc
+            mine = (ipc.export(rk_all), ipc.export(rv_all) if rv_all is not None else None)
+            allh = [None] * self.world
+            dist.all_gather_object(allh, mine, group=self.group)
+            kw, vw = [], []
+            for r, (hk, hv) in enumerate(allh):
+                if r == self.rank:
+                    kw.append(rk_all.data_ptr())
+                    vw.append(rv_all.data_ptr() if rv_all is not None else 0)
+                else:
+                    kw.append(ipc.open(hk))
+                    vw.append(ipc.open(hv) if hv is not None else 0)
+            self._windows_cache = (key, kw, vw)
+        return list(self._windows_cache[1]), list(self._windows_cache[2])
+
+    def _barrier_after_device_work(self):
+        """Every rank's device work so far (the fused stores into peers' buffers) is done
+        before any rank goes on."""
+        if self.keys.is_cuda:
+            torch.cuda.current_stream().synchronize()
+        if self.world > 1:
+            dist.barrier(group=self.group)
 
     def _gather(self, rows):
         """all_gather of this rank's histogram rows ([k][r] ints) -> [k][rank][r]."""

@@ -25,7 +25,7 @@ def _free_port():
     return p
 
 
-def _worker(rank, world, port, n_per, kbits, vbits, dist_name, q):
+def _worker(rank, world, port, n_per, kbits, vbits, dist_name, q, exchange="grouped", steps=1):
     os.environ["MASTER_ADDR"] = "127.0.0.1"
     os.environ["MASTER_PORT"] = str(port)
     dist.init_process_group("gloo", rank=rank, world_size=world)
@@ -33,8 +33,9 @@ def _worker(rank, world, port, n_per, kbits, vbits, dist_name, q):
         from paper_1611_01137_b200 import dist as hdist
         k = gen.keys(n_per, kbits, dist_name, start=rank * n_per, device="cuda:0")
         v = gen.values(n_per, vbits, "index", start=rank * n_per, device="cuda:0") if vbits else None
-        sorter = hdist.DistributedSorter(k, v)
-        ko, vo, off = sorter.step()
+        sorter = hdist.DistributedSorter(k, v, exchange=exchange)
+        for _ in range(steps):  # (later steps reuse every buffer and, fused, the IPC windows)
+            ko, vo, off = sorter.step()
         torch.cuda.synchronize()
         q.put((rank, off, oracle._u64(ko.cpu()).tolist(),
                oracle._u64(vo.cpu()).tolist() if vo is not None else None, sorter.last))
@@ -42,14 +43,21 @@ def _worker(rank, world, port, n_per, kbits, vbits, dist_name, q):
         dist.destroy_process_group()
 
 
-@pytest.mark.parametrize("world,n_per,kbits,vbits,dist_name", [
-    (2, 100003, 32, 32, "uniform"), (3, 50001, 32, 32, "and4"), (2, 30000, 64, 64, "and3"),
-    (3, 20000, 32, 0, "const"), (2, 40000, 64, 32, "const")])
-def test_distributed_cuda_matches_oracle(world, n_per, kbits, vbits, dist_name):
+@pytest.mark.parametrize("world,n_per,kbits,vbits,dist_name,exchange", [
+    (2, 100003, 32, 32, "uniform", "grouped"), (3, 50001, 32, 32, "and4", "grouped"),
+    (2, 30000, 64, 64, "and3", "grouped"), (3, 20000, 32, 0, "const", "grouped"),
+    (2, 40000, 64, 32, "const", "grouped"), (2, 30011, 32, 32, "and3", "a2a"),
+    (2, 100003, 32, 32, "uniform", "fused"), (3, 50001, 32, 32, "and4", "fused"),
+    (2, 30000, 64, 64, "and2", "fused"), (3, 20000, 64, 0, "const", "fused"), (1, 70001, 32, 32, "uniform", "fused")])
+def test_distributed_cuda_matches_oracle(world, n_per, kbits, vbits, dist_name, exchange):
+    """Grouped (bucket-major P2P) and all-to-all exchanges, and the fused exchange: the
+    partition scatter writes every owned bucket straight into the receiving process's buffer
+    through a CUDA IPC mapping (hrs_partition_pass_to; on a node these are NVLink peer
+    writes), the boundary buckets are refined locally and sent.  Two steps per run."""
     ctx = mp.get_context("spawn")
     q = ctx.Queue()
     port = _free_port()
-    procs = [ctx.Process(target=_worker, args=(r, world, port, n_per, kbits, vbits, dist_name, q))
+    procs = [ctx.Process(target=_worker, args=(r, world, port, n_per, kbits, vbits, dist_name, q, exchange, 2))
              for r in range(world)]
     for p in procs:
         p.start()

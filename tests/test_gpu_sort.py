@@ -550,3 +550,34 @@ def _conditional_graph_replays():
             assert np.array_equal(_np(ko), ek), (n, dist, i)
             if vbits:
                 assert np.array_equal(_np(vo), ev), (n, dist, i)
+
+
+@pytest.mark.parametrize("kbits,vbits", TYPES)
+def test_partition_pass_to_windows(kbits, vbits):
+    """hrs_partition_pass_to (the fused exchange's scatter): every digit's
+    run goes to its own window at its own offset -- here three separate device buffers in a
+    scrambled bucket order with gaps -- and must equal the oracle's stable partition."""
+    import paper_1611_01137_b200 as hrs
+    rng = np.random.default_rng(kbits + vbits)
+    for n, dist, (lo, hi) in ((300001, "and2", (kbits - 8, kbits)), (70001, "uniform", (3, 9)), (1, "uniform", (0, 8))):
+        k, v = _inputs(n, kbits, vbits, dist, seed=n)
+        ek, ev, eo = oracle.partition_pass(k, v, lo, hi)
+        r = 1 << (hi - lo)
+        cnt = np.diff(eo.astype(np.int64))
+        win = rng.integers(0, 3, size=r)
+        order = rng.permutation(r)
+        sizes, offs = [0, 0, 0], [0] * r
+        for d in order:  # place the runs window by window in a scrambled order, with gaps
+            offs[d] = (int(win[d]) << 48) | (sizes[win[d]] + 7)
+            sizes[win[d]] += int(cnt[d]) + 7
+        kd = k.to(DEV)
+        vd = v.to(DEV) if v is not None else None
+        kwin = [torch.zeros(sz + 8, dtype=kd.dtype, device=DEV) for sz in sizes]
+        vwin = [torch.zeros(sz + 8, dtype=vd.dtype, device=DEV) for sz in sizes] if v is not None else None
+        hrs.partition_pass_to(kd, vd, lo, hi, offs, kwin, vwin)
+        torch.cuda.synchronize()
+        for d in range(r):
+            w, o, c = offs[d] >> 48, offs[d] & ((1 << 48) - 1), int(cnt[d])
+            assert np.array_equal(_np(kwin[w][o:o + c]), ek[int(eo[d]):int(eo[d]) + c]), (n, d)
+            if v is not None:
+                assert np.array_equal(_np(vwin[w][o:o + c]), ev[int(eo[d]):int(eo[d]) + c]), (n, d)
