@@ -208,7 +208,7 @@ class DistributedSorter:
                 # the receive buffer is not in use before the exchange: it is the scratch of
                 # the refinement passes (a refined sub-range larger than it gets its own)
                 big = max(it[5][me] for it in todo)
-                if big <= rk_all.numel():
+                if big <= rk_all.numel() and not fused:  # (fused: peers are writing the receive buffer)
                     scratch_k, scratch_v = rk_all, rv_all
                 else:
                     scratch_k = torch.empty(big, dtype=kp.dtype, device=kp.device)
