@@ -1382,6 +1382,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
     static_assert(THREADS % RADIX == 0 && THREADS <= 4 * RADIX, "threads 0..255 fold one digit each");
     static_assert(32 * KPT < (1 << 16), "the in-warp rank is packed above the digit");
     using L = ScatterSmem<K, V, THREADS, KPT, NBUF, DST>;
+    static_assert(!DST || THREADS * KPT < (1 << 16), "DST packs a tile slot and a window into 32 bits");
     constexpr int W = THREADS / 32;
     constexpr bool HV = HasVal<V>::value;
     using VT = ValT<V>;
@@ -1573,9 +1574,10 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
 #pragma unroll
                     for (int w = 0; w < RADIX / 32; ++w) run += w < warp ? wsum[w] : 0u;
                     if constexpr (DST) {
-                        const uint64_t v = (gdst & ~DST_OFF_MASK) | ((gdst & DST_OFF_MASK) + gbase - run);
+                        // element offset of slot 0 of digit d (mod 2^64: slot `run` onward is in range)
+                        const uint64_t v = (gdst & DST_OFF_MASK) + gbase - static_cast<uint64_t>(run);
                         gs[tid] = make_uint2(static_cast<uint32_t>(v), static_cast<uint32_t>(v >> 32));
-                        sstart[tid] = run;
+                        sstart[tid] = run | (static_cast<uint32_t>(gdst >> 48) << 16);  // start | window << 16
                     } else {
                         gs[tid] = make_uint2(gbase - run, run);
                     }
@@ -1619,12 +1621,12 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
                             const uint32_t i = sidx[j];
                             const uint32_t d = digit_of(k, lo, mask);
                             const uint2 g = gs[d];
-                            const uint64_t v = (static_cast<uint64_t>(g.y) << 32) | g.x;
-                            const uint64_t pos = (v & DST_OFF_MASK) + j;
-                            const uint32_t w = static_cast<uint32_t>(v >> 48);
+                            const uint32_t sw = sstart[d];
+                            const uint64_t pos = ((static_cast<uint64_t>(g.y) << 32) | g.x) + j;
+                            const uint32_t w = sw >> 16;
                             reinterpret_cast<K *>(prm.dst_kwin[w])[pos] = k;
                             if (HV) reinterpret_cast<VT *>(prm.dst_vwin[w])[pos] = vb[i];
-                            if (check && j > sstart[d]) bad |= sidx[j - 1] > i;
+                            if (check && j > (sw & 0xFFFFu)) bad |= sidx[j - 1] > i;
                         } else if constexpr (DIRECT) {
                             const uint32_t pos = gs[digit_of(k, lo, mask)].x + j;
                             kdst[pos] = unmap ? key_map(k, prm.kind, true) : k;
