@@ -381,6 +381,8 @@ class DistributedSorter:
             else:
                 offs[b] = (j << 48) | int(C[b] - t[j] + before[b])
         kw, vw = self._windows(rk_all, rv_all)
+        # every receiver is done with its buffer (the previous step's local sort read it)
+        self._barrier_after_device_work()
         self.ops.partition_pass_to(keys, vals, lo, hi, offs, kw + [kp.data_ptr()],
                                    (vw + [vp.data_ptr()]) if vals is not None else None)
         return boundary
