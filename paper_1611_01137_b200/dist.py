@@ -323,35 +323,36 @@ class DistributedSorter:
 
     def _p2p(self, rbuf, sbuf, sends, recvs):
         """The pieces as one batch of point-to-point messages (NCCL groups them; NVLink),
-        this rank's own pieces as device copies."""
+        this rank's own pieces as device copies (one launch).  With gloo (tests) the
+        messages go through host copies and only the received ranges are copied back."""
         me = self.rank
         staged = _host_staged(self.group, sbuf)
-        sb = sbuf.cpu() if staged else sbuf
-        rb = torch.empty_like(rbuf, device="cpu") if staged else rbuf
-        sbv, rbv = _bits(sb), _bits(rb)
-        ops, own = [], []
+        own = []
         for peer, a, ln, d, *_ in sends:
             if peer == me:
                 if own and own[-1][0] + own[-1][2] == a and own[-1][1] + own[-1][2] == d:
                     own[-1] = (own[-1][0], own[-1][1], own[-1][2] + ln)  # contiguous on both sides
                 else:
                     own.append((a, d, ln))
-            else:
-                ops.append(dist.P2POp(dist.isend, sbv[a:a + ln], peer, self.group))
         if own:
-            if hasattr(self.ops, "copy_pieces") and not staged:
-                self.ops.copy_pieces(rbv, sbv, own)  # one launch for all own pieces
+            if hasattr(self.ops, "copy_pieces"):
+                self.ops.copy_pieces(_bits(rbuf), _bits(sbuf), own)
             else:
                 for a, d, ln in own:
-                    rbv[d:d + ln].copy_(sbv[a:a + ln])
-        for peer, d, ln, *_ in recvs:
-            if peer != me:
-                ops.append(dist.P2POp(dist.irecv, rbv[d:d + ln], peer, self.group))
-        if ops:
-            for req in dist.batch_isend_irecv(ops):
-                req.wait()
+                    _bits(rbuf)[d:d + ln].copy_(_bits(sbuf)[a:a + ln])
+        peer_sends = [x for x in sends if x[0] != me]
+        peer_recvs = [x for x in recvs if x[0] != me]
+        if not peer_sends and not peer_recvs:
+            return
+        sbv = _bits(sbuf.cpu() if staged else sbuf)
+        rbv = _bits(torch.empty_like(rbuf, device="cpu")) if staged else _bits(rbuf)
+        ops = [dist.P2POp(dist.isend, sbv[a:a + ln], peer, self.group) for peer, a, ln, d, *_ in peer_sends]
+        ops += [dist.P2POp(dist.irecv, rbv[d:d + ln], peer, self.group) for peer, d, ln, *_ in peer_recvs]
+        for req in dist.batch_isend_irecv(ops):
+            req.wait()
         if staged:
-            rbuf.copy_(rb)
+            for peer, d, ln, *_ in peer_recvs:
+                _bits(rbuf)[d:d + ln].copy_(rbv[d:d + ln])
 
     def _fused_partition(self, keys, vals, hists, N, lo, hi, kp, vp, rk_all, rv_all):
         """The fused exchange's partition (hrs_partition_pass_to): bucket b that lies inside
