@@ -193,7 +193,7 @@ def run_hrs(args):
 
     if use_dist:
         from paper_1611_01137_b200 import dist as hdist
-        sorter = hdist.DistributedSorter(keys, vals, group=pg)
+        sorter = hdist.DistributedSorter(keys, vals, group=pg, exchange=args.exchange)
         step = sorter.step
     else:
         keys_out = torch.empty_like(keys)
@@ -242,6 +242,7 @@ def run_hrs(args):
            "config": {"workload": f"{args.config}:{desc}, {dist_name}", "n_per_gpu": n, "key_bits": kbits,
                       "value_bits": vbits, "bits": [0, kbits], "values": "input index",
                       "parallelism": f"dp{world}" if world > 1 else "single",
+                      "exchange": args.exchange if use_dist else None,
                       "l2": "inputs (>= 2 GiB) larger than the 126 MB L2; no flush"},
            "gpu_launches": launches, "clocks": clocks,
            "step_ms": {"median": statistics.median(step_ms), "min": min(step_ms), "max": max(step_ms)}}
@@ -518,6 +519,9 @@ def main(argv=None):
     ap.add_argument("--no-e2e", action="store_true")
     ap.add_argument("--force-dist", action="store_true",
                     help="run the distributed path (NCCL) even at world size 1 (tests the N>1 code path on one GPU)")
+    ap.add_argument("--exchange", default="grouped", choices=["grouped", "fused", "a2a"],
+                    help="distributed exchange: bucket-major NCCL P2P (default), the fused scatter into the "
+                         "receivers' buffers (CUDA IPC / NVLink peer memory, SURVEY N2), or one all-to-all")
     ap.add_argument("--no-cpu", action="store_true")
     ap.add_argument("--cpu-log2", type=int, default=24)
     ap.add_argument("--ref-log2", type=int, default=24)
