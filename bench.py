@@ -183,7 +183,9 @@ def run_hrs(args):
                 os.environ.setdefault("MASTER_PORT", str(sk.getsockname()[1]))
             os.environ.update(RANK="0", WORLD_SIZE="1", LOCAL_RANK="0")
             os.environ.setdefault("MASTER_ADDR", "127.0.0.1")
-        dist.init_process_group("nccl", device_id=dev)
+        import datetime
+        # a hung collective (a dead peer) fails the run after this long instead of blocking it
+        dist.init_process_group("nccl", device_id=dev, timeout=datetime.timedelta(seconds=args.nccl_timeout))
         pg = dist.group.WORLD
 
     seed = gen.SEEDS[0]
@@ -522,6 +524,7 @@ def main(argv=None):
     ap.add_argument("--exchange", default="grouped", choices=["grouped", "fused", "a2a"],
                     help="distributed exchange: bucket-major NCCL P2P (default), the fused scatter into the "
                          "receivers' buffers (CUDA IPC / NVLink peer memory, SURVEY N2), or one all-to-all")
+    ap.add_argument("--nccl-timeout", type=int, default=300, help="seconds before a stuck collective aborts")
     ap.add_argument("--no-cpu", action="store_true")
     ap.add_argument("--cpu-log2", type=int, default=24)
     ap.add_argument("--ref-log2", type=int, default=24)

@@ -14,6 +14,8 @@
 #include <unordered_map>
 #include <vector>
 
+#include <nvtx3/nvToolsExt.h>
+
 #include "hrs_device.cuh"
 
 namespace hrs_host {
@@ -42,12 +44,39 @@ inline cudaEvent_t prof_event() {
     return e;
 }
 
+// NVTX ranges around every launch, opt-in (HRS_NVTX=1 in the environment): named by kind
+// (hist, classify, scatter, local, ...) so a timeline tool shows the pass structure
+inline bool nvtx_enabled() {
+    static const bool on = [] {
+        const char *e = std::getenv("HRS_NVTX");
+        return e && e[0] == '1';
+    }();
+    return on;
+}
+inline const char *kind_name(int kind) {
+    static const char *const names[] = {"hrs:init", "hrs:hist", "hrs:scatter", "hrs:local", "hrs:copy", "hrs:classify"};
+    return (kind >= 0 && kind < 6) ? names[kind] : "hrs:other";
+}
+
 // RAII bracket around one launch: counts it and, when profiling, records events
 struct LaunchScope {
     cudaStream_t st;
     ProfRec rec;
+    bool nvtx = false;
     LaunchScope(cudaStream_t s, int kind, int pass) : st(s) {
         ++g_launches;
+        if (nvtx_enabled()) {
+            nvtx = true;
+            nvtxEventAttributes_t a;
+            std::memset(&a, 0, sizeof(a));
+            a.version = NVTX_VERSION;
+            a.size = NVTX_EVENT_ATTRIB_STRUCT_SIZE;
+            a.messageType = NVTX_MESSAGE_TYPE_ASCII;
+            a.message.ascii = kind_name(kind);
+            a.payloadType = NVTX_PAYLOAD_TYPE_INT32;
+            a.payload.iValue = pass;
+            nvtxRangePushEx(&a);
+        }
         if (g_prof) {
             rec.kind = kind;
             rec.pass = pass;
@@ -57,6 +86,7 @@ struct LaunchScope {
         }
     }
     ~LaunchScope() {
+        if (nvtx) nvtxRangePop();
         if (g_prof) {
             cudaEventRecord(rec.b, st);
             g_prof_recs.push_back(rec);
