@@ -157,6 +157,27 @@ template <> struct LocalCfg<4> { static constexpr int THREADS = 128, KPT = 16; }
 template <> struct LocalCfg<5> { static constexpr int THREADS = 256, KPT = 16; };
 template <> struct LocalCfg<6> { static constexpr int THREADS = 288, KPT = 16; };
 template <> struct LocalCfg<7> { static constexpr int THREADS = 512, KPT = 16; };
+// the counting local sort's CTA shape for classes 5 and 6 (same capacity as LocalCfg)
+#ifndef HRS_LCC5_T
+#define HRS_LCC5_T 256
+#endif
+#ifndef HRS_LCC5_K
+#define HRS_LCC5_K 16
+#endif
+#ifndef HRS_LCC6_T
+#define HRS_LCC6_T 288
+#endif
+#ifndef HRS_LCC6_K
+#define HRS_LCC6_K 16
+#endif
+#ifndef HRS_LCC_OCC
+#define HRS_LCC_OCC 4
+#endif
+template <int C>
+struct LocalCntCfg : LocalCfg<C> {};
+template <> struct LocalCntCfg<5> { static constexpr int THREADS = HRS_LCC5_T, KPT = HRS_LCC5_K; };
+template <> struct LocalCntCfg<6> { static constexpr int THREADS = HRS_LCC6_T, KPT = HRS_LCC6_K; };
+static_assert(HRS_LCC5_T * HRS_LCC5_K == 4096 && HRS_LCC6_T * HRS_LCC6_K == 4608, "class capacities");
 
 // two-stage TMA prefetch where it fits next to a second resident CTA, else one stage
 // two-stage TMA prefetch when three CTAs still fit per SM, else one stage; the
@@ -199,7 +220,7 @@ struct LocalStages {
 constexpr int CNT_LO = 5, CNT_HI = 6;
 template <typename K, typename V, int C, bool RECON>
 struct LocalCntStages {
-    using LC = LocalCfg<C>;
+    using LC = LocalCntCfg<C>;
     static constexpr int VBYTES = HasVal<V>::value ? static_cast<int>(sizeof(V)) : 0;
     static constexpr int CB = static_cast<int>(sizeof(K)) + VBYTES <= 8 ? HRS_LC_CB8 : 14;
     static constexpr size_t SM_BUDGET = 228 * 1024;
@@ -211,7 +232,7 @@ struct LocalCntStages {
     static constexpr int by_smem = static_cast<int>(SM_BUDGET / (bytes + 1024));
     static constexpr int by_threads = 2048 / LC::THREADS;
     static constexpr int OCC0 = by_smem < by_threads ? by_smem : by_threads;
-    static constexpr int OCC = OCC0 < 1 ? 1 : (OCC0 > 4 ? 4 : OCC0);
+    static constexpr int OCC = OCC0 < 1 ? 1 : (OCC0 > HRS_LCC_OCC ? HRS_LCC_OCC : OCC0);
 };
 
 template <typename K, typename V>
@@ -771,7 +792,7 @@ struct Runner {
         if constexpr (!LST::fits) {
             return HRS_ERROR_INVALID_VALUE;
         } else {
-            using LC = LocalCfg<C>;
+            using LC = LocalCntCfg<C>;
             LocalParams lp;
             local_params(lp, pl, temp, kin, kout, vin, vout);
             Ctl *ctl = at<Ctl>(temp, 0);
