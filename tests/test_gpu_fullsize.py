@@ -143,3 +143,39 @@ def test_more_than_2_31_records():
         ok = (sk[:-1] < sk[1:]) | ((sk[:-1] == sk[1:]) & (idx[:-1] < idx[1:]))
         assert bool(ok.all()), f"order/stability violated near {a}"
         del idx, sk, ok
+
+
+@pytest.mark.parametrize("exchange", ["grouped", "fused"])
+def test_distributed_fullsize_world1(exchange):
+    """The distributed driver at the BASELINE size (2^28 u32/u32 AND-2, a process group of
+    one): partition (or fused partition into the receive window), exchange, grouped local
+    sort -- checked with the O(n) stable-sort certificate in a fresh process."""
+    import os
+    import subprocess
+    import sys
+    root = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+    code = r"""
+import os, socket, torch, torch.distributed as dist
+with socket.socket() as s:
+    s.bind(("127.0.0.1", 0)); port = s.getsockname()[1]
+os.environ.update(MASTER_ADDR="127.0.0.1", MASTER_PORT=str(port))
+dist.init_process_group("gloo", rank=0, world_size=1)
+import importlib.util, gen
+spec = importlib.util.spec_from_file_location("fs", "tests/test_gpu_fullsize.py")
+m = importlib.util.module_from_spec(spec); spec.loader.exec_module(m)
+from paper_1611_01137_b200 import dist as hdist
+n = 1 << 28
+k = gen.keys(n, 32, "and2", device="cuda:0")
+v = gen.values(n, 32, "index", device="cuda:0")
+s = hdist.DistributedSorter(k, v, exchange="%s")
+for _ in range(2):
+    ko, vo, off = s.step()
+torch.cuda.synchronize()
+assert off == 0 and ko.numel() == n
+m.certificate(k, ko, vo, 0, 32)
+print("dist fullsize ok")
+""" % exchange
+    r = subprocess.run([sys.executable, "-c", code], cwd=root, env=dict(os.environ, PYTHONPATH=root),
+                       capture_output=True, text=True, timeout=900)
+    assert r.returncode == 0, r.stdout[-2000:] + r.stderr[-4000:]
+    assert "dist fullsize ok" in r.stdout
