@@ -94,6 +94,9 @@ def build(force: bool = False, verbose: bool = False, out: str | None = None, de
         sys.stderr.write(r.stderr[-8000:])
         raise RuntimeError(f"link failed (exit {r.returncode})")
     os.replace(lib + ".tmp", lib)
+    if out is not None:  # experiment builds: keep only the library
+        import shutil
+        shutil.rmtree(objdir, ignore_errors=True)
     if verbose:
         for _, _, rr in results:
             if rr is not None:
