@@ -35,6 +35,29 @@ std::unordered_map<uint64_t, KernelInfo> g_kinfo;
 std::unordered_map<int, int> g_dev_ok;
 std::unordered_map<int, int> g_dev_sms;
 thread_local GraphCtx *g_gx = nullptr;
+
+cudaStream_t side_stream(int dev, int i) {
+    // per thread: a stream being captured into one thread's graph must not receive another
+    // thread's launches
+    thread_local std::unordered_map<int, std::vector<cudaStream_t>> streams;
+    auto &v = streams[dev];
+    while (static_cast<int>(v.size()) <= i) {
+        cudaStream_t s = nullptr;
+        if (cudaStreamCreateWithFlags(&s, cudaStreamNonBlocking) != cudaSuccess) return nullptr;
+        v.push_back(s);
+    }
+    return v[i];
+}
+
+cudaEvent_t fork_event(int i) {
+    thread_local std::vector<cudaEvent_t> ev;
+    while (static_cast<int>(ev.size()) <= i) {
+        cudaEvent_t e = nullptr;
+        if (cudaEventCreateWithFlags(&e, cudaEventDisableTiming) != cudaSuccess) return nullptr;
+        ev.push_back(e);
+    }
+    return ev[i];
+}
 }  // namespace hrs_host
 
 namespace {
