@@ -55,6 +55,9 @@
 #define HRS_WO_UNROLL 4
 #endif
 namespace hrs { constexpr int WO_UNROLL = HRS_WO_UNROLL; }
+#ifndef HRS_SC_VSPLIT
+#define HRS_SC_VSPLIT 1  // one value staging buffer (two key buffers): larger tiles (0: two of each)
+#endif
 #ifndef HRS_SC_DIRECT
 #define HRS_SC_DIRECT 0  // experiment: values placed from registers, no slot index, no stability check
 #endif
@@ -1340,8 +1343,12 @@ struct ScatterSmem {
     static constexpr bool HV = HasVal<V>::value;
     static constexpr size_t kst_elems = KPB + 32 / sizeof(K);
     static constexpr size_t vst_elems = KPB + 32 / sizeof(VT);
-    static constexpr size_t off_bar = 0;
-    static constexpr size_t off_info = 16;
+    // VS: the values are staged in ONE buffer (own barrier), loaded after the previous
+    // tile's write-out, while the keys keep two: the freed buffer buys a larger tile
+    static constexpr bool VS = HRS_SC_VSPLIT && !HRS_SC_DIRECT && NBUF == 2 && HV;
+    static constexpr size_t off_bar = 0;  // [3]: key stages, value stage
+    static constexpr size_t off_vinfo = 24;
+    static constexpr size_t off_info = 48;
     static constexpr size_t off_cnt = align16(off_info + NBUF * sizeof(StageInfo));
     static constexpr size_t off_wsum = align16(off_cnt + sizeof(uint32_t) * W * RADIX);
     static constexpr size_t off_gs = align16(off_wsum + sizeof(uint32_t) * 16);
@@ -1351,7 +1358,7 @@ struct ScatterSmem {
     static constexpr size_t kst_bytes = align16(sizeof(K) * kst_elems);
     static constexpr size_t off_vst = off_kst + NBUF * kst_bytes;
     static constexpr size_t vst_bytes = HV ? align16(sizeof(VT) * vst_elems) : 0;
-    static constexpr size_t bytes = off_vst + NBUF * vst_bytes;
+    static constexpr size_t bytes = off_vst + (VS ? 1 : NBUF) * vst_bytes;
 };
 
 // One counting pass over the tiles of every bucket of pass p, stable.
@@ -1382,6 +1389,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
     static_assert(THREADS % RADIX == 0 && THREADS <= 4 * RADIX, "threads 0..255 fold one digit each");
     static_assert(32 * KPT < (1 << 16), "the in-warp rank is packed above the digit");
     using L = ScatterSmem<K, V, THREADS, KPT, NBUF, DST>;
+    constexpr bool VS = L::VS;
     static_assert(!DST || THREADS * KPT < (1 << 16), "DST packs a tile slot and a window into 32 bits");
     constexpr int W = THREADS / 32;
     constexpr bool HV = HasVal<V>::value;
@@ -1389,6 +1397,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
     extern __shared__ __align__(16) unsigned char smem[];
     uint64_t *bar = reinterpret_cast<uint64_t *>(smem + L::off_bar);
     StageInfo *info = reinterpret_cast<StageInfo *>(smem + L::off_info);
+    Seg *vinfo = reinterpret_cast<Seg *>(smem + L::off_vinfo);  // VS: the value stage's segment
     uint32_t *cnt = reinterpret_cast<uint32_t *>(smem + L::off_cnt);    // [W][256]
     uint32_t *wsum = reinterpret_cast<uint32_t *>(smem + L::off_wsum);  // [W] digit-total partial sums
     // gs[d] = {destination of slot 0 of digit d relative to the bucket (may wrap), first slot of d}
@@ -1440,7 +1449,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
         in.kpad = sk.pad;
         in.k0 = static_cast<uint32_t>(sk.i0);
         in.k1 = static_cast<uint32_t>(sk.i1);
-        if (HV) {
+        if (HV && !VS) {
             bytes += seg_plan(vin + td.offs, td.count, vin, vin + prm.n, sv);
             in.vpad = sv.pad;
             in.v0 = static_cast<uint32_t>(sv.i0);
@@ -1448,12 +1457,24 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
         }
         mbar_arrive_expect_tx(&bar[s], bytes);
         seg_issue(kst(s), kin + td.offs, sk, &bar[s], pol);
-        if (HV) seg_issue(vst(s), vin + td.offs, sv, &bar[s], pol);
+        if (HV && !VS) seg_issue(vst(s), vin + td.offs, sv, &bar[s], pol);
+    };
+    // VS: the values of a tile whose keys are staged (the segment is published through
+    // the barrier: written before the arrive, read after the wait)
+    auto vissue = [&](const StageInfo &in) {
+        if (!in.valid) return;
+        const VT *vin = vin_of(in.src);
+        Seg sv;
+        const uint32_t bytes = seg_plan(vin + in.offs, in.count, vin, vin + prm.n, sv);
+        *vinfo = sv;
+        mbar_arrive_expect_tx(&bar[NBUF], bytes);
+        seg_issue(vst(0), vin + in.offs, sv, &bar[NBUF], pol);
     };
     if (tid == 0) {
-        for (int b = 0; b < NBUF; ++b) mbar_init(&bar[b], 1);
+        for (int b = 0; b < NBUF + (VS ? 1 : 0); ++b) mbar_init(&bar[b], 1);
         mbar_fence_init();
         for (int b = 0; b < NBUF; ++b) issue(b, atomicAdd(&prm.ctl->claim[prm.p], 1u));
+        if constexpr (VS) vissue(info[0]);
     }
     __syncthreads();
 
@@ -1496,19 +1517,31 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
         const K *ksrc = kin_of(in.src) + in.offs;
         const VT *vsrc = HV ? vin_of(in.src) + in.offs : nullptr;
         K *const ks = kst(s);
-        VT *const vs = HV ? vst(s) : nullptr;
+        VT *const vs = HV ? vst(VS ? 0 : s) : nullptr;
         mbar_wait(&bar[s], par);
-        const bool full = count == static_cast<uint32_t>(L::KPB) && seg_full(sk, count) && (!HV || seg_full(sv, count));
+        const bool full = count == static_cast<uint32_t>(L::KPB) && seg_full(sk, count) && (!HV || VS || seg_full(sv, count));
         const bool mapin = TY && prm.kind != 0 && in.src == SRC_IN;     // records still in the input
         const bool unmap = TY && prm.kind != 0 && prm.final_pass != 0;  // their final place
-        const VT *const vb = HV ? vs + sv.pad : nullptr;
+        const VT *vb = HV ? vs + sv.pad : nullptr;
+        // VS: wait for this tile's values (issued after the previous tile's write-out)
+        auto vwait = [&]() {
+            if constexpr (VS) {
+                mbar_wait(&bar[NBUF], it & 1u);
+                const Seg s2 = *vinfo;
+                vb = vs + s2.pad;
+                if (!seg_full(s2, count)) {  // (only at the ends of the buffer)
+                    seg_fill_edges<VT, THREADS>(vs, vsrc, s2, count);
+                    __syncthreads();
+                }
+            }
+        };
 
         auto body = [&](auto full_tag) {
             constexpr bool FULL = decltype(full_tag)::value;
             // the values of the elements the bulk copy did not cover (segments at the ends
             // of the buffer) into shared memory, read by the write-out after the barriers
             constexpr bool DIRECT = HRS_SC_DIRECT && HV;
-            if (!DIRECT && !FULL && HV) seg_fill_edges<VT, THREADS>(vs, vsrc, sv, count);
+            if (!DIRECT && !VS && !FULL && HV) seg_fill_edges<VT, THREADS>(vs, vsrc, sv, count);
             const K *const kb = ks + sk.pad;
             [[maybe_unused]] VT val[DIRECT ? KPT : 1];
             // the keys stay in registers from here to the placement; the in-warp ranks are
@@ -1661,6 +1694,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
             // the next tile's metadata (info[s ^ 1] was published by the issue after the
             // previous tile, before this tile's barriers); the loads overlap the write-out
             if (NBUF == 2) meta_load(info[s ^ 1]);
+            vwait();
             const bool bad = write_out(fast && !DIRECT);
             if (__syncthreads_or(bad || (fast && prm.force_redo))) {
                 // the atomics did not serve the lanes of a warp in order: rank the tile
@@ -1681,6 +1715,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
         // ---- the staging buffer is free again (barrier above): claim the next tile into it
         if (tid == 0) {
             fence_proxy_async();
+            if constexpr (VS) vissue(info[s ^ 1]);
             issue(s, atomicAdd(&prm.ctl->claim[prm.p], 1u));
         }
         if (NBUF == 1) {

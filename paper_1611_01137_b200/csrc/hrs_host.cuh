@@ -101,7 +101,8 @@ constexpr uint32_t DEFAULT_MT_DIV = 4;
 #define HRS_SC_THREADS 256
 #endif
 #ifndef HRS_SC_KPT
-#define HRS_SC_KPT 22  // measured on B200 (c2 uniform, both passes): 13 x 3 CTAs/SM 2.51 ms, 16 x 2 2.24, 20 x 2 2.15, 22 x 2 2.10, 32 x 1 2.41
+#define HRS_SC_KPT 28  // measured on B200 (c2 uniform, both passes): 13 x 3 CTAs/SM 2.51 ms, 16 x 2 2.24, 20 x 2 2.15, 22 x 2 2.10, 32 x 1 2.41;
+                       // one value buffer (HRS_SC_VSPLIT): 22 x 2 2.15, 26 x 2 2.09, 28 x 2 2.07 (AND-3 step 6.20 -> 6.00 ms)
 #endif
 #ifndef HRS_SC_NBUF
 #define HRS_SC_NBUF 2
@@ -115,7 +116,8 @@ constexpr uint32_t DEFAULT_MT_DIV = 4;
 #define HRS_SC64_THREADS 256
 #endif
 #ifndef HRS_SC64_KPT
-#define HRS_SC64_KPT 12  // measured (c4 uniform / AND-3 step): 16 x 1 buffer 7.80 / 17.5 ms, 12 x 2 7.66 / 16.1, 22 x 1 7.52 / 17.2
+#define HRS_SC64_KPT 14  // measured (c4 uniform / AND-3 step): 16 x 1 buffer 7.80 / 17.5 ms, 12 x 2 7.66 / 16.1, 22 x 1 7.52 / 17.2;
+                         // one value buffer: 12 x 2 7.82 / 15.9, 14 x 2 7.56 / 15.6, 16 x 2 7.77 / 17.6
 #endif
 #ifndef HRS_SC64_MINB
 #define HRS_SC64_MINB 2
@@ -131,7 +133,7 @@ template <int KB, int VB>
 struct ScatterCfg {
     static constexpr bool SMALL = (KB == 4 && VB <= 4);
     static constexpr int THREADS = SMALL ? HRS_SC_THREADS : HRS_SC64_THREADS;
-    static constexpr int KPT = SMALL ? HRS_SC_KPT : HRS_SC64_KPT;  // 256 x 22: two staging buffers + the slot index for two CTAs per SM
+    static constexpr int KPT = SMALL ? HRS_SC_KPT : HRS_SC64_KPT;  // 256 x 28: two key buffers, one value buffer + the slot index for two CTAs per SM
     static constexpr int MINB = SMALL ? HRS_SC_MINB : HRS_SC64_MINB;
     static constexpr int NBUF = SMALL ? HRS_SC_NBUF : HRS_SC64_NBUF;
 };
@@ -139,10 +141,9 @@ struct ScatterCfg {
 #define HRS_HIST_THREADS 256
 #endif
 #ifndef HRS_HIST_STAGES
-#define HRS_HIST_STAGES 3
+#define HRS_HIST_STAGES 0  // 0: 2 for the 32-bit scatter shape (28 KB stages, 3 CTAs / SM), else 3
 #endif
 constexpr int HIST_THREADS = HRS_HIST_THREADS;
-constexpr int HIST_STAGES = HRS_HIST_STAGES;
 constexpr int CLASSIFY_THREADS = 256;
 constexpr uint32_t RANGE_MAX = 1024;  // >= SMs x resident scatter CTAs per SM
 constexpr size_t SMEM_LIMIT = 227 * 1024;
@@ -603,6 +604,7 @@ struct Runner {
     static constexpr int VB = HasVal<V>::value ? sizeof(V) : 0;
     // histogram staging = one scatter tile (the largest KPB of this key/value type)
     static constexpr int HIST_CAP = ScatterCfg<KB, VB>::THREADS * ScatterCfg<KB, VB>::KPT;
+    static constexpr int HIST_STAGES = HRS_HIST_STAGES > 0 ? HRS_HIST_STAGES : (ScatterCfg<KB, VB>::SMALL ? 2 : 3);
     using SC = ScatterCfg<KB, (VB == 0 ? 4 : VB)>;
 
     static hrs_status init(const Plan &pl, void *temp, cudaStream_t st, int sms, int root_class, int counting,
