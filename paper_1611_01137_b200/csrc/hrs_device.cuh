@@ -320,6 +320,12 @@ __device__ __forceinline__ void bulk_g2s(void *dst, const void *src, uint32_t by
         "l"(src), "r"(bytes), "r"(smem_u32(bar)), "l"(pol)
         : "memory");
 }
+// 16-byte asynchronous copy global -> shared (a work-list entry fetched ahead of its use)
+__device__ __forceinline__ void cp_async16(void *dst, const void *src) {
+    asm volatile("cp.async.ca.shared.global [%0], [%1], 16;\ncp.async.commit_group;" ::"r"(smem_u32(dst)), "l"(src)
+                 : "memory");
+}
+__device__ __forceinline__ void cp_async_wait_all() { asm volatile("cp.async.wait_all;" ::: "memory"); }
 
 // A staged segment of `count` elements starting at global `src`, inside a buffer
 // [base, limit): one bulk copy moves the 16-byte aligned SUPERSET of the segment (up to
@@ -2287,6 +2293,14 @@ struct CntGeom {
     __device__ __forceinline__ static uint32_t phys(uint32_t w) { return w ^ ((w >> 5) & (PW - 1u)); }
 };
 
+// a copy the compiler cannot see through: values recomputed after a barrier are not
+// kept live across it (register pressure)
+__device__ __forceinline__ uint32_t opaque(uint32_t x) {
+    uint32_t y;
+    asm volatile("mov.b32 %0, %1;" : "=r"(y) : "r"(x));
+    return y;
+}
+
 // sum of the eight 4-bit fields of x
 __device__ __forceinline__ uint32_t nib_sum(uint32_t x) {
     x = (x & 0x0F0F0F0Fu) + ((x >> 4) & 0x0F0F0F0Fu);
@@ -2306,7 +2320,11 @@ struct LocalCntSmem {
     static constexpr size_t off_wsum = align16(off_red + sizeof(K) * 2 * W);
     static constexpr size_t off_cnt = align16(off_wsum + sizeof(uint32_t) * 16);
     static constexpr size_t off_pref = off_cnt + sizeof(uint32_t) * G::NW;
-    static constexpr size_t off_comp = align16(off_pref + sizeof(uint16_t) * G::NW);
+    // tie runs sorted before the write-out: runs of two or more records (at most CAP / 2),
+    // with RECON only runs of three or more (the composite holds every sort bit, pairs are
+    // ordered at the write-out; at most CAP / 3)
+    static constexpr size_t off_runs = align16(off_pref + sizeof(uint16_t) * G::NW);
+    static constexpr size_t off_comp = align16(off_runs + sizeof(uint32_t) * (RECON ? CAP / 3 : CAP / 2));
     // RECON: the composites overwrite the key staging buffer (the keys are in registers)
     static constexpr size_t off_kst = align16(off_comp + (RECON ? 0 : sizeof(uint32_t) * CAP));
     static constexpr size_t kst_bytes = align16(sizeof(K) * (CAP + 32 / sizeof(K)));
@@ -2337,6 +2355,8 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
     uint32_t *wsum = reinterpret_cast<uint32_t *>(smem + L::off_wsum);
     uint32_t *cnt = reinterpret_cast<uint32_t *>(smem + L::off_cnt);
     uint16_t *pref = reinterpret_cast<uint16_t *>(smem + L::off_pref);
+    uint32_t *runs = reinterpret_cast<uint32_t *>(smem + L::off_runs);
+    uint32_t *nruns = wsum + 15;  // entries in runs[] (wsum[0 .. LC_SCAN / 32) hold the scan)
     auto kst = [&](int s) { return reinterpret_cast<K *>(smem + L::off_kst + s * L::kst_bytes); };
     auto vst = [&](int s) { return reinterpret_cast<VT *>(smem + L::off_vst + s * L::vst_bytes); };
     const int tid = threadIdx.x, lane = tid & 31, warp = tid >> 5;
@@ -2358,14 +2378,15 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
                                                          : prm.src_vals[SRC_OUT]);
     };
     // info[s]: 0 entry, 1 count, 2 hi_bit, 3 src, 4..5 offs, 6..8 key seg, 9..11 value seg
-    auto issue = [&](int s, uint32_t e) {
+    // the next entry of the list, fetched while the current bucket is sorted
+    LocalEntry *const ahead = reinterpret_cast<LocalEntry *>(info + 16 * NSTAGE + 4);
+    auto issue = [&](int s, uint32_t e, const LocalEntry &en) {
         uint32_t *in = info + 16 * s;
         in[0] = e;
         if (e >= nent) {
             mbar_arrive_expect_tx(&bar[s], 0);  // completes the phase: the waiters see the end
             return;
         }
-        const LocalEntry en = prm.list[e];
         in[1] = en.count;
         in[2] = en.hi_bit;
         in[3] = en.src;
@@ -2403,8 +2424,14 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
     if (tid == 0) {
         for (int s = 0; s < NSTAGE; ++s) mbar_init(&bar[s], 1);
         mbar_fence_init();
-        for (int s = 0; s < NSTAGE; ++s) issue(s, blockIdx.x + s * gridDim.x);
+        for (int s = 0; s < NSTAGE; ++s) {
+            const uint32_t e = blockIdx.x + s * gridDim.x;
+            LocalEntry en{};
+            if (e < nent) en = prm.list[e];
+            issue(s, e, en);
+        }
         info[16 * NSTAGE] = blockIdx.x + NSTAGE * gridDim.x;  // next entry to issue
+        *nruns = 0;
     }
     __syncthreads();
 
@@ -2419,6 +2446,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
         __syncthreads();
         const uint32_t e_id = in[0];
         if (e_id >= nent) break;
+        if (tid == 0 && info[16 * NSTAGE] < nent) cp_async16(ahead, prm.list + info[16 * NSTAGE]);
         const uint32_t count = in[1];
         const int hi_bit = static_cast<int>(in[2]);
         const uint32_t src = in[3];
@@ -2559,73 +2587,80 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
                 uint32_t *comp = RECON ? reinterpret_cast<uint32_t *>(ks)
                                        : reinterpret_cast<uint32_t *>(smem + L::off_comp);
                 // slot = prefix of the word + counts of the smaller values in the word + the
-                // record's own rank among the ties; the record that counted first (on == 0)
-                // of a value held by r > 1 records owns that tie run: run[c] = start | r << 16
-                uint32_t run[KPT];
+                // record's own rank among the ties.  The record that counted first (on == 0)
+                // of a value held by r > 1 records owns that tie run.  When the composite holds
+                // every sort bit (!low) a pair is put in order at the write-out (min / max of the
+                // two neighbours); longer runs, and every run when key bits below the composite
+                // decide (low), go to a list that the whole CTA sorts before the write-out
+                const bool low = clo > begin_bit;
+                const uint32_t r0 = low ? 2u : 3u;
 #pragma unroll
                 for (int c = 0; c < KPT; ++c) {
                     const uint32_t e = c * THREADS + tid;
-                    run[c] = 0;
                     if (e < count) {
                         const uint32_t ph = rec[c] & 0xFFFFu, sh = (rec[c] >> 16) & 31u, on = rec[c] >> 24;
                         const uint32_t w = cnt[ph];
                         const uint32_t slot = pref[ph] + nib_sum(w & ((1u << sh) - 1u)) + on;
                         comp[slot] = cv[c];
                         const uint32_t r = (w >> sh) & 15u;
-                        if (on == 0 && r > 1) run[c] = slot | (r << 16);
+                        if (on == 0 && r >= r0) runs[atomicAdd(nruns, 1u)] = slot | (r << 16);
                     }
                 }
                 __syncthreads();  // B5
                 for (int i = tid; i < G::NW; i += THREADS) cnt[i] = 0;
-                // tie runs (equal counted value, at most 15 records): insertion sort by the
-                // rest of the composite, then the key bits below it, then the index
-                const bool low = clo > begin_bit;
-                const int lb = clo - begin_bit;
-                const K lmask = lb >= KBITS ? ~K(0) : ((K(1) << lb) - 1);
-                auto less = [&](uint32_t x, uint32_t y) -> bool {
-                    if ((x >> IB) != (y >> IB)) return x < y;
-                    if (low) {
-                        const K lx = (kin_map(ksp[x & IMASK]) >> begin_bit) & lmask,
-                                ly = (kin_map(ksp[y & IMASK]) >> begin_bit) & lmask;
-                        if (lx != ly) return lx < ly;
-                    }
-                    return x < y;
-                };
-#pragma unroll
-                for (int c = 0; c < KPT; ++c) {
-                    if (run[c]) {
-                        uint32_t *rb = comp + (run[c] & 0xFFFFu);
-                        const uint32_t r = run[c] >> 16;
-                        if (r == 2) {  // most tie runs are pairs
-                            const uint32_t x = rb[0], y = rb[1];
-                            if (low ? less(y, x) : y < x) {
-                                rb[0] = y;
-                                rb[1] = x;
-                            }
-                            continue;
+                const uint32_t nr = *nruns;
+                if (nr) {
+                    // tie runs (equal counted value, at most 15 records): insertion sort by the
+                    // rest of the composite, then the key bits below it, then the index
+                    const int lb = clo - begin_bit;
+                    const K lmask = lb >= KBITS ? ~K(0) : ((K(1) << lb) - 1);
+                    auto less = [&](uint32_t x, uint32_t y) -> bool {
+                        if ((x >> IB) != (y >> IB)) return x < y;
+                        if (low) {
+                            const K lx = (kin_map(ksp[x & IMASK]) >> begin_bit) & lmask,
+                                    ly = (kin_map(ksp[y & IMASK]) >> begin_bit) & lmask;
+                            if (lx != ly) return lx < ly;
                         }
+                        return x < y;
+                    };
+                    for (uint32_t q = tid; q < nr; q += THREADS) {
+                        const uint32_t rn = runs[q];
+                        uint32_t *rb = comp + (rn & 0xFFFFu);
+                        const uint32_t r = rn >> 16;
                         for (uint32_t i = 1; i < r; ++i) {
                             const uint32_t x = rb[i];
                             int j = static_cast<int>(i) - 1;
                             while (j >= 0) {
                                 const uint32_t y = rb[j];
-                                if (low ? !less(x, y) : !(x < y)) break;
+                                if (!less(x, y)) break;
                                 rb[j + 1] = y;
                                 --j;
                             }
                             rb[j + 1] = x;
                         }
                     }
+                    __syncthreads();  // B6
                 }
-                __syncthreads();  // B6
                 // write-out: RECON rebuilds the key from the bits above thi (common to
                 // the bucket) and the composite's sort field; otherwise it is gathered
                 const K khigh = thi >= KBITS ? K(0) : (aa & ~((K(1) << thi) - 1));
+                const uint32_t fs2 = opaque(static_cast<uint32_t>(FS));
 #pragma unroll
                 for (int c = 0; c < KPT; ++c) {
                     const uint32_t e = c * THREADS + tid;
                     if (e < count) {
-                        const uint32_t x = comp[e], ix = x & IMASK;
+                        uint32_t x = comp[e];
+                        if (!low) {
+                            // first of a run: the smaller of itself and its successor; last: the
+                            // larger of its predecessor and itself; inside a (sorted) longer run
+                            // or alone: itself
+                            const uint32_t xp = comp[e > 0 ? e - 1 : 0], xn = comp[e + 1 < L::CAP ? e + 1 : e];
+                            const uint32_t v = x >> fs2;
+                            const bool sp = e > 0 && (xp >> fs2) == v, sn = e + 1 < count && (xn >> fs2) == v;
+                            if (sn && !sp) x = min(x, xn);
+                            if (sp && !sn) x = max(x, xp);
+                        }
+                        const uint32_t ix = x & IMASK;
                         kd[e] = RECON ? kout_map(khigh | static_cast<K>(x >> IB)) : kout_raw(ksp[ix]);
                         if (HV) vd[e] = vsp[ix];
                     }
@@ -2633,10 +2668,12 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
             }
         }
     next_entry:
-        __syncthreads();  // staging buffer s, info[s], red[], comp are free
+        __syncthreads();  // staging buffer s, info[s], red[], comp, the run list are free
         if (tid == 0) {
+            *nruns = 0;
             fence_proxy_async();
-            issue(s, info[16 * NSTAGE]);
+            cp_async_wait_all();
+            issue(s, info[16 * NSTAGE], *ahead);
             info[16 * NSTAGE] += gridDim.x;
         }
     }
