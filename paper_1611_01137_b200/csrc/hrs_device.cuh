@@ -2280,6 +2280,9 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
 // -- about 30 shared-memory wavefronts per 32 records against about 42 for two LSD passes
 // (profiles/).
 constexpr int LC_SCAN = 256;  // threads that scan the counters
+#ifndef HRS_LC_RUNDIV
+#define HRS_LC_RUNDIV 3
+#endif
 
 template <int CB>
 struct CntGeom {
@@ -2322,9 +2325,10 @@ struct LocalCntSmem {
     static constexpr size_t off_pref = off_cnt + sizeof(uint32_t) * G::NW;
     // tie runs sorted before the write-out: runs of two or more records (at most CAP / 2),
     // with RECON only runs of three or more (the composite holds every sort bit, pairs are
-    // ordered at the write-out; at most CAP / 3)
+    // ordered at the write-out), at most RUNCAP of them (more: the bucket is handed off)
+    static constexpr int RUNCAP = RECON ? CAP / HRS_LC_RUNDIV : CAP / 2;
     static constexpr size_t off_runs = align16(off_pref + sizeof(uint16_t) * G::NW);
-    static constexpr size_t off_comp = align16(off_runs + sizeof(uint32_t) * (RECON ? CAP / 3 : CAP / 2));
+    static constexpr size_t off_comp = align16(off_runs + sizeof(uint32_t) * RUNCAP);
     // RECON: the composites overwrite the key staging buffer (the keys are in registers)
     static constexpr size_t off_kst = align16(off_comp + (RECON ? 0 : sizeof(uint32_t) * CAP));
     static constexpr size_t kst_bytes = align16(sizeof(K) * (CAP + 32 / sizeof(K)));
@@ -2603,12 +2607,19 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
                         const uint32_t slot = pref[ph] + nib_sum(w & ((1u << sh) - 1u)) + on;
                         comp[slot] = cv[c];
                         const uint32_t r = (w >> sh) & 15u;
-                        if (on == 0 && r >= r0) runs[atomicAdd(nruns, 1u)] = slot | (r << 16);
+                        if (on == 0 && r >= r0) {
+                            const uint32_t q = atomicAdd(nruns, 1u);
+                            if (q < L::RUNCAP) runs[q] = slot | (r << 16);
+                        }
                     }
                 }
                 __syncthreads();  // B5
                 for (int i = tid; i < G::NW; i += THREADS) cnt[i] = 0;
                 const uint32_t nr = *nruns;
+                if (nr > L::RUNCAP) {  // more tie runs than the list holds: k_local takes the bucket
+                    if (tid == 0) hand_off(offs, count, hi_bit, src);
+                    goto next_entry;
+                }
                 if (nr) {
                     // tie runs (equal counted value, at most 15 records): insertion sort by the
                     // rest of the composite, then the key bits below it, then the index
