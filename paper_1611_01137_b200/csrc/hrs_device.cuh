@@ -1591,14 +1591,11 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
             // ---- B: fold the warp counters into first slots; digit starts and bases
             auto fold = [&]() {
                 __syncthreads();  // counts complete
-                uint32_t v[W];
+                // (the W counters of digit tid are read twice rather than kept: registers)
                 uint32_t t = 0, incl = 0;
                 if (tid < RADIX) {
 #pragma unroll
-                    for (int w = 0; w < W; ++w) {
-                        v[w] = cnt[w * RADIX + tid];
-                        t += v[w];
-                    }
+                    for (int w = 0; w < W; ++w) t += cnt[w * RADIX + tid];
                     incl = t;
 #pragma unroll
                     for (int o = 1; o < 32; o <<= 1) {
@@ -1622,8 +1619,9 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
                     }
 #pragma unroll
                     for (int w = 0; w < W; ++w) {
+                        const uint32_t x = cnt[w * RADIX + tid];
                         cnt[w * RADIX + tid] = run;
-                        run += v[w];
+                        run += x;
                     }
                 }
                 __syncthreads();  // first slots published
