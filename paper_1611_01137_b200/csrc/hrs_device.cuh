@@ -810,166 +810,118 @@ struct HistParams {
     int kind;  // hrs_key_kind: keys still in the input go through the bijection
 };
 
-template <typename K, int THREADS, int NSTAGE, int CAP>
-struct HistSmem {
-    static constexpr int W = THREADS / 32;
-    static constexpr size_t off_bar = 0;
-    static constexpr size_t off_info = align16(sizeof(uint64_t) * NSTAGE);
-    static constexpr size_t off_wh = align16(off_info + sizeof(uint32_t) * 8 * NSTAGE);
-    static constexpr size_t off_stage = align16(off_wh + sizeof(uint32_t) * 2 * RADIX);
-    static constexpr size_t stage_elems = CAP + 32 / sizeof(K);
-    static constexpr size_t bytes = off_stage + NSTAGE * align16(sizeof(K) * stage_elems);
+// One CTA walks a contiguous run of tiles [tb, te) (the same runs as k_scatter): per tile a
+// block histogram of the digit (plain shared atomics: on B200 they run at the same rate for
+// any skew, profiles/r01_micro_hist.txt), the tile's prefix within its bucket segment and
+// its descriptor for the scatter.  The keys come straight from global memory in 16-byte
+// vectors (no staging: every resident CTA keeps a whole tile of loads in flight), and one
+// barrier per tile suffices: the histograms and the tile records are double-buffered, the
+// counts of tile i are folded in after the barrier that ends its counting.
+#ifndef HRS_HIST_MINB
+#define HRS_HIST_MINB 4
+#endif
+// element q of a 16-byte vector of keys (no address taken: the vector stays in registers)
+template <typename K>
+__device__ __forceinline__ K vec_elem(const uint4 &v, int q) {
+    if constexpr (sizeof(K) == 4) return static_cast<K>(q == 0 ? v.x : q == 1 ? v.y : q == 2 ? v.z : v.w);
+    else return static_cast<K>(q == 0 ? (static_cast<unsigned long long>(v.y) << 32 | v.x)
+                                      : (static_cast<unsigned long long>(v.w) << 32 | v.z));
+}
+struct HistTile {
+    uint64_t offs;
+    uint32_t count, bucket, flush, src;
 };
 
-template <typename K, int THREADS, int NSTAGE, int CAP, bool TY>
-__global__ void __launch_bounds__(THREADS) k_hist(HistParams prm) {
+template <typename K, int THREADS, int CAP, bool TY>
+__global__ void __launch_bounds__(THREADS, HRS_HIST_MINB) k_hist(HistParams prm) {
     pdl_wait();
-    using L = HistSmem<K, THREADS, NSTAGE, CAP>;
     static_assert(THREADS >= RADIX, "one thread per digit for the tile prefixes");
     constexpr int VK = 16 / sizeof(K);
-    extern __shared__ __align__(16) unsigned char smem[];
-    uint64_t *bar = reinterpret_cast<uint64_t *>(smem + L::off_bar);
-    // info[s]: 0 valid, 1 count, 2 bucket, 3 pad, 4 i0, 5 i1, 6 last tile of its bucket segment,
-    //          7 tile index
-    uint32_t *info = reinterpret_cast<uint32_t *>(smem + L::off_info);
-    uint32_t *wh = reinterpret_cast<uint32_t *>(smem + L::off_wh);
-    auto stage = [&](int s) {
-        return reinterpret_cast<K *>(smem + L::off_stage + s * align16(sizeof(K) * L::stage_elems));
-    };
-    __shared__ const K *src_of[NSTAGE];  // key buffer of the tile in stage s
-    const int tid = threadIdx.x, warp = tid >> 5;
+    constexpr int NV = (CAP / VK + THREADS - 1) / THREADS;  // whole vectors of a tile per thread
+    __shared__ uint32_t wh[2][RADIX];
+    __shared__ HistTile ti[2];
+    __shared__ TileCursor cur;
+    const int tid = threadIdx.x;
     const unsigned long long al = prm.ctl->alloc[prm.p];
     const uint32_t T = alloc_tiles(al), NB = alloc_buckets(al);
-    // a contiguous run of tiles per CTA (the same runs as k_scatter): bucket histograms
-    // are flushed once per bucket segment, the last segment is also kept per CTA
     const uint32_t tb = range_begin(T, blockIdx.x, gridDim.x), te = range_begin(T, blockIdx.x + 1, gridDim.x);
     if (tb >= te) {
         if (tid == 0) prm.seg_meta[blockIdx.x] = RangeMeta{EMPTY_RANGE, EMPTY_RANGE};
         return;
     }
-    const uint64_t pol = policy_evict_first();
-    __shared__ TileCursor cur;
-    __shared__ uint64_t offs_of[NSTAGE];
-
-    auto issue = [&](int s) {
-        uint32_t *in = info + 8 * s;
-        in[0] = cur.valid();
-        if (!cur.valid()) return;
-        const uint64_t o = cur.offs();
-        const uint32_t cnt = cur.count();
-        const K *keys = static_cast<const K *>(prm.src_keys[cur.bk.src]);
-        src_of[s] = keys;
-        Seg sg;
-        const uint32_t bytes = seg_plan(keys + o, cnt, keys, keys + prm.n, sg);
-        in[1] = cnt;
-        in[2] = cur.b;
-        in[3] = sg.pad;
-        in[4] = static_cast<uint32_t>(sg.i0);
-        in[5] = static_cast<uint32_t>(sg.i1);
-        in[6] = cur.last_of_bucket() || cur.t + 1 == te;
-        in[7] = cur.t;
-        offs_of[s] = o;
-        mbar_arrive_expect_tx(&bar[s], bytes);
-        seg_issue(stage(s), keys + o, sg, &bar[s], pol);
+    auto publish = [&](int slot) {  // tid 0: the cursor's tile into ti[slot], then advance
+        HistTile h;
+        h.offs = cur.offs();
+        h.count = cur.count();
+        h.bucket = cur.b;
+        h.flush = cur.last_of_bucket() || cur.t + 1 == te;
+        h.src = cur.bk.src;
+        ti[slot] = h;
         cur.next();
     };
     if (tid == 0) {
-        for (int s = 0; s < NSTAGE; ++s) mbar_init(&bar[s], 1);
-        mbar_fence_init();
         cur.start(prm.buckets, NB, tb, te, prm.kpb);
-        const uint32_t fb = cur.b;
-        for (int s = 0; s < NSTAGE; ++s) issue(s);
-        prm.seg_meta[blockIdx.x].first_bucket = fb;
+        prm.seg_meta[blockIdx.x].first_bucket = cur.b;
+        publish(0);
     }
-    for (int i = tid; i < 2 * RADIX; i += THREADS) wh[i] = 0;
+    for (int i = tid; i < 2 * RADIX; i += THREADS) (&wh[0][0])[i] = 0;
     __syncthreads();
-    uint32_t seg_run = 0;            // digit tid: count of the current bucket segment before this tile
-    bool first_seg = true;           // inside the CTA's first bucket segment (its carry applies)
+    uint32_t seg_run = 0;   // digit tid: count of the current bucket segment before this tile
+    bool first_seg = true;  // inside the CTA's first bucket segment (its carry applies)
     for (uint32_t t = tb, it = 0; t < te; ++t, ++it) {
-        const int s = static_cast<int>(it % NSTAGE);
-        const uint32_t par = (it / NSTAGE) & 1u;
-        const uint32_t *in = info + 8 * s;
-        const uint32_t count = in[1], bucket = in[2];
-        const bool flush = in[6] != 0;
-        Seg sg;
-        sg.pad = in[3];
-        sg.i0 = static_cast<int32_t>(in[4]);
-        sg.i1 = static_cast<int32_t>(in[5]);
-        const uint64_t toffs = offs_of[s];
-        const K *src = src_of[s] + toffs;
-        const bool mapin = TY && prm.kind != 0 && src_of[s] == static_cast<const K *>(prm.src_keys[SRC_IN]);
-        // one block histogram per tile, double-buffered: the counts of tile i are read
-        // and cleared while tile i + 1 is counted into the other buffer
-        uint32_t *my = wh + (it & 1u) * RADIX;
+        const HistTile in = ti[it & 1u];
+        // (selected, not indexed: a dynamic index would copy the parameters to local memory)
+        const void *kb = in.src == SRC_IN ? prm.src_keys[SRC_IN] : in.src == SRC_AUX ? prm.src_keys[SRC_AUX] : prm.src_keys[SRC_OUT];
+        const K *src = static_cast<const K *>(kb) + in.offs;
+        const bool mapin = TY && prm.kind != 0 && in.src == SRC_IN;
+        // [0, h0) before the first 16-byte boundary, nvec whole vectors, the tail after them
+        const uint32_t mis = static_cast<uint32_t>(reinterpret_cast<uintptr_t>(src) / sizeof(K)) % VK;
+        const uint32_t h0 = min(in.count, (VK - mis) % VK);
+        const uint32_t nvec = (in.count - h0) / VK, tail0 = h0 + nvec * VK;
+        const uint4 *vp = reinterpret_cast<const uint4 *>(src + h0);
+        uint4 w[NV];
+#pragma unroll
+        for (int j = 0; j < NV; ++j) {
+            const uint32_t v = tid + j * THREADS;
+            if (v < nvec) w[j] = __ldcs(vp + v);
+        }
+        const uint32_t ne = h0 + (in.count - tail0);  // edge elements (< 2 VK)
+        K ek = K(0);
+        if (static_cast<uint32_t>(tid) < ne) ek = src[static_cast<uint32_t>(tid) < h0 ? tid : tail0 + (tid - h0)];
+        if (tid == 0 && t + 1 < te) publish((it + 1) & 1u);
         // tile descriptor and tile-ordered prefix for the scatter
         if (tid < RADIX) prm.tile_pref[static_cast<uint64_t>(t) * RADIX + tid] = seg_run;
         if (tid == 0) {
             TileDesc td;
-            td.offs = toffs;
-            td.count = count;
-            td.bucket = bucket;
+            td.offs = in.offs;
+            td.count = in.count;
+            td.bucket = in.bucket;
             td.carry_row = first_seg ? blockIdx.x : EMPTY_RANGE;
             td.pad = 0;
             prm.tiles[t] = td;
         }
-        if (!HRS_WAIT1 || warp == 0) mbar_wait(&bar[s], par);  // one warp waits, the barrier releases the rest
-        if (HRS_WAIT1) __syncthreads();
-        const K *sb = stage(s);
-        // 16-byte vectors over the staged superset: vector v holds elements ibase + v*VK
-        // .. + VK - 1 (element i = position - pad); the vectors wholly inside [0, count)
-        // are counted without checks, the (at most two) partial edge vectors per element
-        if (sg.i1 > sg.i0) {
-            const int32_t q0 = (static_cast<int32_t>(sg.pad) + sg.i0) / VK;
-            const int32_t nq = (sg.i1 - sg.i0) / VK;
-            const uint4 *vb = reinterpret_cast<const uint4 *>(sb) + q0;
-            const int32_t ibase = q0 * VK - static_cast<int32_t>(sg.pad);
-            const int32_t vlo = ibase < 0 ? 1 : 0;
-            const int32_t vhi = min(nq, (static_cast<int32_t>(count) - ibase) / VK);
-#pragma unroll 4
-            for (int32_t v = vlo + tid; v < vhi; v += THREADS) {
-                const uint4 w = vb[v];
-                const K *kk = reinterpret_cast<const K *>(&w);
+        uint32_t *my = wh[it & 1u];
+        auto dig = [&](K k) { return digit_of(mapin ? key_map(k, prm.kind, false) : k, prm.lo, prm.mask); };
 #pragma unroll
-                for (int j = 0; j < VK; ++j) atomicAdd(&my[digit_of(mapin ? key_map(kk[j], prm.kind, false) : kk[j], prm.lo, prm.mask)], 1u);
-            }
-            // edge vectors: v = 0 when it starts before element 0, v = vhi when partial
-            const int32_t ve = tid == 0 ? (vlo ? 0 : -1) : (tid == 1 && vhi < nq && vhi >= vlo ? vhi : -1);
-            if (ve >= 0) {
-                const uint4 w = vb[ve];
-                const K *kk = reinterpret_cast<const K *>(&w);
-                const int32_t i = ibase + ve * VK;
+        for (int j = 0; j < NV; ++j) {
+            if (tid + j * THREADS < nvec) {
 #pragma unroll
-                for (int j = 0; j < VK; ++j)
-                    if (i + j >= 0 && i + j < static_cast<int32_t>(count))
-                        atomicAdd(&my[digit_of(mapin ? key_map(kk[j], prm.kind, false) : kk[j], prm.lo, prm.mask)], 1u);
+                for (int q = 0; q < VK; ++q) atomicAdd(&my[dig(vec_elem<K>(w[j], q))], 1u);
             }
         }
-        // elements the copy did not cover (segments at the ends of the buffer) from global
-        if (!seg_full(sg, count)) {
-            const uint32_t h = sg.i1 > sg.i0 ? static_cast<uint32_t>(max(sg.i0, 0)) : count;
-            const uint32_t tl = sg.i1 > sg.i0 ? static_cast<uint32_t>(min(sg.i1, static_cast<int32_t>(count))) : count;
-            for (uint32_t j = tid; j < h + (count - tl); j += THREADS) {
-                const uint32_t i = j < h ? j : tl + (j - h);
-                atomicAdd(&my[digit_of(mapin ? key_map(src[i], prm.kind, false) : src[i], prm.lo, prm.mask)], 1u);
-            }
-        }
-        __syncthreads();
-        if (tid == 0) {
-            fence_proxy_async();
-            issue(s);
-        }
-        // segment count so far
+        if (static_cast<uint32_t>(tid) < ne) atomicAdd(&my[dig(ek)], 1u);
+        __syncthreads();  // the tile's counts are complete; ti[(it + 1) & 1] is published
         if (tid < RADIX) {
             seg_run += my[tid];
-            my[tid] = 0;
+            my[tid] = 0;  // (counted into again two tiles on, after the next barrier)
         }
-        if (flush) {
+        if (in.flush) {
             const bool last_seg = t + 1 == te;
             if (tid < RADIX) {
-                if (seg_run) atomicAdd(&prm.tot[static_cast<uint64_t>(bucket) * RADIX + tid], seg_run);
+                if (seg_run) atomicAdd(&prm.tot[static_cast<uint64_t>(in.bucket) * RADIX + tid], seg_run);
                 if (last_seg) prm.seg_last[static_cast<uint64_t>(blockIdx.x) * RADIX + tid] = seg_run;
             }
-            if (last_seg && tid == 0) prm.seg_meta[blockIdx.x].last_bucket = bucket;
+            if (last_seg && tid == 0) prm.seg_meta[blockIdx.x].last_bucket = in.bucket;
             seg_run = 0;
             first_seg = false;
         }
@@ -1245,22 +1197,48 @@ __device__ void classify_bucket(const ClassifyParams &prm, const Bucket &bk, uin
 // Carry of every hist/scatter CTA: the digit counts of the tiles of its first bucket
 // that precede its range (an exclusive scan over CTAs, segmented by bucket).  One
 // thread per digit walks the CTAs; the loads are batched so their latencies overlap.
+// The carry of every CTA range (the digit counts of the tiles of its first bucket that lie
+// in earlier ranges): a scan over the ranges, segmented where a bucket ends, one per digit.
+// CARRY_CTAS blocks split the digits; inside a block the ranges are cut into
+// THREADS / (RADIX / CARRY_CTAS) chunks scanned in parallel: first each chunk's outgoing run
+// assuming none comes in (and whether an incoming run would flow through it), then the runs
+// entering the chunks in chunk order, then each chunk's scan again from its true incoming
+// run, writing the carries.
+constexpr int CARRY_CTAS = 8;
 template <int THREADS>
-__device__ void range_carries(const ClassifyParams &prm) {
+__device__ void range_carries(const ClassifyParams &prm, uint32_t part) {
+    constexpr int DPB = RADIX / CARRY_CTAS;  // digits per block
+    constexpr int NQ = THREADS / DPB;        // chunks of ranges
     constexpr int B = 32;
+    static_assert(THREADS % DPB == 0 && NQ >= 1, "carry geometry");
+    __shared__ uint32_t out_run[NQ][DPB], out_pass[NQ][DPB];
     const RangeMeta *__restrict__ meta = prm.seg_meta;
     const uint32_t *__restrict__ segl = prm.seg_last;
     uint32_t *__restrict__ carry = prm.carry;
-    for (int d = threadIdx.x; d < RADIX; d += THREADS) {
-        uint32_t run = 0, prev_last = EMPTY_RANGE;
-        for (uint32_t c0 = 0; c0 < prm.ranges; c0 += B) {
+    const uint32_t dl = threadIdx.x % DPB, d = part * DPB + dl, q = threadIdx.x / DPB;
+    const uint32_t R = prm.ranges;
+    const uint32_t c0 = static_cast<uint32_t>((static_cast<uint64_t>(R) * q) / NQ);
+    const uint32_t c1 = static_cast<uint32_t>((static_cast<uint64_t>(R) * (q + 1)) / NQ);
+    uint32_t last0 = EMPTY_RANGE;  // last bucket of the last non-empty range before c0
+    for (uint32_t c = c0; c-- > 0;) {
+        const RangeMeta m = meta[c];
+        if (m.first_bucket != EMPTY_RANGE) {
+            last0 = m.last_bucket;
+            break;
+        }
+    }
+    // scan of the chunk from run `in`; WRITE: store the carries
+    auto scan = [&](uint32_t in, bool write, bool &pass) -> uint32_t {
+        uint32_t run = in, prev_last = last0;
+        pass = true;
+        for (uint32_t cb = c0; cb < c1; cb += B) {
             RangeMeta m[B];
             uint32_t sl[B];
 #pragma unroll
             for (int i = 0; i < B; ++i) {
-                if (c0 + i < prm.ranges) {
-                    m[i] = meta[c0 + i];
-                    sl[i] = segl[static_cast<uint64_t>(c0 + i) * RADIX + d];
+                if (cb + i < c1) {
+                    m[i] = meta[cb + i];
+                    sl[i] = segl[static_cast<uint64_t>(cb + i) * RADIX + d];
                 } else {
                     m[i].first_bucket = EMPTY_RANGE;
                     m[i].last_bucket = EMPTY_RANGE;
@@ -1270,13 +1248,25 @@ __device__ void range_carries(const ClassifyParams &prm) {
 #pragma unroll
             for (int i = 0; i < B; ++i) {
                 if (m[i].first_bucket == EMPTY_RANGE) continue;
-                const uint32_t car = m[i].first_bucket == prev_last ? run : 0u;
-                carry[static_cast<uint64_t>(c0 + i) * RADIX + d] = car;
+                const bool cont = m[i].first_bucket == prev_last;
+                const uint32_t car = cont ? run : 0u;
+                if (write) carry[static_cast<uint64_t>(cb + i) * RADIX + d] = car;
+                pass = pass && cont && m[i].first_bucket == m[i].last_bucket;
                 run = (m[i].first_bucket == m[i].last_bucket) ? car + sl[i] : sl[i];
                 prev_last = m[i].last_bucket;
             }
         }
+        return run;
+    };
+    bool pass;
+    uint32_t inc = 0;  // the run entering chunk q
+    if (NQ > 1) {
+        out_run[q][dl] = scan(0u, false, pass);
+        out_pass[q][dl] = pass;
+        __syncthreads();
+        for (uint32_t r = 0; r < q; ++r) inc = out_run[r][dl] + (out_pass[r][dl] ? inc : 0u);
     }
+    scan(inc, true, pass);
 }
 
 template <int THREADS>
@@ -1285,11 +1275,12 @@ __global__ void __launch_bounds__(THREADS) k_classify(ClassifyParams prm) {
     __shared__ uint32_t scratch[11 * NBINS];  // classify_bucket: 7 rows, merge_groups: 3 rows + 8 words
     const uint32_t nb = alloc_buckets(prm.ctl->alloc[prm.p]);
     if (nb == 0) return;  // nothing reached this pass
-    if (blockIdx.x == gridDim.x - 1) {
-        range_carries<THREADS>(prm);
-        if (gridDim.x > 1) return;
+    // the last CARRY_CTAS blocks compute the range carries, the others classify buckets
+    const uint32_t nblk = gridDim.x - CARRY_CTAS;
+    if (blockIdx.x >= nblk) {
+        range_carries<THREADS>(prm, blockIdx.x - nblk);
+        return;
     }
-    const uint32_t nblk = gridDim.x > 1 ? gridDim.x - 1 : 1;
     for (uint32_t b = blockIdx.x; b < nb; b += nblk) {
         const Bucket bk = prm.buckets[b];
         classify_bucket<THREADS>(prm, bk, b, scratch);

@@ -140,9 +140,6 @@ struct ScatterCfg {
 #ifndef HRS_HIST_THREADS
 #define HRS_HIST_THREADS 256
 #endif
-#ifndef HRS_HIST_STAGES
-#define HRS_HIST_STAGES 0  // 0: 2 for the 32-bit scatter shape (28 KB stages, 3 CTAs / SM), else 3
-#endif
 constexpr int HIST_THREADS = HRS_HIST_THREADS;
 constexpr int CLASSIFY_THREADS = 256;
 constexpr uint32_t RANGE_MAX = 1024;  // >= SMs x resident scatter CTAs per SM
@@ -604,7 +601,6 @@ struct Runner {
     static constexpr int VB = HasVal<V>::value ? sizeof(V) : 0;
     // histogram staging = one scatter tile (the largest KPB of this key/value type)
     static constexpr int HIST_CAP = ScatterCfg<KB, VB>::THREADS * ScatterCfg<KB, VB>::KPT;
-    static constexpr int HIST_STAGES = HRS_HIST_STAGES > 0 ? HRS_HIST_STAGES : (ScatterCfg<KB, VB>::SMALL ? 2 : 3);
     using SC = ScatterCfg<KB, (VB == 0 ? 4 : VB)>;
 
     static hrs_status init(const Plan &pl, void *temp, cudaStream_t st, int sms, int root_class, int counting,
@@ -631,10 +627,9 @@ struct Runner {
     // the hist / classify grid of a pass (CTAs = contiguous tile runs): the hist
     // kernel's persistent grid, capped by the temp layout
     static hrs_status range_grid(const Plan &pl, int dev, int sms, uint32_t *G) {
-        auto fn = k_hist<K, HIST_THREADS, HIST_STAGES, HIST_CAP, TY>;
-        const size_t smem = HistSmem<K, HIST_THREADS, HIST_STAGES, HIST_CAP>::bytes;
+        auto fn = k_hist<K, HIST_THREADS, HIST_CAP, TY>;
         int grid = 0;
-        hrs_status s = grid_for(fn, HIST_THREADS, smem, dev, sms, &grid);
+        hrs_status s = grid_for(fn, HIST_THREADS, 0, dev, sms, &grid);
         if (s) return s;
         *G = std::min<uint32_t>(static_cast<uint32_t>(grid), pl.range_cap);
         return HRS_SUCCESS;
@@ -674,13 +669,9 @@ struct Runner {
         hp.tiles = at<TileDesc>(temp, pl.off_tiles);
         hp.tile_pref = at<uint32_t>(temp, pl.off_tile_pref);
         hp.ctl = at<Ctl>(temp, 0);
-        auto fn = k_hist<K, HIST_THREADS, HIST_STAGES, HIST_CAP, TY>;
-        const size_t smem = HistSmem<K, HIST_THREADS, HIST_STAGES, HIST_CAP>::bytes;
-        int grid = 0;
-        hrs_status s = grid_for(fn, HIST_THREADS, smem, dev, sms, &grid);  // sets the smem attribute
-        if (s) return s;
+        auto fn = k_hist<K, HIST_THREADS, HIST_CAP, TY>;
         LaunchScope ls(st, 1, p);
-        launch_pdl(fn, dim3(G), dim3(HIST_THREADS), smem, st, hp);
+        launch_pdl(fn, dim3(G), dim3(HIST_THREADS), 0, st, hp);
         return last_launch();
     }
 
@@ -720,7 +711,7 @@ struct Runner {
         hrs_status s = grid_for(fn, CLASSIFY_THREADS, 0, dev, sms, &grid);
         if (s) return s;
         // one block per bucket (up to the resident limit) plus the carry block
-        grid = static_cast<int>(std::min<uint64_t>(grid, std::max<uint64_t>(pl.bucket_cap, 1))) + 1;
+        grid = static_cast<int>(std::min<uint64_t>(grid, std::max<uint64_t>(pl.bucket_cap, 1))) + CARRY_CTAS;
         LaunchScope ls(st, 5, p);
         launch_pdl(fn, dim3(grid), dim3(CLASSIFY_THREADS), 0, st, cp);
         return last_launch();
