@@ -2557,12 +2557,19 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
         } else {
             const int FS = IB + (flo - clo);  // composite >> FS = counted value
             const uint32_t cmask = (1u << (thi - clo)) - 1u;
+            // the composites' buffer (RECON: the key staging buffer, whose keys are now in
+            // registers); low: key bits below the composite decide ties
+            uint32_t *const comp = RECON ? reinterpret_cast<uint32_t *>(ks) : reinterpret_cast<uint32_t *>(smem + L::off_comp);
+            const bool low = clo > begin_bit;
+            constexpr uint32_t SENT = 0xFFFFFFFFu;  // no composite (index bits 8191 > CAP)
+            static_assert(L::CAP < (1 << IB) - 1, "SENT is not a composite");
             uint32_t cv[KPT], rec[KPT];
 #pragma unroll
             for (int c = 0; c < KPT; ++c) {
                 const uint32_t e = c * THREADS + tid;
                 cv[c] = ((static_cast<uint32_t>(key[c] >> clo) & cmask) << IB) | e;
                 if (e < count) {
+                    if constexpr (RECON) comp[e] = SENT;  // (tie pairs swap into their first slot)
                     const uint32_t v = cv[c] >> FS;
                     const uint32_t ph = G::phys(v >> 3), sh = (v & 7u) * 4u;
                     const uint32_t on = (atomicAdd(&cnt[ph], 1u << sh) >> sh) & 15u;
@@ -2611,15 +2618,13 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
                     }
                 }
                 __syncthreads();  // B4
-                uint32_t *comp = RECON ? reinterpret_cast<uint32_t *>(ks)
-                                       : reinterpret_cast<uint32_t *>(smem + L::off_comp);
                 // slot = prefix of the word + counts of the smaller values in the word + the
                 // record's own rank among the ties.  The record that counted first (on == 0)
                 // of a value held by r > 1 records owns that tie run.  When the composite holds
-                // every sort bit (!low) a pair is put in order at the write-out (min / max of the
-                // two neighbours); longer runs, and every run when key bits below the composite
+                // every sort bit (!low) a pair is ordered without the list: here (RECON, atomic
+                // exchange into its first slot) or at the write-out (min / max of the two
+                // neighbours); longer runs, and every run when key bits below the composite
                 // decide (low), go to a list that the whole CTA sorts before the write-out
-                const bool low = clo > begin_bit;
                 const uint32_t r0 = low ? 2u : 3u;
 #pragma unroll
                 for (int c = 0; c < KPT; ++c) {
@@ -2628,8 +2633,19 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
                         const uint32_t ph = rec[c] & 0xFFFFu, sh = (rec[c] >> 16) & 31u, on = rec[c] >> 24;
                         const uint32_t w = cnt[ph];
                         const uint32_t slot = pref[ph] + nib_sum(w & ((1u << sh) - 1u)) + on;
-                        comp[slot] = cv[c];
                         const uint32_t r = (w >> sh) & 15u;
+                        if (RECON && r == 2u) {
+                            // (RECON: the composite holds every sort bit) a tie pair orders
+                            // itself: the second record to arrive swaps its composite in and
+                            // writes the two in order (the slots start as SENT)
+                            const uint32_t b0 = slot - on, old = atomicExch(&comp[b0], cv[c]);
+                            if (old != SENT) {
+                                comp[b0] = min(old, cv[c]);
+                                comp[b0 + 1] = max(old, cv[c]);
+                            }
+                        } else {
+                            comp[slot] = cv[c];
+                        }
                         if (on == 0 && r >= r0) {
                             const uint32_t q = atomicAdd(nruns, 1u);
                             if (q < L::RUNCAP) runs[q] = slot | (r << 16);
@@ -2684,7 +2700,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
                     const uint32_t e = c * THREADS + tid;
                     if (e < count) {
                         uint32_t x = comp[e];
-                        if (!low) {
+                        if (!RECON && !low) {
                             // first of a run: the smaller of itself and its successor; last: the
                             // larger of its predecessor and itself; inside a (sorted) longer run
                             // or alone: itself
