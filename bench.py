@@ -275,8 +275,10 @@ def run_hrs(args):
             per.setdefault(key, []).append(ms)
         kern = {k2: sum(v2) / args.steps for k2, v2 in per.items()}
         out["kernels_ms_per_step"] = {k2: round(v2, 4) for k2, v2 in sorted(kern.items())}
-        # dominant kernel: the scatter (2(K+V) bytes per record of every counting pass)
-        sc_bytes = sum(r * 2 * (kb + vb) for r in st["recs_in_pass"])
+        # dominant kernel: the scatter (2(K+V) bytes per record it moves: the records of every
+        # counting pass minus those of skipped buckets, reading #22)
+        skipped = st.get("skipped_recs_in_pass", [0] * len(st["recs_in_pass"]))
+        sc_bytes = sum((r - sk) * 2 * (kb + vb) for r, sk in zip(st["recs_in_pass"], skipped))
         sc_ms = sum(v2 for k2, v2 in kern.items() if k2.startswith("scatter"))
         traffic = None
         tpath = os.path.join(ROOT, "profiles", "traffic.json")
