@@ -116,8 +116,9 @@ constexpr uint32_t DEFAULT_MT_DIV = 4;
 #define HRS_SC64_THREADS 256
 #endif
 #ifndef HRS_SC64_KPT
-#define HRS_SC64_KPT 14  // measured (c4 uniform / AND-3 step): 16 x 1 buffer 7.80 / 17.5 ms, 12 x 2 7.66 / 16.1, 22 x 1 7.52 / 17.2;
-                         // one value buffer: 12 x 2 7.82 / 15.9, 14 x 2 7.56 / 15.6, 16 x 2 7.77 / 17.6
+#define HRS_SC64_KPT 15  // measured (c4 uniform / AND-3 step): 16 x 1 buffer 7.80 / 17.5 ms, 12 x 2 7.66 / 16.1, 22 x 1 7.52 / 17.2;
+                         // one value buffer: 12 x 2 7.82 / 15.9, 14 x 2 7.56 / 15.6, 16 x 2 7.77 / 17.6;
+                         // with the address table (PTR): 14 x 2 6.91, 15 x 2 6.86 (16 no longer fits two CTAs)
 #endif
 #ifndef HRS_SC64_MINB
 #define HRS_SC64_MINB 2
