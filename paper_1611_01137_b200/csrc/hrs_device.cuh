@@ -2306,6 +2306,11 @@ constexpr int LC_SCAN = 256;  // threads that scan the counters
 #ifndef HRS_LC_RUNDIV
 #define HRS_LC_RUNDIV 3
 #endif
+// the values of a bucket complete on their own barrier, waited for just before the
+// write-out: their load overlaps the count, scan and placement of the bucket
+#ifndef HRS_LC_VSPLIT
+#define HRS_LC_VSPLIT 1
+#endif
 
 template <int CB>
 struct CntGeom {
@@ -2340,8 +2345,9 @@ struct LocalCntSmem {
     using VT = ValT<V>;
     static constexpr bool HV = HasVal<V>::value;
     using G = CntGeom<CB>;
+    static constexpr bool VSPLIT = HRS_LC_VSPLIT && HV;  // [NSTAGE + s]: values of stage s
     static constexpr size_t off_bar = 0;
-    static constexpr size_t off_info = align16(sizeof(uint64_t) * NSTAGE);
+    static constexpr size_t off_info = align16(sizeof(uint64_t) * NSTAGE * (VSPLIT ? 2 : 1));
     static constexpr size_t off_red = align16(off_info + sizeof(uint32_t) * 16 * (NSTAGE + 1));
     static constexpr size_t off_wsum = align16(off_red + sizeof(K) * 2 * W);
     static constexpr size_t off_cnt = align16(off_wsum + sizeof(uint32_t) * 16);
@@ -2367,6 +2373,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
     using G = CntGeom<CB>;
     constexpr int IB = 13;     // index bits of a composite
     constexpr int CBITS = 19;  // sort bits of a composite
+    static_assert(CBITS <= 24, "a record's register holds the composite's key field below bit 24");
     constexpr uint32_t IMASK = (1u << IB) - 1u;
     constexpr int W = THREADS / 32;
     constexpr int KBITS = 8 * static_cast<int>(sizeof(K));
@@ -2412,6 +2419,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
         in[0] = e;
         if (e >= nent) {
             mbar_arrive_expect_tx(&bar[s], 0);  // completes the phase: the waiters see the end
+            if constexpr (L::VSPLIT) mbar_arrive_expect_tx(&bar[NSTAGE + s], 0);
             return;
         }
         in[1] = en.count;
@@ -2425,16 +2433,18 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
         in[6] = sk.pad;
         in[7] = static_cast<uint32_t>(sk.i0);
         in[8] = static_cast<uint32_t>(sk.i1);
+        uint32_t vbytes = 0;
         if (HV) {
             const VT *vbuf = srcv(en.src);
-            bytes += seg_plan(vbuf + en.offs, en.count, vbuf, vbuf + prm.n, sv);
+            vbytes = seg_plan(vbuf + en.offs, en.count, vbuf, vbuf + prm.n, sv);
             in[9] = sv.pad;
             in[10] = static_cast<uint32_t>(sv.i0);
             in[11] = static_cast<uint32_t>(sv.i1);
         }
-        mbar_arrive_expect_tx(&bar[s], bytes);
+        mbar_arrive_expect_tx(&bar[s], L::VSPLIT ? bytes : bytes + vbytes);
         seg_issue(kst(s), kbuf + en.offs, sk, &bar[s], pol);
-        if (HV) seg_issue(vst(s), srcv(en.src) + en.offs, sv, &bar[s], pol);
+        if constexpr (L::VSPLIT) mbar_arrive_expect_tx(&bar[NSTAGE + s], vbytes);
+        if (HV) seg_issue(vst(s), srcv(en.src) + en.offs, sv, &bar[L::VSPLIT ? NSTAGE + s : s], pol);
     };
     auto hand_off = [&](uint64_t offs, uint32_t count, int hi_bit, uint32_t src) {
         const uint32_t slot = atomicAdd(prm.fb_count, 1u);
@@ -2449,7 +2459,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
     };
     for (int i = tid; i < G::NW; i += THREADS) cnt[i] = 0;  // cleared again after every bucket
     if (tid == 0) {
-        for (int s = 0; s < NSTAGE; ++s) mbar_init(&bar[s], 1);
+        for (int s = 0; s < NSTAGE * (L::VSPLIT ? 2 : 1); ++s) mbar_init(&bar[s], 1);
         mbar_fence_init();
         for (int s = 0; s < NSTAGE; ++s) {
             const uint32_t e = blockIdx.x + s * gridDim.x;
@@ -2497,6 +2507,10 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
         const VT *vsrc = HV ? srcv(src) + offs : nullptr;
         K *ks = kst(s);
         VT *vs = HV ? vst(s) : nullptr;
+        // VSPLIT: every thread waits for the values itself before it reads them
+        auto vwait = [&]() {
+            if constexpr (L::VSPLIT) mbar_wait(&bar[NSTAGE + s], par);
+        };
         // elements the bulk copy did not cover (entries at the ends of a buffer): into
         // shared memory before anything is written (the entry may be sorted in place)
         if (!seg_full(sk, count) || (HV && !seg_full(sv, count))) {
@@ -2543,6 +2557,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
         if (nosort) {
             // every record has the same sort bits: the stable order is the input order
             if (src != SRC_OUT || typed) {
+                vwait();
 #pragma unroll
                 for (int c = 0; c < KPT; ++c) {
                     const uint32_t e = c * THREADS + tid;
@@ -2563,17 +2578,22 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
             const bool low = clo > begin_bit;
             constexpr uint32_t SENT = 0xFFFFFFFFu;  // no composite (index bits 8191 > CAP)
             static_assert(L::CAP < (1 << IB) - 1, "SENT is not a composite");
-            uint32_t cv[KPT], rec[KPT];
+            // one register per record from the count to the placement: the composite's key
+            // field (<= CBITS bits) and the record's rank among its ties (bits 24..27); the
+            // composite, counted value, word and nibble are recomputed from them (registers:
+            // five CTAs per SM where the shared memory allows)
+            const int VSH = flo - clo;  // key field >> VSH = counted value
+            uint32_t rec[KPT];
 #pragma unroll
             for (int c = 0; c < KPT; ++c) {
                 const uint32_t e = c * THREADS + tid;
-                cv[c] = ((static_cast<uint32_t>(key[c] >> clo) & cmask) << IB) | e;
+                const uint32_t kf = static_cast<uint32_t>(key[c] >> clo) & cmask;
                 if (e < count) {
                     if constexpr (RECON) comp[e] = SENT;  // (tie pairs swap into their first slot)
-                    const uint32_t v = cv[c] >> FS;
+                    const uint32_t v = kf >> VSH;
                     const uint32_t ph = G::phys(v >> 3), sh = (v & 7u) * 4u;
                     const uint32_t on = (atomicAdd(&cnt[ph], 1u << sh) >> sh) & 15u;
-                    rec[c] = ph | (sh << 16) | (on << 24);
+                    rec[c] = kf | (on << 24);
                 }
             }
             __syncthreads();  // B2 (counts complete)
@@ -2630,7 +2650,9 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
                 for (int c = 0; c < KPT; ++c) {
                     const uint32_t e = c * THREADS + tid;
                     if (e < count) {
-                        const uint32_t ph = rec[c] & 0xFFFFu, sh = (rec[c] >> 16) & 31u, on = rec[c] >> 24;
+                        const uint32_t kf = rec[c] & 0xFFFFFFu, on = rec[c] >> 24;
+                        const uint32_t cvc = (kf << IB) | e, v = kf >> VSH;
+                        const uint32_t ph = G::phys(v >> 3), sh = (v & 7u) * 4u;
                         const uint32_t w = cnt[ph];
                         const uint32_t slot = pref[ph] + nib_sum(w & ((1u << sh) - 1u)) + on;
                         const uint32_t r = (w >> sh) & 15u;
@@ -2638,13 +2660,13 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
                             // (RECON: the composite holds every sort bit) a tie pair orders
                             // itself: the second record to arrive swaps its composite in and
                             // writes the two in order (the slots start as SENT)
-                            const uint32_t b0 = slot - on, old = atomicExch(&comp[b0], cv[c]);
+                            const uint32_t b0 = slot - on, old = atomicExch(&comp[b0], cvc);
                             if (old != SENT) {
-                                comp[b0] = min(old, cv[c]);
-                                comp[b0 + 1] = max(old, cv[c]);
+                                comp[b0] = min(old, cvc);
+                                comp[b0 + 1] = max(old, cvc);
                             }
                         } else {
-                            comp[slot] = cv[c];
+                            comp[slot] = cvc;
                         }
                         if (on == 0 && r >= r0) {
                             const uint32_t q = atomicAdd(nruns, 1u);
@@ -2695,6 +2717,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
                 // the bucket) and the composite's sort field; otherwise it is gathered
                 const K khigh = thi >= KBITS ? K(0) : (aa & ~((K(1) << thi) - 1));
                 const uint32_t fs2 = opaque(static_cast<uint32_t>(FS));
+                vwait();
 #pragma unroll
                 for (int c = 0; c < KPT; ++c) {
                     const uint32_t e = c * THREADS + tid;
@@ -2721,6 +2744,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
         __syncthreads();  // staging buffer s, info[s], red[], comp, the run list are free
         if (tid == 0) {
             *nruns = 0;
+            vwait();  // (a bucket handed off never waited: the phase completes before the re-arm)
             fence_proxy_async();
             cp_async_wait_all();
             issue(s, info[16 * NSTAGE], *ahead);

@@ -172,6 +172,12 @@ template <> struct LocalCfg<7> { static constexpr int THREADS = 512, KPT = 16; }
 #ifndef HRS_LCC_OCC
 #define HRS_LCC_OCC 4
 #endif
+#ifndef HRS_LCC5_OCC
+#define HRS_LCC5_OCC HRS_LCC_OCC
+#endif
+#ifndef HRS_LCC6_OCC
+#define HRS_LCC6_OCC HRS_LCC_OCC
+#endif
 template <int C>
 struct LocalCntCfg : LocalCfg<C> {};
 template <> struct LocalCntCfg<5> { static constexpr int THREADS = HRS_LCC5_T, KPT = HRS_LCC5_K; };
@@ -231,7 +237,8 @@ struct LocalCntStages {
     static constexpr int by_smem = static_cast<int>(SM_BUDGET / (bytes + 1024));
     static constexpr int by_threads = 2048 / LC::THREADS;
     static constexpr int OCC0 = by_smem < by_threads ? by_smem : by_threads;
-    static constexpr int OCC = OCC0 < 1 ? 1 : (OCC0 > HRS_LCC_OCC ? HRS_LCC_OCC : OCC0);
+    static constexpr int OCC_CAP = C == 5 ? HRS_LCC5_OCC : HRS_LCC6_OCC;
+    static constexpr int OCC = OCC0 < 1 ? 1 : (OCC0 > OCC_CAP ? OCC_CAP : OCC0);
 };
 
 template <typename K, typename V>
