@@ -6,31 +6,34 @@
 // P:517-541), so each pass costs a constant number of launches and the host never
 // reads device memory:
 //
-//   k_hist<p>      streams the keys of every tile through a TMA bulk-copy ring into
-//                  shared memory and counts the digit with per-warp shared-memory
-//                  atomics (on B200 plain smem atomics run at full HBM
-//                  read rate even for a constant digit -- profiles/r01_micro_hist.txt
-//                  -- so the paper's sorting-network thread reduction, is
-//                  not needed).  Each CTA owns a contiguous run of tiles and adds the
-//                  bucket histograms to global memory once per bucket run.
+//   k_hist<p>      reads the keys of every tile straight from global memory in 16-byte
+//                  vectors and counts the digit into one block histogram per tile with
+//                  plain shared-memory atomics (on B200 they run at full HBM
+//                  read rate even for a constant digit -- profiles/r01_micro_hist.txt --
+//                  so neither warp aggregation nor the paper's sorting-network thread
+//                  reduction, is needed).  Each CTA owns a contiguous run of
+//                  tiles, records each tile's prefix within its bucket segment and adds
+//                  the bucket histograms to global memory once per bucket run.
 //   k_classify<p>  one CTA per bucket: exclusive prefix sum of the bucket histogram
 //                  into sub-bucket offsets and classification of the
 //                  sub-buckets (R1-R3 P:805-811, merging P:552-561) into next-pass
-//                  buckets/tiles and local-sort lists.
-//   k_scatter<p>   per tile, with the next tile already in flight through TMA: a
-//                  STABLE in-tile rank, staging in shared memory and write-combined
-//                  stores of every digit run (Fig 3); values follow their
-//                  keys.  The tile-ordered offset of every tile inside
-//                  its sub-bucket is known before the scatter starts: k_hist walks a
-//                  contiguous run of tiles per CTA and records each tile's prefix
-//                  within the run, k_classify scans the runs into per-CTA carries.
-//                  Deterministic, no look-back, and it replaces the atomicAdd chunk
-//                  reservation of P:696-703 (which is not stable).
+//                  buckets/tiles and local-sort lists; 8 more CTAs scan the CTA runs
+//                  into per-run carries.
+//   k_scatter<p>   per tile, with the next tile's keys already in flight through TMA: a
+//                  STABLE in-tile rank (per-warp digit counters), staging in shared
+//                  memory and write-combined stores of every digit run (P:704-722,
+//                  Fig 3); values follow their keys.  The tile-ordered
+//                  offset of every tile inside its sub-bucket is known before the
+//                  scatter starts (k_hist prefixes + k_classify carries): deterministic,
+//                  no look-back, and it replaces the atomicAdd chunk reservation of
+//                  P:696-703 (which is not stable).
 //
-// then one k_local launch per size class sorts every bucket of at most
-// ∂ˆ records on chip: a stable LSD radix sort of (key, index) pairs over the
-// remaining bits, skipping digits that are constant across the bucket,
-// and a final gather of the values.
+// then the buckets of at most ∂ˆ records are sorted on chip, one launch per size class
+// (P:562-577): the two largest classes by k_local_cnt (one counting sort on the top
+// varying sort bits, ties ordered afterwards), the others -- and every bucket the
+// counting sort hands off -- by k_local, a stable LSD radix sort of (key, index)
+// composites over the remaining bits that skips digits constant across the
+// bucket and gathers the values once at the end.
 //
 // Stability everywhere (ties keep input order) is the one deliberate departure
 // from the paper: the output is the unique stable sort.
@@ -820,6 +823,9 @@ struct HistParams {
 #ifndef HRS_HIST_MINB
 #define HRS_HIST_MINB 4
 #endif
+#ifndef HRS_HIST_PF
+#define HRS_HIST_PF 1
+#endif
 // element q of a 16-byte vector of keys (no address taken: the vector stays in registers)
 template <typename K>
 __device__ __forceinline__ K vec_elem(const uint4 &v, int q) {
@@ -838,8 +844,12 @@ __global__ void __launch_bounds__(THREADS, HRS_HIST_MINB) k_hist(HistParams prm)
     static_assert(THREADS >= RADIX, "one thread per digit for the tile prefixes");
     constexpr int VK = 16 / sizeof(K);
     constexpr int NV = (CAP / VK + THREADS - 1) / THREADS;  // whole vectors of a tile per thread
+    // HRS_HIST_PF: the loads of tile t + 1 are issued as soon as tile t's keys are counted,
+    // before the barrier that ends tile t (its descriptor was published a tile earlier:
+    // three descriptor slots), so they overlap the barrier and the fold
+    constexpr int NTI = HRS_HIST_PF ? 3 : 2;
     __shared__ uint32_t wh[2][RADIX];
-    __shared__ HistTile ti[2];
+    __shared__ HistTile ti[NTI];
     __shared__ TileCursor cur;
     const int tid = threadIdx.x;
     const unsigned long long al = prm.ctl->alloc[prm.p];
@@ -863,32 +873,49 @@ __global__ void __launch_bounds__(THREADS, HRS_HIST_MINB) k_hist(HistParams prm)
         cur.start(prm.buckets, NB, tb, te, prm.kpb);
         prm.seg_meta[blockIdx.x].first_bucket = cur.b;
         publish(0);
+        if (HRS_HIST_PF && tb + 1 < te) publish(1);
     }
     for (int i = tid; i < 2 * RADIX; i += THREADS) (&wh[0][0])[i] = 0;
     __syncthreads();
-    uint32_t seg_run = 0;   // digit tid: count of the current bucket segment before this tile
-    bool first_seg = true;  // inside the CTA's first bucket segment (its carry applies)
-    for (uint32_t t = tb, it = 0; t < te; ++t, ++it) {
-        const HistTile in = ti[it & 1u];
+    // a tile's key vectors: [0, h0) before the first 16-byte boundary, nvec whole vectors,
+    // the tail after them (edge elements: ne < 2 VK, one per thread)
+    struct Geo {
+        const K *src;
+        uint32_t h0, nvec, tail0, ne;
+        bool mapin;
+    };
+    auto geo = [&](const HistTile &in) {
+        Geo g;
         // (selected, not indexed: a dynamic index would copy the parameters to local memory)
         const void *kb = in.src == SRC_IN ? prm.src_keys[SRC_IN] : in.src == SRC_AUX ? prm.src_keys[SRC_AUX] : prm.src_keys[SRC_OUT];
-        const K *src = static_cast<const K *>(kb) + in.offs;
-        const bool mapin = TY && prm.kind != 0 && in.src == SRC_IN;
-        // [0, h0) before the first 16-byte boundary, nvec whole vectors, the tail after them
-        const uint32_t mis = static_cast<uint32_t>(reinterpret_cast<uintptr_t>(src) / sizeof(K)) % VK;
-        const uint32_t h0 = min(in.count, (VK - mis) % VK);
-        const uint32_t nvec = (in.count - h0) / VK, tail0 = h0 + nvec * VK;
-        const uint4 *vp = reinterpret_cast<const uint4 *>(src + h0);
-        uint4 w[NV];
+        g.src = static_cast<const K *>(kb) + in.offs;
+        g.mapin = TY && prm.kind != 0 && in.src == SRC_IN;
+        const uint32_t mis = static_cast<uint32_t>(reinterpret_cast<uintptr_t>(g.src) / sizeof(K)) % VK;
+        g.h0 = min(in.count, (VK - mis) % VK);
+        g.nvec = (in.count - g.h0) / VK;
+        g.tail0 = g.h0 + g.nvec * VK;
+        g.ne = g.h0 + (in.count - g.tail0);
+        return g;
+    };
+    uint4 w[NV];
+    K ek = K(0);
+    auto load = [&](const Geo &g) {
+        const uint4 *vp = reinterpret_cast<const uint4 *>(g.src + g.h0);
 #pragma unroll
         for (int j = 0; j < NV; ++j) {
             const uint32_t v = tid + j * THREADS;
-            if (v < nvec) w[j] = __ldcs(vp + v);
+            if (v < g.nvec) w[j] = __ldcs(vp + v);
         }
-        const uint32_t ne = h0 + (in.count - tail0);  // edge elements (< 2 VK)
-        K ek = K(0);
-        if (static_cast<uint32_t>(tid) < ne) ek = src[static_cast<uint32_t>(tid) < h0 ? tid : tail0 + (tid - h0)];
-        if (tid == 0 && t + 1 < te) publish((it + 1) & 1u);
+        if (static_cast<uint32_t>(tid) < g.ne) ek = g.src[static_cast<uint32_t>(tid) < g.h0 ? tid : g.tail0 + (tid - g.h0)];
+    };
+    if constexpr (HRS_HIST_PF) load(geo(ti[0]));
+    uint32_t seg_run = 0;   // digit tid: count of the current bucket segment before this tile
+    bool first_seg = true;  // inside the CTA's first bucket segment (its carry applies)
+    for (uint32_t t = tb, it = 0; t < te; ++t, ++it) {
+        const HistTile in = ti[it % NTI];
+        const Geo g = geo(in);
+        if constexpr (!HRS_HIST_PF) load(g);
+        if (tid == 0 && t + (NTI - 1) < te) publish((it + NTI - 1) % NTI);
         // tile descriptor and tile-ordered prefix for the scatter
         if (tid < RADIX) prm.tile_pref[static_cast<uint64_t>(t) * RADIX + tid] = seg_run;
         if (tid == 0) {
@@ -901,16 +928,18 @@ __global__ void __launch_bounds__(THREADS, HRS_HIST_MINB) k_hist(HistParams prm)
             prm.tiles[t] = td;
         }
         uint32_t *my = wh[it & 1u];
-        auto dig = [&](K k) { return digit_of(mapin ? key_map(k, prm.kind, false) : k, prm.lo, prm.mask); };
+        auto dig = [&](K k) { return digit_of(g.mapin ? key_map(k, prm.kind, false) : k, prm.lo, prm.mask); };
 #pragma unroll
         for (int j = 0; j < NV; ++j) {
-            if (tid + j * THREADS < nvec) {
+            if (tid + j * THREADS < g.nvec) {
 #pragma unroll
                 for (int q = 0; q < VK; ++q) atomicAdd(&my[dig(vec_elem<K>(w[j], q))], 1u);
             }
         }
-        if (static_cast<uint32_t>(tid) < ne) atomicAdd(&my[dig(ek)], 1u);
-        __syncthreads();  // the tile's counts are complete; ti[(it + 1) & 1] is published
+        if (static_cast<uint32_t>(tid) < g.ne) atomicAdd(&my[dig(ek)], 1u);
+        // (PF: ti[(it + 1) % 3] was published before the previous barrier)
+        if (HRS_HIST_PF && t + 1 < te) load(geo(ti[(it + 1) % NTI]));
+        __syncthreads();  // the tile's counts are complete; the next descriptor is published
         if (tid < RADIX) {
             seg_run += my[tid];
             my[tid] = 0;  // (counted into again two tiles on, after the next barrier)
