@@ -164,10 +164,10 @@ template <> struct LocalCfg<7> { static constexpr int THREADS = 512, KPT = 16; }
 #define HRS_LCC5_K 16
 #endif
 #ifndef HRS_LCC6_T
-#define HRS_LCC6_T 288
+#define HRS_LCC6_T 256
 #endif
 #ifndef HRS_LCC6_K
-#define HRS_LCC6_K 16
+#define HRS_LCC6_K 18
 #endif
 #ifndef HRS_LCC_OCC
 #define HRS_LCC_OCC 4
