@@ -1010,7 +1010,8 @@ __device__ __forceinline__ uint32_t block_suffix_min256(uint32_t v, uint32_t *wb
 // (it holds the candidates of [i, gend), size P[gend] - P[i]) and the next group
 // starts at the first candidate >= gend.  The groups are the chain of starts from the
 // first candidate, marked by pointer doubling (8 rounds for 256 digits).
-// Writes glead[i] = group size and gmulti[i] = (>= 2 members) at every group start i.
+// Writes glead[i] = group size and gmulti[i] = (>= 2 members ? group end : 0) at every
+// group start i.
 template <int THREADS>
 __device__ void merge_groups(const ClassifyParams &prm, const uint32_t *tot, const uint32_t *P, uint32_t *glead,
                              uint32_t *gmulti, uint32_t *ws) {
@@ -1068,7 +1069,7 @@ __device__ void merge_groups(const ClassifyParams &prm, const uint32_t *tot, con
     }
     if (cand && flag[d]) {
         glead[d] = size;
-        gmulti[d] = multi ? 1u : 0u;
+        gmulti[d] = multi ? gend : 0u;  // (> d: the group's digits are [d, gend))
     }
 }
 
@@ -1080,7 +1081,7 @@ __device__ void classify_bucket(const ClassifyParams &prm, const Bucket &bk, uin
     uint32_t *ct = sm + 2 * NBINS;      // child tiles per digit -> exclusive
     uint32_t *cb = sm + 3 * NBINS;      // child flag per digit -> exclusive
     uint32_t *glead = sm + 4 * NBINS;   // local group size at the leader digit (0 = none)
-    uint32_t *gmulti = sm + 5 * NBINS;  // 1 if the group merged >= 2 sub-buckets
+    uint32_t *gmulti = sm + 5 * NBINS;  // group end if the group merged >= 2 sub-buckets, else 0
     uint32_t *misc = sm + 6 * NBINS;    // [0] base tile, [1] base bucket, [2..9] class counts, [10..17] class bases
     const int tid = threadIdx.x;
     for (int d = tid; d < NBINS; d += THREADS) {
@@ -1168,7 +1169,7 @@ __device__ void classify_bucket(const ClassifyParams &prm, const Bucket &bk, uin
         const uint32_t s = tot[tid];
         if (s > prm.lt) recs_next = s;
         lrecs = glead[tid];
-        merged = gmulti[tid];
+        merged = gmulti[tid] ? 1u : 0u;
     }
 #pragma unroll
     for (int o = 16; o > 0; o >>= 1) {
@@ -1189,14 +1190,22 @@ __device__ void classify_bucket(const ClassifyParams &prm, const Bucket &bk, uin
         misc[10 + tid] = base;
     }
     __syncthreads();
-    const int hi_p = prm.lo + prm.width;
     if (my_cls >= 0) {
         const uint32_t slot = misc[10 + my_cls] + my_slot;
         if (slot < prm.local_cap[my_cls]) {
             LocalEntry e;
             e.offs = boffs + start[tid];
             e.count = glead[tid];
-            e.hi_bit = static_cast<uint16_t>(gmulti[tid] ? hi_p : prm.lo);
+            // a merged group sorts the digit bits in which its members differ (reading #6: the
+            // bits of [hi_bit, hi_p) are common to digits tid .. last): the local sort's
+            // counted bits start at its top varying bit
+            int hb = prm.lo;
+            if (gmulti[tid]) {
+                uint32_t last = gmulti[tid] - 1u;
+                while (last > static_cast<uint32_t>(tid) && tot[last] == 0u) --last;  // last non-empty member
+                hb = prm.lo + (32 - __clz(static_cast<int>(static_cast<uint32_t>(tid) ^ last)));
+            }
+            e.hi_bit = static_cast<uint16_t>(hb);
             e.src = child_src;
             prm.local[my_cls][slot] = e;
         }
@@ -2337,6 +2346,11 @@ constexpr int LC_SCAN = 256;  // threads that scan the counters
 #endif
 // the values of a bucket complete on their own barrier, waited for just before the
 // write-out: their load overlaps the count, scan and placement of the bucket
+// the top varying sort bit of a bucket is taken from its entry (hi_bit) instead of an
+// AND/OR reduction over the bucket's keys (one barrier less per bucket)
+#ifndef HRS_LC_NORED
+#define HRS_LC_NORED 1
+#endif
 #ifndef HRS_LC_VSPLIT
 #define HRS_LC_VSPLIT 1
 #endif
@@ -2402,6 +2416,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
     using G = CntGeom<CB>;
     constexpr int IB = 13;     // index bits of a composite
     constexpr int CBITS = 19;  // sort bits of a composite
+    constexpr bool NORED = HRS_LC_NORED;
     static_assert(CBITS <= 24, "a record's register holds the composite's key field below bit 24");
     constexpr uint32_t IMASK = (1u << IB) - 1u;
     constexpr int W = THREADS / 32;
@@ -2554,30 +2569,48 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
         for (int c = 0; c < KPT; ++c) {
             const uint32_t e = c * THREADS + tid;
             key[c] = kin_map(ksp[e < count ? e : 0u]);  // past the end: a copy of key 0 (neutral for and/or)
-            a &= key[c];
-            o |= key[c];
+            if constexpr (!NORED) {
+                a &= key[c];
+                o |= key[c];
+            }
         }
-        a = warp_and(a);
-        o = warp_or(o);
-        if (lane == 0) {
-            red[warp] = a;
-            red[W + warp] = o;
-        }
-        __syncthreads();  // B1: red[], filled edges
-        K aa = ~K(0), oo = K(0);
-#pragma unroll
-        for (int w = 0; w < W; ++w) {
-            aa &= red[w];
-            oo |= red[W + w];
-        }
-        const K diff = aa ^ oo;
-        const K rmask = (hi_bit >= KBITS ? ~K(0) : ((K(1) << hi_bit) - 1)) & ~((K(1) << begin_bit) - 1);
-        const K dv = diff & rmask;  // sort bits that vary across the bucket
+        // thi: the top sort bit that varies across the bucket (counted bits [thi - CB, thi)).
+        // NORED: the entry's hi_bit -- every key bit at or above it is common to the bucket
+        // (its partitioned digits; a merged group's hi_bit is the top bit in which its digits
+        // differ) and the next bit below varies in practice for buckets of > 2048 records;
+        // were it constant, the counted values would tie more (overflow: hand-off), never a
+        // different result.  Saves the AND/OR reduction and its barrier.
+        K aa, diff;
         int thi = 0;
-        if (dv != 0) thi = KBITS - (sizeof(K) == 8 ? __clzll(static_cast<long long>(dv)) : __clz(static_cast<int>(dv)));
+        bool nosort;
+        if constexpr (NORED) {
+            thi = hi_bit;
+            aa = key[0];  // (bits >= thi: common to the bucket)
+            diff = K(0);
+            nosort = false;
+        } else {
+            a = warp_and(a);
+            o = warp_or(o);
+            if (lane == 0) {
+                red[warp] = a;
+                red[W + warp] = o;
+            }
+            __syncthreads();  // B1: red[], filled edges
+            aa = ~K(0);
+            K oo = K(0);
+#pragma unroll
+            for (int w = 0; w < W; ++w) {
+                aa &= red[w];
+                oo |= red[W + w];
+            }
+            diff = aa ^ oo;
+            const K rmask = (hi_bit >= KBITS ? ~K(0) : ((K(1) << hi_bit) - 1)) & ~((K(1) << begin_bit) - 1);
+            const K dv = diff & rmask;  // sort bits that vary across the bucket
+            if (dv != 0) thi = KBITS - (sizeof(K) == 8 ? __clzll(static_cast<long long>(dv)) : __clz(static_cast<int>(dv)));
+            nosort = dv == 0;
+        }
         const int clo = max(begin_bit, thi - CBITS);  // composite: key bits [clo, thi)
         const int flo = max(clo, thi - CB);           // counted: key bits [flo, thi)
-        const bool nosort = dv == 0;
         bool take = !nosort && thi - begin_bit > 8;
         if (RECON) take = take && begin_bit == 0 && clo == 0 && (thi >= KBITS || (diff >> thi) == 0);
         K *const kd = kout + offs;
@@ -2618,7 +2651,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
                 const uint32_t e = c * THREADS + tid;
                 const uint32_t kf = static_cast<uint32_t>(key[c] >> clo) & cmask;
                 if (e < count) {
-                    if constexpr (RECON) comp[e] = SENT;  // (tie pairs swap into their first slot)
+                    if constexpr (RECON && !NORED) comp[e] = SENT;  // (tie pairs swap into their first slot)
                     const uint32_t v = kf >> VSH;
                     const uint32_t ph = G::phys(v >> 3), sh = (v & 7u) * 4u;
                     const uint32_t on = (atomicAdd(&cnt[ph], 1u << sh) >> sh) & 15u;
@@ -2626,6 +2659,15 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
                 }
             }
             __syncthreads();  // B2 (counts complete)
+            if constexpr (RECON && NORED) {
+                // (after B2: without B1 another thread may read its key from the staging buffer,
+                // which the composites overwrite, until then)
+#pragma unroll
+                for (int c = 0; c < KPT; ++c) {
+                    const uint32_t e = c * THREADS + tid;
+                    if (e < count) comp[e] = SENT;  // (tie pairs swap into their first slot)
+                }
+            }
             {
                 // exclusive prefix of the word totals: 256 threads own PW consecutive words.
                 // A counter that passed 15 wrapped (-16, +1 carried into its neighbour or
