@@ -2351,6 +2351,9 @@ constexpr int LC_SCAN = 256;  // threads that scan the counters
 #ifndef HRS_LC_NORED
 #define HRS_LC_NORED 1
 #endif
+#ifndef HRS_LC_ALLWAIT
+#define HRS_LC_ALLWAIT 1
+#endif
 #ifndef HRS_LC_VSPLIT
 #define HRS_LC_VSPLIT 1
 #endif
@@ -2520,11 +2523,11 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
         const int s = static_cast<int>(it % NSTAGE);
         const uint32_t par = (it / NSTAGE) & 1u;
         const uint32_t *in = info + 16 * s;
-        // one warp waits for the bulk copies (the producer wrote info[s] before its arrive:
-        // the wait acquires it); the barrier passes both on to the other warps, which
-        // meanwhile do not take issue slots from the other resident CTAs
-        if (warp == 0) mbar_wait(&bar[s], par);
-        __syncthreads();
+        // the bulk copies of the keys (the producer wrote info[s] before its arrive: the wait
+        // acquires it).  ALLWAIT: every thread waits on the barrier itself (no CTA barrier);
+        // else one warp waits and a CTA barrier passes both on to the other warps
+        if (HRS_LC_ALLWAIT || warp == 0) mbar_wait(&bar[s], par);
+        if (!HRS_LC_ALLWAIT) __syncthreads();
         const uint32_t e_id = in[0];
         if (e_id >= nent) break;
         if (tid == 0 && info[16 * NSTAGE] < nent) cp_async16(ahead, prm.list + info[16 * NSTAGE]);
