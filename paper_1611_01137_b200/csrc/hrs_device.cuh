@@ -300,6 +300,9 @@ __device__ __forceinline__ void mbar_arrive_expect_tx(uint64_t *bar, uint32_t by
     asm volatile("mbarrier.arrive.expect_tx.shared::cta.b64 _, [%0], %1;" ::"r"(smem_u32(bar)), "r"(bytes)
                  : "memory");
 }
+__device__ __forceinline__ void mbar_arrive(uint64_t *bar) {
+    asm volatile("mbarrier.arrive.shared::cta.b64 _, [%0];" ::"r"(smem_u32(bar)) : "memory");
+}
 __device__ __forceinline__ void mbar_wait(uint64_t *bar, uint32_t parity) {
     asm volatile(
         "{\n"
@@ -2351,6 +2354,9 @@ constexpr int LC_SCAN = 256;  // threads that scan the counters
 #ifndef HRS_LC_NORED
 #define HRS_LC_NORED 1
 #endif
+#ifndef HRS_LC_EARLYK
+#define HRS_LC_EARLYK 1
+#endif
 #ifndef HRS_LC_ALLWAIT
 #define HRS_LC_ALLWAIT 1
 #endif
@@ -2392,8 +2398,13 @@ struct LocalCntSmem {
     static constexpr bool HV = HasVal<V>::value;
     using G = CntGeom<CB>;
     static constexpr bool VSPLIT = HRS_LC_VSPLIT && HV;  // [NSTAGE + s]: values of stage s
+    // EARLYK: the next bucket's keys are loaded while this bucket's values are written out
+    // (the key staging buffer holds the composites, read into registers first; RECON only:
+    // nothing else reads the key staging buffer in the write-out); [2 NSTAGE]: the
+    // composites are consumed (one arrival per warp)
+    static constexpr bool EARLYK = HRS_LC_EARLYK && RECON && (VSPLIT || !HV);
     static constexpr size_t off_bar = 0;
-    static constexpr size_t off_info = align16(sizeof(uint64_t) * NSTAGE * (VSPLIT ? 2 : 1));
+    static constexpr size_t off_info = align16(sizeof(uint64_t) * (2 * NSTAGE + 1));
     static constexpr size_t off_red = align16(off_info + sizeof(uint32_t) * 16 * (NSTAGE + 1));
     static constexpr size_t off_wsum = align16(off_red + sizeof(K) * 2 * W);
     static constexpr size_t off_cnt = align16(off_wsum + sizeof(uint32_t) * 16);
@@ -2461,12 +2472,28 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
     // info[s]: 0 entry, 1 count, 2 hi_bit, 3 src, 4..5 offs, 6..8 key seg, 9..11 value seg
     // the next entry of the list, fetched while the current bucket is sorted
     LocalEntry *const ahead = reinterpret_cast<LocalEntry *>(info + 16 * NSTAGE + 4);
-    auto issue = [&](int s, uint32_t e, const LocalEntry &en) {
+    // mode bit 0: the keys (and info[s]), bit 1: the values (VSPLIT; else they come with the keys)
+    auto issue = [&](int s, uint32_t e, const LocalEntry &en, int mode) {
         uint32_t *in = info + 16 * s;
+        if (!(mode & 1)) {  // the values of the entry whose keys were issued earlier
+            if constexpr (L::VSPLIT) {
+                if (e >= nent) {
+                    mbar_arrive_expect_tx(&bar[NSTAGE + s], 0);
+                    return;
+                }
+                Seg sv;
+                sv.pad = in[9];
+                sv.i0 = static_cast<int32_t>(in[10]);
+                sv.i1 = static_cast<int32_t>(in[11]);
+                mbar_arrive_expect_tx(&bar[NSTAGE + s], sv.i1 > sv.i0 ? static_cast<uint32_t>(sv.i1 - sv.i0) * static_cast<uint32_t>(sizeof(VT)) : 0u);
+                seg_issue(vst(s), srcv(en.src) + en.offs, sv, &bar[NSTAGE + s], pol);
+            }
+            return;
+        }
         in[0] = e;
         if (e >= nent) {
             mbar_arrive_expect_tx(&bar[s], 0);  // completes the phase: the waiters see the end
-            if constexpr (L::VSPLIT) mbar_arrive_expect_tx(&bar[NSTAGE + s], 0);
+            if constexpr (L::VSPLIT) if (mode & 2) mbar_arrive_expect_tx(&bar[NSTAGE + s], 0);
             return;
         }
         in[1] = en.count;
@@ -2490,6 +2517,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
         }
         mbar_arrive_expect_tx(&bar[s], L::VSPLIT ? bytes : bytes + vbytes);
         seg_issue(kst(s), kbuf + en.offs, sk, &bar[s], pol);
+        if (L::VSPLIT && !(mode & 2)) return;
         if constexpr (L::VSPLIT) mbar_arrive_expect_tx(&bar[NSTAGE + s], vbytes);
         if (HV) seg_issue(vst(s), srcv(en.src) + en.offs, sv, &bar[L::VSPLIT ? NSTAGE + s : s], pol);
     };
@@ -2506,18 +2534,21 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
     };
     for (int i = tid; i < G::NW; i += THREADS) cnt[i] = 0;  // cleared again after every bucket
     if (tid == 0) {
-        for (int s = 0; s < NSTAGE * (L::VSPLIT ? 2 : 1); ++s) mbar_init(&bar[s], 1);
+        for (int s = 0; s < 2 * NSTAGE; ++s) mbar_init(&bar[s], 1);
+        mbar_init(&bar[2 * NSTAGE], W);
         mbar_fence_init();
         for (int s = 0; s < NSTAGE; ++s) {
             const uint32_t e = blockIdx.x + s * gridDim.x;
             LocalEntry en{};
             if (e < nent) en = prm.list[e];
-            issue(s, e, en);
+            issue(s, e, en, 3);
         }
         info[16 * NSTAGE] = blockIdx.x + NSTAGE * gridDim.x;  // next entry to issue
         *nruns = 0;
     }
     __syncthreads();
+    bool keys_early = false;  // (tid 0) the next entry's keys are already in flight
+    uint32_t cf_par = 0;      // (tid 0) phase of the composites-consumed barrier
 
     for (uint32_t it = 0;; ++it) {
         const int s = static_cast<int>(it % NSTAGE);
@@ -2792,6 +2823,36 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
                 const K khigh = thi >= KBITS ? K(0) : (aa & ~((K(1) << thi) - 1));
                 const uint32_t fs2 = opaque(static_cast<uint32_t>(FS));
                 vwait();
+                if constexpr (L::EARLYK) {
+                    // composites into registers, the key staging buffer is free: the next
+                    // entry's keys load while the values are gathered and written
+                    uint32_t xs[KPT];
+#pragma unroll
+                    for (int c = 0; c < KPT; ++c) {
+                        const uint32_t e = c * THREADS + tid;
+                        xs[c] = e < count ? comp[e] : 0u;
+                    }
+                    __syncwarp();
+                    if (lane == 0) mbar_arrive(&bar[2 * NSTAGE]);
+                    if (tid == 0) {
+                        mbar_wait(&bar[2 * NSTAGE], cf_par);
+                        cf_par ^= 1u;
+                        fence_proxy_async();
+                        cp_async_wait_all();
+                        issue(s, info[16 * NSTAGE], *ahead, 1);
+                        keys_early = true;
+                    }
+#pragma unroll
+                    for (int c = 0; c < KPT; ++c) {
+                        const uint32_t e = c * THREADS + tid;
+                        if (e < count) {
+                            const uint32_t x = xs[c];
+                            kd[e] = kout_map(khigh | static_cast<K>(x >> IB));
+                            if (HV) vd[e] = vsp[x & IMASK];
+                        }
+                    }
+                    goto next_entry;
+                }
 #pragma unroll
                 for (int c = 0; c < KPT; ++c) {
                     const uint32_t e = c * THREADS + tid;
@@ -2821,8 +2882,9 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
             vwait();  // (a bucket handed off never waited: the phase completes before the re-arm)
             fence_proxy_async();
             cp_async_wait_all();
-            issue(s, info[16 * NSTAGE], *ahead);
+            issue(s, info[16 * NSTAGE], *ahead, keys_early ? 2 : 3);
             info[16 * NSTAGE] += gridDim.x;
+            keys_early = false;
         }
     }
 }
