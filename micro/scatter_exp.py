@@ -54,7 +54,7 @@ def run(name, dist="uniform", kbits=32):
         a, b = kk[:-1] ^ (-(2 ** 63)), kk[1:] ^ (-(2 ** 63))  # unsigned order as signed
         ok = ok and bool(((a < b) | ((a == b) & (vv[:-1] < vv[1:]))).all())
     print(f"{name:12s} {dist:8s} k{kbits} {'OK ' if ok else 'BAD'} step={tot:.3f} ms " + " ".join(
-        f"{k2}={sum(x) / len(x):.3f}" for k2, x in sorted(per.items()) if sum(x) / len(x) > 0.02), flush=True)
+        f"{k2}={sum(x) / len(x):.3f}" for k2, x in sorted(per.items()) if sum(x) / len(x) > 0.009), flush=True)
 
 
 if __name__ == "__main__":
