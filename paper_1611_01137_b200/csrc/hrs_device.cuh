@@ -58,6 +58,9 @@
 #define HRS_WO_UNROLL 4
 #endif
 namespace hrs { constexpr int WO_UNROLL = HRS_WO_UNROLL; }
+#ifndef HRS_SC_STHINT
+#define HRS_SC_STHINT 0  // measured: evict_last stores on pass 1 only slow pass 2 (0.99 -> 1.08 ms), on every pass no change
+#endif
 #ifndef HRS_SC_VSPLIT
 #define HRS_SC_VSPLIT 1  // one value staging buffer (two key buffers): larger tiles (0: two of each)
 #endif
@@ -318,6 +321,15 @@ __device__ __forceinline__ uint64_t policy_evict_first() {
     uint64_t p;
     asm volatile("createpolicy.fractional.L2::evict_first.b64 %0, 1.0;" : "=l"(p));
     return p;
+}
+__device__ __forceinline__ uint64_t policy_evict_last() {
+    uint64_t p;
+    asm volatile("createpolicy.fractional.L2::evict_last.b64 %0, 1.0;" : "=l"(p));
+    return p;
+}
+// 4-byte global store with an L2 cache-eviction hint
+__device__ __forceinline__ void st_hint(uint32_t *p, uint32_t v, uint64_t pol) {
+    asm volatile("st.global.L2::cache_hint.b32 [%0], %1, %2;" ::"l"(p), "r"(v), "l"(pol) : "memory");
 }
 __device__ __forceinline__ void bulk_g2s(void *dst, const void *src, uint32_t bytes, uint64_t *bar, uint64_t pol) {
     asm volatile(
@@ -1465,6 +1477,10 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
         cudaGraphSetConditional(prm.next_cond, alloc_buckets(prm.ctl->alloc[prm.p + 1]) != 0u ? 1u : 0u);
     if (blockIdx.x >= T) return;
     const uint64_t pol = policy_evict_first();
+    // HRS_SC_STHINT: the write-out's stores carry an L2 evict_last hint (1: first pass only,
+    // whose write frontiers are spread over the whole output; 2: every pass)
+    const bool sthint = HRS_SC_STHINT == 2 || (HRS_SC_STHINT == 1 && prm.p == 1);
+    const uint64_t spol = HRS_SC_STHINT ? policy_evict_last() : 0ull;
     uint32_t *const ca = cnt + warp * RADIX;  // this warp's counters
     for (int i = tid; i < W * RADIX; i += THREADS) cnt[i] = 0;
 
@@ -1741,6 +1757,14 @@ __global__ void __launch_bounds__(THREADS, MINB) k_scatter(ScatterParams prm) {
                             const uint32_t i = sidx[j];
                             const uint2 g = gs[digit_of(k, lo, mask)];
                             const uint32_t pos = g.x + j;
+                            if constexpr (HRS_SC_STHINT && sizeof(K) == 4 && (!HV || sizeof(VT) == 4)) {
+                                if (sthint) {
+                                    st_hint(reinterpret_cast<uint32_t *>(kdst + pos), static_cast<uint32_t>(unmap ? key_map(k, prm.kind, true) : k), spol);
+                                    if (HV) st_hint(reinterpret_cast<uint32_t *>(vdst + pos), static_cast<uint32_t>(vb[i]), spol);
+                                    if (check && j > g.y) bad |= sidx[j - 1] > i;
+                                    continue;
+                                }
+                            }
                             kdst[pos] = unmap ? key_map(k, prm.kind, true) : k;
                             if (HV) vdst[pos] = vb[i];
                             if (check && j > g.y) bad |= sidx[j - 1] > i;
