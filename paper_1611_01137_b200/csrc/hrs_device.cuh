@@ -2398,6 +2398,9 @@ constexpr int LC_SCAN = 256;  // threads that scan the counters
 #ifndef HRS_LC_NORED
 #define HRS_LC_NORED 1
 #endif
+#ifndef HRS_LC_PL2
+#define HRS_LC_PL2 0  // measured slower (spills at 64 registers): c2 local 0.647 + 0.648 -> 0.695 + 0.769 ms
+#endif
 #ifndef HRS_LC_EARLYK
 #define HRS_LC_EARLYK 0  // (measured slower: c2 local 0.646 + 0.659 -> 0.653 + 0.671 ms)
 #endif
@@ -2728,6 +2731,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
             for (int c = 0; c < KPT; ++c) {
                 const uint32_t e = c * THREADS + tid;
                 const uint32_t kf = static_cast<uint32_t>(key[c] >> clo) & cmask;
+                rec[c] = kf;  // (past the end: a valid counter word for the placement's loads)
                 if (e < count) {
                     if constexpr (RECON && !NORED) comp[e] = SENT;  // (tie pairs swap into their first slot)
                     const uint32_t v = kf >> VSH;
@@ -2795,16 +2799,37 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local_cnt(LocalParams prm) {
                 // neighbours); longer runs, and every run when key bits below the composite
                 // decide (low), go to a list that the whole CTA sorts before the write-out
                 const uint32_t r0 = low ? 2u : 3u;
+                // PL2: every record's slot and tie count first (loads of all records in flight
+                // together, no branches), then the stores
+                [[maybe_unused]] uint32_t sr[HRS_LC_PL2 ? KPT : 1];
+                if constexpr (HRS_LC_PL2) {
+#pragma unroll
+                    for (int c = 0; c < KPT; ++c) {
+                        const uint32_t kf = rec[c] & 0xFFFFFFu, on = rec[c] >> 24;
+                        const uint32_t v = kf >> VSH;
+                        const uint32_t ph = G::phys(v >> 3), sh = (v & 7u) * 4u;
+                        const uint32_t w = cnt[ph];
+                        const uint32_t slot = pref[ph] + nib_sum(w & ((1u << sh) - 1u)) + on;
+                        sr[c] = slot | (((w >> sh) & 15u) << 16);
+                    }
+                }
 #pragma unroll
                 for (int c = 0; c < KPT; ++c) {
                     const uint32_t e = c * THREADS + tid;
                     if (e < count) {
                         const uint32_t kf = rec[c] & 0xFFFFFFu, on = rec[c] >> 24;
-                        const uint32_t cvc = (kf << IB) | e, v = kf >> VSH;
-                        const uint32_t ph = G::phys(v >> 3), sh = (v & 7u) * 4u;
-                        const uint32_t w = cnt[ph];
-                        const uint32_t slot = pref[ph] + nib_sum(w & ((1u << sh) - 1u)) + on;
-                        const uint32_t r = (w >> sh) & 15u;
+                        const uint32_t cvc = (kf << IB) | e;
+                        uint32_t slot, r;
+                        if constexpr (HRS_LC_PL2) {
+                            slot = sr[c] & 0xFFFFu;
+                            r = sr[c] >> 16;
+                        } else {
+                            const uint32_t v = kf >> VSH;
+                            const uint32_t ph = G::phys(v >> 3), sh = (v & 7u) * 4u;
+                            const uint32_t w = cnt[ph];
+                            slot = pref[ph] + nib_sum(w & ((1u << sh) - 1u)) + on;
+                            r = (w >> sh) & 15u;
+                        }
                         if (RECON && r == 2u) {
                             // (RECON: the composite holds every sort bit) a tie pair orders
                             // itself: the second record to arrive swaps its composite in and
