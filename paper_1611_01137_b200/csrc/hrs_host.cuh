@@ -182,7 +182,7 @@ template <int C>
 struct LocalCntCfg : LocalCfg<C> {};
 template <> struct LocalCntCfg<5> { static constexpr int THREADS = HRS_LCC5_T, KPT = HRS_LCC5_K; };
 template <> struct LocalCntCfg<6> { static constexpr int THREADS = HRS_LCC6_T, KPT = HRS_LCC6_K; };
-static_assert(HRS_LCC5_T * HRS_LCC5_K == 4096 && HRS_LCC6_T * HRS_LCC6_K == 4608, "class capacities");
+static_assert(HRS_LCC5_T * HRS_LCC5_K >= 4096 && HRS_LCC6_T * HRS_LCC6_K >= 4608, "class capacities");
 
 // two-stage TMA prefetch where it fits next to a second resident CTA, else one stage
 // two-stage TMA prefetch when three CTAs still fit per SM, else one stage; the
