@@ -152,7 +152,14 @@ template <> struct LocalCfg<0> { static constexpr int THREADS = 32, KPT = 4; };
 template <> struct LocalCfg<1> { static constexpr int THREADS = 64, KPT = 4; };
 template <> struct LocalCfg<2> { static constexpr int THREADS = 64, KPT = 8; };
 template <> struct LocalCfg<3> { static constexpr int THREADS = 128, KPT = 8; };
-template <> struct LocalCfg<4> { static constexpr int THREADS = 128, KPT = 16; };
+#ifndef HRS_LC4_T
+#define HRS_LC4_T 128
+#endif
+#ifndef HRS_LC4_K
+#define HRS_LC4_K 16
+#endif
+template <> struct LocalCfg<4> { static constexpr int THREADS = HRS_LC4_T, KPT = HRS_LC4_K; };
+static_assert(HRS_LC4_T * HRS_LC4_K >= 2048, "class 4 capacity");
 template <> struct LocalCfg<5> { static constexpr int THREADS = 256, KPT = 16; };
 template <> struct LocalCfg<6> { static constexpr int THREADS = 288, KPT = 16; };
 template <> struct LocalCfg<7> { static constexpr int THREADS = 512, KPT = 16; };
