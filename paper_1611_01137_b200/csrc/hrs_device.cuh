@@ -2371,8 +2371,10 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
 //
 // The local sort of a bucket as ONE counting pass instead of
 // ceil(bits / 8) LSD passes: a counting sort (histogram -> exclusive prefix -> placement,
-// the same three steps as a counting pass) on the top CB <= 15 sort bits that
-// vary across the bucket, with 2^CB four-bit counters packed eight to a word.  2^CB is
+// the same three steps as a counting pass) on the CB <= 15 sort bits below the
+// entry's top bit (hi_bit: the bits above it are common to the bucket; HRS_LC_NORED=0
+// finds the top varying bit with an AND/OR reduction instead), with 2^CB four-bit
+// counters packed eight to a word.  2^CB is
 // many times the bucket size (<= 4608), so the counted values are nearly distinct; the
 // records that tie on them (about one in eight for uniform keys) are put in order by a
 // short insertion sort of each tie run, on the remaining sort bits and then the input
@@ -2381,7 +2383,7 @@ __global__ void __launch_bounds__(THREADS, MINB) k_local(LocalParams prm) {
 // own counter increment (any order among the ties: the fix-up orders them).
 //
 // Buckets it does not take go to a hand-off list sorted afterwards by k_local:
-//   * at most 8 varying sort bits (one LSD pass is cheaper);
+//   * at most 8 sort bits (one LSD pass is cheaper);
 //   * a counted value held by more than 15 records (four-bit counter overflow: skewed keys);
 //   * RECON: more than 19 varying sort bits (the keys are rebuilt from the composites).
 // Per record: one shared atomic, two lookups, one composite store and the value gather
